@@ -1,0 +1,156 @@
+"""CPU oracle for A&R over BWD columns -- TEST INFRASTRUCTURE ONLY.
+
+Plain, slow, obviously correct definitions of what the hot path computes,
+written from the paper (PAPER.md = H. Pirk, S. Manegold, M. Kersten, "Waste
+Not... Efficient Co-Processing of Relational Data", ICDE 2014).  The arithmetic
+lives in plain C (`oracle.c`, compiled with gcc on demand); this module only
+marshals numpy arrays.
+
+Only tests/, __graft_entry__.smoke() and bench.py's cpu_baseline and
+`--impl reference` legs may import this package.  The product package
+(paper_conf_icde_pirkmk14_b200) never imports it, and the two share no code.
+
+Pins (tests/test_oracle_*.py):
+  decompose       Fig. 2 worked value, round trip, non-redundancy
+  bucket_flags    Fig. 4, Fig. 6, brute-force
+                  exists/forall over residuals, printed f(x) superset
+  select_sum      brute force on tiny tables, closed-form sums, thread-count invariance
+  sum_at          closed forms
+No function is "parity unpinned".
+"""
+from __future__ import annotations
+
+import ctypes
+import os
+import subprocess
+import threading
+
+import numpy as np
+
+_HERE = os.path.dirname(os.path.abspath(__file__))
+_SRC = os.path.join(_HERE, "oracle.c")
+_LIB = os.path.join(_HERE, "liboracle.so")
+_lock = threading.Lock()
+_lib = None
+
+OPS = {"==": 0, ">": 1, ">=": 2, "<": 3, "<=": 4}
+
+
+def build(force: bool = False) -> str:
+    """Compile liboracle.so in-tree with gcc (plain C, pthreads)."""
+    with _lock:
+        if force or not os.path.exists(_LIB) or os.path.getmtime(_LIB) < os.path.getmtime(_SRC):
+            tmp = _LIB + f".tmp{os.getpid()}"
+            subprocess.check_call(["gcc", "-O2", "-fPIC", "-shared", "-pthread", "-o", tmp, _SRC])
+            os.replace(tmp, _LIB)
+    return _LIB
+
+
+def _load():
+    global _lib
+    if _lib is None:
+        lib = ctypes.CDLL(build())
+        p, i64, i32, u32 = ctypes.c_void_p, ctypes.c_int64, ctypes.c_int, ctypes.c_uint32
+        lib.or_decompose.argtypes = [p, i64, i32, u32, p, p]
+        lib.or_decompose.restype = i32
+        lib.or_bucket_flags.argtypes = [p, i64, i32, u32, u32, u32, p, p]
+        lib.or_paper_f_flags.argtypes = [p, i64, i32, i32, u32, p]
+        lib.or_select_sum.argtypes = [i64, i32, p, p, p, i32, p, p, p, p, i32]
+        lib.or_select_sum.restype = i32
+        lib.or_sum_at.argtypes = [p, i64, i32, p, p]
+        lib.or_sum_at.restype = i32
+        lib.or_threads_default.restype = i32
+        _lib = lib
+    return _lib
+
+
+def _u32(a):
+    a = np.ascontiguousarray(a, dtype=np.uint32)
+    return a
+
+
+def _ptr(a):
+    return a.ctypes.data_as(ctypes.c_void_p)
+
+
+def _ptr_array(arrs):
+    arr = (ctypes.c_void_p * max(1, len(arrs)))(*[a.ctypes.data for a in arrs])
+    return arr
+
+
+def default_threads() -> int:
+    return int(_load().or_threads_default())
+
+
+def decompose(v, k: int, base: int = 0):
+    """(major, residual, w_M) of the BWD split with k residual bits (Fig. 2)."""
+    v = _u32(v)
+    major = np.empty_like(v)
+    residual = np.empty_like(v)
+    w = _load().or_decompose(_ptr(v), v.size, k, base, _ptr(major), _ptr(residual))
+    return major, residual, int(w)
+
+
+def bucket_flags(major, k: int, lo: int, hi: int, base: int = 0):
+    """(cand, def) bool flags of lo <= v <= hi on the approximation."""
+    major = _u32(major)
+    cand = np.empty(major.size, dtype=np.uint8)
+    dfn = np.empty(major.size, dtype=np.uint8)
+    _load().or_bucket_flags(_ptr(major), major.size, k, base, lo, hi, _ptr(cand), _ptr(dfn))
+    return cand.astype(bool), dfn.astype(bool)
+
+
+def paper_f_flags(v, k: int, op: str, x: int):
+    """Candidate flags under the printed relaxation f(x)."""
+    v = _u32(v)
+    flag = np.empty(v.size, dtype=np.uint8)
+    _load().or_paper_f_flags(_ptr(v), v.size, k, OPS[op], x, _ptr(flag))
+    return flag.astype(bool)
+
+
+def approx_select(values, ks, los, his, base=None):
+    """Reference intermediates of the approximate selection (conjunction of predicates):
+    returns (cand_positions int64, definite flags at those positions).  Each predicate
+    column is decomposed with its own k; cand/def of a row are the ANDs over predicates."""
+    n = len(values[0])
+    cand = np.ones(n, dtype=bool)
+    dfn = np.ones(n, dtype=bool)
+    for c, v in enumerate(values):
+        b = 0 if base is None else base[c]
+        major, _, _ = decompose(v, ks[c], b)
+        cf, df = bucket_flags(major, ks[c], los[c], his[c], b)
+        cand &= cf
+        dfn &= df
+    pos = np.nonzero(cand)[0].astype(np.int64)
+    return pos, dfn[pos]
+
+
+def select_sum(pred_cols, los, his, agg_cols=(), threads: int = 1, positions: bool = True):
+    """Exact select + product SUM (the plain definition): returns (positions|None, count, sum)."""
+    pred_cols = [_u32(c) for c in pred_cols]
+    agg_cols = [_u32(c) for c in agg_cols]
+    n = pred_cols[0].size if pred_cols else (agg_cols[0].size if agg_cols else 0)
+    lo = np.asarray(los, dtype=np.uint32)
+    hi = np.asarray(his, dtype=np.uint32)
+    out = np.empty(n if positions else 1, dtype=np.int64)
+    cnt = ctypes.c_int64(0)
+    s = ctypes.c_int64(0)
+    pc, ac = _ptr_array(pred_cols), _ptr_array(agg_cols)
+    ovf = _load().or_select_sum(n, len(pred_cols), ctypes.cast(pc, ctypes.c_void_p), _ptr(lo), _ptr(hi),
+                                len(agg_cols), ctypes.cast(ac, ctypes.c_void_p),
+                                _ptr(out) if positions else None, ctypes.byref(cnt), ctypes.byref(s),
+                                threads)
+    if ovf:
+        raise OverflowError("exact SUM does not fit in int64")
+    return (out[: cnt.value] if positions else None), int(cnt.value), int(s.value)
+
+
+def sum_at(pos, agg_cols):
+    """Exact product SUM at given positions (SUM(refine), Fig. 3 / Fig. 7)."""
+    pos = np.ascontiguousarray(pos, dtype=np.int64)
+    agg_cols = [_u32(c) for c in agg_cols]
+    s = ctypes.c_int64(0)
+    ac = _ptr_array(agg_cols)
+    if _load().or_sum_at(_ptr(pos), pos.size, len(agg_cols), ctypes.cast(ac, ctypes.c_void_p), ctypes.byref(s)):
+        raise OverflowError("exact SUM does not fit in int64")
+    return int(s.value)

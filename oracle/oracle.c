@@ -1,0 +1,246 @@
+/*
+ * oracle.c -- TEST INFRASTRUCTURE ONLY.
+ *
+ * A plain, slow, obviously correct CPU statement of what Approximate & Refine
+ * (A&R) over bitwise-distributed (BWD) columns computes, written from
+ * H. Pirk, S. Manegold, M. Kersten, "Waste Not... Efficient Co-Processing of
+ * Relational Data", ICDE 2014 (cited as PAPER.md:<line>, s<section>).
+ *
+ * Only tests/, __graft_entry__.smoke() and bench.py's cpu_baseline /
+ * `--impl reference` legs may load this library.  The product path
+ * (paper_conf_icde_pirkmk14_b200/) never imports, links or calls it, and this
+ * file shares no code, header, table or constant with the CUDA path.
+ *
+ * Because A&R is exact (the approximation is a superset; the
+ * refined result is correct), the oracle for the final
+ * result is the plain definition over the undecomposed columns:
+ *   R = [ i ascending : for all predicates c, lo_c <= v_c[i] <= hi_c ]
+ *   S = sum_{i in R} prod_{c in agg} v_c[i]              (exact, int64)
+ * The intermediates (decomposition, candidate / definite flags) are written
+ * out from their definitions too.
+ *
+ * Every function is pinned by tests/test_oracle_*.py against the paper's
+ * worked examples (Fig. 2, 4, 6), closed forms, and brute force.
+ */
+#include <stdint.h>
+#include <stdlib.h>
+#include <string.h>
+#include <pthread.h>
+#include <unistd.h>
+
+/* ----------------------------------------------------------------- threads */
+
+typedef void (*or_chunk_fn)(void* ctx, int t, int64_t begin, int64_t end);
+typedef struct { or_chunk_fn fn; void* ctx; int t; int64_t b, e; } or_job;
+
+static void* or_run(void* p) { or_job* j = (or_job*)p; j->fn(j->ctx, j->t, j->b, j->e); return NULL; }
+
+int or_threads_default(void) {
+    long c = sysconf(_SC_NPROCESSORS_ONLN);
+    return c > 0 ? (int)c : 1;
+}
+
+#define OR_MAX_THREADS 256
+
+/* T threads over contiguous row chunks; chunk t is [t*chunk, (t+1)*chunk). */
+static int or_parallel(int64_t n, int threads, or_chunk_fn fn, void* ctx, int64_t* bounds) {
+    if (threads <= 0) threads = or_threads_default();
+    if (threads > OR_MAX_THREADS) threads = OR_MAX_THREADS;
+    int64_t chunk = threads > 0 ? (n + threads - 1) / threads : n;
+    if (chunk == 0) chunk = 1;
+    pthread_t tid[OR_MAX_THREADS];
+    or_job jobs[OR_MAX_THREADS];
+    int started[OR_MAX_THREADS];
+    for (int t = 0; t < threads; ++t) {
+        int64_t b = (int64_t)t * chunk, e = b + chunk;
+        if (b > n) b = n;
+        if (e > n) e = n;
+        bounds[2 * t] = b; bounds[2 * t + 1] = e;
+        jobs[t] = (or_job){fn, ctx, t, b, e};
+        started[t] = (threads > 1) && pthread_create(&tid[t], NULL, or_run, &jobs[t]) == 0;
+        if (!started[t]) fn(ctx, t, b, e);
+    }
+    for (int t = 0; t < threads; ++t) if (started[t]) pthread_join(tid[t], NULL);
+    return threads;
+}
+
+/* --------------------------------------------------------- decomposition */
+
+/*
+ * BWD decomposition, PAPER.md:143-160 (s II-A) and Fig. 2:
+ * the value is split at bit granularity into major bits (the approximation)
+ * and minor bits (the residual), non-redundantly; leading zeros are removed.
+ * With k residual bits (k = 32 - major_bits) and prefix base b
+ * (b = 0 in v1):
+ *     u = v - b,   major = u >> k,   residual = u mod 2^k.
+ * Returns the stored major width w_M = bit length of max(major) (the leading
+ * zeros the paper removes).  Either output pointer may be NULL.
+ */
+int or_decompose(const uint32_t* v, int64_t n, int k, uint32_t base,
+                 uint32_t* major, uint32_t* residual) {
+    uint64_t two_k = (uint64_t)1 << k;               /* k in [0, 32] */
+    uint64_t maxmajor = 0;
+    for (int64_t i = 0; i < n; ++i) {
+        uint64_t u = (uint64_t)(uint32_t)(v[i] - base);
+        uint64_t m = u / two_k;
+        uint64_t r = u % two_k;
+        if (major) major[i] = (uint32_t)m;
+        if (residual) residual[i] = (uint32_t)r;
+        if (m > maxmajor) maxmajor = m;
+    }
+    int w = 0;
+    while (w < 64 && (maxmajor >> w) != 0) ++w;
+    return w;
+}
+
+/* ---------------------------------------------- approximate select flags */
+
+/*
+ * Candidate / definite flags of one predicate lo <= v <= hi evaluated on the
+ * approximation alone (s IV-B; tight reading SURVEY A2/A6).
+ * A major value m stands for its bucket, the 2^k exact values it can hold:
+ *     bucket(m) = [ b + m*2^k , b + m*2^k + 2^k - 1 ]
+ *   cand(m) <=> bucket(m) intersects [lo, hi]   (superset of the hits)
+ *   def(m)  <=> bucket(m) is contained in [lo, hi]  (certain hits)
+ * cand / def are byte flags (0/1), either may be NULL.
+ */
+void or_bucket_flags(const uint32_t* major, int64_t n, int k, uint32_t base,
+                     uint32_t lo, uint32_t hi, uint8_t* cand, uint8_t* def) {
+    uint64_t two_k = (uint64_t)1 << k;
+    for (int64_t i = 0; i < n; ++i) {
+        uint64_t first = (uint64_t)base + (uint64_t)major[i] * two_k;
+        uint64_t last = first + two_k - 1;
+        int c = (first <= (uint64_t)hi) && (last >= (uint64_t)lo) && (lo <= hi);
+        int d = (first >= (uint64_t)lo) && (last <= (uint64_t)hi);
+        if (cand) cand[i] = (uint8_t)c;
+        if (def) def[i] = (uint8_t)d;
+    }
+}
+
+/*
+ * The relaxation function f(x) exactly as printed, with the
+ * lost shift operator restored as "<<":
+ *     appr(x) = x & ~((1 << resbits) - 1)
+ *     '==' : appr(x)               '>=' : appr(x)
+ *     '>'  : appr(x) - 1           '<=' : appr(x) + (1 << resbits)
+ *     '<'  : appr(x) + (1 << resbits) + 1
+ * and the scan keeps the operator: flag = appr(v) op f(x).  Used by tests only,
+ * to check printed-f candidates contain the tight candidates.
+ * op: 0 '==', 1 '>', 2 '>=', 3 '<', 4 '<='.
+ */
+void or_paper_f_flags(const uint32_t* v, int64_t n, int k, int op, uint32_t x, uint8_t* flag) {
+    int64_t two_k = (int64_t)1 << k;
+    int64_t ax = (int64_t)((uint64_t)x & ~(uint64_t)(two_k - 1));
+    int64_t fx;
+    switch (op) {
+        case 0: fx = ax; break;
+        case 1: fx = ax - 1; break;
+        case 2: fx = ax; break;
+        case 3: fx = ax + two_k + 1; break;
+        default: fx = ax + two_k; break;
+    }
+    for (int64_t i = 0; i < n; ++i) {
+        int64_t av = (int64_t)((uint64_t)v[i] & ~(uint64_t)(two_k - 1));
+        int f;
+        switch (op) {
+            case 0: f = av == fx; break;
+            case 1: f = av > fx; break;
+            case 2: f = av >= fx; break;
+            case 3: f = av < fx; break;
+            default: f = av <= fx; break;
+        }
+        flag[i] = (uint8_t)f;
+    }
+}
+
+/* ------------------------------------------------ exact select and SUM */
+
+typedef struct {
+    int npred;
+    const uint32_t* const* pcols;
+    const uint32_t* lo;
+    const uint32_t* hi;
+    int nagg;
+    const uint32_t* const* acols;
+    int64_t* out_pos;            /* may be NULL                      */
+    int64_t count[OR_MAX_THREADS];
+    __int128 sum[OR_MAX_THREADS];
+    int64_t* bounds;
+    int pass;                    /* 0: count+sum, 1: write positions */
+    int64_t offset[OR_MAX_THREADS];
+} sel_ctx;
+
+static int row_qualifies(const sel_ctx* c, int64_t i) {
+    for (int p = 0; p < c->npred; ++p) {
+        uint32_t v = c->pcols[p][i];
+        if (!(c->lo[p] <= v && v <= c->hi[p])) return 0;
+    }
+    return 1;
+}
+
+static void sel_chunk(void* p, int t, int64_t b, int64_t e) {
+    sel_ctx* c = (sel_ctx*)p;
+    if (c->pass == 0) {
+        int64_t cnt = 0;
+        __int128 s = 0;
+        for (int64_t i = b; i < e; ++i) {
+            if (!row_qualifies(c, i)) continue;
+            ++cnt;
+            if (c->nagg > 0) {
+                __int128 prod = 1;
+                for (int a = 0; a < c->nagg; ++a) prod *= (__int128)c->acols[a][i];
+                s += prod;
+            }
+        }
+        c->count[t] = cnt;
+        c->sum[t] = s;
+    } else {
+        int64_t o = c->offset[t];
+        for (int64_t i = b; i < e; ++i)
+            if (row_qualifies(c, i)) c->out_pos[o++] = i;
+    }
+}
+
+/*
+ * Exact conjunctive range select + product SUM over the full-precision
+ * columns: the plain definition the A&R plan must reproduce (Fig. 3 / Fig. 7,
+ * PAPER.md:333-359, 879-893; Q6 shape PAPER.md:1291-1309).
+ *   out_pos (optional): ascending positions of qualifying rows
+ *   *out_count       : |R|
+ *   *out_sum         : sum over R of prod_a acols[a][i]  (0 if nagg == 0)
+ * Rows are split over `threads` contiguous chunks and chunk results are
+ * concatenated / added in chunk order, so the result does not depend on T.
+ * Returns 0, or 1 if the exact sum does not fit in int64.
+ */
+int or_select_sum(int64_t n, int npred, const uint32_t* const* pcols,
+                  const uint32_t* lo, const uint32_t* hi,
+                  int nagg, const uint32_t* const* acols,
+                  int64_t* out_pos, int64_t* out_count, int64_t* out_sum, int threads) {
+    sel_ctx* c = (sel_ctx*)calloc(1, sizeof(sel_ctx));
+    int64_t bounds[2 * OR_MAX_THREADS];
+    c->npred = npred; c->pcols = pcols; c->lo = lo; c->hi = hi;
+    c->nagg = nagg; c->acols = acols; c->out_pos = out_pos; c->bounds = bounds;
+    c->pass = 0;
+    int T = or_parallel(n, threads, sel_chunk, c, bounds);
+    int64_t total = 0;
+    __int128 s = 0;
+    for (int t = 0; t < T; ++t) { c->offset[t] = total; total += c->count[t]; s += c->sum[t]; }
+    if (out_pos) { c->pass = 1; or_parallel(n, T, sel_chunk, c, bounds); }
+    if (out_count) *out_count = total;
+    int overflow = (s > (__int128)INT64_MAX) || (s < (__int128)INT64_MIN);
+    if (out_sum) *out_sum = (int64_t)s;
+    free(c);
+    return overflow;
+}
+
+/* Product SUM over given positions (SUM(refine) of Fig. 3/7), exact; returns 1 on int64 overflow. */
+int or_sum_at(const int64_t* pos, int64_t npos, int nagg, const uint32_t* const* acols, int64_t* out_sum) {
+    __int128 s = 0;
+    for (int64_t j = 0; j < npos; ++j) {
+        __int128 prod = 1;
+        for (int a = 0; a < nagg; ++a) prod *= (__int128)acols[a][pos[j]];
+        s += prod;
+    }
+    *out_sum = (int64_t)s;
+    return (s > (__int128)INT64_MAX) || (s < (__int128)INT64_MIN);
+}
