@@ -1,0 +1,296 @@
+/*
+ * ar.h -- C ABI of the B200-native Approximate & Refine (A&R) hot path over
+ * bitwise-distributed (BWD) integer columns.
+ *
+ * Method: H. Pirk, S. Manegold, M. Kersten, "Waste Not... Efficient
+ * Co-Processing of Relational Data", ICDE 2014.  Citations "PAPER.md:<line>"
+ * refer to the text of that paper; "SURVEY s8" to /root/repo/SURVEY.md s8 (the
+ * hot-path scope table), "DESIGN" to /root/repo/DESIGN.md.
+ *
+ * Conventions (all calls):
+ *  - Plain pointers and sizes only.  A "device pointer" is CUDA device memory
+ *    (e.g. a torch CUDA tensor's data_ptr); a "host-pinned pointer" is page-
+ *    locked host memory (cudaHostAlloc / torch pin_memory) the GPU reads over
+ *    the host link.  `stream` is a cudaStream_t passed as void*.
+ *  - Every call that takes a stream is asynchronous on it, except
+ *    ar_decompose_plan (documented below).  Results that live in device memory
+ *    (counts, sums) are valid once the stream reaches that point.
+ *  - The library never allocates device memory: the caller owns every buffer
+ *    and workspace.  Handles (ar_column, ar_dist) are small host objects.
+ *  - No call aborts or throws.  Each returns an ar_status; on failure
+ *    ar_last_error() (thread-local) describes the cause.
+ *  - Values are uint32 (signed callers map v -> v ^ 0x80000000).
+ *    Positions are uint32 row indices local to the column (a shard), counts
+ *    and sums are int64.  There is no floating point anywhere on the path.
+ */
+#ifndef AR_H
+#define AR_H
+
+#include <stddef.h>
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+typedef enum {
+    AR_OK = 0,
+    AR_ERR_INVALID = 1,      /* bad argument (null pointer, bad width, mismatched columns) */
+    AR_ERR_RANGE = 2,        /* a buffer / workspace / capacity is too small, or overflow possible */
+    AR_ERR_CUDA = 3,         /* CUDA runtime error (launch failure, bad pointer, no device) */
+    AR_ERR_NCCL = 4,         /* NCCL error in an ar_dist_* call */
+    AR_ERR_UNSUPPORTED = 5   /* valid but outside what this build implements (e.g. too many planes) */
+} ar_status;
+
+/* Where a part of a column lives. */
+typedef enum {
+    AR_LOC_DEVICE = 0,       /* HBM of the current device */
+    AR_LOC_HOST_PINNED = 1   /* pinned host memory, read by kernels over the host link (zero-copy) */
+} ar_loc;
+
+/*
+ * Physical layout of the major (approximation) part.  The paper leaves the
+ * physical representation inside a bitwise partition open (PAPER.md:219-221,
+ * s II-A); this build offers two (DESIGN "Data layout in HBM"):
+ *  AR_LAYOUT_SLICED: rows are grouped in blocks of 32; block b stores w_major
+ *    uint32 words, word j holding bit j of the majors of rows 32b..32b+31
+ *    (bit l of the word = row 32b+l).  Scan-optimised: a range test costs a
+ *    few bitwise ops per bit plane per 32 rows.  Required for ar_approx_select.
+ *  AR_LAYOUT_PACKED: LSB-first bitstream, row i occupies bits [i*w, i*w+w) of
+ *    the little-endian uint32 word stream.  Gather-optimised (one sector per
+ *    value): use it for columns that are only aggregated (l_extendedprice).
+ * Residuals (minor bits) are always AR_LAYOUT_PACKED with width k.
+ */
+typedef enum {
+    AR_LAYOUT_SLICED = 0,
+    AR_LAYOUT_PACKED = 1
+} ar_layout;
+
+#define AR_MAX_PRED 8          /* predicates per conjunctive select            */
+#define AR_MAX_AGG 2           /* factors of the SUM product    */
+#define AR_MAX_PLANES 64       /* sum of w_major over the predicates of a scan */
+
+/*
+ * Decomposition descriptor, the "extended BAT" metadata of PAPER.md:908-916
+ * (s V-C): number and significance of the bits on each device (which also
+ * encodes the error of the approximation) and the prefix-compression base.
+ * Filled by ar_decompose_plan; plain old data, caller-owned.
+ */
+typedef struct {
+    int64_t n;                 /* rows                                                    */
+    int32_t major_bits;        /* M of bwdecompose(A, M); k = 32 - M   */
+    int32_t k;                 /* residual (minor) bits, 0..31                            */
+    int32_t w_major;           /* stored major width after leading-zero removal, 0..M     */
+    int32_t major_layout;      /* ar_layout of the major part                             */
+    int32_t residual_loc;      /* ar_loc of the residual part                             */
+    uint32_t base;             /* prefix base b: value = ((major << k) | residual) + b    */
+    uint64_t major_bytes;      /* bytes the major buffer must provide (device memory)     */
+    uint64_t residual_bytes;   /* bytes the residual buffer must provide (0 if k == 0)    */
+} ar_column_desc;
+
+typedef struct ar_column ar_column;   /* opaque: desc + part pointers (host object) */
+
+/* One conjunct lo <= value <= hi (inclusive, exact bounds; lo > hi selects nothing).
+ * Operators normalise to this form: <x -> [0,x-1], >x -> [x+1,2^32-1],
+ * ==x -> [x,x], between a and b -> [a,b]. */
+typedef struct {
+    const ar_column* col;
+    uint32_t lo;
+    uint32_t hi;
+} ar_pred;
+
+/*
+ * Candidate relation: the output of the approximate selection, a superset of
+ * the exact result (Fig. 4 "sigma(Approx A <= 4)" yields
+ * (ID, Approx A) pairs).  Entry j (0 <= j < *count) is
+ *   pos[j]: the row position (ascending in j: the compaction is stable, so
+ *           every refine join is a positional "invisible" join)
+ *   aux[j]: bit 31 = definite (the row's whole bucket satisfies every
+ *           predicate, so it needs no residual); bits 0..30 = the
+ *           approximation tuple, i.e. the predicate columns' majors
+ *           concatenated LSB-first in predicate order, present iff
+ *           appr_bits > 0 (ar_approx_select flag AR_SELECT_CARRY_APPR).
+ * pos, aux and count are caller-owned device buffers of `capacity` entries
+ * (capacity >= n is always sufficient).
+ */
+typedef struct {
+    uint32_t* pos;
+    uint32_t* aux;
+    int64_t* count;            /* device int64 */
+    int64_t capacity;
+    int32_t appr_bits;         /* set by ar_approx_select */
+    int32_t reserved;
+} ar_cands;
+
+#define AR_AUX_DEFINITE 0x80000000u
+
+/* Refined positions: ascending row positions of the exact result. Caller-owned device buffers. */
+typedef struct {
+    uint32_t* pos;
+    int64_t* count;            /* device int64 */
+    int64_t capacity;
+} ar_positions;
+
+/* ---------------------------------------------------------------- errors */
+
+const char* ar_status_str(ar_status s);
+const char* ar_last_error(void);     /* thread-local detail of the last failure */
+const char* ar_version(void);
+
+/* --------------------------------------------------- a1: decomposition */
+
+/* Workspace (device memory, >= this many bytes) for ar_decompose_plan. */
+size_t ar_decompose_ws_bytes(void);
+
+/*
+ * Plan a BWD decomposition of column `col` (n uint32 values, device pointer or
+ * host-pinned pointer) into `major_bits` major bits and k = 32 - major_bits
+ * residual bits, the split of bwdecompose(A, bits) (s V-A).
+ * Computes w_major = bit length of max((v - base) >> k) (leading zeros are
+ * removed) with a max-reduction kernel, then the byte sizes of
+ * both parts.  SYNCHRONISES `stream` once (the sizing pass).
+ * Errors: AR_ERR_INVALID if col == NULL && n > 0, n < 0, n >= 2^32,
+ * major_bits outside [1,32], bad layout / location, ws too small or desc NULL.
+ */
+ar_status ar_decompose_plan(const uint32_t* col, int64_t n, int32_t major_bits,
+                            int32_t major_layout, int32_t residual_loc, uint32_t base,
+                            void* ws, size_t ws_bytes, ar_column_desc* desc, void* stream);
+
+/*
+ * Decompose and pack `col` per `desc`: the major part is written to
+ * `major_buf` (device memory, desc->major_bytes bytes, padding zeroed) and the
+ * residual part to `residual_buf` (device memory, or pinned host memory when
+ * desc->residual_loc == AR_LOC_HOST_PINNED; desc->residual_bytes bytes).
+ * The buffers must outlive the returned handle, which is freed with
+ * ar_column_free.  Values larger than the plan's maximum are not detected:
+ * plan and decompose the same column.
+ * Errors: AR_ERR_INVALID (null pointers, bad desc), AR_ERR_RANGE (buffer too
+ * small), AR_ERR_CUDA (launch failure or unmappable host pointer).
+ */
+ar_status ar_decompose(const uint32_t* col, const ar_column_desc* desc,
+                       void* major_buf, uint64_t major_buf_bytes,
+                       void* residual_buf, uint64_t residual_buf_bytes,
+                       void* stream, ar_column** out);
+
+/* Wrap already-decomposed parts (e.g. a copy of the buffers ar_decompose wrote) in a new handle. */
+ar_status ar_column_wrap(const ar_column_desc* desc, const void* major_buf, const void* residual_buf,
+                         ar_column** out);
+ar_status ar_column_get_desc(const ar_column* col, ar_column_desc* desc);
+void ar_column_free(ar_column* col);
+
+/* ------------------------------------- a2 + a3: approximate selection */
+
+#define AR_SELECT_CARRY_APPR 1   /* write the approximation tuple into aux bits 0..30 */
+
+/* Workspace (device memory) for ar_approx_select over n rows. */
+size_t ar_select_ws_bytes(int64_t n);
+
+/*
+ * Approximate selection (s IV-B) of the conjunction of
+ * `npred` predicates over columns of equal n (all major parts AR_LAYOUT_SLICED
+ * in device memory).  Host side (a2): each exact [lo, hi] is relaxed to the
+ * major ranges cand = [lo>>k, hi>>k] (bucket intersects [lo,hi]) and
+ * def = [ceil(lo/2^k), floor((hi+1)/2^k) - 1] (bucket inside [lo,hi]), with
+ * b = base subtracted first (DESIGN "Readings").  Device side
+ * (a3): one pass over the packed majors, stable compaction (warp ballot /
+ * popc, block scan, decoupled look-back) into out->pos / out->aux /
+ * *out->count.  npred == 0 selects every row.  A predicate with lo > hi makes
+ * the result empty (AR_OK).
+ * Errors: AR_ERR_INVALID (npred > AR_MAX_PRED, null / mismatched columns,
+ * non-SLICED or host-resident majors), AR_ERR_RANGE (capacity < n, ws too
+ * small, AR_SELECT_CARRY_APPR with sum of w_major > 31), AR_ERR_UNSUPPORTED
+ * (sum of w_major > AR_MAX_PLANES).
+ */
+ar_status ar_approx_select(const ar_pred* preds, int32_t npred, int32_t flags, ar_cands* out,
+                           void* ws, size_t ws_bytes, void* stream);
+
+/* ----------------------------------------------------- a5: refinement */
+
+/* Workspace (device memory) for ar_refine over up to `capacity` candidates. */
+size_t ar_refine_ws_bytes(int64_t capacity);
+
+/*
+ * Selection refinement (Algorithm 2 SELECTREFINE):
+ * for every candidate in `in` (ascending), definite candidates are kept
+ * without touching residuals; the others are joined positionally with the
+ * residual of every predicate column with k > 0 (device or host-pinned), the
+ * exact value is rebuilt by bitwise concatenation ((major << k) | residual) +
+ * base, and the exact predicate re-evaluated.  Output: ascending positions of
+ * the exact result (stable compaction) and its count.  `preds` must be the
+ * same list (same order) given to the ar_approx_select that produced `in`.
+ * Errors: AR_ERR_INVALID (mismatch with in->appr_bits, null pointers),
+ * AR_ERR_RANGE (out->capacity < in->capacity, ws too small).
+ */
+ar_status ar_refine(const ar_cands* in, const ar_pred* preds, int32_t npred, ar_positions* out,
+                    void* ws, size_t ws_bytes, void* stream);
+
+/* ----------------------------------------------------- a6: aggregation */
+
+/*
+ * SUM over the positions of `pos` of prod_c value_c(p), c < ncols (ncols in
+ * {1, 2}), exact in int64 (SUM(refine), Fig. 3 / Fig. 7, PAPER.md:884-889;
+ * destructive distributivity, is why the exact values are
+ * rebuilt before multiplying).  Result written to *out_sum_dev (device int64).
+ * Errors: AR_ERR_INVALID (ncols not in {1,2}, null pointers, column shorter
+ * than a position), AR_ERR_RANGE if sum of (w_major + k) + ceil(log2 n) > 63
+ * (the exact sum could overflow int64).
+ */
+ar_status ar_sum(const ar_positions* pos, const ar_column* const* cols, int32_t ncols,
+                 int64_t* out_sum_dev, void* stream);
+
+/*
+ * Fused refine + SUM (a5 + a6): the refinement of ar_refine without
+ * materialising positions, then the product SUM of ar_sum over the refined
+ * rows.  Aggregated columns that are also predicate columns reuse the carried
+ * approximation (and residual) instead of re-gathering.  Writes
+ * *out_sum_dev and *out_count_dev (refined row count); either may be NULL.
+ * Errors: as ar_refine and ar_sum.
+ */
+ar_status ar_refine_sum(const ar_cands* in, const ar_pred* preds, int32_t npred,
+                        const ar_column* const* cols, int32_t ncols,
+                        int64_t* out_sum_dev, int64_t* out_count_dev, void* stream);
+
+/*
+ * One-pass A&R (a3 + a5 + a6 fused, SURVEY s8(a) "Fusion note"): scan the
+ * majors, decide candidate / definite per row, refine the non-definite
+ * candidates inline from the residuals and add the product SUM of `cols` over
+ * the exact result.  No candidate list is materialised.  out_dev[0] = SUM,
+ * out_dev[1] = |exact result|, out_dev[2] = |candidates|, out_dev[3] =
+ * |definite| (device int64[4]; out_dev[2..3] give the approximate COUNT
+ * interval [#definite, #candidates] before refinement).
+ * Returns results identical to ar_approx_select -> ar_refine_sum.
+ * Errors: as ar_approx_select and ar_sum (ncols may be 0: COUNT only).
+ */
+ar_status ar_select_refine_sum(const ar_pred* preds, int32_t npred,
+                               const ar_column* const* cols, int32_t ncols,
+                               int64_t* out_dev, void* stream);
+
+/* -------------------------------- a4: row-sharded multi-GPU exchange */
+
+typedef struct ar_dist ar_dist;
+
+/* Size of the opaque NCCL unique id blob (rank 0 creates it; the caller broadcasts it). */
+size_t ar_dist_unique_id_bytes(void);
+ar_status ar_dist_get_unique_id(void* id_out);
+
+/* One communicator per rank over the current device (NCCL over NVLink / NVSwitch). */
+ar_status ar_dist_init(ar_dist** d, const void* unique_id, int32_t rank, int32_t world);
+
+/*
+ * Count exchange: ncclAllGather of each rank's *local_count_dev into
+ * all_counts_dev[world], then *global_offset_dev = sum of the counts of lower
+ * ranks (the rank's slice of the concatenated, globally ordered result starts
+ * there; global position = shard_row_base + local position).  Device pointers.
+ */
+ar_status ar_dist_offsets(ar_dist* d, const int64_t* local_count_dev, int64_t* all_counts_dev,
+                          int64_t* global_offset_dev, void* stream);
+
+/* In-place ncclAllReduce(int64, sum) of `n` device int64 values (the Q6 SUM and counts). */
+ar_status ar_dist_sum(ar_dist* d, int64_t* values_dev, int32_t n, void* stream);
+
+void ar_dist_free(ar_dist* d);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* AR_H */

@@ -1,0 +1,183 @@
+"""Torch plumbing around the C ABI: device / pinned buffers, streams, handles.
+
+PyTorch only supplies memory and streams here; every step of the A&R path
+runs in libar_b200.so.  Names follow the paper: a column is decomposed
+(bwdecompose) into an approximation (major bits) and a
+residual (minor bits); the approximate selection yields a candidate relation
+(PAPER.md:368-374), the refinement the exact positions and
+SUM(refine) the aggregate (Fig. 7).
+"""
+from __future__ import annotations
+
+import numpy as np
+import torch
+
+from . import _ar
+from ._ar import (AR_LAYOUT_PACKED, AR_LAYOUT_SLICED, AR_LOC_DEVICE, AR_LOC_HOST_PINNED,  # noqa: F401
+                  AR_SELECT_CARRY_APPR, Cands, Positions)
+
+
+def _stream(stream=None) -> int:
+    s = stream if stream is not None else torch.cuda.current_stream()
+    return s.cuda_stream
+
+
+def _nbytes_tensor(nbytes: int, device, pinned: bool = False) -> torch.Tensor:
+    nbytes = max(int(nbytes), 16)
+    if pinned:
+        return torch.empty(nbytes, dtype=torch.uint8, pin_memory=True)
+    return torch.empty(nbytes, dtype=torch.uint8, device=device)
+
+
+def as_u32_device(values, device="cuda") -> torch.Tensor:
+    """uint32 numpy array / int32 tensor -> contiguous int32 CUDA tensor holding the same bits."""
+    if isinstance(values, np.ndarray):
+        values = torch.from_numpy(np.ascontiguousarray(values, dtype=np.uint32).view(np.int32))
+    return values.to(device=device, dtype=torch.int32).contiguous()
+
+
+class BWDColumn:
+    """A bitwise-decomposed column (major part in HBM, residual in HBM or pinned host memory)."""
+
+    def __init__(self, values, major_bits: int, layout: int = AR_LAYOUT_SLICED,
+                 residual_loc: int = AR_LOC_DEVICE, base: int = 0, device="cuda", stream=None,
+                 _wrap=None):
+        self.device = torch.device(device)
+        if _wrap is not None:
+            self.desc, self.major, self.residual = _wrap
+            self.handle = _ar.ar_column_wrap(self.desc, self.major.data_ptr(),
+                                             self.residual.data_ptr() if self.desc.residual_bytes else None)
+            return
+        col = as_u32_device(values, self.device)
+        s = _stream(stream)
+        ws = torch.empty(_ar.ar_decompose_ws_bytes(), dtype=torch.uint8, device=self.device)
+        n = col.numel()
+        self.desc = _ar.ar_decompose_plan(col.data_ptr() if n else None, n, major_bits, layout, residual_loc, base,
+                                          ws.data_ptr(), ws.numel(), s)
+        self.major = _nbytes_tensor(self.desc.major_bytes, self.device)
+        self.residual = _nbytes_tensor(self.desc.residual_bytes, self.device,
+                                       pinned=(residual_loc == AR_LOC_HOST_PINNED))
+        self.handle = _ar.ar_decompose(col.data_ptr() if n else None, self.desc, self.major.data_ptr(),
+                                       self.major.numel(), self.residual.data_ptr(), self.residual.numel(), s)
+        torch.cuda.current_stream(self.device).synchronize() if stream is None else stream.synchronize()
+        del col
+
+    # -- metadata (decomposition + compression base)
+    @property
+    def n(self) -> int:
+        return int(self.desc.n)
+
+    @property
+    def k(self) -> int:
+        return int(self.desc.k)
+
+    @property
+    def w_major(self) -> int:
+        return int(self.desc.w_major)
+
+    def nbytes(self) -> dict:
+        return {"major": int(self.desc.major_bytes), "residual": int(self.desc.residual_bytes)}
+
+    def copy(self, residual_loc=None) -> "BWDColumn":
+        """A second handle over copies of the buffers (used to rotate inputs past L2 in the bench)."""
+        major = self.major.clone()
+        residual = self.residual.clone() if self.residual.device.type == "cuda" else self.residual.clone().pin_memory()
+        return BWDColumn(None, 0, _wrap=(self.desc, major, residual), device=self.device)
+
+    def free(self):
+        if getattr(self, "handle", None):
+            _ar.ar_column_free(self.handle)
+            self.handle = None
+
+    def __del__(self):
+        try:
+            self.free()
+        except Exception:
+            pass
+
+
+class CandidateList:
+    """Device buffers of an ar_cands (positions, aux words, count)."""
+
+    def __init__(self, capacity: int, device="cuda"):
+        cap = max(int(capacity), 1)
+        self.pos = torch.empty(cap + 8, dtype=torch.int32, device=device)
+        self.aux = torch.empty(cap + 8, dtype=torch.int32, device=device)
+        self.count_t = torch.zeros(1, dtype=torch.int64, device=device)
+        self.c = Cands(self.pos.data_ptr(), self.aux.data_ptr(), self.count_t.data_ptr(), int(capacity), 0, 0)
+
+    def count(self) -> int:
+        return int(self.count_t.item())
+
+    def positions(self) -> np.ndarray:
+        n = self.count()
+        return self.pos[:n].cpu().numpy().view(np.uint32).astype(np.int64)
+
+    def aux_words(self) -> np.ndarray:
+        n = self.count()
+        return self.aux[:n].cpu().numpy().view(np.uint32)
+
+    def definite(self) -> np.ndarray:
+        return (self.aux_words() & _ar.AR_AUX_DEFINITE) != 0
+
+
+class PositionList:
+    def __init__(self, capacity: int, device="cuda"):
+        cap = max(int(capacity), 1)
+        self.pos = torch.empty(cap + 8, dtype=torch.int32, device=device)
+        self.count_t = torch.zeros(1, dtype=torch.int64, device=device)
+        self.p = Positions(self.pos.data_ptr(), self.count_t.data_ptr(), int(capacity))
+
+    def count(self) -> int:
+        return int(self.count_t.item())
+
+    def positions(self) -> np.ndarray:
+        n = self.count()
+        return self.pos[:n].cpu().numpy().view(np.uint32).astype(np.int64)
+
+
+def _pred_tuples(preds):
+    return [(c.handle, int(lo), int(hi)) for c, lo, hi in preds]
+
+
+class Workspace:
+    """Caller-owned device workspace (the library never allocates device memory)."""
+
+    def __init__(self, nbytes: int, device="cuda"):
+        self.t = torch.empty(max(int(nbytes), 16), dtype=torch.uint8, device=device)
+
+    @property
+    def ptr(self):
+        return self.t.data_ptr()
+
+    @property
+    def nbytes(self):
+        return self.t.numel()
+
+
+def approx_select(preds, cands: CandidateList, ws: Workspace, carry: bool = True, stream=None):
+    """Steps a2+a3: preds = [(BWDColumn, lo, hi), ...] -> candidate relation in `cands`."""
+    _ar.ar_approx_select(_pred_tuples(preds), AR_SELECT_CARRY_APPR if carry else 0, cands.c, ws.ptr, ws.nbytes,
+                         _stream(stream))
+
+
+def refine(cands: CandidateList, preds, out: PositionList, ws: Workspace, stream=None):
+    """Step a5 (Algorithm 2): candidate relation -> exact ascending positions."""
+    _ar.ar_refine(cands.c, _pred_tuples(preds), out.p, ws.ptr, ws.nbytes, _stream(stream))
+
+
+def sum_at(pos: PositionList, cols, out: torch.Tensor, stream=None):
+    """Step a6: out[0] = SUM over pos of prod(cols)."""
+    _ar.ar_sum(pos.p, [c.handle for c in cols], out.data_ptr(), _stream(stream))
+
+
+def refine_sum(cands: CandidateList, preds, cols, out_sum: torch.Tensor, out_count: torch.Tensor = None,
+               stream=None):
+    """Steps a5+a6 fused: out_sum[0] = SUM(prod(cols)) over the refined rows, out_count[0] = their number."""
+    _ar.ar_refine_sum(cands.c, _pred_tuples(preds), [c.handle for c in cols], out_sum.data_ptr(),
+                      out_count.data_ptr() if out_count is not None else None, _stream(stream))
+
+
+def select_refine_sum(preds, cols, out4: torch.Tensor, stream=None):
+    """Steps a3+a5+a6 in one pass: out4 = [SUM, |result|, |candidates|, |definite|]."""
+    _ar.ar_select_refine_sum(_pred_tuples(preds), [c.handle for c in cols], out4.data_ptr(), _stream(stream))

@@ -1,0 +1,569 @@
+// api.cu -- the C ABI (include/ar.h): argument validation, relaxation of the
+// predicates (step a2, host scalars), workspace sizing and kernel launches.
+#include <algorithm>
+#include <cstring>
+#include <new>
+
+#include "kernels.cuh"
+
+namespace ar {
+
+static thread_local std::string g_err;
+
+void set_error(const char* fmt, ...) {
+    char buf[512];
+    va_list ap;
+    va_start(ap, fmt);
+    vsnprintf(buf, sizeof(buf), fmt, ap);
+    va_end(ap);
+    g_err = buf;
+}
+
+ar_status cuda_fail(cudaError_t e, const char* where) {
+    set_error("%s: %s (%s)", where, cudaGetErrorString(e), cudaGetErrorName(e));
+    return AR_ERR_CUDA;
+}
+
+int num_sms() {
+    static thread_local int cached_dev = -1, cached_sms = 0;
+    int dev = 0, sms = 0;
+    if (cudaGetDevice(&dev) != cudaSuccess) return 148;
+    if (dev == cached_dev) return cached_sms;
+    if (cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev) != cudaSuccess || sms <= 0) return 148;
+    cached_dev = dev;
+    cached_sms = sms;
+    return sms;
+}
+
+// Step a2: exact [lo, hi] -> candidate / definite major ranges.
+// In u = v - base units, bucket(m) = [m 2^k, m 2^k + 2^k - 1]:
+//   cand(m) <=> m 2^k <= uhi && m 2^k + 2^k - 1 >= ulo  <=>  ulo >> k <= m <= uhi >> k
+//   def(m)  <=> m 2^k >= ulo && m 2^k + 2^k - 1 <= uhi  <=>  ceil(ulo/2^k) <= m <= floor((uhi+1)/2^k) - 1
+// Both ranges are clamped to the stored width (m <= 2^w - 1).
+Relaxed relax(uint32_t lo, uint32_t hi, uint32_t base, int k, int w) {
+    Relaxed R{};
+    R.empty = true;
+    if (lo > hi || hi < base) return R;
+    const uint64_t ulo = lo < base ? 0 : (uint64_t)(lo - base);
+    const uint64_t uhi = (uint64_t)(hi - base);
+    const uint64_t maxm = w >= 32 ? 0xffffffffull : ((1ull << w) - 1);
+    const uint64_t clo = ulo >> k, chi = std::min<uint64_t>(uhi >> k, maxm);
+    if (clo > chi) return R;
+    R.empty = false;
+    R.clo = (uint32_t)clo;
+    R.chi = (uint32_t)chi;
+    const uint64_t two_k = 1ull << k;
+    const uint64_t dlo = (ulo + two_k - 1) >> k;
+    const uint64_t dtop = (uhi + 1) >> k;      // floor((uhi + 1) / 2^k)
+    R.def_any = false;
+    if (dtop >= 1) {
+        const uint64_t dhi = std::min<uint64_t>(dtop - 1, maxm);
+        if (dlo <= dhi) {
+            R.def_any = true;
+            R.dlo = (uint32_t)dlo;
+            R.dhi = (uint32_t)dhi;
+        }
+    }
+    return R;
+}
+
+static bool valid_col(const ar_column* c) { return c && (c->d.w_major == 0 || c->major); }
+
+// Rough pipeline sizing: aim for ~3 CTAs per SM and >= 3 stages each.
+static uint32_t pick_stages_uncached(uint32_t stage_words, bool staging, int* ctas_per_sm) {
+    uint32_t best = 2;
+    int best_occ = 0;
+    for (uint32_t st = 8; st >= 2; --st) {
+        const size_t smem = select_smem_bytes(stage_words, st, staging);
+        if (smem > 227 * 1024) continue;
+        const int occ = select_occupancy(smem, !staging);
+        // bytes in flight per SM ~ occ * (st - 1) * stage bytes; prefer more CTAs at similar depth
+        if (occ <= 0) continue;
+        if (occ * (int)(st - 1) > best_occ * (int)(best - 1) || best_occ == 0) {
+            best_occ = occ;
+            best = st;
+        }
+        if (occ >= 3 && st >= 3) break;
+    }
+    if (ctas_per_sm) *ctas_per_sm = best_occ > 0 ? best_occ : 1;
+    return best;
+}
+
+// Memoised per (stage_words, staging): the occupancy queries stay out of the launch path.
+static uint32_t pick_stages(uint32_t stage_words, bool staging, int* ctas_per_sm) {
+    struct Entry { uint32_t words; bool staging; uint32_t stages; int occ; };
+    static thread_local Entry cache[16];
+    static thread_local int used = 0;
+    for (int i = 0; i < used; ++i)
+        if (cache[i].words == stage_words && cache[i].staging == staging) {
+            *ctas_per_sm = cache[i].occ;
+            return cache[i].stages;
+        }
+    const uint32_t st = pick_stages_uncached(stage_words, staging, ctas_per_sm);
+    if (used < 16) cache[used++] = Entry{stage_words, staging, st, *ctas_per_sm};
+    return st;
+}
+
+}  // namespace ar
+
+using namespace ar;
+
+extern "C" {
+
+const char* ar_status_str(ar_status s) {
+    switch (s) {
+        case AR_OK: return "AR_OK";
+        case AR_ERR_INVALID: return "AR_ERR_INVALID";
+        case AR_ERR_RANGE: return "AR_ERR_RANGE";
+        case AR_ERR_CUDA: return "AR_ERR_CUDA";
+        case AR_ERR_NCCL: return "AR_ERR_NCCL";
+        case AR_ERR_UNSUPPORTED: return "AR_ERR_UNSUPPORTED";
+    }
+    return "AR_ERR_?";
+}
+
+const char* ar_last_error(void) { return g_err.c_str(); }
+const char* ar_version(void) { return "ar-b200 0.1 (sm_100a)"; }
+
+// ------------------------------------------------------------------ a1
+
+size_t ar_decompose_ws_bytes(void) { return 256; }
+
+ar_status ar_decompose_plan(const uint32_t* col, int64_t n, int32_t major_bits, int32_t major_layout,
+                            int32_t residual_loc, uint32_t base, void* ws, size_t ws_bytes, ar_column_desc* desc,
+                            void* stream) {
+    if (!desc || n < 0 || n >= (int64_t)1 << 32 || (n > 0 && !col)) {
+        set_error("ar_decompose_plan: bad column pointer / size (n=%lld)", (long long)n);
+        return AR_ERR_INVALID;
+    }
+    if (major_bits < 1 || major_bits > 32) {
+        set_error("ar_decompose_plan: major_bits=%d outside [1,32]", major_bits);
+        return AR_ERR_INVALID;
+    }
+    if ((major_layout != AR_LAYOUT_SLICED && major_layout != AR_LAYOUT_PACKED) ||
+        (residual_loc != AR_LOC_DEVICE && residual_loc != AR_LOC_HOST_PINNED)) {
+        set_error("ar_decompose_plan: bad layout (%d) or residual location (%d)", major_layout, residual_loc);
+        return AR_ERR_INVALID;
+    }
+    if (!ws || ws_bytes < ar_decompose_ws_bytes()) {
+        set_error("ar_decompose_plan: workspace of %zu bytes < %zu", ws_bytes, ar_decompose_ws_bytes());
+        return AR_ERR_INVALID;
+    }
+    cudaStream_t s = (cudaStream_t)stream;
+    const int k = 32 - major_bits;
+    uint32_t maxu = 0;
+    if (n > 0) {
+        AR_TRY_CUDA(cudaMemsetAsync(ws, 0, 4, s));
+        ar_status st = launch_decompose_max(col, n, base, (uint32_t*)ws, s);
+        if (st != AR_OK) return st;
+        AR_TRY_CUDA(cudaMemcpyAsync(&maxu, ws, 4, cudaMemcpyDeviceToHost, s));
+        AR_TRY_CUDA(cudaStreamSynchronize(s));
+    }
+    const uint32_t maxm = k >= 32 ? 0 : (maxu >> k);
+    int w = 0;
+    while (w < 32 && (maxm >> w) != 0) ++w;
+    memset(desc, 0, sizeof(*desc));
+    desc->n = n;
+    desc->major_bits = major_bits;
+    desc->k = k;
+    desc->w_major = w;
+    desc->major_layout = major_layout;
+    desc->residual_loc = residual_loc;
+    desc->base = base;
+    desc->major_bytes = major_layout == AR_LAYOUT_SLICED ? sliced_bytes(n, w) : packed_bytes(n, w);
+    desc->residual_bytes = packed_bytes(n, k);
+    return AR_OK;
+}
+
+static ar_status check_desc(const ar_column_desc* d) {
+    if (!d || d->n < 0 || d->n >= (int64_t)1 << 32 || d->major_bits < 1 || d->major_bits > 32 ||
+        d->k != 32 - d->major_bits || d->w_major < 0 || d->w_major > d->major_bits ||
+        (d->major_layout != AR_LAYOUT_SLICED && d->major_layout != AR_LAYOUT_PACKED) ||
+        (d->residual_loc != AR_LOC_DEVICE && d->residual_loc != AR_LOC_HOST_PINNED)) {
+        set_error("invalid ar_column_desc");
+        return AR_ERR_INVALID;
+    }
+    return AR_OK;
+}
+
+static ar_status device_alias(const void* p, int loc, const uint32_t** out) {
+    if (!p || loc == AR_LOC_DEVICE) {
+        *out = (const uint32_t*)p;
+        return AR_OK;
+    }
+    void* dp = nullptr;
+    cudaError_t e = cudaHostGetDevicePointer(&dp, const_cast<void*>(p), 0);
+    if (e != cudaSuccess) {
+        cudaGetLastError();
+        set_error("residual buffer is not mapped pinned host memory (%s)", cudaGetErrorString(e));
+        return AR_ERR_CUDA;
+    }
+    *out = (const uint32_t*)dp;
+    return AR_OK;
+}
+
+ar_status ar_column_wrap(const ar_column_desc* desc, const void* major_buf, const void* residual_buf,
+                         ar_column** out) {
+    ar_status st = check_desc(desc);
+    if (st != AR_OK) return st;
+    if (!out || (desc->major_bytes > 0 && !major_buf) || (desc->residual_bytes > 0 && !residual_buf)) {
+        set_error("ar_column_wrap: null buffer or output");
+        return AR_ERR_INVALID;
+    }
+    const uint32_t* res = nullptr;
+    st = device_alias(residual_buf, desc->residual_loc, &res);
+    if (st != AR_OK) return st;
+    ar_column* c = new (std::nothrow) ar_column;
+    if (!c) {
+        set_error("out of host memory");
+        return AR_ERR_RANGE;
+    }
+    c->d = *desc;
+    c->major = (const uint32_t*)major_buf;
+    c->residual = desc->k > 0 ? res : nullptr;
+    *out = c;
+    return AR_OK;
+}
+
+ar_status ar_decompose(const uint32_t* col, const ar_column_desc* desc, void* major_buf, uint64_t major_buf_bytes,
+                       void* residual_buf, uint64_t residual_buf_bytes, void* stream, ar_column** out) {
+    ar_status st = check_desc(desc);
+    if (st != AR_OK) return st;
+    if (!out || (desc->n > 0 && !col)) {
+        set_error("ar_decompose: null column or output handle");
+        return AR_ERR_INVALID;
+    }
+    if (major_buf_bytes < desc->major_bytes || residual_buf_bytes < desc->residual_bytes) {
+        set_error("ar_decompose: buffers (%llu, %llu bytes) smaller than planned (%llu, %llu)",
+                  (unsigned long long)major_buf_bytes, (unsigned long long)residual_buf_bytes,
+                  (unsigned long long)desc->major_bytes, (unsigned long long)desc->residual_bytes);
+        return AR_ERR_RANGE;
+    }
+    ar_column* c = nullptr;
+    st = ar_column_wrap(desc, major_buf, residual_buf, &c);
+    if (st != AR_OK) return st;
+    cudaStream_t s = (cudaStream_t)stream;
+    const int64_t n = desc->n;
+    const int w = desc->w_major, k = desc->k;
+    if (w > 0) {
+        if (desc->major_layout == AR_LAYOUT_SLICED)
+            st = launch_pack_sliced(col, n, k, desc->base, w, (uint32_t*)major_buf, s);
+        else
+            st = launch_pack_packed(col, n, k, 0xffffffffu, desc->base, w, desc->major_bytes / 4,
+                                    (uint32_t*)major_buf, s);
+    }
+    if (st == AR_OK && k > 0)
+        st = launch_pack_packed(col, n, 0, (1u << k) - 1u, desc->base, k, desc->residual_bytes / 4,
+                                const_cast<uint32_t*>(c->residual), s);
+    if (st != AR_OK) {
+        delete c;
+        return st;
+    }
+    *out = c;
+    return AR_OK;
+}
+
+ar_status ar_column_get_desc(const ar_column* col, ar_column_desc* desc) {
+    if (!col || !desc) {
+        set_error("ar_column_get_desc: null argument");
+        return AR_ERR_INVALID;
+    }
+    *desc = col->d;
+    return AR_OK;
+}
+
+void ar_column_free(ar_column* col) { delete col; }
+
+// ------------------------------------------------------------- a2 + a3
+
+size_t ar_select_ws_bytes(int64_t n) {
+    const uint64_t tiles = ceil_div_u64((uint64_t)std::max<int64_t>(n, 0), ard::kSelTileRows);
+    return 16 + 8 * tiles;
+}
+
+// Shared predicate setup of ar_approx_select / ar_select_refine_sum.
+static ar_status setup_scan(const ar_pred* preds, int32_t npred, ard::SelParams& P, bool& empty, int64_t& n) {
+    if (npred < 0 || npred > AR_MAX_PRED || (npred > 0 && !preds)) {
+        set_error("npred=%d outside [0,%d] or preds == NULL", npred, AR_MAX_PRED);
+        return AR_ERR_INVALID;
+    }
+    if (npred == 0) {
+        set_error("npred == 0: a scan needs at least one predicate column (use [0, 2^32-1] to keep all rows)");
+        return AR_ERR_INVALID;
+    }
+    memset(&P, 0, sizeof(P));
+    empty = false;
+    n = preds[0].col ? preds[0].col->d.n : -1;
+    uint32_t words = 0, ashift = 0;
+    for (int c = 0; c < npred; ++c) {
+        const ar_column* col = preds[c].col;
+        if (!valid_col(col) || col->d.n != n) {
+            set_error("predicate %d: null column or n differs from predicate 0", c);
+            return AR_ERR_INVALID;
+        }
+        if (col->d.major_layout != AR_LAYOUT_SLICED) {
+            set_error("predicate %d: the approximate scan needs AR_LAYOUT_SLICED majors", c);
+            return AR_ERR_INVALID;
+        }
+        const int w = col->d.w_major, k = col->d.k;
+        const Relaxed R = relax(preds[c].lo, preds[c].hi, col->d.base, k, w);
+        if (R.empty) empty = true;
+        ard::SelPred& p = P.p[c];
+        p.planes = col->major;
+        p.w = (uint32_t)w;
+        p.mode = k == 0 ? 0u : (R.def_any ? 1u : 2u);
+        p.clo = R.clo;
+        p.chi = R.chi;
+        p.dlo = R.dlo;
+        p.dhi = R.dhi;
+        p.soff = words;
+        p.ashift = ashift;
+        p.residual = col->residual;
+        p.k = (uint32_t)k;
+        p.base = col->d.base;
+        p.lo = preds[c].lo;
+        p.hi = preds[c].hi;
+        words += (uint32_t)(ard::kSelTileRows / 32) * (uint32_t)w;
+        ashift += (uint32_t)w;
+    }
+    uint32_t planes = 0;
+    for (int c = 0; c < npred; ++c) planes += P.p[c].w;
+    if (planes > AR_MAX_PLANES) {
+        set_error("sum of w_major over predicates = %u > AR_MAX_PLANES (%d)", planes, AR_MAX_PLANES);
+        return AR_ERR_UNSUPPORTED;
+    }
+    P.npred = npred;
+    P.n = n;
+    P.num_tiles = (int64_t)ceil_div_u64((uint64_t)n, ard::kSelTileRows);
+    P.stage_words = std::max<uint32_t>(words, 4);
+    return AR_OK;
+}
+
+ar_status ar_approx_select(const ar_pred* preds, int32_t npred, int32_t flags, ar_cands* out, void* ws,
+                           size_t ws_bytes, void* stream) {
+    ard::SelParams P;
+    bool empty = false;
+    int64_t n = 0;
+    ar_status st = setup_scan(preds, npred, P, empty, n);
+    if (st != AR_OK) return st;
+    if (!out || !out->pos || !out->aux || !out->count) {
+        set_error("ar_approx_select: null output buffer");
+        return AR_ERR_INVALID;
+    }
+    if (out->capacity < n) {
+        set_error("ar_approx_select: capacity %lld < n %lld", (long long)out->capacity, (long long)n);
+        return AR_ERR_RANGE;
+    }
+    if (!ws || ws_bytes < ar_select_ws_bytes(n)) {
+        set_error("ar_approx_select: workspace %zu < %zu bytes", ws_bytes, ar_select_ws_bytes(n));
+        return AR_ERR_RANGE;
+    }
+    const bool carry = (flags & AR_SELECT_CARRY_APPR) != 0;
+    uint32_t abits = 0;
+    for (int c = 0; c < npred; ++c) abits += P.p[c].w;
+    if (carry && abits > 31) {
+        set_error("AR_SELECT_CARRY_APPR: approximation tuple of %u bits does not fit aux bits 0..30", abits);
+        return AR_ERR_RANGE;
+    }
+    out->appr_bits = carry ? (int32_t)std::max<uint32_t>(abits, 1) : 0;
+    cudaStream_t s = (cudaStream_t)stream;
+    AR_TRY_CUDA(cudaMemsetAsync(out->count, 0, sizeof(int64_t), s));
+    if (empty || n == 0) return AR_OK;
+    AR_TRY_CUDA(cudaMemsetAsync(ws, 0, 16 + 8 * (size_t)P.num_tiles, s));
+    P.carry = carry ? 1 : 0;
+    P.out_pos = out->pos;
+    P.out_aux = out->aux;
+    P.out_count = (long long*)out->count;
+    P.ticket = (unsigned int*)ws;
+    P.status = (unsigned long long*)((char*)ws + 16);
+    int occ = 1;
+    P.nstages = pick_stages(P.stage_words, true, &occ);
+    const size_t smem = select_smem_bytes(P.stage_words, P.nstages, true);
+    const int grid = (int)std::min<int64_t>(P.num_tiles, (int64_t)num_sms() * occ);
+    return launch_select(P, grid, smem, s);
+}
+
+// ------------------------------------------------------------------ a5
+
+size_t ar_refine_ws_bytes(int64_t capacity) {
+    return 16 + 8 * ceil_div_u64((uint64_t)std::max<int64_t>(capacity, 0), ard::kRefTile);
+}
+
+static ar_status setup_refine(const ar_cands* in, const ar_pred* preds, int32_t npred, ard::RefParams& P) {
+    if (!in || !in->pos || !in->aux || !in->count || npred < 1 || npred > AR_MAX_PRED || !preds) {
+        set_error("refine: null candidates or bad predicate list (npred=%d)", npred);
+        return AR_ERR_INVALID;
+    }
+    memset(&P, 0, sizeof(P));
+    uint32_t ashift = 0, abits = 0;
+    for (int c = 0; c < npred; ++c) {
+        const ar_column* col = preds[c].col;
+        if (!valid_col(col)) {
+            set_error("refine: predicate %d has a null column", c);
+            return AR_ERR_INVALID;
+        }
+        ard::RefPred& p = P.p[c];
+        p.major = col->major;
+        p.residual = col->residual;
+        p.w = (uint32_t)col->d.w_major;
+        p.k = (uint32_t)col->d.k;
+        p.layout = (uint32_t)col->d.major_layout;
+        p.base = col->d.base;
+        p.lo = preds[c].lo;
+        p.hi = preds[c].hi;
+        p.ashift = ashift;
+        p.carried = in->appr_bits > 0 ? 1u : 0u;
+        p.check = col->d.k > 0 ? 1u : 0u;
+        ashift += p.w;
+        abits += p.w;
+    }
+    if (in->appr_bits > 0 && (uint32_t)std::max<uint32_t>(abits, 1) != (uint32_t)in->appr_bits) {
+        set_error("refine: predicates do not match the select that produced the candidates (%u vs %d bits)", abits,
+                  in->appr_bits);
+        return AR_ERR_INVALID;
+    }
+    P.npred = npred;
+    P.in_pos = in->pos;
+    P.in_aux = in->aux;
+    P.in_count = (const long long*)in->count;
+    return AR_OK;
+}
+
+ar_status ar_refine(const ar_cands* in, const ar_pred* preds, int32_t npred, ar_positions* out, void* ws,
+                    size_t ws_bytes, void* stream) {
+    ard::RefParams P;
+    ar_status st = setup_refine(in, preds, npred, P);
+    if (st != AR_OK) return st;
+    if (!out || !out->pos || !out->count) {
+        set_error("ar_refine: null output buffer");
+        return AR_ERR_INVALID;
+    }
+    if (out->capacity < in->capacity) {
+        set_error("ar_refine: output capacity %lld < candidate capacity %lld", (long long)out->capacity,
+                  (long long)in->capacity);
+        return AR_ERR_RANGE;
+    }
+    if (!ws || ws_bytes < ar_refine_ws_bytes(in->capacity)) {
+        set_error("ar_refine: workspace %zu < %zu bytes", ws_bytes, ar_refine_ws_bytes(in->capacity));
+        return AR_ERR_RANGE;
+    }
+    cudaStream_t s = (cudaStream_t)stream;
+    AR_TRY_CUDA(cudaMemsetAsync(out->count, 0, sizeof(int64_t), s));
+    const uint64_t max_tiles = ceil_div_u64((uint64_t)std::max<int64_t>(in->capacity, 0), ard::kRefTile);
+    if (max_tiles == 0) return AR_OK;
+    AR_TRY_CUDA(cudaMemsetAsync(ws, 0, 16 + 8 * max_tiles, s));
+    P.out_pos = out->pos;
+    P.out_count = (long long*)out->count;
+    P.ticket = (unsigned int*)ws;
+    P.status = (unsigned long long*)((char*)ws + 16);
+    const int grid = (int)std::min<uint64_t>(max_tiles, (uint64_t)num_sms() * 8);
+    return launch_refine(P, grid, s);
+}
+
+// ------------------------------------------------------------------ a6
+
+static ar_status setup_aggs(const ar_column* const* cols, int32_t ncols, const ar_pred* preds, int32_t npred,
+                            int64_t n, ard::AggCol* a, int32_t min_cols) {
+    if (ncols < min_cols || ncols > AR_MAX_AGG || (ncols > 0 && !cols)) {
+        set_error("sum: ncols=%d outside [%d,%d]", ncols, min_cols, AR_MAX_AGG);
+        return AR_ERR_INVALID;
+    }
+    uint32_t bits = 0;
+    for (int i = 0; i < ncols; ++i) {
+        const ar_column* c = cols[i];
+        if (!valid_col(c) || (n >= 0 && c->d.n != n)) {
+            set_error("sum: aggregate column %d is null or has n != %lld", i, (long long)n);
+            return AR_ERR_INVALID;
+        }
+        a[i].major = c->major;
+        a[i].residual = c->residual;
+        a[i].w = (uint32_t)c->d.w_major;
+        a[i].k = (uint32_t)c->d.k;
+        a[i].layout = (uint32_t)c->d.major_layout;
+        a[i].base = c->d.base;
+        a[i].pred = -1;
+        for (int p = 0; p < npred; ++p)
+            if (preds[p].col == c) { a[i].pred = p; break; }
+        uint32_t vb = (uint32_t)(c->d.w_major + c->d.k);
+        if (c->d.base) vb = 32;   // value may use every bit
+        bits += vb;
+    }
+    const int64_t rows = n >= 0 ? n : 1;
+    uint32_t lg = 0;
+    while (lg < 63 && ((int64_t)1 << lg) < rows) ++lg;
+    if (ncols > 0 && bits + lg > 63) {
+        set_error("sum: %u value bits + %u count bits > 63: the exact int64 sum could overflow", bits, lg);
+        return AR_ERR_RANGE;
+    }
+    return AR_OK;
+}
+
+ar_status ar_sum(const ar_positions* pos, const ar_column* const* cols, int32_t ncols, int64_t* out_sum_dev,
+                 void* stream) {
+    if (!pos || !pos->pos || !pos->count || !out_sum_dev) {
+        set_error("ar_sum: null argument");
+        return AR_ERR_INVALID;
+    }
+    ard::SumParams P;
+    memset(&P, 0, sizeof(P));
+    const int64_t n = (cols && ncols > 0 && cols[0]) ? cols[0]->d.n : -1;
+    ar_status st = setup_aggs(cols, ncols, nullptr, 0, n, P.a, 1);
+    if (st != AR_OK) return st;
+    P.pos = pos->pos;
+    P.count = (const long long*)pos->count;
+    P.nagg = ncols;
+    P.out_sum = (unsigned long long*)out_sum_dev;
+    cudaStream_t s = (cudaStream_t)stream;
+    AR_TRY_CUDA(cudaMemsetAsync(out_sum_dev, 0, sizeof(int64_t), s));
+    if (pos->capacity <= 0) return AR_OK;
+    const int grid = (int)std::min<int64_t>((pos->capacity + 255) / 256, (int64_t)num_sms() * 8);
+    return launch_sum(P, grid, s);
+}
+
+ar_status ar_refine_sum(const ar_cands* in, const ar_pred* preds, int32_t npred, const ar_column* const* cols,
+                        int32_t ncols, int64_t* out_sum_dev, int64_t* out_count_dev, void* stream) {
+    ard::RefParams P;
+    ar_status st = setup_refine(in, preds, npred, P);
+    if (st != AR_OK) return st;
+    st = setup_aggs(cols, ncols, preds, npred, preds[0].col->d.n, P.a, 0);
+    if (st != AR_OK) return st;
+    P.nagg = ncols;
+    P.out_sum = (unsigned long long*)out_sum_dev;
+    P.out_cnt = (unsigned long long*)out_count_dev;
+    cudaStream_t s = (cudaStream_t)stream;
+    if (out_sum_dev) AR_TRY_CUDA(cudaMemsetAsync(out_sum_dev, 0, sizeof(int64_t), s));
+    if (out_count_dev) AR_TRY_CUDA(cudaMemsetAsync(out_count_dev, 0, sizeof(int64_t), s));
+    const uint64_t max_tiles = ceil_div_u64((uint64_t)std::max<int64_t>(in->capacity, 0), ard::kRefTile);
+    if (max_tiles == 0) return AR_OK;
+    const int grid = (int)std::min<uint64_t>(max_tiles, (uint64_t)num_sms() * 8);
+    return launch_refine_sum(P, grid, s);
+}
+
+// ----------------------------------------------------------- fused a3+a5+a6
+
+ar_status ar_select_refine_sum(const ar_pred* preds, int32_t npred, const ar_column* const* cols, int32_t ncols,
+                               int64_t* out_dev, void* stream) {
+    ard::SelParams P;
+    bool empty = false;
+    int64_t n = 0;
+    ar_status st = setup_scan(preds, npred, P, empty, n);
+    if (st != AR_OK) return st;
+    if (!out_dev) {
+        set_error("ar_select_refine_sum: null output");
+        return AR_ERR_INVALID;
+    }
+    st = setup_aggs(cols, ncols, preds, npred, n, P.a, 0);
+    if (st != AR_OK) return st;
+    P.nagg = ncols;
+    P.out4 = (unsigned long long*)out_dev;
+    cudaStream_t s = (cudaStream_t)stream;
+    AR_TRY_CUDA(cudaMemsetAsync(out_dev, 0, 4 * sizeof(int64_t), s));
+    if (empty || n == 0) return AR_OK;
+    int occ = 1;
+    P.nstages = pick_stages(P.stage_words, false, &occ);
+    const size_t smem = select_smem_bytes(P.stage_words, P.nstages, false);
+    const int grid = (int)std::min<int64_t>(P.num_tiles, (int64_t)num_sms() * occ);
+    return launch_fused(P, grid, smem, s);
+}
+
+}  // extern "C"

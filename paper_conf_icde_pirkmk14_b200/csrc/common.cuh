@@ -1,0 +1,240 @@
+// common.cuh -- shared internals of the A&R CUDA library (sm_100a).
+// Column handle, host error plumbing, device bit-extraction / gather helpers,
+// mbarrier + cp.async.bulk (TMA bulk copy) PTX wrappers, decoupled look-back.
+#pragma once
+
+#include <cuda_runtime.h>
+#include <stdint.h>
+#include <stdio.h>
+#include <stdarg.h>
+#include <string>
+#include <algorithm>
+
+#include "../../include/ar.h"
+
+struct ar_column {
+    ar_column_desc d;
+    const uint32_t* major;      // device pointer (SLICED or PACKED, width d.w_major)
+    const uint32_t* residual;   // device pointer, or device alias of pinned host memory (PACKED, width d.k)
+};
+
+// ------------------------------------------------------------------ host side
+
+namespace ar {
+
+void set_error(const char* fmt, ...);
+ar_status cuda_fail(cudaError_t e, const char* where);
+int num_sms();
+
+inline uint64_t ceil_div_u64(uint64_t a, uint64_t b) { return (a + b - 1) / b; }
+
+// Bytes of a SLICED major part: blocks of 32 rows, padded to 128-row groups so
+// that every 4096-row tile (and every 128-row shard boundary) is 16-B aligned.
+inline uint64_t sliced_bytes(int64_t n, int w) {
+    return w == 0 ? 0 : ceil_div_u64((uint64_t)n, 128) * 16ull * (uint64_t)w;
+}
+// Bytes of a PACKED bitstream of width w: ceil(n*w/32) words + 1 guard word
+// (a straddling value may read word i+1), rounded up to 16 B.
+inline uint64_t packed_bytes(int64_t n, int w) {
+    if (w == 0) return 0;
+    uint64_t words = ceil_div_u64((uint64_t)n * (uint64_t)w, 32) + 1;
+    return ceil_div_u64(words * 4, 16) * 16;
+}
+
+// Relaxation of one exact conjunct [lo, hi] to the major domain (step a2).
+// Tight reading (DESIGN "Readings"):
+//   u = v - base;  cand(m) <=> [m 2^k, m 2^k + 2^k - 1] meets [ulo, uhi]
+//                  def(m)  <=> [m 2^k, m 2^k + 2^k - 1] inside [ulo, uhi]
+struct Relaxed {
+    bool empty;          // no row can qualify
+    uint32_t clo, chi;   // candidate major range (inclusive, <= 2^w - 1)
+    bool def_any;        // definite range non-empty
+    uint32_t dlo, dhi;   // definite major range
+};
+Relaxed relax(uint32_t lo, uint32_t hi, uint32_t base, int k, int w);
+
+}  // namespace ar
+
+#define AR_TRY_CUDA(expr)                                         \
+    do {                                                          \
+        cudaError_t _e = (expr);                                  \
+        if (_e != cudaSuccess) return ar::cuda_fail(_e, #expr);   \
+    } while (0)
+
+#define AR_CHECK_LAUNCH(name)                                     \
+    do {                                                          \
+        cudaError_t _e = cudaGetLastError();                      \
+        if (_e != cudaSuccess) return ar::cuda_fail(_e, name);    \
+    } while (0)
+
+// ---------------------------------------------------------------- device side
+
+namespace ard {
+
+__device__ __forceinline__ uint32_t smem_u32(const void* p) {
+    return static_cast<uint32_t>(__cvta_generic_to_shared(p));
+}
+
+// --- mbarrier (Hopper+) -------------------------------------------------------
+__device__ __forceinline__ void mbar_init(uint64_t* bar, uint32_t count) {
+    asm volatile("mbarrier.init.shared::cta.b64 [%0], %1;" ::"r"(smem_u32(bar)), "r"(count) : "memory");
+}
+__device__ __forceinline__ void fence_mbar_init() {
+    asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+}
+__device__ __forceinline__ void mbar_arrive_expect_tx(uint64_t* bar, uint32_t bytes) {
+    asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(smem_u32(bar)), "r"(bytes)
+                 : "memory");
+}
+__device__ __forceinline__ void mbar_arrive(uint64_t* bar) {
+    asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(smem_u32(bar)) : "memory");
+}
+__device__ __forceinline__ void mbar_wait(uint64_t* bar, uint32_t parity) {
+    asm volatile(
+        "{\n\t.reg .pred p;\n"
+        "AR_WAIT_%=:\n\t"
+        "mbarrier.try_wait.parity.shared::cta.b64 p, [%0], %1;\n\t"
+        "@!p bra AR_WAIT_%=;\n}" ::"r"(smem_u32(bar)),
+        "r"(parity)
+        : "memory");
+}
+
+// --- TMA bulk copy global -> shared (1-D, no tensor map), completes on an mbarrier
+__device__ __forceinline__ void bulk_g2s(void* dst, const void* src, uint32_t bytes, uint64_t* bar,
+                                         uint64_t policy) {
+    asm volatile(
+        "cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes.L2::cache_hint [%0], [%1], %2, [%3], %4;" ::
+            "r"(smem_u32(dst)),
+        "l"(src), "r"(bytes), "r"(smem_u32(bar)), "l"(policy)
+        : "memory");
+}
+__device__ __forceinline__ uint64_t policy_evict_first() {
+    uint64_t p;
+    asm volatile("createpolicy.fractional.L2::evict_first.b64 %0, 1.0;" : "=l"(p));
+    return p;
+}
+
+// --- named barrier among the consumer warps only (id 1; id 0 is __syncthreads)
+__device__ __forceinline__ void bar_sync(uint32_t id, uint32_t nthreads) {
+    asm volatile("bar.sync %0, %1;" ::"r"(id), "r"(nthreads) : "memory");
+}
+
+// --- relaxed / acquire-release 64-bit status words for decoupled look-back
+__device__ __forceinline__ void st_release(unsigned long long* p, unsigned long long v) {
+    asm volatile("st.release.gpu.global.u64 [%0], %1;" ::"l"(p), "l"(v) : "memory");
+}
+__device__ __forceinline__ unsigned long long ld_acquire(const unsigned long long* p) {
+    unsigned long long v;
+    asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+    return v;
+}
+
+constexpr unsigned long long kFlagAgg = 1ull << 62;
+constexpr unsigned long long kFlagPrefix = 2ull << 62;
+constexpr unsigned long long kValueMask = (1ull << 62) - 1;
+
+// Decoupled look-back (Merrill & Garland 2016), run by one full warp for tile
+// `t` (t > 0) whose aggregate is already published: returns the exclusive
+// prefix of all tiles < t.  Lane i inspects tile (t-1-i) of each 32-tile window.
+__device__ __forceinline__ unsigned long long lookback(const unsigned long long* status, long long t,
+                                                       unsigned lane) {
+    unsigned long long excl = 0;
+    long long base = t - 1;
+    while (true) {
+        long long idx = base - (long long)lane;
+        unsigned long long s;
+        while (true) {
+            s = idx >= 0 ? ld_acquire(status + idx) : kFlagPrefix;  // before tile 0: prefix 0
+            if (__all_sync(0xffffffffu, (s >> 62) != 0)) break;
+        }
+        unsigned prefix_lanes = __ballot_sync(0xffffffffu, (s >> 62) == 2);
+        unsigned long long v = s & kValueMask;
+        if (prefix_lanes) {
+            unsigned first = __ffs(prefix_lanes) - 1;   // nearest tile holding an inclusive prefix
+            if (lane > first) v = 0;
+            for (int o = 16; o > 0; o >>= 1) v += __shfl_xor_sync(0xffffffffu, v, o);
+            return excl + v;
+        }
+        for (int o = 16; o > 0; o >>= 1) v += __shfl_xor_sync(0xffffffffu, v, o);
+        excl += v;
+        base -= 32;
+    }
+}
+
+// --- value extraction ----------------------------------------------------------
+
+// Value of row p from a PACKED LSB-first bitstream of width w (1..32).
+__device__ __forceinline__ uint32_t packed_get(const uint32_t* __restrict__ s, uint64_t p, int w) {
+    uint64_t bit = p * (uint64_t)w;
+    uint64_t wi = bit >> 5;
+    uint32_t sh = (uint32_t)(bit & 31);
+    uint32_t lo = __ldg(s + wi);
+    uint32_t v = lo >> sh;
+    if (sh + (uint32_t)w > 32u) v = __funnelshift_r(lo, __ldg(s + wi + 1), sh);
+    return w == 32 ? v : (v & ((1u << w) - 1u));
+}
+// Same, for residuals that may live in pinned host memory (no read-only cache path assumption).
+__device__ __forceinline__ uint32_t packed_get_any(const uint32_t* s, uint64_t p, int w) {
+    uint64_t bit = p * (uint64_t)w;
+    uint64_t wi = bit >> 5;
+    uint32_t sh = (uint32_t)(bit & 31);
+    uint32_t lo = s[wi];
+    uint32_t v = lo >> sh;
+    if (sh + (uint32_t)w > 32u) v = __funnelshift_r(lo, s[wi + 1], sh);
+    return w == 32 ? v : (v & ((1u << w) - 1u));
+}
+
+// Major of row p from a SLICED part of width w (w words per 32-row block).
+__device__ __forceinline__ uint32_t sliced_get(const uint32_t* __restrict__ s, uint64_t p, int w) {
+    const uint32_t* blk = s + (p >> 5) * (uint64_t)w;
+    uint32_t l = (uint32_t)(p & 31);
+    uint32_t m = 0;
+    for (int j = 0; j < w; ++j) m |= ((__ldg(blk + j) >> l) & 1u) << j;
+    return m;
+}
+
+__device__ __forceinline__ uint32_t major_get(const uint32_t* __restrict__ s, uint64_t p, int w, int layout) {
+    if (w == 0) return 0;
+    return layout == AR_LAYOUT_SLICED ? sliced_get(s, p, w) : packed_get(s, p, w);
+}
+
+// Exact value of row p of a column (major and residual joined).
+__device__ __forceinline__ uint32_t value_get(const uint32_t* major, const uint32_t* residual, uint64_t p,
+                                              int w, int k, int layout, uint32_t base) {
+    uint32_t m = major_get(major, p, w, layout);
+    uint32_t r = k ? packed_get_any(residual, p, k) : 0u;
+    uint32_t u = k == 32 ? r : ((m << k) | r);
+    return u + base;
+}
+
+// Valid-row mask of the 32-row block starting at row r0 of an n-row column.
+__device__ __forceinline__ uint32_t valid_mask(int64_t r0, int64_t n) {
+    int64_t rem = n - r0;
+    return rem >= 32 ? 0xffffffffu : (rem <= 0 ? 0u : ((1u << rem) - 1u));
+}
+
+// Block-wide exclusive scan of one uint32 per thread over NT threads (consumer
+// warps only, named barrier `bar`).  `warp_tot` is smem of NT/32 words.
+template <int NT>
+__device__ __forceinline__ uint32_t block_excl_scan(uint32_t x, uint32_t* warp_tot, uint32_t& total, uint32_t bar) {
+    const unsigned lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+    uint32_t incl = x;
+#pragma unroll
+    for (int o = 1; o < 32; o <<= 1) {
+        uint32_t y = __shfl_up_sync(0xffffffffu, incl, o);
+        if (lane >= (unsigned)o) incl += y;
+    }
+    if (lane == 31) warp_tot[warp] = incl;
+    bar_sync(bar, NT);
+    uint32_t before = 0, all = 0;
+#pragma unroll
+    for (int i = 0; i < NT / 32; ++i) {
+        uint32_t t = warp_tot[i];
+        before += (i < (int)warp) ? t : 0u;
+        all += t;
+    }
+    total = all;
+    return before + incl - x;
+}
+
+}  // namespace ard

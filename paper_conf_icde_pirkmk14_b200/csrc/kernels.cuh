@@ -1,0 +1,107 @@
+// kernels.cuh -- parameter blocks and launchers shared by api.cu and the kernel files.
+#pragma once
+#include "common.cuh"
+
+namespace ard {
+
+// Approximate-select predicate, already relaxed to the major domain (step a2).
+struct SelPred {
+    const uint32_t* planes;   // SLICED major part (device)
+    uint32_t w;               // planes per 32-row block (w_major)
+    uint32_t mode;            // 0: k == 0 (def == cand); 1: approximate with a definite range; 2: no definite range
+    uint32_t clo, chi;        // candidate major range
+    uint32_t dlo, dhi;        // definite major range (mode 1)
+    uint32_t soff;            // word offset of this predicate's planes inside one pipeline stage
+    uint32_t ashift;          // bit offset of this major inside the approximation word
+    // refine-side data, used by the fused kernel
+    const uint32_t* residual; // PACKED width k (device or host-mapped), null if k == 0
+    uint32_t k, base, lo, hi; // exact predicate on v = ((m << k) | r) + base
+};
+
+// Aggregate factor of the SUM product.
+struct AggCol {
+    const uint32_t* major;
+    const uint32_t* residual;
+    uint32_t w, k, layout, base;
+    int32_t pred;             // index of the predicate over the same column, or -1
+};
+
+constexpr int kSelWarps = 4;                      // consumer warps per CTA
+constexpr int kSelThreads = kSelWarps * 32;       // one 32-row block per consumer thread
+constexpr int kSelTileRows = kSelThreads * 32;    // 4096 rows per tile
+
+struct SelParams {
+    SelPred p[AR_MAX_PRED];
+    int32_t npred;
+    int32_t carry;            // write the approximation word into aux
+    int64_t n;
+    int64_t num_tiles;
+    uint32_t stage_words;     // uint32 words per pipeline stage (all predicates)
+    uint32_t nstages;
+    uint32_t* out_pos;
+    uint32_t* out_aux;
+    long long* out_count;
+    unsigned long long* status;   // [num_tiles] look-back words
+    unsigned int* ticket;         // dynamic tile counter
+    // fused kernel only
+    AggCol a[AR_MAX_AGG];
+    int32_t nagg;
+    unsigned long long* out4;     // sum, |result|, |cand|, |def|
+};
+
+struct RefPred {
+    const uint32_t* major;
+    const uint32_t* residual;
+    uint32_t w, k, layout, base, lo, hi;
+    uint32_t ashift;
+    uint32_t carried;         // major available in aux
+    uint32_t check;           // k > 0: must be re-evaluated on the exact value
+};
+
+constexpr int kRefThreads = 256;
+constexpr int kRefPerThread = 8;
+constexpr int kRefTile = kRefThreads * kRefPerThread;   // 2048 candidates per tile
+
+struct RefParams {
+    RefPred p[AR_MAX_PRED];
+    int32_t npred;
+    const uint32_t* in_pos;
+    const uint32_t* in_aux;
+    const long long* in_count;
+    uint32_t* out_pos;
+    long long* out_count;
+    unsigned long long* status;
+    unsigned int* ticket;
+    AggCol a[AR_MAX_AGG];
+    int32_t nagg;
+    unsigned long long* out_sum;
+    unsigned long long* out_cnt;
+};
+
+struct SumParams {
+    const uint32_t* pos;
+    const long long* count;
+    AggCol a[AR_MAX_AGG];
+    int32_t nagg;
+    unsigned long long* out_sum;
+};
+
+}  // namespace ard
+
+namespace ar {
+// launchers (return AR_OK or the CUDA failure)
+size_t select_smem_bytes(uint32_t stage_words, uint32_t nstages, bool staging);
+ar_status launch_select(const ard::SelParams& P, int grid, size_t smem, cudaStream_t s);
+ar_status launch_fused(const ard::SelParams& P, int grid, size_t smem, cudaStream_t s);
+ar_status launch_refine(const ard::RefParams& P, int grid, cudaStream_t s);
+ar_status launch_refine_sum(const ard::RefParams& P, int grid, cudaStream_t s);
+ar_status launch_sum(const ard::SumParams& P, int grid, cudaStream_t s);
+ar_status launch_decompose_max(const uint32_t* col, int64_t n, uint32_t base, uint32_t* out_max, cudaStream_t s);
+ar_status launch_pack_sliced(const uint32_t* col, int64_t n, int k, uint32_t base, int w, uint32_t* out,
+                             cudaStream_t s);
+ar_status launch_pack_packed(const uint32_t* col, int64_t n, int shift, uint32_t mask, uint32_t base, int w,
+                             uint64_t out_words, uint32_t* out, cudaStream_t s);
+ar_status launch_exclusive_offset(const long long* all_counts, int world, int rank, long long* out,
+                                  cudaStream_t s);
+int select_occupancy(size_t smem, bool fused);
+}  // namespace ar

@@ -1,0 +1,196 @@
+// refine.cu -- step a5 (selection refinement, Algorithm 2)
+// and step a6 (SUM over exact values).
+//
+// The candidate list is ascending (stable compaction in a3), so the join with
+// the residual is a positional ("invisible") lookup: each
+// candidate's residual is gathered at its row position, from HBM or, for
+// host-resident residuals, straight over the host link through a mapped
+// pointer.  Each thread owns 8 consecutive candidates (two 16-B loads of
+// positions and of aux words), so its residual gathers are independent loads
+// in flight together.  Refine keeps order with the same decoupled look-back
+// as a3; refine+SUM needs no order (integer sums are exact in any order).
+#include "kernels.cuh"
+
+namespace ard {
+
+// Exact re-evaluation of a non-definite candidate (Alg. 2: join with the
+// residual, "+bw" concatenation, CONDITION).
+__device__ __forceinline__ bool refine_keep(const RefParams& P, uint32_t pos, uint32_t aux) {
+    if (aux & AR_AUX_DEFINITE) return true;
+    bool ok = true;
+    for (int c = 0; c < P.npred; ++c) {
+        const RefPred& p = P.p[c];
+        if (!p.check) continue;
+        const uint32_t m = p.carried ? ((aux >> p.ashift) & (p.w == 32 ? 0xffffffffu : ((1u << p.w) - 1u)))
+                                     : major_get(p.major, pos, p.w, p.layout);
+        const uint32_t r = packed_get_any(p.residual, pos, p.k);
+        const uint32_t v = ((m << p.k) | r) + p.base;
+        ok = ok && (v >= p.lo) && (v <= p.hi);
+    }
+    return ok;
+}
+
+__device__ __forceinline__ uint32_t agg_value_at(const RefParams& P, const AggCol& a, uint32_t pos, uint32_t aux) {
+    if (a.pred >= 0 && P.p[a.pred].carried) {
+        const RefPred& p = P.p[a.pred];
+        const uint32_t m = (aux >> p.ashift) & (p.w == 32 ? 0xffffffffu : ((1u << p.w) - 1u));
+        const uint32_t r = a.k ? packed_get_any(a.residual, pos, a.k) : 0u;
+        return ((m << a.k) | r) + a.base;
+    }
+    return value_get(a.major, a.residual, pos, a.w, a.k, a.layout, a.base);
+}
+
+__device__ __forceinline__ void load8(const uint32_t* base, uint64_t j0, long long count, uint32_t (&v)[8]) {
+    if (j0 + 8 <= (uint64_t)count) {
+        const uint4 a = *reinterpret_cast<const uint4*>(base + j0);
+        const uint4 b = *reinterpret_cast<const uint4*>(base + j0 + 4);
+        v[0] = a.x; v[1] = a.y; v[2] = a.z; v[3] = a.w;
+        v[4] = b.x; v[5] = b.y; v[6] = b.z; v[7] = b.w;
+    } else {
+#pragma unroll
+        for (int i = 0; i < 8; ++i) v[i] = (j0 + i < (uint64_t)count) ? base[j0 + i] : 0u;
+    }
+}
+
+__global__ void __launch_bounds__(kRefThreads) refine_kernel(const __grid_constant__ RefParams P) {
+    __shared__ uint32_t st_pos[kRefTile];
+    __shared__ uint32_t warp_tot[kRefThreads / 32];
+    __shared__ long long s_tile;
+    __shared__ unsigned long long s_off;
+    const unsigned warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    const long long count = *P.in_count;
+    const long long num_tiles = (count + kRefTile - 1) / kRefTile;
+
+    while (true) {
+        if (threadIdx.x == 0) s_tile = (long long)atomicAdd(P.ticket, 1u);
+        __syncthreads();
+        const long long t = s_tile;
+        if (t >= num_tiles) break;
+        const uint64_t j0 = (uint64_t)t * kRefTile + threadIdx.x * kRefPerThread;
+        uint32_t pos[8], aux[8];
+        load8(P.in_pos, j0, count, pos);
+        load8(P.in_aux, j0, count, aux);
+        uint32_t keep = 0;
+#pragma unroll
+        for (int i = 0; i < 8; ++i)
+            if (j0 + i < (uint64_t)count && refine_keep(P, pos[i], aux[i])) keep |= 1u << i;
+
+        const uint32_t cnt = __popc(keep);
+        uint32_t total;
+        const uint32_t excl = block_excl_scan<kRefThreads>(cnt, warp_tot, total, 1);
+        if (warp == 0) {
+            unsigned long long prefix = 0;
+            if (t == 0) {
+                if (lane == 0) st_release(P.status, kFlagPrefix | total);
+            } else {
+                if (lane == 0) st_release(P.status + t, kFlagAgg | total);
+                prefix = lookback(P.status, t, lane);
+                if (lane == 0) st_release(P.status + t, kFlagPrefix | (prefix + total));
+            }
+            if (lane == 0) {
+                s_off = prefix;
+                if (t == num_tiles - 1) *P.out_count = (long long)(prefix + total);
+            }
+        }
+        uint32_t o = excl;
+#pragma unroll
+        for (int i = 0; i < 8; ++i)
+            if (keep & (1u << i)) st_pos[o++] = pos[i];
+        __syncthreads();
+        const unsigned long long off = s_off;
+        for (uint32_t j = threadIdx.x; j < total; j += kRefThreads) P.out_pos[off + j] = st_pos[j];
+        __syncthreads();
+    }
+}
+
+template <typename T>
+__device__ __forceinline__ void block_add(T v, unsigned long long* out) {
+    __shared__ unsigned long long red[32];
+    unsigned long long x = (unsigned long long)v;
+#pragma unroll
+    for (int o = 16; o > 0; o >>= 1) x += __shfl_xor_sync(0xffffffffu, x, o);
+    const unsigned warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    __syncthreads();
+    if (lane == 0) red[warp] = x;
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        unsigned long long s = 0;
+        for (unsigned i = 0; i < (blockDim.x + 31) / 32; ++i) s += red[i];
+        if (s) atomicAdd(out, s);
+    }
+}
+
+__global__ void __launch_bounds__(kRefThreads) refine_sum_kernel(const __grid_constant__ RefParams P) {
+    const long long count = *P.in_count;
+    const long long num_tiles = (count + kRefTile - 1) / kRefTile;
+    unsigned long long sum = 0, kept = 0;
+    for (long long t = blockIdx.x; t < num_tiles; t += gridDim.x) {
+        const uint64_t j0 = (uint64_t)t * kRefTile + threadIdx.x * kRefPerThread;
+        uint32_t pos[8], aux[8];
+        load8(P.in_pos, j0, count, pos);
+        load8(P.in_aux, j0, count, aux);
+#pragma unroll
+        for (int i = 0; i < 8; ++i) {
+            if (j0 + i < (uint64_t)count && refine_keep(P, pos[i], aux[i])) {
+                ++kept;
+                if (P.nagg > 0) {
+                    unsigned long long prod = agg_value_at(P, P.a[0], pos[i], aux[i]);
+                    if (P.nagg > 1) prod *= agg_value_at(P, P.a[1], pos[i], aux[i]);
+                    sum += prod;
+                }
+            }
+        }
+    }
+    if (P.out_sum) block_add(sum, P.out_sum);
+    if (P.out_cnt) block_add(kept, P.out_cnt);
+}
+
+__global__ void __launch_bounds__(kRefThreads) sum_kernel(const __grid_constant__ SumParams P) {
+    const long long count = *P.count;
+    unsigned long long sum = 0;
+    const long long stride = (long long)gridDim.x * kRefThreads;
+    for (long long j = (long long)blockIdx.x * kRefThreads + threadIdx.x; j < count; j += stride) {
+        const uint32_t pos = P.pos[j];
+        unsigned long long prod = 1;
+        for (int c = 0; c < P.nagg; ++c) {
+            const AggCol& a = P.a[c];
+            prod *= value_get(a.major, a.residual, pos, a.w, a.k, a.layout, a.base);
+        }
+        sum += prod;
+    }
+    block_add(sum, P.out_sum);
+}
+
+__global__ void exclusive_offset_kernel(const long long* all, int world, int rank, long long* out) {
+    long long s = 0;
+    for (int r = 0; r < rank && r < world; ++r) s += all[r];
+    *out = s;
+}
+
+}  // namespace ard
+
+namespace ar {
+
+ar_status launch_refine(const ard::RefParams& P, int grid, cudaStream_t s) {
+    ard::refine_kernel<<<grid, ard::kRefThreads, 0, s>>>(P);
+    AR_CHECK_LAUNCH("refine_kernel");
+    return AR_OK;
+}
+ar_status launch_refine_sum(const ard::RefParams& P, int grid, cudaStream_t s) {
+    ard::refine_sum_kernel<<<grid, ard::kRefThreads, 0, s>>>(P);
+    AR_CHECK_LAUNCH("refine_sum_kernel");
+    return AR_OK;
+}
+ar_status launch_sum(const ard::SumParams& P, int grid, cudaStream_t s) {
+    ard::sum_kernel<<<grid, ard::kRefThreads, 0, s>>>(P);
+    AR_CHECK_LAUNCH("sum_kernel");
+    return AR_OK;
+}
+ar_status launch_exclusive_offset(const long long* all_counts, int world, int rank, long long* out,
+                                  cudaStream_t s) {
+    ard::exclusive_offset_kernel<<<1, 1, 0, s>>>(all_counts, world, rank, out);
+    AR_CHECK_LAUNCH("exclusive_offset_kernel");
+    return AR_OK;
+}
+
+}  // namespace ar
