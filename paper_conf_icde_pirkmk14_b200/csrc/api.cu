@@ -69,38 +69,51 @@ Relaxed relax(uint32_t lo, uint32_t hi, uint32_t base, int k, int w) {
 
 static bool valid_col(const ar_column* c) { return c && (c->d.w_major == 0 || c->major); }
 
-// Rough pipeline sizing: aim for ~3 CTAs per SM and >= 3 stages each.
-static uint32_t pick_stages_uncached(uint32_t stage_words, bool staging, int* ctas_per_sm) {
-    uint32_t best = 2;
-    int best_occ = 0;
-    for (uint32_t st = 8; st >= 2; --st) {
-        const size_t smem = select_smem_bytes(stage_words, st, staging);
-        if (smem > 227 * 1024) continue;
-        const int occ = select_occupancy(smem, !staging);
-        // bytes in flight per SM ~ occ * (st - 1) * stage bytes; prefer more CTAs at similar depth
-        if (occ <= 0) continue;
-        if (occ * (int)(st - 1) > best_occ * (int)(best - 1) || best_occ == 0) {
-            best_occ = occ;
-            best = st;
-        }
-        if (occ >= 3 && st >= 3) break;
-    }
-    if (ctas_per_sm) *ctas_per_sm = best_occ > 0 ? best_occ : 1;
-    return best;
+// Tuning knobs (read once): AR_STAGES (pipeline stages), AR_CTAS (CTAs per SM).
+static int env_int(const char* name, int dflt) {
+    const char* v = getenv(name);
+    return (v && *v) ? atoi(v) : dflt;
+}
+static int knob(int which) {
+    static int vals[2] = {-2, -2};
+    static const char* names[2] = {"AR_STAGES", "AR_CTAS"};
+    if (vals[which] == -2) vals[which] = env_int(names[which], 0);
+    return vals[which];
 }
 
-// Memoised per (stage_words, staging): the occupancy queries stay out of the launch path.
-static uint32_t pick_stages(uint32_t stage_words, bool staging, int* ctas_per_sm) {
-    struct Entry { uint32_t words; bool staging; uint32_t stages; int occ; };
-    static thread_local Entry cache[16];
+// Pipeline sizing: the most CTAs per SM (up to 4) that still allow >= 3 stages
+// (>= 2 at one CTA per SM), and for that occupancy the deepest ring (<= 8 stages).
+static uint32_t pick_stages_uncached(const void* fn, uint32_t stage_words, bool fused, int* ctas_per_sm) {
+    const int force_st = knob(0), force_occ = knob(1);
+    for (int occ_target = force_occ > 0 ? force_occ : 4; occ_target >= 1; --occ_target) {
+        for (int st = 8; st >= 2; --st) {
+            if (force_st > 0 && st != force_st) continue;
+            const size_t smem = select_smem_bytes(stage_words, (uint32_t)st, !fused);
+            if (smem > 227 * 1024) continue;
+            const int occ = select_occupancy(fn, smem, fused);
+            if (occ >= occ_target && (st >= 3 || occ_target == 1 || force_st > 0)) {
+                *ctas_per_sm = occ_target;
+                return (uint32_t)st;
+            }
+        }
+        if (force_occ > 0) break;
+    }
+    *ctas_per_sm = 1;
+    return 2;
+}
+
+// Memoised per (kernel, stage_words): the occupancy queries stay out of the launch path.
+static uint32_t pick_stages(const void* fn, uint32_t stage_words, bool fused, int* ctas_per_sm) {
+    struct Entry { const void* fn; uint32_t words; uint32_t stages; int occ; };
+    static thread_local Entry cache[32];
     static thread_local int used = 0;
     for (int i = 0; i < used; ++i)
-        if (cache[i].words == stage_words && cache[i].staging == staging) {
+        if (cache[i].fn == fn && cache[i].words == stage_words) {
             *ctas_per_sm = cache[i].occ;
             return cache[i].stages;
         }
-    const uint32_t st = pick_stages_uncached(stage_words, staging, ctas_per_sm);
-    if (used < 16) cache[used++] = Entry{stage_words, staging, st, *ctas_per_sm};
+    const uint32_t st = pick_stages_uncached(fn, stage_words, fused, ctas_per_sm);
+    if (used < 32) cache[used++] = Entry{fn, stage_words, st, *ctas_per_sm};
     return st;
 }
 
@@ -277,12 +290,13 @@ void ar_column_free(ar_column* col) { delete col; }
 // ------------------------------------------------------------- a2 + a3
 
 size_t ar_select_ws_bytes(int64_t n) {
-    const uint64_t tiles = ceil_div_u64((uint64_t)std::max<int64_t>(n, 0), ard::kSelTileRows);
+    const uint64_t tiles = ceil_div_u64((uint64_t)std::max<int64_t>(n, 0), ard::kSelMinTileRows);
     return 16 + 8 * tiles;
 }
 
 // Shared predicate setup of ar_approx_select / ar_select_refine_sum.
-static ar_status setup_scan(const ar_pred* preds, int32_t npred, ard::SelParams& P, bool& empty, int64_t& n) {
+static ar_status setup_scan(const ar_pred* preds, int32_t npred, ard::SelParams& P, bool& empty, int64_t& n,
+                            bool fused) {
     if (npred < 0 || npred > AR_MAX_PRED || (npred > 0 && !preds)) {
         set_error("npred=%d outside [0,%d] or preds == NULL", npred, AR_MAX_PRED);
         return AR_ERR_INVALID;
@@ -294,6 +308,8 @@ static ar_status setup_scan(const ar_pred* preds, int32_t npred, ard::SelParams&
     memset(&P, 0, sizeof(P));
     empty = false;
     n = preds[0].col ? preds[0].col->d.n : -1;
+    P.bpt = (uint32_t)kernel_bpt(fused);
+    P.tile_rows = (uint32_t)kernel_warps(fused) * 32u * 32u * P.bpt;
     uint32_t words = 0, ashift = 0;
     for (int c = 0; c < npred; ++c) {
         const ar_column* col = preds[c].col;
@@ -323,7 +339,7 @@ static ar_status setup_scan(const ar_pred* preds, int32_t npred, ard::SelParams&
         p.base = col->d.base;
         p.lo = preds[c].lo;
         p.hi = preds[c].hi;
-        words += (uint32_t)(ard::kSelTileRows / 32) * (uint32_t)w;
+        words += (P.tile_rows / 32) * (uint32_t)w;
         ashift += (uint32_t)w;
     }
     uint32_t planes = 0;
@@ -334,7 +350,7 @@ static ar_status setup_scan(const ar_pred* preds, int32_t npred, ard::SelParams&
     }
     P.npred = npred;
     P.n = n;
-    P.num_tiles = (int64_t)ceil_div_u64((uint64_t)n, ard::kSelTileRows);
+    P.num_tiles = (int64_t)ceil_div_u64((uint64_t)n, P.tile_rows);
     P.stage_words = std::max<uint32_t>(words, 4);
     return AR_OK;
 }
@@ -344,7 +360,7 @@ ar_status ar_approx_select(const ar_pred* preds, int32_t npred, int32_t flags, a
     ard::SelParams P;
     bool empty = false;
     int64_t n = 0;
-    ar_status st = setup_scan(preds, npred, P, empty, n);
+    ar_status st = setup_scan(preds, npred, P, empty, n, false);
     if (st != AR_OK) return st;
     if (!out || !out->pos || !out->aux || !out->count) {
         set_error("ar_approx_select: null output buffer");
@@ -377,10 +393,11 @@ ar_status ar_approx_select(const ar_pred* preds, int32_t npred, int32_t flags, a
     P.ticket = (unsigned int*)ws;
     P.status = (unsigned long long*)((char*)ws + 16);
     int occ = 1;
-    P.nstages = pick_stages(P.stage_words, true, &occ);
+    const void* fn = select_kernel_fn(P, false);
+    P.nstages = pick_stages(fn, P.stage_words, false, &occ);
     const size_t smem = select_smem_bytes(P.stage_words, P.nstages, true);
     const int grid = (int)std::min<int64_t>(P.num_tiles, (int64_t)num_sms() * occ);
-    return launch_select(P, grid, smem, s);
+    return launch_scan(fn, P, grid, smem, false, s);
 }
 
 // ------------------------------------------------------------------ a5
@@ -546,7 +563,7 @@ ar_status ar_select_refine_sum(const ar_pred* preds, int32_t npred, const ar_col
     ard::SelParams P;
     bool empty = false;
     int64_t n = 0;
-    ar_status st = setup_scan(preds, npred, P, empty, n);
+    ar_status st = setup_scan(preds, npred, P, empty, n, true);
     if (st != AR_OK) return st;
     if (!out_dev) {
         set_error("ar_select_refine_sum: null output");
@@ -560,10 +577,11 @@ ar_status ar_select_refine_sum(const ar_pred* preds, int32_t npred, const ar_col
     AR_TRY_CUDA(cudaMemsetAsync(out_dev, 0, 4 * sizeof(int64_t), s));
     if (empty || n == 0) return AR_OK;
     int occ = 1;
-    P.nstages = pick_stages(P.stage_words, false, &occ);
+    const void* fn = select_kernel_fn(P, true);
+    P.nstages = pick_stages(fn, P.stage_words, true, &occ);
     const size_t smem = select_smem_bytes(P.stage_words, P.nstages, false);
     const int grid = (int)std::min<int64_t>(P.num_tiles, (int64_t)num_sms() * occ);
-    return launch_fused(P, grid, smem, s);
+    return launch_scan(fn, P, grid, smem, true, s);
 }
 
 }  // extern "C"

@@ -89,13 +89,17 @@ __device__ __forceinline__ void mbar_arrive_expect_tx(uint64_t* bar, uint32_t by
 __device__ __forceinline__ void mbar_arrive(uint64_t* bar) {
     asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(smem_u32(bar)) : "memory");
 }
+// Blocking wait on an mbarrier phase.  The suspend-time hint lets the hardware
+// park the thread until the phase completes instead of returning after its short
+// default window: without it a waiting warp spins (YIELD / TRYWAIT / BRA) and
+// steals issue slots from the warps doing the work.
 __device__ __forceinline__ void mbar_wait(uint64_t* bar, uint32_t parity) {
     asm volatile(
         "{\n\t.reg .pred p;\n"
         "AR_WAIT_%=:\n\t"
-        "mbarrier.try_wait.parity.shared::cta.b64 p, [%0], %1;\n\t"
+        "mbarrier.try_wait.parity.shared::cta.b64 p, [%0], %1, %2;\n\t"
         "@!p bra AR_WAIT_%=;\n}" ::"r"(smem_u32(bar)),
-        "r"(parity)
+        "r"(parity), "r"(1000000u)
         : "memory");
 }
 
@@ -119,13 +123,15 @@ __device__ __forceinline__ void bar_sync(uint32_t id, uint32_t nthreads) {
     asm volatile("bar.sync %0, %1;" ::"r"(id), "r"(nthreads) : "memory");
 }
 
-// --- relaxed / acquire-release 64-bit status words for decoupled look-back
-__device__ __forceinline__ void st_release(unsigned long long* p, unsigned long long v) {
-    asm volatile("st.release.gpu.global.u64 [%0], %1;" ::"l"(p), "l"(v) : "memory");
+// --- 64-bit status words for decoupled look-back.  Each word carries its own
+// flag and value, and no other data is published through it, so relaxed
+// gpu-scope single-copy-atomic accesses are sufficient.
+__device__ __forceinline__ void st_relaxed(unsigned long long* p, unsigned long long v) {
+    asm volatile("st.relaxed.gpu.global.u64 [%0], %1;" ::"l"(p), "l"(v) : "memory");
 }
-__device__ __forceinline__ unsigned long long ld_acquire(const unsigned long long* p) {
+__device__ __forceinline__ unsigned long long ld_relaxed(const unsigned long long* p) {
     unsigned long long v;
-    asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+    asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
     return v;
 }
 
@@ -144,7 +150,7 @@ __device__ __forceinline__ unsigned long long lookback(const unsigned long long*
         long long idx = base - (long long)lane;
         unsigned long long s;
         while (true) {
-            s = idx >= 0 ? ld_acquire(status + idx) : kFlagPrefix;  // before tile 0: prefix 0
+            s = idx >= 0 ? ld_relaxed(status + idx) : kFlagPrefix;  // before tile 0: prefix 0
             if (__all_sync(0xffffffffu, (s >> 62) != 0)) break;
         }
         unsigned prefix_lanes = __ballot_sync(0xffffffffu, (s >> 62) == 2);
@@ -158,6 +164,55 @@ __device__ __forceinline__ unsigned long long lookback(const unsigned long long*
         for (int o = 16; o > 0; o >>= 1) v += __shfl_xor_sync(0xffffffffu, v, o);
         excl += v;
         base -= 32;
+    }
+}
+
+// Wide variant: each lane inspects kLookV consecutive predecessors, so one
+// round trip covers 32 * kLookV tiles and the prefix frontier advances that
+// many tiles per L2 latency.  Entry (lane, j) is tile base - kLookV*lane - j.
+constexpr int kLookV = 16;
+__device__ __forceinline__ unsigned long long lookback_wide(const unsigned long long* status, long long t,
+                                                            unsigned lane) {
+    unsigned long long excl = 0;
+    long long base = t - 1;
+    while (true) {
+        unsigned long long s[kLookV];
+#pragma unroll
+        for (int j = 0; j < kLookV; ++j) {
+            const long long idx = base - (long long)(kLookV * lane + j);
+            s[j] = idx >= 0 ? ld_relaxed(status + idx) : kFlagPrefix;   // before tile 0: prefix 0
+        }
+        while (true) {
+            bool ready = true;
+#pragma unroll
+            for (int j = 0; j < kLookV; ++j) ready &= (s[j] >> 62) != 0;
+            if (__all_sync(0xffffffffu, ready)) break;
+            __nanosleep(64);
+#pragma unroll
+            for (int j = 0; j < kLookV; ++j) {
+                const long long idx = base - (long long)(kLookV * lane + j);
+                if ((s[j] >> 62) == 0) s[j] = ld_relaxed(status + idx);
+            }
+        }
+        int first_j = kLookV;   // nearest predecessor of this lane holding an inclusive prefix
+#pragma unroll
+        for (int j = kLookV - 1; j >= 0; --j)
+            if ((s[j] >> 62) == 2) first_j = j;
+        const unsigned has = __ballot_sync(0xffffffffu, first_j < kLookV);
+        unsigned long long v = 0;
+        if (has) {
+            const unsigned first_lane = __ffs(has) - 1;
+#pragma unroll
+            for (int j = 0; j < kLookV; ++j)
+                if (lane < first_lane || (lane == first_lane && j <= first_j)) v += s[j] & kValueMask;
+            for (int o = 16; o > 0; o >>= 1) v += __shfl_xor_sync(0xffffffffu, v, o);
+            return excl + v;
+        }
+#pragma unroll
+        for (int j = 0; j < kLookV; ++j) v += s[j] & kValueMask;
+        for (int o = 16; o > 0; o >>= 1) v += __shfl_xor_sync(0xffffffffu, v, o);
+        excl += v;
+        base -= 32 * kLookV;
     }
 }
 
@@ -185,7 +240,9 @@ __device__ __forceinline__ uint32_t packed_get_any(const uint32_t* s, uint64_t p
 }
 
 // Major of row p from a SLICED part of width w (w words per 32-row block).
-__device__ __forceinline__ uint32_t sliced_get(const uint32_t* __restrict__ s, uint64_t p, int w) {
+// Off the hot path (majors of predicate columns travel in the aux word), so
+// kept out of line to keep the kernels' instruction footprint small.
+static __device__ __noinline__ uint32_t sliced_get(const uint32_t* __restrict__ s, uint64_t p, int w) {
     const uint32_t* blk = s + (p >> 5) * (uint64_t)w;
     uint32_t l = (uint32_t)(p & 31);
     uint32_t m = 0;
@@ -199,7 +256,8 @@ __device__ __forceinline__ uint32_t major_get(const uint32_t* __restrict__ s, ui
 }
 
 // Exact value of row p of a column (major and residual joined).
-__device__ __forceinline__ uint32_t value_get(const uint32_t* major, const uint32_t* residual, uint64_t p,
+// Generic (any layout, any k): out of line; kernels inline only their hot case.
+static __device__ __noinline__ uint32_t value_get(const uint32_t* major, const uint32_t* residual, uint64_t p,
                                               int w, int k, int layout, uint32_t base) {
     uint32_t m = major_get(major, p, w, layout);
     uint32_t r = k ? packed_get_any(residual, p, k) : 0u;

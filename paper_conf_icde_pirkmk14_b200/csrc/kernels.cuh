@@ -26,9 +26,18 @@ struct AggCol {
     int32_t pred;             // index of the predicate over the same column, or -1
 };
 
+// Value of aggregate column a at row p.  Hot case inline (a bit-packed column
+// without residual, e.g. l_extendedprice: one or two loads from one sector),
+// everything else through the out-of-line generic path.
+__device__ __forceinline__ uint32_t agg_gather(const AggCol& a, uint64_t p) {
+    if (a.k == 0 && a.layout == AR_LAYOUT_PACKED && a.w > 0) return packed_get(a.major, p, (int)a.w) + a.base;
+    return value_get(a.major, a.residual, p, (int)a.w, (int)a.k, (int)a.layout, a.base);
+}
+
 constexpr int kSelWarps = 4;                      // consumer warps per CTA
-constexpr int kSelThreads = kSelWarps * 32;       // one 32-row block per consumer thread
-constexpr int kSelTileRows = kSelThreads * 32;    // 4096 rows per tile
+constexpr int kSelThreads = kSelWarps * 32;       // each consumer thread owns BPT consecutive 32-row blocks
+constexpr int kSelMinTileRows = kSelThreads * 32; // tile rows = 4096 * BPT (BPT in {1, 2, 4})
+constexpr int kStageEntries = 2048;               // output staging entries (pos + aux) per round
 
 struct SelParams {
     SelPred p[AR_MAX_PRED];
@@ -38,6 +47,8 @@ struct SelParams {
     int64_t num_tiles;
     uint32_t stage_words;     // uint32 words per pipeline stage (all predicates)
     uint32_t nstages;
+    uint32_t bpt;             // 32-row blocks per consumer thread (template parameter of the launch)
+    uint32_t tile_rows;       // kSelMinTileRows * bpt
     uint32_t* out_pos;
     uint32_t* out_aux;
     long long* out_count;
@@ -91,8 +102,11 @@ struct SumParams {
 namespace ar {
 // launchers (return AR_OK or the CUDA failure)
 size_t select_smem_bytes(uint32_t stage_words, uint32_t nstages, bool staging);
-ar_status launch_select(const ard::SelParams& P, int grid, size_t smem, cudaStream_t s);
-ar_status launch_fused(const ard::SelParams& P, int grid, size_t smem, cudaStream_t s);
+int kernel_warps(bool fused);
+int kernel_bpt(bool fused);
+const void* select_kernel_fn(const ard::SelParams& P, bool fused);
+int select_occupancy(const void* fn, size_t smem, bool fused);
+ar_status launch_scan(const void* fn, const ard::SelParams& P, int grid, size_t smem, bool fused, cudaStream_t s);
 ar_status launch_refine(const ard::RefParams& P, int grid, cudaStream_t s);
 ar_status launch_refine_sum(const ard::RefParams& P, int grid, cudaStream_t s);
 ar_status launch_sum(const ard::SumParams& P, int grid, cudaStream_t s);
@@ -103,5 +117,4 @@ ar_status launch_pack_packed(const uint32_t* col, int64_t n, int shift, uint32_t
                              uint64_t out_words, uint32_t* out, cudaStream_t s);
 ar_status launch_exclusive_offset(const long long* all_counts, int world, int rank, long long* out,
                                   cudaStream_t s);
-int select_occupancy(size_t smem, bool fused);
 }  // namespace ar

@@ -37,7 +37,7 @@ __device__ __forceinline__ uint32_t agg_value_at(const RefParams& P, const AggCo
         const uint32_t r = a.k ? packed_get_any(a.residual, pos, a.k) : 0u;
         return ((m << a.k) | r) + a.base;
     }
-    return value_get(a.major, a.residual, pos, a.w, a.k, a.layout, a.base);
+    return agg_gather(a, pos);
 }
 
 __device__ __forceinline__ void load8(const uint32_t* base, uint64_t j0, long long count, uint32_t (&v)[8]) {
@@ -81,11 +81,11 @@ __global__ void __launch_bounds__(kRefThreads) refine_kernel(const __grid_consta
         if (warp == 0) {
             unsigned long long prefix = 0;
             if (t == 0) {
-                if (lane == 0) st_release(P.status, kFlagPrefix | total);
+                if (lane == 0) st_relaxed(P.status, kFlagPrefix | total);
             } else {
-                if (lane == 0) st_release(P.status + t, kFlagAgg | total);
-                prefix = lookback(P.status, t, lane);
-                if (lane == 0) st_release(P.status + t, kFlagPrefix | (prefix + total));
+                if (lane == 0) st_relaxed(P.status + t, kFlagAgg | total);
+                prefix = lookback_wide(P.status, t, lane);
+                if (lane == 0) st_relaxed(P.status + t, kFlagPrefix | (prefix + total));
             }
             if (lane == 0) {
                 s_off = prefix;
@@ -154,7 +154,7 @@ __global__ void __launch_bounds__(kRefThreads) sum_kernel(const __grid_constant_
         unsigned long long prod = 1;
         for (int c = 0; c < P.nagg; ++c) {
             const AggCol& a = P.a[c];
-            prod *= value_get(a.major, a.residual, pos, a.w, a.k, a.layout, a.base);
+            prod *= agg_gather(a, pos);
         }
         sum += prod;
     }

@@ -2,65 +2,59 @@
 // majors (s IV-B), and the one-pass fused A&R kernel
 // (a3 + a5 + a6).
 //
-// Structure (both kernels): persistent CTAs, one producer warp + kSelWarps
-// consumer warps.  The producer streams 4096-row tiles of every predicate's
-// bit planes into a ring of shared-memory stages with 1-D TMA bulk copies
-// (cp.async.bulk, completion on an mbarrier), so several tiles of HBM traffic
-// are always in flight per SM.  Each consumer thread owns one 32-row block of
-// the tile and evaluates every range predicate on the bit planes with borrow
-// chains: per plane and per bound one 3-input logic op decides 32 rows at once
-// (DESIGN "Kernel a3").  The select kernel then compacts candidate rows in
-// ascending order: per-thread popc, block scan, decoupled look-back across
-// tiles (dynamic tile tickets), shared-memory staging and coalesced stores.
+// Structure (both kernels): persistent CTAs, one producer warp + NW consumer
+// warps.  The producer streams tiles (NW * 32 threads * BPT blocks * 32 rows)
+// of every predicate's bit planes into a ring of shared-memory stages with 1-D
+// TMA bulk copies (cp.async.bulk, completion on an mbarrier), so several tiles
+// of HBM traffic are in flight per SM.  Each consumer thread owns BPT
+// consecutive 32-row blocks and evaluates every range predicate on the bit
+// planes with borrow chains: per plane and per bound one 3-input logic op
+// decides 32 rows at once (DESIGN "Kernel a3").
+//
+// Like the paper's operators, which are JIT-generated per data type and
+// decomposition, the kernels are specialised on the
+// decomposition: FixedPlanes<BPT, W...> holds the thread's planes in registers
+// with compile-time widths (tight, unrolled code); DynPlanes<BPT> is the
+// generic runtime-width path for any other shape.
+//
+// select_kernel: ordered compaction.  popc per thread, block scan, decoupled
+// look-back across tiles with a 256-tile window, then the tile's (pos, aux)
+// entries are staged in shared memory in rounds of kStageEntries and written
+// with coalesced stores.  Cooperative launch + round-robin tiles.
+//
+// fused_kernel: no candidate list in HBM.  Non-definite candidates are refined
+// in place (residual gathers issued kBatch at a time per thread so they
+// overlap), then the SUM factors of the exact rows are gathered the same way.
+#include <type_traits>
+
 #include "kernels.cuh"
 
 namespace ard {
 
-// Range test lo <= v <= hi of the 32 rows of one block whose W bit planes are
-// x[0..W) (x[j] = bit j of the 32 values).  v < lo iff subtracting lo borrows
-// out of the top bit; v > hi iff hi - v borrows.  One LOP3 per plane and bound.
+// ------------------------------------------------------------ bit-plane tests
+
+// For one 32-row block with W planes x[0..W) (x[j] = bit j of the 32 values,
+// LSB first), lo <= v <= hi is decided by two borrow chains run from the LSB:
+// v < lo iff v - lo borrows out of the top bit, v > hi iff hi - v does.  Per
+// plane and bound the borrow update is one 3-input logic op (LOP3); the bound's
+// bit j is a warp-uniform all-0 / all-1 mask.
+__device__ __forceinline__ uint32_t borrow_sub(uint32_t x, uint32_t cbit, uint32_t b) {   // borrow of x - c
+    return (~x & (cbit | b)) | (x & cbit & b);
+}
+__device__ __forceinline__ uint32_t borrow_rsub(uint32_t x, uint32_t cbit, uint32_t b) {  // borrow of c - x
+    return (~cbit & (x | b)) | (cbit & x & b);
+}
+__device__ __forceinline__ uint32_t bitmask(uint32_t v, uint32_t j) { return 0u - ((v >> j) & 1u); }
+
 template <int W>
 __device__ __forceinline__ uint32_t range_mask(const uint32_t* x, uint32_t lo, uint32_t hi) {
     uint32_t bl = 0, bh = 0;
 #pragma unroll
     for (int j = 0; j < W; ++j) {
-        const uint32_t L = 0u - ((lo >> j) & 1u);
-        const uint32_t H = 0u - ((hi >> j) & 1u);
-        bl = (~x[j] & (L | bl)) | (x[j] & L & bl);   // borrow of v - lo
-        bh = (~H & (x[j] | bh)) | (H & x[j] & bh);   // borrow of hi - v
+        bl = borrow_sub(x[j], bitmask(lo, j), bl);
+        bh = borrow_rsub(x[j], bitmask(hi, j), bh);
     }
     return ~(bl | bh);
-}
-
-template <int W>
-__device__ __forceinline__ void eval_pred_w(const uint32_t* __restrict__ pl, const SelPred& p, uint32_t& cm,
-                                            uint32_t& dm) {
-    uint32_t x[W > 0 ? W : 1];
-#pragma unroll
-    for (int j = 0; j < W; ++j) x[j] = pl[j];
-    const uint32_t c = range_mask<W>(x, p.clo, p.chi);
-    cm &= c;
-    if (p.mode == 0) {
-        dm &= c;
-    } else if (p.mode == 1) {
-        dm &= range_mask<W>(x, p.dlo, p.dhi);
-    } else {
-        dm = 0;
-    }
-}
-
-__device__ __forceinline__ void eval_pred(const uint32_t* __restrict__ pl, const SelPred& p, uint32_t& cm,
-                                          uint32_t& dm) {
-    switch (p.w) {
-#define AR_W(W) \
-    case W: eval_pred_w<W>(pl, p, cm, dm); break;
-        AR_W(0) AR_W(1) AR_W(2) AR_W(3) AR_W(4) AR_W(5) AR_W(6) AR_W(7) AR_W(8)
-        AR_W(9) AR_W(10) AR_W(11) AR_W(12) AR_W(13) AR_W(14) AR_W(15) AR_W(16)
-        AR_W(17) AR_W(18) AR_W(19) AR_W(20) AR_W(21) AR_W(22) AR_W(23) AR_W(24)
-        AR_W(25) AR_W(26) AR_W(27) AR_W(28) AR_W(29) AR_W(30) AR_W(31) AR_W(32)
-#undef AR_W
-        default: break;
-    }
 }
 
 // Major of row l (0..31) of a block from its bit planes in shared memory.
@@ -69,6 +63,176 @@ __device__ __forceinline__ uint32_t plane_value(const uint32_t* pl, uint32_t w, 
     for (uint32_t j = 0; j < w; ++j) m |= ((pl[j] >> l) & 1u) << j;
     return m;
 }
+
+// ------------------------------------------------------------ plane sources
+
+template <int... Ws>
+__host__ __device__ constexpr int wid(int c) {
+    constexpr int a[] = {Ws..., 0};
+    return a[c];
+}
+template <int... Ws>
+__host__ __device__ constexpr int woff(int c) {
+    constexpr int a[] = {Ws..., 0};
+    int o = 0;
+    for (int i = 0; i < c; ++i) o += a[i];
+    return o;
+}
+
+// Compile-time decomposition shape: the thread's planes live in registers.
+template <int BPT, int... Ws>
+struct FixedPlanes {
+    static constexpr int N = sizeof...(Ws);
+    static constexpr int TOTAL = (0 + ... + Ws);
+    uint32_t x[BPT][TOTAL > 0 ? TOTAL : 1];
+
+    template <int C>
+    __device__ __forceinline__ void load_c(const SelParams& P, const uint32_t* stg) {
+        if constexpr (C < N) {
+            constexpr int w = wid<Ws...>(C), o = woff<Ws...>(C);
+            const uint32_t* pl = stg + P.p[C].soff + threadIdx.x * (BPT * w);
+            if constexpr ((BPT * w) % 4 == 0) {
+#pragma unroll
+                for (int q = 0; q < BPT * w / 4; ++q) {
+                    const uint4 v = reinterpret_cast<const uint4*>(pl)[q];
+                    const uint32_t vv[4] = {v.x, v.y, v.z, v.w};
+#pragma unroll
+                    for (int e = 0; e < 4; ++e) x[(4 * q + e) / w][o + (4 * q + e) % w] = vv[e];
+                }
+            } else {
+#pragma unroll
+                for (int b = 0; b < BPT; ++b)
+#pragma unroll
+                    for (int j = 0; j < w; ++j) x[b][o + j] = pl[b * w + j];
+            }
+            load_c<C + 1>(P, stg);
+        }
+    }
+    __device__ __forceinline__ void load(const SelParams& P, const uint32_t* stg) { load_c<0>(P, stg); }
+
+    template <int C>
+    __device__ __forceinline__ void eval_c(const SelParams& P, uint32_t (&cm)[BPT], uint32_t (&dm)[BPT]) const {
+        if constexpr (C < N) {
+            constexpr int w = wid<Ws...>(C), o = woff<Ws...>(C);
+            const SelPred& p = P.p[C];
+#pragma unroll
+            for (int b = 0; b < BPT; ++b) {
+                const uint32_t c = range_mask<w>(&x[b][o], p.clo, p.chi);
+                cm[b] &= c;
+                if (p.mode == 0)
+                    dm[b] &= c;
+                else if (p.mode == 1)
+                    dm[b] &= range_mask<w>(&x[b][o], p.dlo, p.dhi);
+                else
+                    dm[b] = 0;
+            }
+            eval_c<C + 1>(P, cm, dm);
+        }
+    }
+    __device__ __forceinline__ void eval(const SelParams& P, uint32_t (&cm)[BPT], uint32_t (&dm)[BPT]) const {
+        eval_c<0>(P, cm, dm);
+    }
+
+    // major of predicate C at row l of block B
+    template <int B, int C>
+    __device__ __forceinline__ uint32_t value(uint32_t l) const {
+        constexpr int w = wid<Ws...>(C), o = woff<Ws...>(C);
+        uint32_t m = 0;
+#pragma unroll
+        for (int j = 0; j < w; ++j) m |= ((x[B][o + j] >> l) & 1u) << j;
+        return m;
+    }
+    template <int B, int C = 0>
+    __device__ __forceinline__ uint32_t value_rt(int c, uint32_t l) const {
+        if constexpr (C < N) {
+            if (c == C) return value<B, C>(l);
+            return value_rt<B, C + 1>(c, l);
+        } else {
+            return 0u;
+        }
+    }
+    // approximation tuple: all majors concatenated LSB-first in predicate order
+    template <int B>
+    __device__ __forceinline__ uint32_t appr(const SelParams&, uint32_t l) const {
+        uint32_t a = 0;
+#pragma unroll
+        for (int p = 0; p < TOTAL; ++p) a |= ((x[B][p] >> l) & 1u) << p;
+        return a;
+    }
+};
+
+// Runtime decomposition shape: planes stay in shared memory.
+template <int BPT>
+struct DynPlanes {
+    const uint32_t* stg;
+
+    __device__ __forceinline__ void load(const SelParams&, const uint32_t* s) { stg = s; }
+
+    __device__ __forceinline__ void eval(const SelParams& P, uint32_t (&cm)[BPT], uint32_t (&dm)[BPT]) const {
+        for (int c = 0; c < P.npred; ++c) {
+            const SelPred& p = P.p[c];
+            const uint32_t w = p.w;
+            const uint32_t* pl = stg + p.soff + threadIdx.x * BPT * w;
+            uint32_t cl[BPT], ch[BPT], dl[BPT], dh[BPT];
+#pragma unroll
+            for (int b = 0; b < BPT; ++b) cl[b] = ch[b] = dl[b] = dh[b] = 0;
+            for (uint32_t j = 0; j < w; ++j) {
+                const uint32_t L = bitmask(p.clo, j), H = bitmask(p.chi, j);
+                const uint32_t DL = bitmask(p.dlo, j), DH = bitmask(p.dhi, j);
+#pragma unroll
+                for (int b = 0; b < BPT; ++b) {
+                    const uint32_t x = pl[b * w + j];
+                    cl[b] = borrow_sub(x, L, cl[b]);
+                    ch[b] = borrow_rsub(x, H, ch[b]);
+                    dl[b] = borrow_sub(x, DL, dl[b]);
+                    dh[b] = borrow_rsub(x, DH, dh[b]);
+                }
+            }
+#pragma unroll
+            for (int b = 0; b < BPT; ++b) {
+                const uint32_t c0 = ~(cl[b] | ch[b]);
+                cm[b] &= c0;
+                dm[b] = p.mode == 0 ? (dm[b] & c0) : (p.mode == 1 ? (dm[b] & ~(dl[b] | dh[b])) : 0u);
+            }
+        }
+    }
+    template <int B>
+    __device__ __forceinline__ uint32_t value_rt(const SelParams& P, int c, uint32_t l) const {
+        const uint32_t w = P.p[c].w;
+        return plane_value(stg + P.p[c].soff + (threadIdx.x * BPT + B) * w, w, l);
+    }
+    template <int B>
+    __device__ __forceinline__ uint32_t appr(const SelParams& P, uint32_t l) const {
+        uint32_t a = 0;
+        for (int c = 0; c < P.npred; ++c) a |= value_rt<B>(P, c, l) << P.p[c].ashift;
+        return a;
+    }
+};
+
+template <class T>
+struct requires_params : std::false_type {};
+template <int BPT>
+struct requires_params<DynPlanes<BPT>> : std::true_type {};
+
+template <int I>
+using ic = std::integral_constant<int, I>;
+template <int N, int I = 0, class F>
+__device__ __forceinline__ void static_for(F&& f) {
+    if constexpr (I < N) {
+        f(ic<I>{});
+        static_for<N, I + 1>(f);
+    }
+}
+
+template <class PS, int B>
+__device__ __forceinline__ uint32_t ps_value(const PS& ps, const SelParams& P, int c, uint32_t l) {
+    if constexpr (requires_params<PS>::value)
+        return ps.template value_rt<B>(P, c, l);
+    else
+        return ps.template value_rt<B>(c, l);
+}
+
+// ------------------------------------------------------------ pipeline
 
 struct SmemLayout {
     uint64_t* full;
@@ -91,8 +255,8 @@ __device__ __forceinline__ SmemLayout carve(unsigned char* smem, uint32_t nstage
     unsigned char* p = reinterpret_cast<unsigned char*>(L.misc + 8);
     if (staging) {
         L.st_pos = reinterpret_cast<uint32_t*>(p);
-        L.st_aux = L.st_pos + kSelTileRows;
-        p = reinterpret_cast<unsigned char*>(L.st_aux + kSelTileRows);
+        L.st_aux = L.st_pos + kStageEntries;
+        p = reinterpret_cast<unsigned char*>(L.st_aux + kStageEntries);
     } else {
         L.st_pos = L.st_aux = nullptr;
     }
@@ -101,24 +265,23 @@ __device__ __forceinline__ SmemLayout carve(unsigned char* smem, uint32_t nstage
     return L;
 }
 
-// Producer: one elected lane streams tiles into the stage ring.  Tile order
-// comes from `next_tile` (a ticket for the ordered select, a static stride for
-// the fused kernel); a negative tile index ends the stream.
-template <typename NextTile>
-__device__ __forceinline__ void produce(const SelParams& P, const SmemLayout& L, NextTile next_tile) {
+// Producer: one lane streams tiles (tile = blockIdx + i * gridDim) into the
+// stage ring; a tile index past the end is passed on as -1 and ends the stream.
+__device__ __forceinline__ void produce(const SelParams& P, const SmemLayout& L) {
     const uint64_t pol = policy_evict_first();
+    const uint32_t blocks_per_tile = P.tile_rows / 32;
     for (uint32_t i = 0;; ++i) {
         const uint32_t s = i % P.nstages;
         if (i >= P.nstages) mbar_wait(L.empty + s, ((i / P.nstages) - 1) & 1);
-        const long long t = next_tile(i);
-        if (t < 0) {
+        const long long t = (long long)blockIdx.x + (long long)i * gridDim.x;
+        if (t >= P.num_tiles) {
             L.slot[s] = -1;
             mbar_arrive(L.full + s);
             return;
         }
         L.slot[s] = t;
-        const int64_t r0 = t * (int64_t)kSelTileRows;
-        const int64_t rows = min((int64_t)kSelTileRows, P.n - r0);
+        const int64_t r0 = t * (int64_t)P.tile_rows;
+        const int64_t rows = min((int64_t)P.tile_rows, P.n - r0);
         const uint32_t groups = (uint32_t)((rows + 127) / 128);   // 128-row groups, 16 B per plane
         uint32_t bytes = 0;
         for (int c = 0; c < P.npred; ++c) bytes += groups * 16u * P.p[c].w;
@@ -127,33 +290,39 @@ __device__ __forceinline__ void produce(const SelParams& P, const SmemLayout& L,
         for (int c = 0; c < P.npred; ++c) {
             const uint32_t w = P.p[c].w;
             if (w == 0) continue;
-            const uint32_t* src = P.p[c].planes + (size_t)t * (kSelTileRows / 32) * w;
+            const uint32_t* src = P.p[c].planes + (size_t)t * blocks_per_tile * w;
             bulk_g2s(stg + P.p[c].soff, src, groups * 16u * w, L.full + s, pol);
         }
     }
 }
 
-template <bool kCarry>
-__global__ void __launch_bounds__((kSelWarps + 1) * 32) select_kernel(const __grid_constant__ SelParams P) {
-    extern __shared__ __align__(128) unsigned char smem[];
-    const SmemLayout L = carve(smem, P.nstages, true);
-    const unsigned warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
-
+template <int NW>
+__device__ __forceinline__ void init_barriers(const SelParams& P, const SmemLayout& L) {
     if (threadIdx.x == 0) {
         for (uint32_t s = 0; s < P.nstages; ++s) {
             mbar_init(L.full + s, 1);
-            mbar_init(L.empty + s, kSelWarps);
+            mbar_init(L.empty + s, NW);
         }
         fence_mbar_init();
     }
     __syncthreads();
+}
 
-    if (warp == kSelWarps) {
-        if (lane == 0)
-            produce(P, L, [&](uint32_t) -> long long {
-                const long long t = (long long)atomicAdd(P.ticket, 1u);
-                return t < P.num_tiles ? t : -1;
-            });
+// ------------------------------------------------------------ ordered select
+
+template <class PS, int NW, int BPT, bool kCarry>
+__global__ void __launch_bounds__((NW + 1) * 32) select_kernel(const __grid_constant__ SelParams P) {
+    constexpr int NT = NW * 32;
+    extern __shared__ __align__(128) unsigned char smem[];
+    const SmemLayout L = carve(smem, P.nstages, true);
+    const unsigned warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    init_barriers<NW>(P, L);
+
+    // Tiles are dealt round-robin: all CTAs are co-resident (cooperative launch),
+    // so round i proceeds in lock-step and a tile's look-back window only spans
+    // tiles of its own and the previous round.
+    if (warp == NW) {
+        if (lane == 0) produce(P, L);
         return;
     }
 
@@ -162,89 +331,96 @@ __global__ void __launch_bounds__((kSelWarps + 1) * 32) select_kernel(const __gr
         mbar_wait(L.full + s, (i / P.nstages) & 1);
         const long long t = L.slot[s];
         if (t < 0) break;
-        const uint32_t* stg = L.stages + (size_t)s * P.stage_words;
-        const int64_t r0 = t * (int64_t)kSelTileRows + (int64_t)threadIdx.x * 32;
+        const int64_t r0 = t * (int64_t)P.tile_rows + (int64_t)threadIdx.x * (32 * BPT);
 
-        uint32_t cm = valid_mask(r0, P.n), dm = cm;
-        for (int c = 0; c < P.npred; ++c) eval_pred(stg + P.p[c].soff + threadIdx.x * P.p[c].w, P.p[c], cm, dm);
-
-        const uint32_t cnt = __popc(cm);
+        PS ps;
+        ps.load(P, L.stages + (size_t)s * P.stage_words);
+        uint32_t cm[BPT], dm[BPT];
+#pragma unroll
+        for (int b = 0; b < BPT; ++b) cm[b] = dm[b] = valid_mask(r0 + 32 * b, P.n);
+        ps.eval(P, cm, dm);
+        uint32_t cnt = 0;
+#pragma unroll
+        for (int b = 0; b < BPT; ++b) cnt += __popc(cm[b]);
         uint32_t total;
-        const uint32_t excl = block_excl_scan<kSelThreads>(cnt, L.warp_tot, total, 1);
+        const uint32_t excl = block_excl_scan<NT>(cnt, L.warp_tot, total, 1);
 
         if (warp == 0) {
             unsigned long long prefix = 0;
             if (t == 0) {
-                if (lane == 0) st_release(P.status, kFlagPrefix | total);
+                if (lane == 0) st_relaxed(P.status, kFlagPrefix | total);
             } else {
-                if (lane == 0) st_release(P.status + t, kFlagAgg | total);
-                prefix = lookback(P.status, t, lane);
-                if (lane == 0) st_release(P.status + t, kFlagPrefix | (prefix + total));
+                if (lane == 0) st_relaxed(P.status + t, kFlagAgg | total);
+                prefix = lookback_wide(P.status, t, lane);
+                if (lane == 0) st_relaxed(P.status + t, kFlagPrefix | (prefix + total));
             }
             if (lane == 0) {
                 L.misc[0] = prefix;
                 if (t == P.num_tiles - 1) *P.out_count = (long long)(prefix + total);
             }
         }
-
-        // stage this thread's candidates (ascending) at their tile-local offsets
-        uint32_t m = cm, o = excl;
-        while (m) {
-            const uint32_t l = __ffs(m) - 1;
-            m &= m - 1;
-            uint32_t aux = ((dm >> l) & 1u) << 31;
-            if (kCarry) {
-                for (int c = 0; c < P.npred; ++c)
-                    aux |= plane_value(stg + P.p[c].soff + threadIdx.x * P.p[c].w, P.p[c].w, l) << P.p[c].ashift;
-            }
-            L.st_pos[o] = (uint32_t)(r0 + l);
-            L.st_aux[o] = aux;
-            ++o;
-        }
-        bar_sync(1, kSelThreads);
-        if (lane == 0) mbar_arrive(L.empty + s);   // planes of stage s no longer needed
-
+        bar_sync(1, NT);
         const unsigned long long off = L.misc[0];
-        for (uint32_t j = threadIdx.x; j < total; j += kSelThreads) {
-            P.out_pos[off + j] = L.st_pos[j];
-            P.out_aux[off + j] = L.st_aux[j];
+
+        // write the tile's entries in rounds of kStageEntries through shared memory
+        uint32_t e = excl;
+        for (uint32_t base = 0; base < total; base += kStageEntries) {
+            const uint32_t lim = min(base + (uint32_t)kStageEntries, excl + cnt);
+            auto emit = [&](auto bc) {
+                constexpr int b = decltype(bc)::value;
+                while (cm[b] && e < lim) {
+                    const uint32_t l = __ffs(cm[b]) - 1;
+                    cm[b] &= cm[b] - 1;
+                    uint32_t aux = ((dm[b] >> l) & 1u) << 31;
+                    if (kCarry) aux |= ps.template appr<b>(P, l);
+                    L.st_pos[e - base] = (uint32_t)(r0 + 32 * b + l);
+                    L.st_aux[e - base] = aux;
+                    ++e;
+                }
+            };
+            static_for<BPT>(emit);
+            bar_sync(1, NT);
+            const uint32_t nround = min((uint32_t)kStageEntries, total - base);
+            for (uint32_t j = threadIdx.x; j < nround; j += NT) {
+                P.out_pos[off + base + j] = L.st_pos[j];
+                P.out_aux[off + base + j] = L.st_aux[j];
+            }
+            bar_sync(1, NT);
         }
+        if (lane == 0) mbar_arrive(L.empty + s);   // planes of stage s no longer needed
     }
 }
 
 // ----------------------------------------------------------------- fused a3+a5+a6
 
-__device__ __forceinline__ uint32_t agg_value(const AggCol& a, const SelParams& P, const uint32_t* stg,
-                                              uint32_t bt, uint32_t l, uint64_t row) {
-    if (a.pred >= 0) {
-        const SelPred& p = P.p[a.pred];
-        const uint32_t m = plane_value(stg + p.soff + bt * p.w, p.w, l);
-        const uint32_t r = a.k ? packed_get_any(a.residual, row, a.k) : 0u;
-        return ((m << a.k) | r) + a.base;
-    }
-    return value_get(a.major, a.residual, row, a.w, a.k, a.layout, a.base);
+// Each warp owns a 1024 * BPT-row slice of the tile.  Its candidate rows are
+// compacted into a per-warp list in shared memory (a 16-bit row offset with
+// the definite flag in bit 15 -- the candidate relation of PAPER.md:368-374,
+// kept on chip), then the lanes take kLanesPer consecutive-in-round entries
+// each and refine / aggregate them in parallel, so the residual and aggregate
+// gathers of a whole warp are in flight together (Alg. 2).
+constexpr int kPer = 2;               // list entries per lane per pass
+constexpr uint32_t kDefFlag = 0x8000u;
+
+// Major of predicate c at block-local row l of global block `blk` of the tile.
+__device__ __forceinline__ uint32_t stage_value(const SelParams& P, const uint32_t* stg, int c, uint32_t blk,
+                                                uint32_t l) {
+    const uint32_t w = P.p[c].w;
+    return plane_value(stg + P.p[c].soff + blk * w, w, l);
 }
 
-__global__ void __launch_bounds__((kSelWarps + 1) * 32) fused_kernel(const __grid_constant__ SelParams P) {
+template <class PS, int NW, int BPT>
+__global__ void __launch_bounds__((NW + 1) * 32) fused_kernel(const __grid_constant__ SelParams P) {
+    constexpr int kWarpRows = 32 * 32 * BPT;
     extern __shared__ __align__(128) unsigned char smem[];
     const SmemLayout L = carve(smem, P.nstages, false);
     const unsigned warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    init_barriers<NW>(P, L);
+    // per-warp candidate lists live after the stage ring
+    uint16_t* list = reinterpret_cast<uint16_t*>(L.stages + (size_t)P.nstages * P.stage_words) + warp * kWarpRows;
 
-    if (threadIdx.x == 0) {
-        for (uint32_t s = 0; s < P.nstages; ++s) {
-            mbar_init(L.full + s, 1);
-            mbar_init(L.empty + s, kSelWarps);
-        }
-        fence_mbar_init();
-    }
-    __syncthreads();
-
-    if (warp == kSelWarps) {
-        if (lane == 0)
-            produce(P, L, [&](uint32_t i) -> long long {
-                const long long t = (long long)blockIdx.x + (long long)i * gridDim.x;
-                return t < P.num_tiles ? t : -1;
-            });
+    if (warp == NW) {
+        if (lane == 0) produce(P, L);
         return;
     }
 
@@ -255,39 +431,101 @@ __global__ void __launch_bounds__((kSelWarps + 1) * 32) fused_kernel(const __gri
         const long long t = L.slot[s];
         if (t < 0) break;
         const uint32_t* stg = L.stages + (size_t)s * P.stage_words;
-        const int64_t r0 = t * (int64_t)kSelTileRows + (int64_t)threadIdx.x * 32;
+        const int64_t tile_r0 = t * (int64_t)P.tile_rows;
+        const int64_t r0 = tile_r0 + (int64_t)threadIdx.x * (32 * BPT);
 
-        uint32_t cm = valid_mask(r0, P.n), dm = cm;
-        for (int c = 0; c < P.npred; ++c) eval_pred(stg + P.p[c].soff + threadIdx.x * P.p[c].w, P.p[c], cm, dm);
-        ncand += __popc(cm);
-        ndef += __popc(dm);
-
-        // refine the non-definite candidates inline (Alg. 2 on the fly)
-        uint32_t res = dm, nd = cm & ~dm;
-        while (nd) {
-            const uint32_t l = __ffs(nd) - 1;
-            nd &= nd - 1;
-            bool ok = true;
-            for (int c = 0; c < P.npred && ok; ++c) {
-                const SelPred& p = P.p[c];
-                if (p.k == 0) continue;   // exact already at the approximation
-                const uint32_t m = plane_value(stg + p.soff + threadIdx.x * p.w, p.w, l);
-                const uint32_t r = packed_get_any(p.residual, (uint64_t)(r0 + l), p.k);
-                const uint32_t v = ((m << p.k) | r) + p.base;
-                ok = (v >= p.lo) && (v <= p.hi);
-            }
-            if (ok) res |= 1u << l;
+        // a3: candidate / definite masks of this thread's blocks
+        PS ps;
+        ps.load(P, stg);
+        uint32_t cm[BPT], dm[BPT];
+#pragma unroll
+        for (int b = 0; b < BPT; ++b) cm[b] = dm[b] = valid_mask(r0 + 32 * b, P.n);
+        ps.eval(P, cm, dm);
+        uint32_t cnt = 0;
+#pragma unroll
+        for (int b = 0; b < BPT; ++b) {
+            cnt += __popc(cm[b]);
+            ndef += __popc(dm[b]);
         }
-        nres += __popc(res);
-        if (P.nagg > 0) {
-            uint32_t m = res;
+        ncand += cnt;
+
+        // compact the warp's candidates into its list (ascending row order)
+        uint32_t incl = cnt;
+#pragma unroll
+        for (int o = 1; o < 32; o <<= 1) {
+            const uint32_t y = __shfl_up_sync(0xffffffffu, incl, o);
+            if (lane >= (unsigned)o) incl += y;
+        }
+        const uint32_t total = __shfl_sync(0xffffffffu, incl, 31);
+        uint32_t e = incl - cnt;
+#pragma unroll
+        for (int b = 0; b < BPT; ++b) {
+            uint32_t m = cm[b];
             while (m) {
                 const uint32_t l = __ffs(m) - 1;
                 m &= m - 1;
-                const uint64_t row = (uint64_t)(r0 + l);
-                unsigned long long prod = agg_value(P.a[0], P, stg, threadIdx.x, l, row);
-                if (P.nagg > 1) prod *= agg_value(P.a[1], P, stg, threadIdx.x, l, row);
-                sum += prod;
+                list[e++] = (uint16_t)((((lane * BPT + b) << 5) | l) | (((dm[b] >> l) & 1u) ? kDefFlag : 0u));
+            }
+        }
+        __syncwarp();
+
+        // a5 + a6 over the list: each lane takes kPer entries per pass
+        const uint32_t blk0 = warp * 32 * BPT;          // first tile-block of this warp
+        const uint64_t row_base = (uint64_t)tile_r0 + (uint64_t)warp * kWarpRows;
+        for (uint32_t base = 0; base < total; base += 32 * kPer) {
+            uint32_t ent[kPer];
+            bool ok[kPer];
+#pragma unroll
+            for (int q = 0; q < kPer; ++q) {
+                const uint32_t k = base + q * 32 + lane;
+                ent[q] = k < total ? list[k] : 0u;
+                ok[q] = k < total;
+            }
+            // refine non-definite entries: residual gathers first (all in flight), then the exact test
+            for (int c = 0; c < P.npred; ++c) {
+                const SelPred& p = P.p[c];
+                if (p.k == 0) continue;   // exact already at the approximation
+                uint32_t r[kPer];
+#pragma unroll
+                for (int q = 0; q < kPer; ++q)
+                    r[q] = (ok[q] && !(ent[q] & kDefFlag))
+                               ? packed_get_any(p.residual, row_base + (ent[q] & 0x7fffu), p.k) : 0u;
+#pragma unroll
+                for (int q = 0; q < kPer; ++q) {
+                    if (!ok[q] || (ent[q] & kDefFlag)) continue;
+                    const uint32_t m = stage_value(P, stg, c, blk0 + ((ent[q] & 0x7fffu) >> 5), ent[q] & 31u);
+                    const uint32_t v = ((m << p.k) | r[q]) + p.base;
+                    ok[q] = (v >= p.lo) && (v <= p.hi);
+                }
+            }
+#pragma unroll
+            for (int q = 0; q < kPer; ++q) nres += ok[q];
+            if (P.nagg > 0) {
+                unsigned long long prod[kPer];
+#pragma unroll
+                for (int q = 0; q < kPer; ++q) prod[q] = ok[q] ? 1ull : 0ull;
+                for (int a = 0; a < P.nagg; ++a) {
+                    const AggCol& A = P.a[a];
+                    uint32_t v[kPer];
+#pragma unroll
+                    for (int q = 0; q < kPer; ++q) {
+                        const uint64_t row = row_base + (ent[q] & 0x7fffu);
+                        if (!ok[q]) {
+                            v[q] = 0u;
+                        } else if (A.pred >= 0) {
+                            const uint32_t m =
+                                stage_value(P, stg, A.pred, blk0 + ((ent[q] & 0x7fffu) >> 5), ent[q] & 31u);
+                            const uint32_t r = A.k ? packed_get_any(A.residual, row, A.k) : 0u;
+                            v[q] = ((m << A.k) | r) + A.base;
+                        } else {
+                            v[q] = agg_gather(A, row);
+                        }
+                    }
+#pragma unroll
+                    for (int q = 0; q < kPer; ++q) prod[q] *= v[q];
+                }
+#pragma unroll
+                for (int q = 0; q < kPer; ++q) sum += prod[q];
             }
         }
         __syncwarp();
@@ -312,50 +550,109 @@ __global__ void __launch_bounds__((kSelWarps + 1) * 32) fused_kernel(const __gri
 
 }  // namespace ard
 
+// ------------------------------------------------------------------------ host
+
 namespace ar {
+
+// Kernel configurations: (consumer warps, blocks per thread) of the ordered
+// select and of the fused kernel, and the decomposition shapes with
+// specialised kernels.  Any other shape takes the DynPlanes path.
+constexpr int kSelNW = ard::kSelWarps, kSelBPT = 2;
+constexpr int kFusNW = 8, kFusBPT = 1;
+
+template <int... Ws>
+struct ShapeEntry {
+    static bool match(const ard::SelParams& P) {
+        constexpr int n = sizeof...(Ws);
+        constexpr int w[] = {Ws..., 0};
+        if (P.npred != n) return false;
+        for (int c = 0; c < n; ++c)
+            if ((int)P.p[c].w != w[c]) return false;
+        return true;
+    }
+    static const void* select_fn(bool carry) {
+        using PS = ard::FixedPlanes<kSelBPT, Ws...>;
+        return carry ? (const void*)ard::select_kernel<PS, kSelNW, kSelBPT, true>
+                     : (const void*)ard::select_kernel<PS, kSelNW, kSelBPT, false>;
+    }
+    static const void* fused_fn() {
+        using PS = ard::FixedPlanes<kFusBPT, Ws...>;
+        return (const void*)ard::fused_kernel<PS, kFusNW, kFusBPT>;
+    }
+};
+
+// Q6 (l_shipdate 24/8 -> 4 major bits, l_discount 4, l_quantity 6); single
+// columns at 8 / 16 / 24 / 32 major bits (configs C1, C3); two 24-bit columns
+// (spatial range query).
+template <class... Es>
+struct ShapeList {
+    static bool find(const ard::SelParams& P, bool fused, bool carry, const void** fn) {
+        return (try_one<Es>(P, fused, carry, fn) || ...);
+    }
+    template <class E>
+    static bool try_one(const ard::SelParams& P, bool fused, bool carry, const void** fn) {
+        if (!E::match(P)) return false;
+        *fn = fused ? E::fused_fn() : E::select_fn(carry);
+        return true;
+    }
+};
+using Shapes = ShapeList<ShapeEntry<4, 4, 6>, ShapeEntry<8>, ShapeEntry<16>, ShapeEntry<24>, ShapeEntry<32>,
+                         ShapeEntry<24, 24>>;
+
+int kernel_warps(bool fused) { return fused ? kFusNW : kSelNW; }
+int kernel_bpt(bool fused) { return fused ? kFusBPT : kSelBPT; }
+
+const void* select_kernel_fn(const ard::SelParams& P, bool fused) {
+    const void* fn = nullptr;
+    if (!getenv("AR_FORCE_GENERIC") && Shapes::find(P, fused, P.carry != 0, &fn)) return fn;
+    if (fused) return (const void*)ard::fused_kernel<ard::DynPlanes<kFusBPT>, kFusNW, kFusBPT>;
+    return P.carry ? (const void*)ard::select_kernel<ard::DynPlanes<kSelBPT>, kSelNW, kSelBPT, true>
+                   : (const void*)ard::select_kernel<ard::DynPlanes<kSelBPT>, kSelNW, kSelBPT, false>;
+}
 
 size_t select_smem_bytes(uint32_t stage_words, uint32_t nstages, bool staging) {
     size_t head = nstages * (8 + 8 + 8) + 32 * 4 + 8 * 8;
-    if (staging) head += 2ull * ard::kSelTileRows * 4;
+    if (staging) head += 2ull * ard::kStageEntries * 4;
     head = (head + 127) & ~size_t(127);
-    return head + 128 + (size_t)nstages * stage_words * 4;
+    size_t bytes = head + 128 + (size_t)nstages * stage_words * 4;
+    if (!staging) bytes += (size_t)kFusNW * 32 * 32 * kFusBPT * 2;   // per-warp candidate lists (u16)
+    return bytes;
 }
 
-static bool g_attr_done[3] = {false, false, false};
-
-static void set_max_smem(const void* fn, int idx) {
-    if (!g_attr_done[idx]) {
-        cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, 227 * 1024);
-        g_attr_done[idx] = true;
-    }
+static void set_max_smem(const void* fn) {
+    static thread_local const void* done[64];
+    static thread_local int used = 0;
+    for (int i = 0; i < used; ++i)
+        if (done[i] == fn) return;
+    cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, 227 * 1024);
+    if (used < 64) done[used++] = fn;
 }
 
-int select_occupancy(size_t smem, bool fused) {
+int select_occupancy(const void* fn, size_t smem, bool fused) {
     int blocks = 0;
-    const void* fn = fused ? (const void*)ard::fused_kernel : (const void*)ard::select_kernel<true>;
-    set_max_smem(fn, fused ? 2 : 0);
-    if (!fused) set_max_smem((const void*)ard::select_kernel<false>, 1);
-    cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks, fn, (ard::kSelWarps + 1) * 32, smem);
+    set_max_smem(fn);
+    cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks, fn, (kernel_warps(fused) + 1) * 32, smem);
     return blocks;
 }
 
-ar_status launch_select(const ard::SelParams& P, int grid, size_t smem, cudaStream_t s) {
-    const dim3 block((ard::kSelWarps + 1) * 32);
-    if (P.carry) {
-        set_max_smem((const void*)ard::select_kernel<true>, 0);
-        ard::select_kernel<true><<<grid, block, smem, s>>>(P);
-    } else {
-        set_max_smem((const void*)ard::select_kernel<false>, 1);
-        ard::select_kernel<false><<<grid, block, smem, s>>>(P);
-    }
-    AR_CHECK_LAUNCH("select_kernel");
-    return AR_OK;
-}
-
-ar_status launch_fused(const ard::SelParams& P, int grid, size_t smem, cudaStream_t s) {
-    set_max_smem((const void*)ard::fused_kernel, 2);
-    ard::fused_kernel<<<grid, (ard::kSelWarps + 1) * 32, smem, s>>>(P);
-    AR_CHECK_LAUNCH("fused_kernel");
+// Cooperative launch for the ordered select: guarantees every CTA of the grid
+// is co-resident, which the round-robin look-back relies on (a CTA never waits
+// on a tile of a CTA that is not running).  The grid is sized from the
+// occupancy calculator.
+ar_status launch_scan(const void* fn, const ard::SelParams& P, int grid, size_t smem, bool fused, cudaStream_t s) {
+    set_max_smem(fn);
+    void* args[] = {const_cast<ard::SelParams*>(&P)};
+    cudaLaunchConfig_t cfg = {};
+    cfg.gridDim = dim3(grid);
+    cfg.blockDim = dim3((kernel_warps(fused) + 1) * 32);
+    cfg.dynamicSmemBytes = smem;
+    cfg.stream = s;
+    cudaLaunchAttribute attr[1];
+    attr[0].id = cudaLaunchAttributeCooperative;
+    attr[0].val.cooperative = fused ? 0 : 1;
+    cfg.attrs = attr;
+    cfg.numAttrs = 1;
+    AR_TRY_CUDA(cudaLaunchKernelExC(&cfg, fn, args));
     return AR_OK;
 }
 

@@ -1,0 +1,59 @@
+"""Summarise an ncu report: per kernel launch the time, DRAM bytes, issue activity,
+stall breakdown and the hottest SASS lines (needs -lineinfo + --import-source)."""
+import csv
+import io
+import subprocess
+import sys
+
+
+def ncu_csv(rep, *args):
+    out = subprocess.run(["ncu", "-i", rep, *args, "--csv"], capture_output=True, text=True).stdout
+    return list(csv.reader(io.StringIO(out)))
+
+
+def main(rep, kernel_regex=None, top=12):
+    rows = ncu_csv(rep, "--page", "raw")
+    hdr = rows[0]
+    for row in rows[2:]:
+        d = dict(zip(hdr, row))
+        name = d["Kernel Name"]
+        if kernel_regex and kernel_regex not in name:
+            continue
+        f = lambda k: d.get(k, "?")
+        print(f"== {name[:60]}  id={f('ID')}")
+        print(f"   time {f('gpu__time_duration.sum')} us  dram rd {f('dram__bytes_read.sum')} MB  wr {f('dram__bytes_write.sum')} MB"
+              f"  dram% {f('gpu__dram_throughput.avg.pct_of_peak_sustained_elapsed')}  issue% {f('smsp__issue_active.avg.pct_of_peak_sustained_active')}"
+              f"  warps% {f('sm__warps_active.avg.pct_of_peak_sustained_active')}  inst {f('smsp__inst_executed.sum')}  grid {f('launch__grid_size')}"
+              f"  regs {f('launch__registers_per_thread')}")
+        st = []
+        for h, v in d.items():
+            if h.startswith("smsp__pcsamp_warps_issue_stalled") and not h.endswith("not_issued"):
+                try:
+                    st.append((float(v), h.replace("smsp__pcsamp_warps_issue_stalled_", "")))
+                except ValueError:
+                    pass
+        tot = sum(v for v, _ in st) or 1
+        print("   stalls: " + ", ".join(f"{h} {v / tot * 100:.0f}%" for v, h in sorted(st, reverse=True)[:7]))
+
+
+if __name__ == "__main__":
+    main(sys.argv[1], sys.argv[2] if len(sys.argv) > 2 else None)
+
+
+def hot_lines(rep, kernel_regex, top=25, by="Warp Stall Sampling (All Samples)"):
+    rows = ncu_csv(rep, "--page", "source", "-k", f"regex:{kernel_regex}", "--launch-count", "1",
+                   "--print-source", "sass")
+    hi = [i for i, x in enumerate(rows) if by in x][0]
+    hdr = rows[hi]
+    body = [x for x in rows[hi + 1:] if len(x) == len(hdr)]
+    i_s, i_src, i_ex = hdr.index(by), hdr.index("Source"), hdr.index("Instructions Executed")
+
+    def num(v):
+        try:
+            return float(v)
+        except ValueError:
+            return 0.0
+    tot = sum(num(x[i_s]) for x in body)
+    print(f"   total {by}: {tot:.0f}; instructions executed: {sum(num(x[i_ex]) for x in body):.0f}")
+    for x in sorted(body, key=lambda x: -num(x[i_s]))[:top]:
+        print(f"   {num(x[i_s]):8.0f} {num(x[i_ex]):10.0f}  {x[0][-5:]}  {x[i_src].strip()[:90]}")
