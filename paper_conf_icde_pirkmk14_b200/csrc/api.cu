@@ -341,12 +341,29 @@ static ar_status setup_scan(const ar_pred* preds, int32_t npred, ard::SelParams&
         p.hi = preds[c].hi;
         words += (P.tile_rows / 32) * (uint32_t)w;
         ashift += (uint32_t)w;
+        // the one-pass kernel streams device-resident residual tiles with the majors (dense
+        // 8-bit residuals: streaming ~1.4x the touched bytes beats a dependent gather round trip)
+        if (fused && k > 0 && col->d.residual_loc == AR_LOC_DEVICE && col->residual) {
+            p.res_stream = 1;
+            p.res_soff = words;
+            words += (P.tile_rows / 32) * (uint32_t)k + 4;   // + 16 B: the copy rounds up to 16 B
+        }
     }
     uint32_t planes = 0;
     for (int c = 0; c < npred; ++c) planes += P.p[c].w;
     if (planes > AR_MAX_PLANES) {
         set_error("sum of w_major over predicates = %u > AR_MAX_PLANES (%d)", planes, AR_MAX_PLANES);
         return AR_ERR_UNSUPPORTED;
+    }
+    for (int c = 0; c < npred; ++c) {
+        const ard::SelPred& p = P.p[c];
+        for (uint32_t j = 0; j < p.w; ++j) {
+            uint32_t* m = P.pm[p.ashift + j];
+            m[0] = 0u - ((p.clo >> j) & 1u);
+            m[1] = 0u - ((p.chi >> j) & 1u);
+            m[2] = 0u - ((p.dlo >> j) & 1u);
+            m[3] = 0u - ((p.dhi >> j) & 1u);
+        }
     }
     P.npred = npred;
     P.n = n;

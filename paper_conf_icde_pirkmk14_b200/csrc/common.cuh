@@ -218,22 +218,32 @@ __device__ __forceinline__ unsigned long long lookback_wide(const unsigned long 
 
 // --- value extraction ----------------------------------------------------------
 
-// Value of row p from a PACKED LSB-first bitstream of width w (1..32).
+// Gather load of one word.  On B200 a plain scalar load makes L2 fetch a whole
+// 128-B line from HBM; the .L2::64B prefetch-size hint halves that, which is the
+// smallest gather granularity measured (tools/gather_probe.cu, DESIGN "Gathers").
+__device__ __forceinline__ uint32_t ld_gather(const uint32_t* p) {
+    uint32_t v;
+    asm("ld.global.nc.L2::64B.u32 %0, [%1];" : "=r"(v) : "l"(p));
+    return v;
+}
+
+// Value of row p from a PACKED LSB-first bitstream of width w (1..32) in global memory.
 __device__ __forceinline__ uint32_t packed_get(const uint32_t* __restrict__ s, uint64_t p, int w) {
     uint64_t bit = p * (uint64_t)w;
     uint64_t wi = bit >> 5;
     uint32_t sh = (uint32_t)(bit & 31);
-    uint32_t lo = __ldg(s + wi);
+    uint32_t lo = ld_gather(s + wi);
     uint32_t v = lo >> sh;
-    if (sh + (uint32_t)w > 32u) v = __funnelshift_r(lo, __ldg(s + wi + 1), sh);
+    if (sh + (uint32_t)w > 32u) v = __funnelshift_r(lo, ld_gather(s + wi + 1), sh);
     return w == 32 ? v : (v & ((1u << w) - 1u));
 }
-// Same, for residuals that may live in pinned host memory (no read-only cache path assumption).
-__device__ __forceinline__ uint32_t packed_get_any(const uint32_t* s, uint64_t p, int w) {
-    uint64_t bit = p * (uint64_t)w;
-    uint64_t wi = bit >> 5;
-    uint32_t sh = (uint32_t)(bit & 31);
-    uint32_t lo = s[wi];
+// Residual gather: device memory or pinned host memory through a mapped pointer.
+__device__ __forceinline__ uint32_t packed_get_any(const uint32_t* s, uint64_t p, int w) { return packed_get(s, p, w); }
+
+// Same extraction from a PACKED stream staged in shared memory (bit offset `bit`).
+__device__ __forceinline__ uint32_t packed_get_smem(const uint32_t* s, uint32_t bit, int w) {
+    const uint32_t wi = bit >> 5, sh = bit & 31;
+    const uint32_t lo = s[wi];
     uint32_t v = lo >> sh;
     if (sh + (uint32_t)w > 32u) v = __funnelshift_r(lo, s[wi + 1], sh);
     return w == 32 ? v : (v & ((1u << w) - 1u));

@@ -16,6 +16,8 @@ struct SelPred {
     // refine-side data, used by the fused kernel
     const uint32_t* residual; // PACKED width k (device or host-mapped), null if k == 0
     uint32_t k, base, lo, hi; // exact predicate on v = ((m << k) | r) + base
+    uint32_t res_stream;      // fused kernel: residual tile streamed into the stage (device-resident residuals)
+    uint32_t res_soff;        // word offset of the streamed residual tile inside a stage
 };
 
 // Aggregate factor of the SUM product.
@@ -41,6 +43,7 @@ constexpr int kStageEntries = 2048;               // output staging entries (pos
 
 struct SelParams {
     SelPred p[AR_MAX_PRED];
+    uint32_t pm[AR_MAX_PLANES][4];   // per global plane (ashift + j): cand lo/hi, def lo/hi bit as 0 / ~0
     int32_t npred;
     int32_t carry;            // write the approximation word into aux
     int64_t n;

@@ -46,13 +46,16 @@ __device__ __forceinline__ uint32_t borrow_rsub(uint32_t x, uint32_t cbit, uint3
 }
 __device__ __forceinline__ uint32_t bitmask(uint32_t v, uint32_t j) { return 0u - ((v >> j) & 1u); }
 
-template <int W>
-__device__ __forceinline__ uint32_t range_mask(const uint32_t* x, uint32_t lo, uint32_t hi) {
+// Bound bits come as precomputed all-0 / all-1 words from the kernel parameters
+// (pm[plane][0..3] = candidate lo / hi, definite lo / hi), so with compile-time
+// plane indices each LOP3 takes its bound straight from the constant bank.
+template <int W, int O, int LO, int HI>
+__device__ __forceinline__ uint32_t range_mask_pm(const uint32_t* x, const SelParams& P) {
     uint32_t bl = 0, bh = 0;
 #pragma unroll
     for (int j = 0; j < W; ++j) {
-        bl = borrow_sub(x[j], bitmask(lo, j), bl);
-        bh = borrow_rsub(x[j], bitmask(hi, j), bh);
+        bl = borrow_sub(x[j], P.pm[O + j][LO], bl);
+        bh = borrow_rsub(x[j], P.pm[O + j][HI], bh);
     }
     return ~(bl | bh);
 }
@@ -65,6 +68,17 @@ __device__ __forceinline__ uint32_t plane_value(const uint32_t* pl, uint32_t w, 
 }
 
 // ------------------------------------------------------------ plane sources
+
+template <int I>
+using ic = std::integral_constant<int, I>;
+template <int N, int I = 0, class F>
+__device__ __forceinline__ void static_for(F&& f) {
+    if constexpr (I < N) {
+        f(ic<I>{});
+        static_for<N, I + 1>(f);
+    }
+}
+
 
 template <int... Ws>
 __host__ __device__ constexpr int wid(int c) {
@@ -84,6 +98,15 @@ template <int BPT, int... Ws>
 struct FixedPlanes {
     static constexpr int N = sizeof...(Ws);
     static constexpr int TOTAL = (0 + ... + Ws);
+    // shape ops: compile-time predicate loop and widths
+    template <class F>
+    __device__ __forceinline__ static void for_pred(const SelParams&, F&& f) {
+        static_for<N>(f);
+    }
+    template <int C>
+    __device__ __forceinline__ static constexpr uint32_t pw(const SelParams&, std::integral_constant<int, C>) {
+        return (uint32_t)wid<Ws...>(C);
+    }
     uint32_t x[BPT][TOTAL > 0 ? TOTAL : 1];
 
     template <int C>
@@ -117,12 +140,12 @@ struct FixedPlanes {
             const SelPred& p = P.p[C];
 #pragma unroll
             for (int b = 0; b < BPT; ++b) {
-                const uint32_t c = range_mask<w>(&x[b][o], p.clo, p.chi);
+                const uint32_t c = range_mask_pm<w, o, 0, 1>(&x[b][o], P);
                 cm[b] &= c;
                 if (p.mode == 0)
                     dm[b] &= c;
                 else if (p.mode == 1)
-                    dm[b] &= range_mask<w>(&x[b][o], p.dlo, p.dhi);
+                    dm[b] &= range_mask_pm<w, o, 2, 3>(&x[b][o], P);
                 else
                     dm[b] = 0;
             }
@@ -165,6 +188,11 @@ struct FixedPlanes {
 template <int BPT>
 struct DynPlanes {
     const uint32_t* stg;
+    template <class F>
+    __device__ __forceinline__ static void for_pred(const SelParams& P, F&& f) {
+        for (int c = 0; c < P.npred; ++c) f(c);
+    }
+    __device__ __forceinline__ static uint32_t pw(const SelParams& P, int c) { return P.p[c].w; }
 
     __device__ __forceinline__ void load(const SelParams&, const uint32_t* s) { stg = s; }
 
@@ -214,16 +242,6 @@ struct requires_params : std::false_type {};
 template <int BPT>
 struct requires_params<DynPlanes<BPT>> : std::true_type {};
 
-template <int I>
-using ic = std::integral_constant<int, I>;
-template <int N, int I = 0, class F>
-__device__ __forceinline__ void static_for(F&& f) {
-    if constexpr (I < N) {
-        f(ic<I>{});
-        static_for<N, I + 1>(f);
-    }
-}
-
 template <class PS, int B>
 __device__ __forceinline__ uint32_t ps_value(const PS& ps, const SelParams& P, int c, uint32_t l) {
     if constexpr (requires_params<PS>::value)
@@ -260,8 +278,10 @@ __device__ __forceinline__ SmemLayout carve(unsigned char* smem, uint32_t nstage
     } else {
         L.st_pos = L.st_aux = nullptr;
     }
-    uintptr_t a = (reinterpret_cast<uintptr_t>(p) + 127) & ~uintptr_t(127);
-    L.stages = reinterpret_cast<uint32_t*>(a);
+    // align by offset from the smem base (an integer round trip would lose the
+    // shared address space and turn every stage access into a generic load)
+    const size_t off = (size_t)(p - smem);
+    L.stages = reinterpret_cast<uint32_t*>(smem + ((off + 127) & ~size_t(127)));
     return L;
 }
 
@@ -284,14 +304,23 @@ __device__ __forceinline__ void produce(const SelParams& P, const SmemLayout& L)
         const int64_t rows = min((int64_t)P.tile_rows, P.n - r0);
         const uint32_t groups = (uint32_t)((rows + 127) / 128);   // 128-row groups, 16 B per plane
         uint32_t bytes = 0;
-        for (int c = 0; c < P.npred; ++c) bytes += groups * 16u * P.p[c].w;
+        for (int c = 0; c < P.npred; ++c) {
+            bytes += groups * 16u * P.p[c].w;
+            if (P.p[c].res_stream) bytes += (uint32_t)(((rows * P.p[c].k + 7) / 8 + 15) / 16 * 16);
+        }
         mbar_arrive_expect_tx(L.full + s, bytes);
         uint32_t* stg = L.stages + (size_t)s * P.stage_words;
         for (int c = 0; c < P.npred; ++c) {
             const uint32_t w = P.p[c].w;
-            if (w == 0) continue;
-            const uint32_t* src = P.p[c].planes + (size_t)t * blocks_per_tile * w;
-            bulk_g2s(stg + P.p[c].soff, src, groups * 16u * w, L.full + s, pol);
+            if (w > 0) {
+                const uint32_t* src = P.p[c].planes + (size_t)t * blocks_per_tile * w;
+                bulk_g2s(stg + P.p[c].soff, src, groups * 16u * w, L.full + s, pol);
+            }
+            if (P.p[c].res_stream) {   // the tile's residual bits, a contiguous 16-B aligned byte range
+                const uint32_t k = P.p[c].k;
+                const uint32_t* src = P.p[c].residual + (size_t)t * (P.tile_rows / 32) * k;
+                bulk_g2s(stg + P.p[c].res_soff, src, (uint32_t)(((rows * k + 7) / 8 + 15) / 16 * 16), L.full + s, pol);
+            }
         }
     }
 }
@@ -410,7 +439,7 @@ __device__ __forceinline__ uint32_t stage_value(const SelParams& P, const uint32
 }
 
 template <class PS, int NW, int BPT>
-__global__ void __launch_bounds__((NW + 1) * 32) fused_kernel(const __grid_constant__ SelParams P) {
+__global__ void __launch_bounds__((NW + 1) * 32, 2) fused_kernel(const __grid_constant__ SelParams P) {
     constexpr int kWarpRows = 32 * 32 * BPT;
     extern __shared__ __align__(128) unsigned char smem[];
     const SmemLayout L = carve(smem, P.nstages, false);
@@ -457,7 +486,7 @@ __global__ void __launch_bounds__((NW + 1) * 32) fused_kernel(const __grid_const
             if (lane >= (unsigned)o) incl += y;
         }
         const uint32_t total = __shfl_sync(0xffffffffu, incl, 31);
-        uint32_t e = incl - cnt;
+        uint32_t e = incl - cnt;   // this thread's first slot in the warp list
 #pragma unroll
         for (int b = 0; b < BPT; ++b) {
             uint32_t m = cm[b];
@@ -470,34 +499,45 @@ __global__ void __launch_bounds__((NW + 1) * 32) fused_kernel(const __grid_const
         __syncwarp();
 
         // a5 + a6 over the list: each lane takes kPer entries per pass
-        const uint32_t blk0 = warp * 32 * BPT;          // first tile-block of this warp
-        const uint64_t row_base = (uint64_t)tile_r0 + (uint64_t)warp * kWarpRows;
+        const uint32_t row_in_tile0 = warp * kWarpRows;
+        const uint64_t row_base = (uint64_t)tile_r0 + row_in_tile0;
         for (uint32_t base = 0; base < total; base += 32 * kPer) {
-            uint32_t ent[kPer];
-            bool ok[kPer];
+            uint32_t off[kPer];
+            bool ok[kPer], dfn[kPer];
 #pragma unroll
             for (int q = 0; q < kPer; ++q) {
                 const uint32_t k = base + q * 32 + lane;
-                ent[q] = k < total ? list[k] : 0u;
+                const uint32_t e = k < total ? list[k] : 0u;
                 ok[q] = k < total;
+                dfn[q] = (e & kDefFlag) != 0;
+                off[q] = e & 0x7fffu;   // row offset inside the warp slice
             }
-            // refine non-definite entries: residual gathers first (all in flight), then the exact test
-            for (int c = 0; c < P.npred; ++c) {
-                const SelPred& p = P.p[c];
-                if (p.k == 0) continue;   // exact already at the approximation
+            // refine non-definite entries (Alg. 2): residual + major -> exact value -> predicate
+            PS::for_pred(P, [&](auto cc) {
+                const SelPred& p = P.p[int(cc)];
+                if (p.k == 0) return;   // exact already at the approximation
+                const uint32_t w = PS::pw(P, cc);
                 uint32_t r[kPer];
 #pragma unroll
-                for (int q = 0; q < kPer; ++q)
-                    r[q] = (ok[q] && !(ent[q] & kDefFlag))
-                               ? packed_get_any(p.residual, row_base + (ent[q] & 0x7fffu), p.k) : 0u;
+                for (int q = 0; q < kPer; ++q) {
+                    const bool need = ok[q] && !dfn[q];
+                    if (p.res_stream)
+                        r[q] = need ? packed_get_smem(stg + p.res_soff, (row_in_tile0 + off[q]) * p.k, p.k) : 0u;
+                    else
+                        r[q] = need ? packed_get_any(p.residual, row_base + off[q], p.k) : 0u;
+                }
 #pragma unroll
                 for (int q = 0; q < kPer; ++q) {
-                    if (!ok[q] || (ent[q] & kDefFlag)) continue;
-                    const uint32_t m = stage_value(P, stg, c, blk0 + ((ent[q] & 0x7fffu) >> 5), ent[q] & 31u);
+                    if (!ok[q] || dfn[q]) continue;
+                    const uint32_t* pl = stg + p.soff + ((row_in_tile0 + off[q]) >> 5) * w;
+                    const uint32_t l = off[q] & 31u;
+                    uint32_t m = 0;
+#pragma unroll
+                    for (uint32_t j = 0; j < w; ++j) m |= ((pl[j] >> l) & 1u) << j;
                     const uint32_t v = ((m << p.k) | r[q]) + p.base;
                     ok[q] = (v >= p.lo) && (v <= p.hi);
                 }
-            }
+            });
 #pragma unroll
             for (int q = 0; q < kPer; ++q) nres += ok[q];
             if (P.nagg > 0) {
@@ -508,18 +548,31 @@ __global__ void __launch_bounds__((NW + 1) * 32) fused_kernel(const __grid_const
                     const AggCol& A = P.a[a];
                     uint32_t v[kPer];
 #pragma unroll
-                    for (int q = 0; q < kPer; ++q) {
-                        const uint64_t row = row_base + (ent[q] & 0x7fffu);
-                        if (!ok[q]) {
-                            v[q] = 0u;
-                        } else if (A.pred >= 0) {
-                            const uint32_t m =
-                                stage_value(P, stg, A.pred, blk0 + ((ent[q] & 0x7fffu) >> 5), ent[q] & 31u);
-                            const uint32_t r = A.k ? packed_get_any(A.residual, row, A.k) : 0u;
-                            v[q] = ((m << A.k) | r) + A.base;
-                        } else {
-                            v[q] = agg_gather(A, row);
-                        }
+                    for (int q = 0; q < kPer; ++q) v[q] = 0u;
+                    if (A.pred >= 0) {
+                        // an aggregate that is also a predicate column: its major is in the stage
+                        PS::for_pred(P, [&](auto cc) {
+                            if (int(cc) != A.pred) return;
+                            const SelPred& p = P.p[int(cc)];
+                            const uint32_t w = PS::pw(P, cc);
+#pragma unroll
+                            for (int q = 0; q < kPer; ++q) {
+                                if (!ok[q]) continue;
+                                const uint32_t* pl = stg + p.soff + ((row_in_tile0 + off[q]) >> 5) * w;
+                                const uint32_t l = off[q] & 31u;
+                                uint32_t m = 0;
+#pragma unroll
+                                for (uint32_t j = 0; j < w; ++j) m |= ((pl[j] >> l) & 1u) << j;
+                                uint32_t r = 0u;
+                                if (p.k)
+                                    r = p.res_stream ? packed_get_smem(stg + p.res_soff, (row_in_tile0 + off[q]) * p.k, p.k)
+                                                     : packed_get_any(p.residual, row_base + off[q], p.k);
+                                v[q] = ((m << p.k) | r) + p.base;
+                            }
+                        });
+                    } else {
+#pragma unroll
+                        for (int q = 0; q < kPer; ++q) v[q] = ok[q] ? agg_gather(A, row_base + off[q]) : 0u;
                     }
 #pragma unroll
                     for (int q = 0; q < kPer; ++q) prod[q] *= v[q];

@@ -57,3 +57,35 @@ def hot_lines(rep, kernel_regex, top=25, by="Warp Stall Sampling (All Samples)")
     print(f"   total {by}: {tot:.0f}; instructions executed: {sum(num(x[i_ex]) for x in body):.0f}")
     for x in sorted(body, key=lambda x: -num(x[i_s]))[:top]:
         print(f"   {num(x[i_s]):8.0f} {num(x[i_ex]):10.0f}  {x[0][-5:]}  {x[i_src].strip()[:90]}")
+
+
+def hot_blocks(rep, kernel_regex, top=14, key="inst"):
+    """Group SASS into runs of equal execution count (≈ basic blocks); rank by instructions or stalls."""
+    rows = ncu_csv(rep, "--page", "source", "-k", f"regex:{kernel_regex}", "--launch-count", "1",
+                   "--print-source", "sass")
+    hi = [i for i, x in enumerate(rows) if "Instructions Executed" in x][0]
+    hdr = rows[hi]
+    body = []
+    for x in rows[hi + 1:]:
+        if "Instructions Executed" in x:
+            break                      # next launch's table
+        if len(x) == len(hdr):
+            body.append(x)
+    ie, src = hdr.index("Instructions Executed"), hdr.index("Source")
+    ws = hdr.index("Warp Stall Sampling (All Samples)")
+    blocks = []
+    for x in body:
+        c, s = float(x[ie] or 0), float(x[ws] or 0)
+        if blocks and blocks[-1][0] == c:
+            blocks[-1][1] += 1
+            blocks[-1][3] += s
+            blocks[-1][4].append(x[src].strip())
+        else:
+            blocks.append([c, 1, x[0][-5:], s, [x[src].strip()]])
+    tot = sum(b[0] * b[1] for b in blocks) or 1
+    tws = sum(b[3] for b in blocks) or 1
+    print(f"   instructions {tot:.0f}, stall samples {tws:.0f}")
+    k = (lambda b: -b[0] * b[1]) if key == "inst" else (lambda b: -b[3])
+    for b in sorted(blocks, key=k)[:top]:
+        print(f"   {b[0]:9.0f} x{b[1]:4d} = {b[0] * b[1] / tot * 100:5.1f}% inst {b[3] / tws * 100:5.1f}% stall"
+              f" @{b[2]}: {' | '.join(b[4][:7])[:170]}")
