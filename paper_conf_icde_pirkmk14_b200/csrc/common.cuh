@@ -223,7 +223,7 @@ __device__ __forceinline__ unsigned long long lookback_wide(const unsigned long 
 // smallest gather granularity measured (tools/gather_probe.cu, DESIGN "Gathers").
 __device__ __forceinline__ uint32_t ld_gather(const uint32_t* p) {
     uint32_t v;
-    asm("ld.global.nc.L2::64B.u32 %0, [%1];" : "=r"(v) : "l"(p));
+    asm volatile("ld.global.nc.L2::64B.u32 %0, [%1];" : "=r"(v) : "l"(p));   // volatile: never speculated past its guard
     return v;
 }
 

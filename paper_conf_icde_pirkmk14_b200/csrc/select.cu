@@ -290,9 +290,9 @@ __device__ __forceinline__ SmemLayout carve(unsigned char* smem, uint32_t nstage
 __device__ __forceinline__ void produce(const SelParams& P, const SmemLayout& L) {
     const uint64_t pol = policy_evict_first();
     const uint32_t blocks_per_tile = P.tile_rows / 32;
+    uint32_t s = 0, ph = 0;   // ring slot and its phase parity (no integer division in the loop)
     for (uint32_t i = 0;; ++i) {
-        const uint32_t s = i % P.nstages;
-        if (i >= P.nstages) mbar_wait(L.empty + s, ((i / P.nstages) - 1) & 1);
+        if (i >= P.nstages) mbar_wait(L.empty + s, ph ^ 1u);
         const long long t = (long long)blockIdx.x + (long long)i * gridDim.x;
         if (t >= P.num_tiles) {
             L.slot[s] = -1;
@@ -321,6 +321,10 @@ __device__ __forceinline__ void produce(const SelParams& P, const SmemLayout& L)
                 const uint32_t* src = P.p[c].residual + (size_t)t * (P.tile_rows / 32) * k;
                 bulk_g2s(stg + P.p[c].res_soff, src, (uint32_t)(((rows * k + 7) / 8 + 15) / 16 * 16), L.full + s, pol);
             }
+        }
+        if (++s == P.nstages) {
+            s = 0;
+            ph ^= 1u;
         }
     }
 }
@@ -355,9 +359,9 @@ __global__ void __launch_bounds__((NW + 1) * 32) select_kernel(const __grid_cons
         return;
     }
 
-    for (uint32_t i = 0;; ++i) {
-        const uint32_t s = i % P.nstages;
-        mbar_wait(L.full + s, (i / P.nstages) & 1);
+    uint32_t s = 0, ph = 0;
+    for (;; s = (s + 1 == P.nstages) ? (ph ^= 1u, 0u) : s + 1) {
+        mbar_wait(L.full + s, ph);
         const long long t = L.slot[s];
         if (t < 0) break;
         const int64_t r0 = t * (int64_t)P.tile_rows + (int64_t)threadIdx.x * (32 * BPT);
@@ -454,9 +458,9 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_kernel(const __grid_co
     }
 
     unsigned long long sum = 0, nres = 0, ncand = 0, ndef = 0;
-    for (uint32_t i = 0;; ++i) {
-        const uint32_t s = i % P.nstages;
-        mbar_wait(L.full + s, (i / P.nstages) & 1);
+    uint32_t s = 0, ph = 0;
+    for (;; s = (s + 1 == P.nstages) ? (ph ^= 1u, 0u) : s + 1) {
+        mbar_wait(L.full + s, ph);
         const long long t = L.slot[s];
         if (t < 0) break;
         const uint32_t* stg = L.stages + (size_t)s * P.stage_words;
