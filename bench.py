@@ -12,9 +12,13 @@ SUM(l_extendedprice * l_discount).  With N GPUs each rank holds its own
 60 M-row range of an SF(10 N) table (weak scaling) and the step adds the count
 allgather (a4) and the int64 SUM allreduce over NCCL.
 
-One step = one pass of the whole hot path: a2+a3 approximate select with
-stable compaction (candidate relation materialised), a4 (N > 1), a5+a6 fused
-refine + SUM.  `--variant fused` times the one-pass a3+a5+a6 kernel instead.
+One step = one pass of the whole hot path over the batch.  Headline
+(`--variant fused`, default): ar_select_refine_sum, the one-pass kernel that
+runs a2+a3 (approximate select, candidate relation compacted per warp in shared
+memory), a5 (refine) and a6 (SUM), then (N > 1) the SUM allreduce.  The staged
+pipeline is timed in the same run and reported under "variants": a2+a3
+ar_approx_select with the ordered candidate list in HBM, a4 count allgather
+(N > 1), a5+a6 ar_refine_sum.
 Inputs are resident in HBM; R copies of the decomposed columns are rotated so
 consecutive steps never re-read L2-resident data (R x 345 MB > 126 MB L2).
 The K timed steps are one CUDA-graph replay; per-kernel durations come from
@@ -53,7 +57,9 @@ def parse():
     ap.add_argument("--steps", type=int, default=1000)
     ap.add_argument("--warmup", type=int, default=10)
     ap.add_argument("--impl", choices=["ours", "reference"], default="ours")
-    ap.add_argument("--variant", choices=["staged", "fused"], default="staged")
+    ap.add_argument("--variant", choices=["staged", "fused"], default="fused",
+                    help="headline variant (the other one is timed too and reported under 'variants')")
+    ap.add_argument("--only", action="store_true", help="time the headline variant only")
     ap.add_argument("--sf", type=float, default=SF_PER_GPU, help="scale factor per GPU")
     ap.add_argument("--copies", type=int, default=3, help="rotated input copies (L2 defeat)")
     ap.add_argument("--e2e-steps", type=int, default=10)
@@ -266,7 +272,7 @@ def ours(args):
     s_ptr = stream.cuda_stream
     cands = cu.CandidateList(rows, device=dev)
     ws_sel = cu.Workspace(_ar.ar_select_ws_bytes(rows), device=dev)
-    out = torch.zeros(4, dtype=torch.int64, device=dev)        # sum, count, (fused: cand, def)
+    out = torch.zeros(4, dtype=torch.int64, device=dev)        # SUM, |result|, (fused: |cand|, |def|)
     counts = torch.zeros(world, dtype=torch.int64, device=dev)
     goff = torch.zeros(1, dtype=torch.int64, device=dev)
 
@@ -276,13 +282,24 @@ def ours(args):
     pred_sets = [preds_of(cs) for cs in copies]
     agg_sets = [[cs[3].handle, cs[1].handle] for cs in copies]
 
-    launches_per_step = 0
-    kernel_names = []
+    def new_event():
+        err, e = drv.cuEventCreate(drv.CUevent_flags.CU_EVENT_DEFAULT)
+        assert err == drv.CUresult.CUDA_SUCCESS, err
+        return e
 
-    def step(i, ev=None):
-        """One pass of the hot path on copy i % R; ev = (events) recorded around each kernel."""
+    def rec(e):
+        err, = drv.cuEventRecordWithFlags(e, s_ptr, drv.CUevent_record_flags.CU_EVENT_RECORD_EXTERNAL)
+        assert err == drv.CUresult.CUDA_SUCCESS, err
+
+    def elapsed(a, b):
+        err, ms = drv.cuEventElapsedTime(a, b)
+        assert err == drv.CUresult.CUDA_SUCCESS, err
+        return ms
+
+    def step(variant, i, ev=None):
+        """One pass of the hot path on copy i % R; ev = events recorded around each kernel."""
         r = i % len(copies)
-        if args.variant == "staged":
+        if variant == "staged":
             if ev is not None:
                 rec(ev[0])
             _ar.ar_approx_select(pred_sets[r], _ar.AR_SELECT_CARRY_APPR, cands.c, ws_sel.ptr, ws_sel.nbytes, s_ptr)
@@ -306,81 +323,56 @@ def ours(args):
             if dist_h:
                 _ar.ar_dist_sum(dist_h, out.data_ptr(), 4, s_ptr)
 
-    if args.variant == "staged":
-        launches_per_step = 2 + (1 if dist_h else 0)
-        kernel_names = ["select_kernel", "refine_sum_kernel"] + (["exclusive_offset_kernel"] if dist_h else [])
-        n_ev = 4
-    else:
-        launches_per_step = 1
-        kernel_names = ["fused_kernel"]
-        n_ev = 2
-
-    def new_event():
-        err, e = drv.cuEventCreate(drv.CUevent_flags.CU_EVENT_DEFAULT)
-        assert err == drv.CUresult.CUDA_SUCCESS, err
-        return e
-
-    def rec(e):
-        err, = drv.cuEventRecordWithFlags(e, s_ptr, drv.CUevent_record_flags.CU_EVENT_RECORD_EXTERNAL)
-        assert err == drv.CUresult.CUDA_SUCCESS, err
-
-    def elapsed(a, b):
-        err, ms = drv.cuEventElapsedTime(a, b)
-        assert err == drv.CUresult.CUDA_SUCCESS, err
-        return ms
-
-    # eager warm-up (also primes attribute caches before capture)
-    with torch.cuda.stream(stream):
-        for i in range(max(3, args.warmup)):
-            step(i)
-    stream.synchronize()
-
-    # capture the W warm-up steps and the K timed steps as two graphs
+    KERNELS = {"staged": ["select_kernel", "refine_sum_kernel"] + (["exclusive_offset_kernel"] if dist_h else []),
+               "fused": ["fused_kernel"]}
     K = args.steps
-    evs = [[new_event() for _ in range(n_ev)] for _ in range(K)]
-    g_warm, g_timed = torch.cuda.CUDAGraph(), torch.cuda.CUDAGraph()
-    with torch.cuda.graph(g_warm, stream=stream, capture_error_mode="relaxed"):
-        for i in range(args.warmup):
-            step(i)
-    with torch.cuda.graph(g_timed, stream=stream, capture_error_mode="relaxed"):
-        for i in range(K):
-            step(i + args.warmup, evs[i])
-    torch.cuda.synchronize()
 
-    sampler = ClockSampler(torch.cuda.current_device() if "CUDA_VISIBLE_DEVICES" not in os.environ else local)
-    t_start, t_end = new_event(), new_event()
-    with torch.cuda.stream(stream):
-        g_warm.replay()
+    def time_variant(variant, sampler=None):
+        # eager warm-up (also primes the library's attribute / occupancy caches before capture)
+        with torch.cuda.stream(stream):
+            for i in range(max(3, args.warmup)):
+                step(variant, i)
         stream.synchronize()
+        n_ev = 4 if variant == "staged" else 2
+        evs = [[new_event() for _ in range(n_ev)] for _ in range(K)]
+        g_warm, g_timed = torch.cuda.CUDAGraph(), torch.cuda.CUDAGraph()
+        with torch.cuda.graph(g_warm, stream=stream, capture_error_mode="relaxed"):
+            for i in range(args.warmup):
+                step(variant, i)
+        with torch.cuda.graph(g_timed, stream=stream, capture_error_mode="relaxed"):
+            for i in range(K):
+                step(variant, i + args.warmup, evs[i])
+        torch.cuda.synchronize()
+        t0, t1 = new_event(), new_event()
+        with torch.cuda.stream(stream):
+            g_warm.replay()
+            stream.synchronize()
+            if pg:
+                pg.barrier()
+            torch.cuda.synchronize()
+            ctx = sampler if sampler is not None else _Null()
+            with ctx:
+                drv.cuEventRecord(t0, s_ptr)
+                g_timed.replay()
+                drv.cuEventRecord(t1, s_ptr)
+                stream.synchronize()
+        torch.cuda.synchronize()
         if pg:
             pg.barrier()
-        torch.cuda.synchronize()
-        with sampler:
-            drv.cuEventRecord(t_start, s_ptr)
-            g_timed.replay()
-            drv.cuEventRecord(t_end, s_ptr)
-            stream.synchronize()
-    torch.cuda.synchronize()
-    if pg:
-        pg.barrier()
-    ms_total = elapsed(t_start, t_end)
-    if pg:
-        t = torch.tensor([ms_total], dtype=torch.float64, device=dev)
-        pg.all_reduce(t, op=pg.ReduceOp.MAX)
-        ms_total = float(t.item())
-    ms_step = ms_total / K
-    value = rows * world * K / (ms_total / 1e3)
+        ms_total = elapsed(t0, t1)
+        if pg:
+            t = torch.tensor([ms_total], dtype=torch.float64, device=dev)
+            pg.all_reduce(t, op=pg.ReduceOp.MAX)
+            ms_total = float(t.item())
+        if variant == "staged":
+            kern = {"select_kernel": [elapsed(e[0], e[1]) for e in evs],
+                    "refine_sum_kernel": [elapsed(e[2], e[3]) for e in evs]}
+        else:
+            kern = {"fused_kernel": [elapsed(e[0], e[1]) for e in evs]}
+        res = out.cpu().tolist()
+        del g_warm, g_timed
+        return ms_total, {k: statistics.mean(v) for k, v in kern.items()}, res
 
-    # per-kernel durations inside the timed region
-    if args.variant == "staged":
-        k_sel = [elapsed(e[0], e[1]) for e in evs]
-        k_ref = [elapsed(e[2], e[3]) for e in evs]
-        kernels = {"select_kernel": k_sel, "refine_sum_kernel": k_ref}
-    else:
-        kernels = {"fused_kernel": [elapsed(e[0], e[1]) for e in evs]}
-    kern_ms = {k: statistics.mean(v) for k, v in kernels.items()}
-
-    res = out.cpu().tolist()
     ab = algorithmic_bytes(cols, rows)
     peaks = {}
     try:
@@ -390,26 +382,38 @@ def ours(args):
     hbm_peak = peaks.get("hbm_gbs")
     peak_src = "measured (MEASURED_PEAKS.json hbm_gbs)" if hbm_peak else "fallback (B200_PROFILING.md 6.65 TB/s)"
     hbm_peak = hbm_peak or 6650.0
+    per_kernel_bytes = {
+        "fused_kernel": ab["total"],                                        # majors + touched residual/ep sectors
+        "select_kernel": ab["scan"] + ab["cand_list_bytes"],                # majors read + (pos, aux) written
+        "refine_sum_kernel": ab["cand_list_bytes"] + ab["gather"] + 16.0,   # cands read + sector gathers + out
+    }
 
-    # dominant kernel roofline: algorithmic bytes per launch / mean launch duration
-    if args.variant == "staged":
-        sel_bytes = ab["scan"] + ab["cand_list_bytes"]                       # majors read + (pos, aux) written
-        ref_bytes = ab["cand_list_bytes"] + ab["gather"] + 16.0               # cands read + sector gathers + out
-        per_kernel_bytes = {"select_kernel": sel_bytes, "refine_sum_kernel": ref_bytes}
-    else:
-        per_kernel_bytes = {"fused_kernel": ab["total"]}
-    dom = max(kern_ms, key=lambda k: kern_ms[k])
-    achieved = per_kernel_bytes[dom] / (kern_ms[dom] / 1e3) / 1e9
-    roofline = {"bound": "hbm", "achieved": achieved, "peak": hbm_peak, "unit": "GB/s", "frac": achieved / hbm_peak,
-                "traffic": None, "kernel": dom, "algorithmic_bytes_per_launch": per_kernel_bytes[dom],
-                "kernel_ms": kern_ms[dom], "peak_source": peak_src,
-                "per_kernel": {k: {"ms": kern_ms[k], "bytes": per_kernel_bytes[k],
-                                   "gbs": per_kernel_bytes[k] / (kern_ms[k] / 1e3) / 1e9} for k in kern_ms},
-                "step_bytes": ab["total"], "step_frac": ab["total"] / (ms_step / 1e3) / 1e9 / hbm_peak}
+    variants = [args.variant] + [v for v in ("fused", "staged") if v != args.variant and not args.only]
+    results = {}
+    sampler = ClockSampler(torch.cuda.current_device() if "CUDA_VISIBLE_DEVICES" not in os.environ else local)
+    for v in variants:
+        ms_total, kern_ms, res = time_variant(v, sampler if v == args.variant else None)
+        ms_step = ms_total / K
+        dom = max(kern_ms, key=lambda k: kern_ms[k])
+        achieved = per_kernel_bytes[dom] / (kern_ms[dom] / 1e3) / 1e9
+        results[v] = {
+            "value": rows * world * K / (ms_total / 1e3), "ms_per_step": ms_step, "result": res,
+            "roofline": {"bound": "hbm", "achieved": achieved, "peak": hbm_peak, "unit": "GB/s",
+                         "frac": achieved / hbm_peak, "traffic": None, "kernel": dom,
+                         "algorithmic_bytes_per_launch": per_kernel_bytes[dom], "kernel_ms": kern_ms[dom],
+                         "peak_source": peak_src,
+                         "per_kernel": {k: {"ms": kern_ms[k], "bytes": per_kernel_bytes[k],
+                                            "gbs": per_kernel_bytes[k] / (kern_ms[k] / 1e3) / 1e9} for k in kern_ms},
+                         "step_bytes": ab["total"],
+                         "step_frac": ab["total"] / (ms_step / 1e3) / 1e9 / hbm_peak},
+            "gpu_launches": len(KERNELS[v]) * K, "gpu_kernels": KERNELS[v]}
+    head = results[args.variant]
     traffic_file = os.path.join(ROOT, "profiles", "traffic.json")
     if os.path.exists(traffic_file):
         try:
-            roofline["traffic"] = json.load(open(traffic_file)).get(args.variant, {}).get(dom)
+            tr = json.load(open(traffic_file))
+            for v in results:
+                results[v]["roofline"]["traffic"] = tr.get(v, {}).get(results[v]["roofline"]["kernel"])
         except Exception:
             pass
 
@@ -429,7 +433,7 @@ def ours(args):
             for i in range(args.e2e_steps):
                 for h, d in host_parts:
                     d.copy_(h, non_blocking=True)
-                step(0)
+                step(args.variant, 0)
                 res_host.copy_(out, non_blocking=True)
             drv.cuEventRecord(e1, s_ptr)
             stream.synchronize()
@@ -441,7 +445,7 @@ def ours(args):
         e2e = {"value": rows * world * args.e2e_steps / (ms_e2e / 1e3), "unit": UNIT, "h2d_bytes_per_step": h2d,
                "d2h_bytes_per_step": 32 if args.variant == "fused" else 16,
                "ms_per_step": ms_e2e / args.e2e_steps,
-               "path": "pinned host decomposed columns -> cudaMemcpyAsync H2D -> ar_* calls -> D2H result"}
+               "path": "pinned host decomposed columns -> cudaMemcpyAsync H2D -> ar_* C-ABI calls -> D2H result"}
 
     cpu = None
     if rank == 0 and world == 1 and not args.no_cpu:
@@ -455,27 +459,48 @@ def ours(args):
         return
     parity = None
     if cpu is not None:
-        parity = {"oracle_sum": cpu["sum"], "gpu_sum": res[0], "oracle_count": cpu["count"], "gpu_count": res[1],
-                  "match": cpu["sum"] == res[0] and cpu["count"] == res[1]}
+        parity = {"oracle_sum": cpu["sum"], "oracle_count": cpu["count"],
+                  "gpu": {v: {"sum": results[v]["result"][0], "count": results[v]["result"][1]} for v in results},
+                  "match": all(results[v]["result"][0] == cpu["sum"] and results[v]["result"][1] == cpu["count"]
+                               for v in results)}
         cpu = {k: v for k, v in cpu.items() if k not in ("sum", "count")}
-    line = {"metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world, "steps": K, "warmup": args.warmup,
-            "ms_per_step": ms_step, "higher_is_better": True, "scaling": "weak", "vs_baseline": None,
-            "dtype": "u32", "data": "synthetic",
+    other = {v: {k: results[v][k] for k in ("value", "ms_per_step", "roofline", "gpu_launches", "gpu_kernels")}
+             for v in results if v != args.variant}
+    line = {"metric": METRIC, "value": head["value"], "unit": UNIT, "n_gpus": world, "steps": K,
+            "warmup": args.warmup, "ms_per_step": head["ms_per_step"], "higher_is_better": True, "scaling": "weak",
+            "vs_baseline": None, "dtype": "u32", "data": "synthetic",
             "config": config_dict(args, world, rows, {
                 "variant": args.variant,
+                "variant_desc": VARIANT_DESC[args.variant],
                 "l2": f"inputs rotated over {len(copies)} copies of the decomposed columns "
                       f"({len(copies)} x {bytes_per_copy / 1e6:.0f} MB > 126 MB L2)",
                 "timing": "K steps = one CUDA-graph replay; CUDA events on the launching stream; max over ranks"}),
-            "roofline": roofline, "cpu_baseline": cpu, "e2e": e2e,
-            "gpu_launches": launches_per_step * K, "gpu_kernels": kernel_names,
+            "roofline": head["roofline"], "cpu_baseline": cpu, "e2e": e2e,
+            "gpu_launches": head["gpu_launches"], "gpu_kernels": head["gpu_kernels"],
             "clocks": sampler.result(),
             "counts": {"candidates": ab["n_cand"], "definite": ab["n_def"], "result": ab["n_result"],
-                       "gpu_result_count": res[1], "gpu_sum": res[0]},
+                       "gpu_result_count": head["result"][1], "gpu_sum": head["result"][0]},
             "parity": parity,
+            "variants": other,
             "hbm_roofline_rows_per_s": hbm_peak * 1e9 / (ab["total"] / rows)}
     print(json.dumps(line), flush=True)
     if pg:
         pg.destroy_process_group()
+
+
+class _Null:
+    def __enter__(self):
+        return self
+
+    def __exit__(self, *a):
+        return False
+
+
+VARIANT_DESC = {
+    "fused": "one pass: a3 approximate select (candidate relation compacted per warp in shared memory) + a5 refine "
+             "+ a6 SUM in one kernel (ar_select_refine_sum)",
+    "staged": "ar_approx_select (ordered candidate list in HBM) -> [a4 count allgather] -> ar_refine_sum",
+}
 
 
 def main():
