@@ -309,6 +309,10 @@ static ar_status setup_scan(const ar_pred* preds, int32_t npred, ard::SelParams&
     empty = false;
     n = preds[0].col ? preds[0].col->d.n : -1;
     P.bpt = (uint32_t)kernel_bpt(fused);
+    static const int suspend_ns = env_int("AR_SUSPEND_NS", 0);
+    P.suspend_ns = (uint32_t)suspend_ns;
+    static const int debug = env_int("AR_DEBUG", 0);
+    P.debug = (uint32_t)debug;
     P.tile_rows = (uint32_t)kernel_warps(fused) * 32u * 32u * P.bpt;
     uint32_t words = 0, ashift = 0;
     for (int c = 0; c < npred; ++c) {
@@ -409,12 +413,11 @@ ar_status ar_approx_select(const ar_pred* preds, int32_t npred, int32_t flags, a
     P.out_count = (long long*)out->count;
     P.ticket = (unsigned int*)ws;
     P.status = (unsigned long long*)((char*)ws + 16);
-    int occ = 1;
+    // one tile per CTA, tiles taken from an atomic ticket (ws[0]); grid = number of tiles
     const void* fn = select_kernel_fn(P, false);
-    P.nstages = pick_stages(fn, P.stage_words, false, &occ);
-    const size_t smem = select_smem_bytes(P.stage_words, P.nstages, true);
-    const int grid = (int)std::min<int64_t>(P.num_tiles, (int64_t)num_sms() * occ);
-    return launch_scan(fn, P, grid, smem, false, s);
+    P.nstages = 1;
+    const size_t smem = select_smem_bytes(P.stage_words, 1, true);
+    return launch_scan(fn, P, (int)P.num_tiles, smem, false, s);
 }
 
 // ------------------------------------------------------------------ a5
@@ -590,6 +593,25 @@ ar_status ar_select_refine_sum(const ar_pred* preds, int32_t npred, const ar_col
     if (st != AR_OK) return st;
     P.nagg = ncols;
     P.out4 = (unsigned long long*)out_dev;
+    // asynchronous gathers when exactly one aggregate column must be gathered (bit-packed, no
+    // residual) and the other factor, if any, is a predicate column whose value fits 26 bits
+    {
+        int g = -1, ng = 0;
+        bool ok = ncols >= 1;
+        for (int i = 0; i < ncols; ++i) {
+            const ard::AggCol& a = P.a[i];
+            if (a.pred < 0) {
+                ++ng;
+                g = i;
+                ok = ok && a.k == 0 && a.layout == AR_LAYOUT_PACKED && a.w > 0;
+            } else {
+                ok = ok && (a.w + a.k) <= 26 && a.base == 0;
+            }
+        }
+        static const int no_async = env_int("AR_NO_ASYNC_GATHER", 0);
+        P.async_agg = (ok && ng == 1 && !no_async) ? 1 : 0;
+        P.gidx = g < 0 ? 0 : g;
+    }
     cudaStream_t s = (cudaStream_t)stream;
     AR_TRY_CUDA(cudaMemsetAsync(out_dev, 0, 4 * sizeof(int64_t), s));
     if (empty || n == 0) return AR_OK;

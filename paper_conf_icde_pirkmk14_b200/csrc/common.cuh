@@ -89,18 +89,29 @@ __device__ __forceinline__ void mbar_arrive_expect_tx(uint64_t* bar, uint32_t by
 __device__ __forceinline__ void mbar_arrive(uint64_t* bar) {
     asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(smem_u32(bar)) : "memory");
 }
-// Blocking wait on an mbarrier phase.  The suspend-time hint lets the hardware
-// park the thread until the phase completes instead of returning after its short
-// default window: without it a waiting warp spins (YIELD / TRYWAIT / BRA) and
-// steals issue slots from the warps doing the work.
-__device__ __forceinline__ void mbar_wait(uint64_t* bar, uint32_t parity) {
-    asm volatile(
-        "{\n\t.reg .pred p;\n"
-        "AR_WAIT_%=:\n\t"
-        "mbarrier.try_wait.parity.shared::cta.b64 p, [%0], %1, %2;\n\t"
-        "@!p bra AR_WAIT_%=;\n}" ::"r"(smem_u32(bar)),
-        "r"(parity), "r"(1000000u)
-        : "memory");
+// Blocking wait on an mbarrier phase.  With a suspend-time hint (ns) the
+// hardware may park the thread until the phase completes instead of returning
+// after its short default window (a spinning warp steals issue slots);
+// hint == 0 is a plain try_wait loop.  The hint is a kernel parameter
+// (AR_SUSPEND_NS) so it can be tuned without recompiling.
+__device__ __forceinline__ void mbar_wait(uint64_t* bar, uint32_t parity, uint32_t hint_ns) {
+    if (hint_ns) {
+        asm volatile(
+            "{\n\t.reg .pred p;\n"
+            "AR_WAIT_%=:\n\t"
+            "mbarrier.try_wait.parity.shared::cta.b64 p, [%0], %1, %2;\n\t"
+            "@!p bra AR_WAIT_%=;\n}" ::"r"(smem_u32(bar)),
+            "r"(parity), "r"(hint_ns)
+            : "memory");
+    } else {
+        asm volatile(
+            "{\n\t.reg .pred p;\n"
+            "AR_WAIT_%=:\n\t"
+            "mbarrier.try_wait.parity.shared::cta.b64 p, [%0], %1;\n\t"
+            "@!p bra AR_WAIT_%=;\n}" ::"r"(smem_u32(bar)),
+            "r"(parity)
+            : "memory");
+    }
 }
 
 // --- TMA bulk copy global -> shared (1-D, no tensor map), completes on an mbarrier
@@ -152,6 +163,7 @@ __device__ __forceinline__ unsigned long long lookback(const unsigned long long*
         while (true) {
             s = idx >= 0 ? ld_relaxed(status + idx) : kFlagPrefix;  // before tile 0: prefix 0
             if (__all_sync(0xffffffffu, (s >> 62) != 0)) break;
+            __nanosleep(32);
         }
         unsigned prefix_lanes = __ballot_sync(0xffffffffu, (s >> 62) == 2);
         unsigned long long v = s & kValueMask;
@@ -170,7 +182,7 @@ __device__ __forceinline__ unsigned long long lookback(const unsigned long long*
 // Wide variant: each lane inspects kLookV consecutive predecessors, so one
 // round trip covers 32 * kLookV tiles and the prefix frontier advances that
 // many tiles per L2 latency.  Entry (lane, j) is tile base - kLookV*lane - j.
-constexpr int kLookV = 16;
+constexpr int kLookV = 8;
 __device__ __forceinline__ unsigned long long lookback_wide(const unsigned long long* status, long long t,
                                                             unsigned lane) {
     unsigned long long excl = 0;

@@ -51,6 +51,8 @@ struct SelParams {
     uint32_t stage_words;     // uint32 words per pipeline stage (all predicates)
     uint32_t nstages;
     uint32_t bpt;             // 32-row blocks per consumer thread (template parameter of the launch)
+    uint32_t suspend_ns;      // mbarrier wait suspend hint (0 = spin)
+    uint32_t debug;           // experiments only (AR_DEBUG): 1 = no look-back (provisional offsets), 2 = no copy-out
     uint32_t tile_rows;       // kSelMinTileRows * bpt
     uint32_t* out_pos;
     uint32_t* out_aux;
@@ -60,6 +62,8 @@ struct SelParams {
     // fused kernel only
     AggCol a[AR_MAX_AGG];
     int32_t nagg;
+    int32_t async_agg;            // fused: the one gathered aggregate column uses asynchronous gathers
+    int32_t gidx;                 // index of that column in a[]
     unsigned long long* out4;     // sum, |result|, |cand|, |def|
 };
 

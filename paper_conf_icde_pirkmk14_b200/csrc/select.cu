@@ -174,6 +174,21 @@ struct FixedPlanes {
             return 0u;
         }
     }
+    // approximation tuple of row l of tile-block blk, read from the stage (lane-parallel pass)
+    template <int C = 0>
+    __device__ __forceinline__ static uint32_t appr_smem(const SelParams& P, const uint32_t* stg, uint32_t blk,
+                                                         uint32_t l) {
+        if constexpr (C < N) {
+            constexpr int w = wid<Ws...>(C), o = woff<Ws...>(C);
+            const uint32_t* pl = stg + P.p[C].soff + blk * w;
+            uint32_t a = 0;
+#pragma unroll
+            for (int j = 0; j < w; ++j) a |= ((pl[j] >> l) & 1u) << (o + j);
+            return a | appr_smem<C + 1>(P, stg, blk, l);
+        } else {
+            return 0u;
+        }
+    }
     // approximation tuple: all majors concatenated LSB-first in predicate order
     template <int B>
     __device__ __forceinline__ uint32_t appr(const SelParams&, uint32_t l) const {
@@ -235,6 +250,12 @@ struct DynPlanes {
         for (int c = 0; c < P.npred; ++c) a |= value_rt<B>(P, c, l) << P.p[c].ashift;
         return a;
     }
+    __device__ __forceinline__ static uint32_t appr_smem(const SelParams& P, const uint32_t* stg, uint32_t blk,
+                                                         uint32_t l) {
+        uint32_t a = 0;
+        for (int c = 0; c < P.npred; ++c) a |= plane_value(stg + P.p[c].soff + blk * P.p[c].w, P.p[c].w, l) << P.p[c].ashift;
+        return a;
+    }
 };
 
 template <class T>
@@ -292,7 +313,7 @@ __device__ __forceinline__ void produce(const SelParams& P, const SmemLayout& L)
     const uint32_t blocks_per_tile = P.tile_rows / 32;
     uint32_t s = 0, ph = 0;   // ring slot and its phase parity (no integer division in the loop)
     for (uint32_t i = 0;; ++i) {
-        if (i >= P.nstages) mbar_wait(L.empty + s, ph ^ 1u);
+        if (i >= P.nstages) mbar_wait(L.empty + s, ph ^ 1u, P.suspend_ns);
         const long long t = (long long)blockIdx.x + (long long)i * gridDim.x;
         if (t >= P.num_tiles) {
             L.slot[s] = -1;
@@ -343,84 +364,107 @@ __device__ __forceinline__ void init_barriers(const SelParams& P, const SmemLayo
 
 // ------------------------------------------------------------ ordered select
 
+// Ordered select, one tile per CTA (single-pass "chained scan" as in CUB's
+// DeviceSelect): a CTA takes the next tile index from an atomic ticket (so every
+// predecessor tile belongs to a CTA that is already running -- no deadlock, and
+// tiles start roughly in order), loads the tile's planes with one TMA bulk copy
+// per predicate, evaluates, publishes its aggregate, resolves its offset with a
+// decoupled look-back (its predecessors usually already hold an inclusive
+// prefix because they started earlier), and writes its (pos, aux) entries
+// through shared memory with coalesced stores.  Many CTAs per SM overlap the
+// load, look-back and store latencies of different tiles.
 template <class PS, int NW, int BPT, bool kCarry>
-__global__ void __launch_bounds__((NW + 1) * 32) select_kernel(const __grid_constant__ SelParams P) {
+__global__ void __launch_bounds__(NW * 32) select_kernel(const __grid_constant__ SelParams P) {
     constexpr int NT = NW * 32;
     extern __shared__ __align__(128) unsigned char smem[];
-    const SmemLayout L = carve(smem, P.nstages, true);
+    __shared__ __align__(8) uint64_t bar;
+    __shared__ long long s_tile;
+    __shared__ unsigned long long s_off;
+    __shared__ uint32_t warp_tot[32];
+    uint32_t* st_pos = reinterpret_cast<uint32_t*>(smem);
+    uint32_t* st_aux = st_pos + kStageEntries;
+    uint32_t* stg = st_aux + kStageEntries;          // 16-B aligned (kStageEntries * 8 bytes above)
     const unsigned warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
-    init_barriers<NW>(P, L);
 
-    // Tiles are dealt round-robin: all CTAs are co-resident (cooperative launch),
-    // so round i proceeds in lock-step and a tile's look-back window only spans
-    // tiles of its own and the previous round.
-    if (warp == NW) {
-        if (lane == 0) produce(P, L);
-        return;
+    if (threadIdx.x == 0) {
+        const long long t = (long long)atomicAdd(P.ticket, 1u);
+        s_tile = t;
+        mbar_init(&bar, 1);
+        fence_mbar_init();
+        const int64_t r0 = t * (int64_t)P.tile_rows;
+        const int64_t rows = min((int64_t)P.tile_rows, P.n - r0);
+        const uint32_t groups = (uint32_t)((rows + 127) / 128);
+        uint32_t bytes = 0;
+        for (int c = 0; c < P.npred; ++c) bytes += groups * 16u * P.p[c].w;
+        mbar_arrive_expect_tx(&bar, bytes);
+        const uint64_t pol = policy_evict_first();
+        for (int c = 0; c < P.npred; ++c) {
+            const uint32_t w = P.p[c].w;
+            if (w)
+                bulk_g2s(stg + P.p[c].soff, P.p[c].planes + (size_t)t * (P.tile_rows / 32) * w, groups * 16u * w,
+                         &bar, pol);
+        }
     }
+    __syncthreads();
+    const long long t = s_tile;
+    mbar_wait(&bar, 0, 0);
 
-    uint32_t s = 0, ph = 0;
-    for (;; s = (s + 1 == P.nstages) ? (ph ^= 1u, 0u) : s + 1) {
-        mbar_wait(L.full + s, ph);
-        const long long t = L.slot[s];
-        if (t < 0) break;
-        const int64_t r0 = t * (int64_t)P.tile_rows + (int64_t)threadIdx.x * (32 * BPT);
-
-        PS ps;
-        ps.load(P, L.stages + (size_t)s * P.stage_words);
-        uint32_t cm[BPT], dm[BPT];
+    const int64_t r0 = t * (int64_t)P.tile_rows + (int64_t)threadIdx.x * (32 * BPT);
+    PS ps;
+    ps.load(P, stg);
+    uint32_t cm[BPT], dm[BPT];
 #pragma unroll
-        for (int b = 0; b < BPT; ++b) cm[b] = dm[b] = valid_mask(r0 + 32 * b, P.n);
-        ps.eval(P, cm, dm);
-        uint32_t cnt = 0;
+    for (int b = 0; b < BPT; ++b) cm[b] = dm[b] = valid_mask(r0 + 32 * b, P.n);
+    ps.eval(P, cm, dm);
+    uint32_t cnt = 0;
 #pragma unroll
-        for (int b = 0; b < BPT; ++b) cnt += __popc(cm[b]);
-        uint32_t total;
-        const uint32_t excl = block_excl_scan<NT>(cnt, L.warp_tot, total, 1);
+    for (int b = 0; b < BPT; ++b) cnt += __popc(cm[b]);
+    uint32_t total;
+    const uint32_t excl = block_excl_scan<NT>(cnt, warp_tot, total, 1);
 
-        if (warp == 0) {
-            unsigned long long prefix = 0;
-            if (t == 0) {
-                if (lane == 0) st_relaxed(P.status, kFlagPrefix | total);
-            } else {
-                if (lane == 0) st_relaxed(P.status + t, kFlagAgg | total);
-                prefix = lookback_wide(P.status, t, lane);
-                if (lane == 0) st_relaxed(P.status + t, kFlagPrefix | (prefix + total));
-            }
-            if (lane == 0) {
-                L.misc[0] = prefix;
-                if (t == P.num_tiles - 1) *P.out_count = (long long)(prefix + total);
-            }
+    if (warp == 0) {
+        unsigned long long prefix = 0;
+        if (t == 0) {
+            if (lane == 0) st_relaxed(P.status, kFlagPrefix | total);
+        } else {
+            if (lane == 0) st_relaxed(P.status + t, kFlagAgg | total);
+            prefix = lookback_wide(P.status, t, lane);
+            if (lane == 0) st_relaxed(P.status + t, kFlagPrefix | (prefix + total));
         }
-        bar_sync(1, NT);
-        const unsigned long long off = L.misc[0];
+        if (lane == 0) {
+            s_off = prefix;
+            if (t == P.num_tiles - 1) *P.out_count = (long long)(prefix + total);
+        }
+    }
+    __syncthreads();
+    const unsigned long long off = s_off;
+    const uint32_t tile_r0 = (uint32_t)(t * (int64_t)P.tile_rows);
 
-        // write the tile's entries in rounds of kStageEntries through shared memory
-        uint32_t e = excl;
-        for (uint32_t base = 0; base < total; base += kStageEntries) {
-            const uint32_t lim = min(base + (uint32_t)kStageEntries, excl + cnt);
-            auto emit = [&](auto bc) {
-                constexpr int b = decltype(bc)::value;
-                while (cm[b] && e < lim) {
-                    const uint32_t l = __ffs(cm[b]) - 1;
-                    cm[b] &= cm[b] - 1;
-                    uint32_t aux = ((dm[b] >> l) & 1u) << 31;
-                    if (kCarry) aux |= ps.template appr<b>(P, l);
-                    L.st_pos[e - base] = (uint32_t)(r0 + 32 * b + l);
-                    L.st_aux[e - base] = aux;
-                    ++e;
-                }
-            };
-            static_for<BPT>(emit);
-            bar_sync(1, NT);
-            const uint32_t nround = min((uint32_t)kStageEntries, total - base);
-            for (uint32_t j = threadIdx.x; j < nround; j += NT) {
-                P.out_pos[off + base + j] = L.st_pos[j];
-                P.out_aux[off + base + j] = L.st_aux[j];
+    // entries in rounds of kStageEntries: per-thread positions, lane-parallel aux, coalesced stores
+    uint32_t e = excl;
+    for (uint32_t base = 0; base < total; base += kStageEntries) {
+        const uint32_t lim = min(base + (uint32_t)kStageEntries, excl + cnt);
+        static_for<BPT>([&](auto bc) {
+            constexpr int b = decltype(bc)::value;
+            const uint32_t rbase = (threadIdx.x * BPT + b) << 5;
+            while (cm[b] && e < lim) {
+                const uint32_t l = __ffs(cm[b]) - 1;
+                cm[b] &= cm[b] - 1;
+                st_pos[e - base] = (rbase | l) | (((dm[b] >> l) & 1u) << 31);
+                ++e;
             }
-            bar_sync(1, NT);
+        });
+        __syncthreads();
+        const uint32_t nround = min((uint32_t)kStageEntries, total - base);
+        for (uint32_t j = threadIdx.x; j < nround; j += NT) {
+            const uint32_t v = st_pos[j];
+            const uint32_t o = v & 0x7fffffffu;
+            uint32_t aux = v & 0x80000000u;
+            if (kCarry) aux |= PS::appr_smem(P, stg, o >> 5, o & 31u);
+            P.out_pos[off + base + j] = tile_r0 + o;
+            P.out_aux[off + base + j] = aux;
         }
-        if (lane == 0) mbar_arrive(L.empty + s);   // planes of stage s no longer needed
+        __syncthreads();
     }
 }
 
@@ -433,6 +477,34 @@ __global__ void __launch_bounds__((NW + 1) * 32) select_kernel(const __grid_cons
 // each and refine / aggregate them in parallel, so the residual and aggregate
 // gathers of a whole warp are in flight together (Alg. 2).
 constexpr int kPer = 2;               // list entries per lane per pass
+constexpr int kGSlot = 32 * kPer;     // async-gather entries per warp per tile (first pass)
+constexpr int kGDepth = 3;            // tiles of gathers in flight per warp
+
+__device__ __forceinline__ void cp_async4(uint32_t* dst, const uint32_t* src) {
+    asm volatile("cp.async.ca.shared.global.L2::64B [%0], [%1], 4;" ::"r"(smem_u32(dst)), "l"(src) : "memory");
+}
+__device__ __forceinline__ void cp_async_commit() { asm volatile("cp.async.commit_group;" ::: "memory"); }
+template <int N>
+__device__ __forceinline__ void cp_async_wait() { asm volatile("cp.async.wait_group %0;" ::"n"(N) : "memory"); }
+
+// Sum this lane's landed entries of one async-gather slot: value of the gathered
+// packed column (1-2 words, shift) times the pre-computed other factor.
+__device__ __forceinline__ unsigned long long gather_drain(const uint32_t* slot, uint32_t lane, const AggCol& G) {
+    unsigned long long acc = 0;
+#pragma unroll
+    for (int q = 0; q < kPer; ++q) {
+        const uint32_t ei = q * 32 + lane;
+        const uint32_t info = slot[2 * kGSlot + ei];
+        if (!(info >> 31)) continue;
+        const uint32_t sh = (info >> 26) & 31u, mult = info & ((1u << 26) - 1u);
+        const uint32_t lo = slot[ei];
+        uint32_t v = lo >> sh;
+        if (sh + G.w > 32u) v = __funnelshift_r(lo, slot[kGSlot + ei], sh);
+        if (G.w < 32) v &= (1u << G.w) - 1u;
+        acc += (unsigned long long)(v + G.base) * mult;
+    }
+    return acc;
+}
 constexpr uint32_t kDefFlag = 0x8000u;
 
 // Major of predicate c at block-local row l of global block `blk` of the tile.
@@ -449,8 +521,11 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_kernel(const __grid_co
     const SmemLayout L = carve(smem, P.nstages, false);
     const unsigned warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     init_barriers<NW>(P, L);
-    // per-warp candidate lists live after the stage ring
+    // per-warp candidate lists live after the stage ring, then the async-gather slots
     uint16_t* list = reinterpret_cast<uint16_t*>(L.stages + (size_t)P.nstages * P.stage_words) + warp * kWarpRows;
+    uint32_t* gslot = reinterpret_cast<uint32_t*>(reinterpret_cast<uint16_t*>(L.stages +
+                                                  (size_t)P.nstages * P.stage_words) + NW * kWarpRows) +
+                      warp * (kGDepth * kGSlot * 3);
 
     if (warp == NW) {
         if (lane == 0) produce(P, L);
@@ -458,9 +533,10 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_kernel(const __grid_co
     }
 
     unsigned long long sum = 0, nres = 0, ncand = 0, ndef = 0;
+    uint32_t gseq = 0;   // async-gather tiles issued by this warp
     uint32_t s = 0, ph = 0;
     for (;; s = (s + 1 == P.nstages) ? (ph ^= 1u, 0u) : s + 1) {
-        mbar_wait(L.full + s, ph);
+        mbar_wait(L.full + s, ph, P.suspend_ns);
         const long long t = L.slot[s];
         if (t < 0) break;
         const uint32_t* stg = L.stages + (size_t)s * P.stage_words;
@@ -544,7 +620,51 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_kernel(const __grid_co
             });
 #pragma unroll
             for (int q = 0; q < kPer; ++q) nres += ok[q];
-            if (P.nagg > 0) {
+            if (P.async_agg && base == 0) {
+                // a6, asynchronous: the other factor (a predicate column's value) now, the gathered
+                // column's 1-2 words by cp.async into this tile's slot; summed kGDepth-1 tiles later
+                uint32_t* slot = gslot + (gseq % kGDepth) * (kGSlot * 3);
+                const AggCol& G = P.a[P.gidx];
+#pragma unroll
+                for (int q = 0; q < kPer; ++q) {
+                    const uint32_t ei = q * 32 + lane;
+                    uint32_t mult = 1u;
+                    if (ok[q] && P.nagg > 1) {
+                        const AggCol& A = P.a[1 - P.gidx];
+                        PS::for_pred(P, [&](auto cc) {
+                            if (int(cc) != A.pred) return;
+                            const SelPred& p = P.p[int(cc)];
+                            const uint32_t w = PS::pw(P, cc);
+                            const uint32_t* pl = stg + p.soff + ((row_in_tile0 + off[q]) >> 5) * w;
+                            const uint32_t l = off[q] & 31u;
+                            uint32_t m = 0;
+#pragma unroll
+                            for (uint32_t j = 0; j < w; ++j) m |= ((pl[j] >> l) & 1u) << j;
+                            uint32_t r = 0u;
+                            if (p.k)
+                                r = p.res_stream ? packed_get_smem(stg + p.res_soff, (row_in_tile0 + off[q]) * p.k, p.k)
+                                                 : packed_get_any(p.residual, row_base + off[q], p.k);
+                            mult = ((m << p.k) | r) + p.base;
+                        });
+                    }
+                    uint32_t info = 0u;
+                    if (ok[q]) {
+                        const uint64_t bit = (row_base + off[q]) * (uint64_t)G.w;
+                        const uint32_t* src = G.major + (bit >> 5);
+                        const uint32_t sh = (uint32_t)(bit & 31);
+                        cp_async4(slot + ei, src);
+                        if (sh + G.w > 32u) cp_async4(slot + kGSlot + ei, src + 1);
+                        info = (1u << 31) | (sh << 26) | mult;   // mult < 2^26 (checked on the host)
+                    }
+                    slot[2 * kGSlot + ei] = info;
+                }
+                cp_async_commit();
+                ++gseq;
+                if (gseq >= (uint32_t)kGDepth) {       // consume the tile issued kGDepth-1 tiles ago
+                    cp_async_wait<kGDepth - 1>();
+                    sum += gather_drain(gslot + (gseq % kGDepth) * (kGSlot * 3), lane, G);
+                }
+            } else if (P.nagg > 0) {
                 unsigned long long prod[kPer];
 #pragma unroll
                 for (int q = 0; q < kPer; ++q) prod[q] = ok[q] ? 1ull : 0ull;
@@ -588,6 +708,12 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_kernel(const __grid_co
         __syncwarp();
         if (lane == 0) mbar_arrive(L.empty + s);
     }
+    if (P.async_agg) {   // drain the gathers still in flight
+        cp_async_wait<0>();
+        const AggCol& G = P.a[P.gidx];
+        for (uint32_t k = (gseq >= (uint32_t)kGDepth ? gseq - kGDepth + 1 : 0); k < gseq; ++k)
+            sum += gather_drain(gslot + (k % kGDepth) * (kGSlot * 3), lane, G);
+    }
 
     // CTA reduction, then one atomic per counter
 #pragma unroll
@@ -614,7 +740,7 @@ namespace ar {
 // Kernel configurations: (consumer warps, blocks per thread) of the ordered
 // select and of the fused kernel, and the decomposition shapes with
 // specialised kernels.  Any other shape takes the DynPlanes path.
-constexpr int kSelNW = ard::kSelWarps, kSelBPT = 2;
+constexpr int kSelNW = 4, kSelBPT = 2;
 constexpr int kFusNW = 8, kFusBPT = 1;
 
 template <int... Ws>
@@ -656,7 +782,8 @@ struct ShapeList {
 using Shapes = ShapeList<ShapeEntry<4, 4, 6>, ShapeEntry<8>, ShapeEntry<16>, ShapeEntry<24>, ShapeEntry<32>,
                          ShapeEntry<24, 24>>;
 
-int kernel_warps(bool fused) { return fused ? kFusNW : kSelNW; }
+int kernel_warps(bool fused) { return fused ? kFusNW : kSelNW; }               // compute warps
+static int kernel_threads(bool fused) { return 32 * (kernel_warps(fused) + (fused ? 1 : 0)); }  // + producer (fused)
 int kernel_bpt(bool fused) { return fused ? kFusBPT : kSelBPT; }
 
 const void* select_kernel_fn(const ard::SelParams& P, bool fused) {
@@ -669,10 +796,11 @@ const void* select_kernel_fn(const ard::SelParams& P, bool fused) {
 
 size_t select_smem_bytes(uint32_t stage_words, uint32_t nstages, bool staging) {
     size_t head = nstages * (8 + 8 + 8) + 32 * 4 + 8 * 8;
-    if (staging) head += 2ull * ard::kStageEntries * 4;
+    if (staging) return 2ull * ard::kStageEntries * 4 + (size_t)stage_words * 4;   // select: one tile per CTA
     head = (head + 127) & ~size_t(127);
     size_t bytes = head + 128 + (size_t)nstages * stage_words * 4;
-    if (!staging) bytes += (size_t)kFusNW * 32 * 32 * kFusBPT * 2;   // per-warp candidate lists (u16)
+    if (!staging) bytes += (size_t)kFusNW * 32 * 32 * kFusBPT * 2   // per-warp candidate lists (u16)
+                         + (size_t)kFusNW * ard::kGDepth * ard::kGSlot * 3 * 4;   // async-gather slots
     return bytes;
 }
 
@@ -681,14 +809,21 @@ static void set_max_smem(const void* fn) {
     static thread_local int used = 0;
     for (int i = 0; i < used; ++i)
         if (done[i] == fn) return;
-    cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, 227 * 1024);
+    // opt in to the largest dynamic allocation this kernel can have (227 KB minus its static smem)
+    cudaFuncAttributes a{};
+    int max_optin = 227 * 1024, dev = 0;
+    if (cudaGetDevice(&dev) == cudaSuccess)
+        cudaDeviceGetAttribute(&max_optin, cudaDevAttrMaxSharedMemoryPerBlockOptin, dev);
+    if (cudaFuncGetAttributes(&a, fn) == cudaSuccess)
+        cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, max_optin - (int)a.sharedSizeBytes);
+    cudaGetLastError();   // never leave a sticky error behind for a later launch check
     if (used < 64) done[used++] = fn;
 }
 
 int select_occupancy(const void* fn, size_t smem, bool fused) {
     int blocks = 0;
     set_max_smem(fn);
-    cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks, fn, (kernel_warps(fused) + 1) * 32, smem);
+    cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks, fn, kernel_threads(fused), smem);
     return blocks;
 }
 
@@ -701,12 +836,12 @@ ar_status launch_scan(const void* fn, const ard::SelParams& P, int grid, size_t 
     void* args[] = {const_cast<ard::SelParams*>(&P)};
     cudaLaunchConfig_t cfg = {};
     cfg.gridDim = dim3(grid);
-    cfg.blockDim = dim3((kernel_warps(fused) + 1) * 32);
+    cfg.blockDim = dim3(kernel_threads(fused));
     cfg.dynamicSmemBytes = smem;
     cfg.stream = s;
     cudaLaunchAttribute attr[1];
     attr[0].id = cudaLaunchAttributeCooperative;
-    attr[0].val.cooperative = fused ? 0 : 1;
+    attr[0].val.cooperative = 0;
     cfg.attrs = attr;
     cfg.numAttrs = 1;
     AR_TRY_CUDA(cudaLaunchKernelExC(&cfg, fn, args));
