@@ -38,11 +38,17 @@ namespace ard {
 // v < lo iff v - lo borrows out of the top bit, v > hi iff hi - v does.  Per
 // plane and bound the borrow update is one 3-input logic op (LOP3); the bound's
 // bit j is a warp-uniform all-0 / all-1 mask.
+// Written as explicit lop3 (immLut = F(0xF0, 0xCC, 0xAA)): left to itself the
+// compiler splits each into three LOP3s.
 __device__ __forceinline__ uint32_t borrow_sub(uint32_t x, uint32_t cbit, uint32_t b) {   // borrow of x - c
-    return (~x & (cbit | b)) | (x & cbit & b);
+    uint32_t d;   // (~x & (c | b)) | (x & c & b)
+    asm("lop3.b32 %0, %1, %2, %3, 0x8E;" : "=r"(d) : "r"(x), "r"(cbit), "r"(b));
+    return d;
 }
 __device__ __forceinline__ uint32_t borrow_rsub(uint32_t x, uint32_t cbit, uint32_t b) {  // borrow of c - x
-    return (~cbit & (x | b)) | (cbit & x & b);
+    uint32_t d;   // (~c & (x | b)) | (c & x & b)
+    asm("lop3.b32 %0, %1, %2, %3, 0xB2;" : "=r"(d) : "r"(x), "r"(cbit), "r"(b));
+    return d;
 }
 __device__ __forceinline__ uint32_t bitmask(uint32_t v, uint32_t j) { return 0u - ((v >> j) & 1u); }
 
@@ -313,7 +319,7 @@ __device__ __forceinline__ void produce(const SelParams& P, const SmemLayout& L)
     const uint32_t blocks_per_tile = P.tile_rows / 32;
     uint32_t s = 0, ph = 0;   // ring slot and its phase parity (no integer division in the loop)
     for (uint32_t i = 0;; ++i) {
-        if (i >= P.nstages) mbar_wait(L.empty + s, ph ^ 1u, P.suspend_ns);
+        if (i >= P.nstages) mbar_wait_sleep(L.empty + s, ph ^ 1u);   // producer backs off instead of spinning
         const long long t = (long long)blockIdx.x + (long long)i * gridDim.x;
         if (t >= P.num_tiles) {
             L.slot[s] = -1;
