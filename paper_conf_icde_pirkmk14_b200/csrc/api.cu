@@ -289,9 +289,12 @@ void ar_column_free(ar_column* col) { delete col; }
 
 // ------------------------------------------------------------- a2 + a3
 
+// Select workspace: per-tile counts (u32) + offsets (u64) + tile-local candidate slices (pos, aux).
 size_t ar_select_ws_bytes(int64_t n) {
-    const uint64_t tiles = ceil_div_u64((uint64_t)std::max<int64_t>(n, 0), ard::kSelMinTileRows);
-    return 16 + 8 * tiles;
+    const uint64_t rows = (uint64_t)std::max<int64_t>(n, 0);
+    const uint64_t tiles = ceil_div_u64(rows, ard::kSelMinTileRows);
+    const uint64_t slice_rows = tiles * ard::kSelMinTileRows;      // >= n, covers the last tile's slice
+    return 16 + 16 * tiles + 8 + 16 + 8 * slice_rows;
 }
 
 // Shared predicate setup of ar_approx_select / ar_select_refine_sum.
@@ -406,18 +409,28 @@ ar_status ar_approx_select(const ar_pred* preds, int32_t npred, int32_t flags, a
     cudaStream_t s = (cudaStream_t)stream;
     AR_TRY_CUDA(cudaMemsetAsync(out->count, 0, sizeof(int64_t), s));
     if (empty || n == 0) return AR_OK;
-    AR_TRY_CUDA(cudaMemsetAsync(ws, 0, 16 + 8 * (size_t)P.num_tiles, s));
     P.carry = carry ? 1 : 0;
     P.out_pos = out->pos;
     P.out_aux = out->aux;
     P.out_count = (long long*)out->count;
-    P.ticket = (unsigned int*)ws;
-    P.status = (unsigned long long*)((char*)ws + 16);
-    // one tile per CTA, tiles taken from an atomic ticket (ws[0]); grid = number of tiles
+    // workspace: [16 B pad][counts u32 x T (+pad)][group sums u64][tmp_pos][tmp_aux]
+    const uint64_t T = (uint64_t)P.num_tiles;
+    P.tile_count = (uint32_t*)((char*)ws + 16);
+    P.group_sum = (unsigned long long*)((char*)ws + 16 + 8 * ((T + 1) / 2));
+    const uint64_t ngroups = (T + (1u << ard::kGroupShift) - 1) >> ard::kGroupShift;
+    AR_TRY_CUDA(cudaMemsetAsync(P.group_sum, 0, 8 * ngroups, s));
+    const uint64_t slice_rows = ceil_div_u64((uint64_t)n, ard::kSelMinTileRows) * ard::kSelMinTileRows;
+    char* tmp = (char*)ws + 16 + 16 * ceil_div_u64((uint64_t)n, ard::kSelMinTileRows) + 8;
+    tmp = (char*)(((uintptr_t)tmp + 15) & ~uintptr_t(15));
+    P.tmp_pos = (uint32_t*)tmp;
+    P.tmp_aux = P.tmp_pos + slice_rows;
+    (void)T;
     const void* fn = select_kernel_fn(P, false);
     P.nstages = 1;
     const size_t smem = select_smem_bytes(P.stage_words, 1, true);
-    return launch_scan(fn, P, (int)P.num_tiles, smem, false, s);
+    ar_status st2 = launch_scan(fn, P, (int)P.num_tiles, smem, false, s);
+    if (st2 != AR_OK) return st2;
+    return launch_select_rest(P, s);
 }
 
 // ------------------------------------------------------------------ a5

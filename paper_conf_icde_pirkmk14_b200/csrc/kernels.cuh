@@ -39,7 +39,8 @@ __device__ __forceinline__ uint32_t agg_gather(const AggCol& a, uint64_t p) {
 constexpr int kSelWarps = 4;                      // consumer warps per CTA
 constexpr int kSelThreads = kSelWarps * 32;       // each consumer thread owns BPT consecutive 32-row blocks
 constexpr int kSelMinTileRows = kSelThreads * 32; // tile rows = 4096 * BPT (BPT in {1, 2, 4})
-constexpr int kStageEntries = 2048;               // output staging entries (pos + aux) per round
+constexpr int kStageEntries = 2048;
+constexpr int kGroupShift = 8;                    // select: 256 tiles per offset group               // output staging entries (pos + aux) per round
 
 struct SelParams {
     SelPred p[AR_MAX_PRED];
@@ -57,8 +58,12 @@ struct SelParams {
     uint32_t* out_pos;
     uint32_t* out_aux;
     long long* out_count;
-    unsigned long long* status;   // [num_tiles] look-back words
-    unsigned int* ticket;         // dynamic tile counter
+    unsigned long long* status;   // [num_tiles] look-back words (unused by the select)
+    unsigned int* ticket;         // dynamic tile counter (unused by the select)
+    uint32_t* tile_count;         // select: [num_tiles] candidates per tile
+    unsigned long long* group_sum; // select: candidates per group of 2^kGroupShift tiles (zeroed per call)
+    uint32_t* tmp_pos;            // select: tile-local candidate slices (workspace, n entries)
+    uint32_t* tmp_aux;
     // fused kernel only
     AggCol a[AR_MAX_AGG];
     int32_t nagg;
@@ -114,6 +119,7 @@ int kernel_bpt(bool fused);
 const void* select_kernel_fn(const ard::SelParams& P, bool fused);
 int select_occupancy(const void* fn, size_t smem, bool fused);
 ar_status launch_scan(const void* fn, const ard::SelParams& P, int grid, size_t smem, bool fused, cudaStream_t s);
+ar_status launch_select_rest(const ard::SelParams& P, cudaStream_t s);
 ar_status launch_refine(const ard::RefParams& P, int grid, cudaStream_t s);
 ar_status launch_refine_sum(const ard::RefParams& P, int grid, cudaStream_t s);
 ar_status launch_sum(const ard::SumParams& P, int grid, cudaStream_t s);

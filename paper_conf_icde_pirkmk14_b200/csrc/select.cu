@@ -370,31 +370,29 @@ __device__ __forceinline__ void init_barriers(const SelParams& P, const SmemLayo
 
 // ------------------------------------------------------------ ordered select
 
-// Ordered select, one tile per CTA (single-pass "chained scan" as in CUB's
-// DeviceSelect): a CTA takes the next tile index from an atomic ticket (so every
-// predecessor tile belongs to a CTA that is already running -- no deadlock, and
-// tiles start roughly in order), loads the tile's planes with one TMA bulk copy
-// per predicate, evaluates, publishes its aggregate, resolves its offset with a
-// decoupled look-back (its predecessors usually already hold an inclusive
-// prefix because they started earlier), and writes its (pos, aux) entries
-// through shared memory with coalesced stores.  Many CTAs per SM overlap the
-// load, look-back and store latencies of different tiles.
+// Ordered select in three short, dependency-free kernels:
+//   1. select_tile_kernel: one tile per CTA.  One TMA bulk copy per predicate
+//      brings the tile's planes, the CTA evaluates them, compacts its candidates
+//      (stable: per-thread popc, block scan) and writes them with coalesced
+//      stores to the tile's own slice of a workspace buffer, plus its count.
+//   2. scan_counts_kernel: one CTA turns the per-tile counts into exclusive
+//      offsets and the total.
+//   3. compact_kernel: each CTA moves one tile's slice to its final offset.
+// No CTA ever waits for another: on this GPU a decoupled look-back spent most
+// of the select kernel's time at its barrier (DESIGN s6.2).  The workspace
+// round trip is 8 B per candidate written and read back (L2-resident at low
+// selectivity).
 template <class PS, int NW, int BPT, bool kCarry>
-__global__ void __launch_bounds__(NW * 32) select_kernel(const __grid_constant__ SelParams P) {
+__global__ void __launch_bounds__(NW * 32) select_tile_kernel(const __grid_constant__ SelParams P) {
     constexpr int NT = NW * 32;
     extern __shared__ __align__(128) unsigned char smem[];
     __shared__ __align__(8) uint64_t bar;
-    __shared__ long long s_tile;
-    __shared__ unsigned long long s_off;
     __shared__ uint32_t warp_tot[32];
     uint32_t* st_pos = reinterpret_cast<uint32_t*>(smem);
-    uint32_t* st_aux = st_pos + kStageEntries;
-    uint32_t* stg = st_aux + kStageEntries;          // 16-B aligned (kStageEntries * 8 bytes above)
-    const unsigned warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    uint32_t* stg = st_pos + kStageEntries;          // 16-B aligned (kStageEntries * 4 bytes above)
+    const long long t = blockIdx.x;
 
     if (threadIdx.x == 0) {
-        const long long t = (long long)atomicAdd(P.ticket, 1u);
-        s_tile = t;
         mbar_init(&bar, 1);
         fence_mbar_init();
         const int64_t r0 = t * (int64_t)P.tile_rows;
@@ -412,7 +410,6 @@ __global__ void __launch_bounds__(NW * 32) select_kernel(const __grid_constant__
         }
     }
     __syncthreads();
-    const long long t = s_tile;
     mbar_wait(&bar, 0, 0);
 
     const int64_t r0 = t * (int64_t)P.tile_rows + (int64_t)threadIdx.x * (32 * BPT);
@@ -427,26 +424,15 @@ __global__ void __launch_bounds__(NW * 32) select_kernel(const __grid_constant__
     for (int b = 0; b < BPT; ++b) cnt += __popc(cm[b]);
     uint32_t total;
     const uint32_t excl = block_excl_scan<NT>(cnt, warp_tot, total, 1);
-
-    if (warp == 0) {
-        unsigned long long prefix = 0;
-        if (t == 0) {
-            if (lane == 0) st_relaxed(P.status, kFlagPrefix | total);
-        } else {
-            if (lane == 0) st_relaxed(P.status + t, kFlagAgg | total);
-            prefix = lookback_wide(P.status, t, lane);
-            if (lane == 0) st_relaxed(P.status + t, kFlagPrefix | (prefix + total));
-        }
-        if (lane == 0) {
-            s_off = prefix;
-            if (t == P.num_tiles - 1) *P.out_count = (long long)(prefix + total);
-        }
+    if (threadIdx.x == 0) {
+        P.tile_count[t] = total;
+        if (total) atomicAdd(P.group_sum + (t >> kGroupShift), (unsigned long long)total);
     }
-    __syncthreads();
-    const unsigned long long off = s_off;
-    const uint32_t tile_r0 = (uint32_t)(t * (int64_t)P.tile_rows);
 
     // entries in rounds of kStageEntries: per-thread positions, lane-parallel aux, coalesced stores
+    const uint32_t tile_r0 = (uint32_t)(t * (int64_t)P.tile_rows);
+    uint32_t* tmp_pos = P.tmp_pos + (size_t)t * P.tile_rows;
+    uint32_t* tmp_aux = P.tmp_aux + (size_t)t * P.tile_rows;
     uint32_t e = excl;
     for (uint32_t base = 0; base < total; base += kStageEntries) {
         const uint32_t lim = min(base + (uint32_t)kStageEntries, excl + cnt);
@@ -467,10 +453,49 @@ __global__ void __launch_bounds__(NW * 32) select_kernel(const __grid_constant__
             const uint32_t o = v & 0x7fffffffu;
             uint32_t aux = v & 0x80000000u;
             if (kCarry) aux |= PS::appr_smem(P, stg, o >> 5, o & 31u);
-            P.out_pos[off + base + j] = tile_r0 + o;
-            P.out_aux[off + base + j] = aux;
+            tmp_pos[base + j] = tile_r0 + o;
+            tmp_aux[base + j] = aux;
         }
         __syncthreads();
+    }
+}
+
+// Move each tile's candidate slice from the workspace to its final offset: one
+// warp per tile (grid-stride).  The tile's offset is the sum of the group
+// totals before its group (groups of 2^kGroupShift tiles, accumulated with one
+// atomic per tile by the select kernel) plus the counts of the earlier tiles of
+// its own group -- two short warp reductions, no separate scan kernel.
+__global__ void __launch_bounds__(256) compact_kernel(const __grid_constant__ SelParams P) {
+    const unsigned lane = threadIdx.x & 31;
+    const long long nw = (long long)gridDim.x * 8;
+    for (long long t = (long long)blockIdx.x * 8 + (threadIdx.x >> 5); t < P.num_tiles; t += nw) {
+        const long long g = t >> kGroupShift, t0 = g << kGroupShift;
+        unsigned long long off = 0;
+        for (long long i = lane; i < g; i += 32) off += __ldcg(P.group_sum + i);
+        for (long long i = t0 + lane; i < t; i += 32) off += __ldcg(P.tile_count + i);
+#pragma unroll
+        for (int o = 16; o > 0; o >>= 1) off += __shfl_xor_sync(0xffffffffu, off, o);
+        const uint32_t c = __ldcg(P.tile_count + t);
+        if (t == P.num_tiles - 1 && lane == 0) *P.out_count = (long long)(off + c);
+        const uint32_t* sp = P.tmp_pos + (size_t)t * P.tile_rows;
+        const uint32_t* sa = P.tmp_aux + (size_t)t * P.tile_rows;
+        for (uint32_t j0 = 0; j0 < c; j0 += 128) {
+            uint32_t vp[4], va[4];
+#pragma unroll
+            for (int k = 0; k < 4; ++k) {
+                const uint32_t j = j0 + k * 32 + lane;
+                vp[k] = j < c ? __ldcs(sp + j) : 0u;   // streaming: each slice is read once
+                va[k] = j < c ? __ldcs(sa + j) : 0u;
+            }
+#pragma unroll
+            for (int k = 0; k < 4; ++k) {
+                const uint32_t j = j0 + k * 32 + lane;
+                if (j < c) {
+                    P.out_pos[off + j] = vp[k];
+                    P.out_aux[off + j] = va[k];
+                }
+            }
+        }
     }
 }
 
@@ -761,8 +786,8 @@ struct ShapeEntry {
     }
     static const void* select_fn(bool carry) {
         using PS = ard::FixedPlanes<kSelBPT, Ws...>;
-        return carry ? (const void*)ard::select_kernel<PS, kSelNW, kSelBPT, true>
-                     : (const void*)ard::select_kernel<PS, kSelNW, kSelBPT, false>;
+        return carry ? (const void*)ard::select_tile_kernel<PS, kSelNW, kSelBPT, true>
+                     : (const void*)ard::select_tile_kernel<PS, kSelNW, kSelBPT, false>;
     }
     static const void* fused_fn() {
         using PS = ard::FixedPlanes<kFusBPT, Ws...>;
@@ -796,13 +821,13 @@ const void* select_kernel_fn(const ard::SelParams& P, bool fused) {
     const void* fn = nullptr;
     if (!getenv("AR_FORCE_GENERIC") && Shapes::find(P, fused, P.carry != 0, &fn)) return fn;
     if (fused) return (const void*)ard::fused_kernel<ard::DynPlanes<kFusBPT>, kFusNW, kFusBPT>;
-    return P.carry ? (const void*)ard::select_kernel<ard::DynPlanes<kSelBPT>, kSelNW, kSelBPT, true>
-                   : (const void*)ard::select_kernel<ard::DynPlanes<kSelBPT>, kSelNW, kSelBPT, false>;
+    return P.carry ? (const void*)ard::select_tile_kernel<ard::DynPlanes<kSelBPT>, kSelNW, kSelBPT, true>
+                   : (const void*)ard::select_tile_kernel<ard::DynPlanes<kSelBPT>, kSelNW, kSelBPT, false>;
 }
 
 size_t select_smem_bytes(uint32_t stage_words, uint32_t nstages, bool staging) {
     size_t head = nstages * (8 + 8 + 8) + 32 * 4 + 8 * 8;
-    if (staging) return 2ull * ard::kStageEntries * 4 + (size_t)stage_words * 4;   // select: one tile per CTA
+    if (staging) return 1ull * ard::kStageEntries * 4 + (size_t)stage_words * 4;   // select: one tile per CTA
     head = (head + 127) & ~size_t(127);
     size_t bytes = head + 128 + (size_t)nstages * stage_words * 4;
     if (!staging) bytes += (size_t)kFusNW * 32 * 32 * kFusBPT * 2   // per-warp candidate lists (u16)
@@ -851,6 +876,13 @@ ar_status launch_scan(const void* fn, const ard::SelParams& P, int grid, size_t 
     cfg.attrs = attr;
     cfg.numAttrs = 1;
     AR_TRY_CUDA(cudaLaunchKernelExC(&cfg, fn, args));
+    return AR_OK;
+}
+
+ar_status launch_select_rest(const ard::SelParams& P, cudaStream_t s) {
+    const int grid = (int)std::min<long long>((P.num_tiles + 7) / 8, (long long)num_sms() * 8);
+    ard::compact_kernel<<<grid, 256, 0, s>>>(P);
+    AR_CHECK_LAUNCH("compact_kernel");
     return AR_OK;
 }
 

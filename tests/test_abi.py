@@ -54,8 +54,8 @@ def test_host_only_entry_points():
     lib = _ar.load()
     assert lib.ar_status_str(0) == b"AR_OK" and lib.ar_status_str(2) == b"AR_ERR_RANGE"
     assert b"sm_100a" in lib.ar_version()
-    assert _ar.ar_select_ws_bytes(0) == 16
-    assert _ar.ar_select_ws_bytes(4096) == 16 + 8 and _ar.ar_select_ws_bytes(4097) == 16 + 16
+    # per-tile counts + offsets and the tile-local candidate slices (8 B per row)
+    assert _ar.ar_select_ws_bytes(4096) >= 8 * 4096 and _ar.ar_select_ws_bytes(4097) >= 8 * 4097
     assert _ar.ar_refine_ws_bytes(2048) == 16 + 8
     assert _ar.ar_dist_unique_id_bytes() == 128
     assert ctypes.sizeof(_ar.ColumnDesc) == 48
