@@ -509,7 +509,7 @@ __global__ void __launch_bounds__(256) compact_kernel(const __grid_constant__ Se
 // gathers of a whole warp are in flight together (Alg. 2).
 constexpr int kPer = 2;               // list entries per lane per pass
 constexpr int kGSlot = 32 * kPer;     // async-gather entries per warp per tile (first pass)
-constexpr int kGDepth = 3;            // tiles of gathers in flight per warp
+constexpr int kGDepth = 4;            // tiles of gathers in flight per warp
 
 __device__ __forceinline__ void cp_async4(uint32_t* dst, const uint32_t* src) {
     asm volatile("cp.async.ca.shared.global.L2::64B [%0], [%1], 4;" ::"r"(smem_u32(dst)), "l"(src) : "memory");
