@@ -84,8 +84,14 @@ typedef struct {
     int32_t major_layout;      /* ar_layout of the major part                             */
     int32_t residual_loc;      /* ar_loc of the residual part                             */
     uint32_t base;             /* prefix base b: value = ((major << k) | residual) + b    */
-    uint64_t major_bytes;      /* bytes the major buffer must provide (device memory)     */
+    uint64_t major_bytes;      /* bytes the major buffer must provide                     */
     uint64_t residual_bytes;   /* bytes the residual buffer must provide (0 if k == 0)    */
+    int32_t major_loc;         /* ar_loc of the major part: AR_LOC_DEVICE (set by the plan);
+                                  a caller may set AR_LOC_HOST_PINNED before ar_decompose /
+                                  ar_column_wrap for a column that is only gathered (an
+                                  aggregate column): kernels then read it over the host link.
+                                  Predicate columns must keep their majors on the device.  */
+    int32_t reserved;
 } ar_column_desc;
 
 typedef struct ar_column ar_column;   /* opaque: desc + part pointers (host object) */

@@ -78,11 +78,18 @@ class BWDColumn:
     def nbytes(self) -> dict:
         return {"major": int(self.desc.major_bytes), "residual": int(self.desc.residual_bytes)}
 
-    def copy(self, residual_loc=None) -> "BWDColumn":
-        """A second handle over copies of the buffers (used to rotate inputs past L2 in the bench)."""
-        major = self.major.clone()
-        residual = self.residual.clone() if self.residual.device.type == "cuda" else self.residual.clone().pin_memory()
-        return BWDColumn(None, 0, _wrap=(self.desc, major, residual), device=self.device)
+    def copy(self, major_loc=None, residual_loc=None) -> "BWDColumn":
+        """A second handle over copies of the buffers, optionally moved between HBM and pinned host
+        memory (used to rotate inputs past L2, and for host-resident parts)."""
+        def place(t, loc):
+            if loc == AR_LOC_HOST_PINNED:
+                return t.cpu().pin_memory()
+            return t.to(self.device).clone() if t.device.type == "cuda" else t.to(self.device)
+        mloc = self.desc.major_loc if major_loc is None else major_loc
+        rloc = self.desc.residual_loc if residual_loc is None else residual_loc
+        desc = _ar.ColumnDesc.from_buffer_copy(self.desc)
+        desc.major_loc, desc.residual_loc = mloc, rloc
+        return BWDColumn(None, 0, _wrap=(desc, place(self.major, mloc), place(self.residual, rloc)), device=self.device)
 
     def free(self):
         if getattr(self, "handle", None):

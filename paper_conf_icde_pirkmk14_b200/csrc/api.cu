@@ -192,7 +192,8 @@ static ar_status check_desc(const ar_column_desc* d) {
     if (!d || d->n < 0 || d->n >= (int64_t)1 << 32 || d->major_bits < 1 || d->major_bits > 32 ||
         d->k != 32 - d->major_bits || d->w_major < 0 || d->w_major > d->major_bits ||
         (d->major_layout != AR_LAYOUT_SLICED && d->major_layout != AR_LAYOUT_PACKED) ||
-        (d->residual_loc != AR_LOC_DEVICE && d->residual_loc != AR_LOC_HOST_PINNED)) {
+        (d->residual_loc != AR_LOC_DEVICE && d->residual_loc != AR_LOC_HOST_PINNED) ||
+        (d->major_loc != AR_LOC_DEVICE && d->major_loc != AR_LOC_HOST_PINNED)) {
         set_error("invalid ar_column_desc");
         return AR_ERR_INVALID;
     }
@@ -226,13 +227,16 @@ ar_status ar_column_wrap(const ar_column_desc* desc, const void* major_buf, cons
     const uint32_t* res = nullptr;
     st = device_alias(residual_buf, desc->residual_loc, &res);
     if (st != AR_OK) return st;
+    const uint32_t* maj = nullptr;
+    st = device_alias(major_buf, desc->major_loc, &maj);
+    if (st != AR_OK) return st;
     ar_column* c = new (std::nothrow) ar_column;
     if (!c) {
         set_error("out of host memory");
         return AR_ERR_RANGE;
     }
     c->d = *desc;
-    c->major = (const uint32_t*)major_buf;
+    c->major = maj;
     c->residual = desc->k > 0 ? res : nullptr;
     *out = c;
     return AR_OK;
@@ -259,11 +263,11 @@ ar_status ar_decompose(const uint32_t* col, const ar_column_desc* desc, void* ma
     const int64_t n = desc->n;
     const int w = desc->w_major, k = desc->k;
     if (w > 0) {
+        uint32_t* mdst = const_cast<uint32_t*>(c->major);   // device alias (mapped when host-resident)
         if (desc->major_layout == AR_LAYOUT_SLICED)
-            st = launch_pack_sliced(col, n, k, desc->base, w, (uint32_t*)major_buf, s);
+            st = launch_pack_sliced(col, n, k, desc->base, w, mdst, s);
         else
-            st = launch_pack_packed(col, n, k, 0xffffffffu, desc->base, w, desc->major_bytes / 4,
-                                    (uint32_t*)major_buf, s);
+            st = launch_pack_packed(col, n, k, 0xffffffffu, desc->base, w, desc->major_bytes / 4, mdst, s);
     }
     if (st == AR_OK && k > 0)
         st = launch_pack_packed(col, n, 0, (1u << k) - 1u, desc->base, k, desc->residual_bytes / 4,
@@ -324,8 +328,8 @@ static ar_status setup_scan(const ar_pred* preds, int32_t npred, ard::SelParams&
             set_error("predicate %d: null column or n differs from predicate 0", c);
             return AR_ERR_INVALID;
         }
-        if (col->d.major_layout != AR_LAYOUT_SLICED) {
-            set_error("predicate %d: the approximate scan needs AR_LAYOUT_SLICED majors", c);
+        if (col->d.major_layout != AR_LAYOUT_SLICED || col->d.major_loc != AR_LOC_DEVICE) {
+            set_error("predicate %d: the approximate scan needs AR_LAYOUT_SLICED majors in device memory", c);
             return AR_ERR_INVALID;
         }
         const int w = col->d.w_major, k = col->d.k;
@@ -616,7 +620,7 @@ ar_status ar_select_refine_sum(const ar_pred* preds, int32_t npred, const ar_col
             if (a.pred < 0) {
                 ++ng;
                 g = i;
-                ok = ok && a.k == 0 && a.layout == AR_LAYOUT_PACKED && a.w > 0;
+                ok = ok && a.k == 0 && a.layout == AR_LAYOUT_PACKED && a.w > 0 && cols[i]->d.major_loc == AR_LOC_DEVICE;
             } else {
                 ok = ok && (a.w + a.k) <= 26 && a.base == 0;
             }

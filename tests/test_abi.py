@@ -58,7 +58,7 @@ def test_host_only_entry_points():
     assert _ar.ar_select_ws_bytes(4096) >= 8 * 4096 and _ar.ar_select_ws_bytes(4097) >= 8 * 4097
     assert _ar.ar_refine_ws_bytes(2048) == 16 + 8
     assert _ar.ar_dist_unique_id_bytes() == 128
-    assert ctypes.sizeof(_ar.ColumnDesc) == 48
+    assert ctypes.sizeof(_ar.ColumnDesc) == 56
 
 
 def test_host_validation_without_gpu():
