@@ -59,7 +59,11 @@ typedef enum {
  *  AR_LAYOUT_PACKED: LSB-first bitstream, row i occupies bits [i*w, i*w+w) of
  *    the little-endian uint32 word stream.  Gather-optimised (one sector per
  *    value): use it for columns that are only aggregated (l_extendedprice).
- * Residuals (minor bits) are always AR_LAYOUT_PACKED with width k.
+ * Residuals (minor bits) use the same two layouts with width k: the plan picks
+ * SLICED for k <= 8 (a block's k residual planes are k*4 <= 32 bytes, one
+ * sector, so a gather costs the same as PACKED, and the one-pass kernel can
+ * evaluate exact predicates on major + residual planes together) and PACKED
+ * for wider residuals (a gather reads one sector instead of k*4 bytes).
  */
 typedef enum {
     AR_LAYOUT_SLICED = 0,
@@ -91,7 +95,7 @@ typedef struct {
                                   ar_column_wrap for a column that is only gathered (an
                                   aggregate column): kernels then read it over the host link.
                                   Predicate columns must keep their majors on the device.  */
-    int32_t reserved;
+    int32_t residual_layout;   /* ar_layout of the residual part (set by the plan, see above) */
 } ar_column_desc;
 
 typedef struct ar_column ar_column;   /* opaque: desc + part pointers (host object) */

@@ -34,7 +34,7 @@ class ColumnDesc(ctypes.Structure):
     _fields_ = [("n", ctypes.c_int64), ("major_bits", ctypes.c_int32), ("k", ctypes.c_int32),
                 ("w_major", ctypes.c_int32), ("major_layout", ctypes.c_int32), ("residual_loc", ctypes.c_int32),
                 ("base", ctypes.c_uint32), ("major_bytes", ctypes.c_uint64), ("residual_bytes", ctypes.c_uint64),
-                ("major_loc", ctypes.c_int32), ("reserved", ctypes.c_int32)]
+                ("major_loc", ctypes.c_int32), ("residual_layout", ctypes.c_int32)]
 
 
 class Pred(ctypes.Structure):

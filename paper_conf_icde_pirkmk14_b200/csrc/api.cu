@@ -184,7 +184,8 @@ ar_status ar_decompose_plan(const uint32_t* col, int64_t n, int32_t major_bits, 
     desc->residual_loc = residual_loc;
     desc->base = base;
     desc->major_bytes = major_layout == AR_LAYOUT_SLICED ? sliced_bytes(n, w) : packed_bytes(n, w);
-    desc->residual_bytes = packed_bytes(n, k);
+    desc->residual_layout = (k >= 1 && k <= 8) ? AR_LAYOUT_SLICED : AR_LAYOUT_PACKED;
+    desc->residual_bytes = desc->residual_layout == AR_LAYOUT_SLICED ? sliced_bytes(n, k) : packed_bytes(n, k);
     return AR_OK;
 }
 
@@ -193,7 +194,8 @@ static ar_status check_desc(const ar_column_desc* d) {
         d->k != 32 - d->major_bits || d->w_major < 0 || d->w_major > d->major_bits ||
         (d->major_layout != AR_LAYOUT_SLICED && d->major_layout != AR_LAYOUT_PACKED) ||
         (d->residual_loc != AR_LOC_DEVICE && d->residual_loc != AR_LOC_HOST_PINNED) ||
-        (d->major_loc != AR_LOC_DEVICE && d->major_loc != AR_LOC_HOST_PINNED)) {
+        (d->major_loc != AR_LOC_DEVICE && d->major_loc != AR_LOC_HOST_PINNED) ||
+        (d->residual_layout != AR_LAYOUT_SLICED && d->residual_layout != AR_LAYOUT_PACKED)) {
         set_error("invalid ar_column_desc");
         return AR_ERR_INVALID;
     }
@@ -265,13 +267,17 @@ ar_status ar_decompose(const uint32_t* col, const ar_column_desc* desc, void* ma
     if (w > 0) {
         uint32_t* mdst = const_cast<uint32_t*>(c->major);   // device alias (mapped when host-resident)
         if (desc->major_layout == AR_LAYOUT_SLICED)
-            st = launch_pack_sliced(col, n, k, desc->base, w, mdst, s);
+            st = launch_pack_sliced(col, n, k, 0xffffffffu, desc->base, w, mdst, s);
         else
             st = launch_pack_packed(col, n, k, 0xffffffffu, desc->base, w, desc->major_bytes / 4, mdst, s);
     }
-    if (st == AR_OK && k > 0)
-        st = launch_pack_packed(col, n, 0, (1u << k) - 1u, desc->base, k, desc->residual_bytes / 4,
-                                const_cast<uint32_t*>(c->residual), s);
+    if (st == AR_OK && k > 0) {
+        uint32_t* rdst = const_cast<uint32_t*>(c->residual);
+        if (desc->residual_layout == AR_LAYOUT_SLICED)
+            st = launch_pack_sliced(col, n, 0, (1u << k) - 1u, desc->base, k, rdst, s);
+        else
+            st = launch_pack_packed(col, n, 0, (1u << k) - 1u, desc->base, k, desc->residual_bytes / 4, rdst, s);
+    }
     if (st != AR_OK) {
         delete c;
         return st;
@@ -350,14 +356,16 @@ static ar_status setup_scan(const ar_pred* preds, int32_t npred, ard::SelParams&
         p.base = col->d.base;
         p.lo = preds[c].lo;
         p.hi = preds[c].hi;
+        p.rlayout = (uint32_t)col->d.residual_layout;
         words += (P.tile_rows / 32) * (uint32_t)w;
         ashift += (uint32_t)w;
-        // the one-pass kernel streams device-resident residual tiles with the majors (dense
-        // 8-bit residuals: streaming ~1.4x the touched bytes beats a dependent gather round trip)
-        if (fused && k > 0 && col->d.residual_loc == AR_LOC_DEVICE && col->residual) {
+        // the one-pass kernel streams device-resident SLICED residual tiles (k <= 8) with the
+        // majors and evaluates the exact predicate on major + residual planes in place
+        if (fused && k > 0 && col->d.residual_loc == AR_LOC_DEVICE && col->residual &&
+            col->d.residual_layout == AR_LAYOUT_SLICED) {
             p.res_stream = 1;
             p.res_soff = words;
-            words += (P.tile_rows / 32) * (uint32_t)k + 4;   // + 16 B: the copy rounds up to 16 B
+            words += (P.tile_rows / 32) * (uint32_t)k;
         }
     }
     uint32_t planes = 0;
@@ -365,6 +373,21 @@ static ar_status setup_scan(const ar_pred* preds, int32_t npred, ard::SelParams&
     if (planes > AR_MAX_PLANES) {
         set_error("sum of w_major over predicates = %u > AR_MAX_PLANES (%d)", planes, AR_MAX_PLANES);
         return AR_ERR_UNSUPPORTED;
+    }
+    // exact-bound masks for the one-pass kernel: bit i of u = v - base over the
+    // concatenated residual (i < k) and major (k <= i < k + w) planes
+    P.exact_mode = fused ? 1 : 0;
+    for (int c = 0; c < npred; ++c) {
+        const ard::SelPred& p = P.p[c];
+        if (p.k > 0 && !p.res_stream) P.exact_mode = 0;
+        if (!p.res_stream) continue;
+        const uint64_t maxu = p.k + p.w >= 32 ? 0xffffffffull : ((1ull << (p.k + p.w)) - 1);
+        const uint64_t ulo = p.lo < p.base ? 0 : (uint64_t)(p.lo - p.base);
+        const uint64_t uhi = std::min<uint64_t>((uint64_t)(p.hi - p.base), maxu);
+        for (uint32_t i = 0; i < p.k + p.w && i < 32; ++i) {
+            P.pmx[c][i][0] = 0u - (uint32_t)((ulo >> i) & 1u);
+            P.pmx[c][i][1] = 0u - (uint32_t)((uhi >> i) & 1u);
+        }
     }
     for (int c = 0; c < npred; ++c) {
         const ard::SelPred& p = P.p[c];
@@ -465,6 +488,7 @@ static ar_status setup_refine(const ar_cands* in, const ar_pred* preds, int32_t 
         p.base = col->d.base;
         p.lo = preds[c].lo;
         p.hi = preds[c].hi;
+        p.rlayout = (uint32_t)col->d.residual_layout;
         p.ashift = ashift;
         p.carried = in->appr_bits > 0 ? 1u : 0u;
         p.check = col->d.k > 0 ? 1u : 0u;
@@ -535,6 +559,7 @@ static ar_status setup_aggs(const ar_column* const* cols, int32_t ncols, const a
         a[i].k = (uint32_t)c->d.k;
         a[i].layout = (uint32_t)c->d.major_layout;
         a[i].base = c->d.base;
+        a[i].rlayout = (uint32_t)c->d.residual_layout;
         a[i].pred = -1;
         for (int p = 0; p < npred; ++p)
             if (preds[p].col == c) { a[i].pred = p; break; }

@@ -118,7 +118,7 @@ __device__ __forceinline__ void mbar_wait(uint64_t* bar, uint32_t parity, uint32
 // producer lane, whose spinning would otherwise take issue slots from the
 // consumer warps of its SM.
 __device__ __forceinline__ void mbar_wait_sleep(uint64_t* bar, uint32_t parity) {
-    uint32_t ns = 32;
+    uint32_t ns = 256;
     while (true) {
         uint32_t done;
         asm volatile(
@@ -130,7 +130,7 @@ __device__ __forceinline__ void mbar_wait_sleep(uint64_t* bar, uint32_t parity) 
             : "memory");
         if (done) return;
         __nanosleep(ns);
-        if (ns < 256) ns <<= 1;
+        if (ns < 2048) ns <<= 1;
     }
 }
 
@@ -269,8 +269,19 @@ __device__ __forceinline__ uint32_t packed_get(const uint32_t* __restrict__ s, u
     if (sh + (uint32_t)w > 32u) v = __funnelshift_r(lo, ld_gather(s + wi + 1), sh);
     return w == 32 ? v : (v & ((1u << w) - 1u));
 }
-// Residual gather: device memory or pinned host memory through a mapped pointer.
-__device__ __forceinline__ uint32_t packed_get_any(const uint32_t* s, uint64_t p, int w) { return packed_get(s, p, w); }
+// Residual of row p (width k) in either layout, from device memory or from
+// pinned host memory through a mapped pointer.  SLICED (k <= 8): the block's k
+// planes sit in one 32-B sector.
+__device__ __forceinline__ uint32_t residual_get(const uint32_t* s, uint64_t p, int k, int layout) {
+    if (layout == AR_LAYOUT_SLICED) {
+        const uint32_t* blk = s + (p >> 5) * (uint64_t)k;
+        const uint32_t l = (uint32_t)(p & 31);
+        uint32_t r = 0;
+        for (int j = 0; j < k; ++j) r |= ((ld_gather(blk + j) >> l) & 1u) << j;
+        return r;
+    }
+    return packed_get(s, p, k);
+}
 
 // Same extraction from a PACKED stream staged in shared memory (bit offset `bit`).
 __device__ __forceinline__ uint32_t packed_get_smem(const uint32_t* s, uint32_t bit, int w) {
@@ -300,9 +311,9 @@ __device__ __forceinline__ uint32_t major_get(const uint32_t* __restrict__ s, ui
 // Exact value of row p of a column (major and residual joined).
 // Generic (any layout, any k): out of line; kernels inline only their hot case.
 static __device__ __noinline__ uint32_t value_get(const uint32_t* major, const uint32_t* residual, uint64_t p,
-                                              int w, int k, int layout, uint32_t base) {
+                                              int w, int k, int layout, uint32_t base, int rlayout) {
     uint32_t m = major_get(major, p, w, layout);
-    uint32_t r = k ? packed_get_any(residual, p, k) : 0u;
+    uint32_t r = k ? residual_get(residual, p, k, rlayout) : 0u;
     uint32_t u = k == 32 ? r : ((m << k) | r);
     return u + base;
 }

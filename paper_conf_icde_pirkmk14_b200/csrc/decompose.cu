@@ -18,13 +18,14 @@ __global__ void max_kernel(const uint32_t* __restrict__ col, int64_t n, uint32_t
 }
 
 // One warp per 32-row block; blocks beyond n (up to the 128-row padding) are zero.
-__global__ void pack_sliced_kernel(const uint32_t* __restrict__ col, int64_t n, int k, uint32_t base, int w,
-                                   int64_t nblocks, uint32_t* __restrict__ out) {
+// Field of row i: ((col[i] - base) >> shift) & mask (major: shift k; residual: mask 2^k - 1).
+__global__ void pack_sliced_kernel(const uint32_t* __restrict__ col, int64_t n, int shift, uint32_t mask,
+                                   uint32_t base, int w, int64_t nblocks, uint32_t* __restrict__ out) {
     const unsigned lane = threadIdx.x & 31;
     const int64_t warps = (int64_t)gridDim.x * (blockDim.x / 32);
     for (int64_t b = (int64_t)blockIdx.x * (blockDim.x / 32) + (threadIdx.x >> 5); b < nblocks; b += warps) {
         const int64_t row = b * 32 + lane;
-        const uint32_t m = row < n ? ((col[row] - base) >> k) : 0u;
+        const uint32_t m = row < n ? (((col[row] - base) >> shift) & mask) : 0u;
         uint32_t mine = 0;
         for (int j = 0; j < w; ++j) {
             const uint32_t plane = __ballot_sync(0xffffffffu, (m >> j) & 1u);
@@ -68,12 +69,12 @@ ar_status launch_decompose_max(const uint32_t* col, int64_t n, uint32_t base, ui
     return AR_OK;
 }
 
-ar_status launch_pack_sliced(const uint32_t* col, int64_t n, int k, uint32_t base, int w, uint32_t* out,
-                             cudaStream_t s) {
+ar_status launch_pack_sliced(const uint32_t* col, int64_t n, int shift, uint32_t mask, uint32_t base, int w,
+                             uint32_t* out, cudaStream_t s) {
     const int64_t nblocks = (int64_t)ceil_div_u64((uint64_t)n, 128) * 4;
     if (w == 0 || nblocks == 0) return AR_OK;
     int grid = (int)std::min<int64_t>((nblocks + 7) / 8, (int64_t)num_sms() * 16);
-    ard::pack_sliced_kernel<<<grid, 256, 0, s>>>(col, n, k, base, w, nblocks, out);
+    ard::pack_sliced_kernel<<<grid, 256, 0, s>>>(col, n, shift, mask, base, w, nblocks, out);
     AR_CHECK_LAUNCH("pack_sliced_kernel");
     return AR_OK;
 }

@@ -16,6 +16,7 @@ struct SelPred {
     // refine-side data, used by the fused kernel
     const uint32_t* residual; // PACKED width k (device or host-mapped), null if k == 0
     uint32_t k, base, lo, hi; // exact predicate on v = ((m << k) | r) + base
+    uint32_t rlayout;         // residual layout (ar_layout)
     uint32_t res_stream;      // fused kernel: residual tile streamed into the stage (device-resident residuals)
     uint32_t res_soff;        // word offset of the streamed residual tile inside a stage
 };
@@ -24,7 +25,7 @@ struct SelPred {
 struct AggCol {
     const uint32_t* major;
     const uint32_t* residual;
-    uint32_t w, k, layout, base;
+    uint32_t w, k, layout, base, rlayout;
     int32_t pred;             // index of the predicate over the same column, or -1
 };
 
@@ -33,7 +34,7 @@ struct AggCol {
 // everything else through the out-of-line generic path.
 __device__ __forceinline__ uint32_t agg_gather(const AggCol& a, uint64_t p) {
     if (a.k == 0 && a.layout == AR_LAYOUT_PACKED && a.w > 0) return packed_get(a.major, p, (int)a.w) + a.base;
-    return value_get(a.major, a.residual, p, (int)a.w, (int)a.k, (int)a.layout, a.base);
+    return value_get(a.major, a.residual, p, (int)a.w, (int)a.k, (int)a.layout, a.base, (int)a.rlayout);
 }
 
 constexpr int kSelWarps = 4;                      // consumer warps per CTA
@@ -67,6 +68,9 @@ struct SelParams {
     // fused kernel only
     AggCol a[AR_MAX_AGG];
     int32_t nagg;
+    int32_t exact_mode;           // fused: every decomposed predicate has its residual planes streamed, so
+                                  // the exact predicate is evaluated on major + residual planes in place
+    uint32_t pmx[AR_MAX_PRED][32][2];   // exact bounds, bit i of (lo - base) / (hi - base) as 0 / ~0
     int32_t async_agg;            // fused: the one gathered aggregate column uses asynchronous gathers
     int32_t gidx;                 // index of that column in a[]
     unsigned long long* out4;     // sum, |result|, |cand|, |def|
@@ -75,7 +79,7 @@ struct SelParams {
 struct RefPred {
     const uint32_t* major;
     const uint32_t* residual;
-    uint32_t w, k, layout, base, lo, hi;
+    uint32_t w, k, layout, base, lo, hi, rlayout;
     uint32_t ashift;
     uint32_t carried;         // major available in aux
     uint32_t check;           // k > 0: must be re-evaluated on the exact value
@@ -124,8 +128,8 @@ ar_status launch_refine(const ard::RefParams& P, int grid, cudaStream_t s);
 ar_status launch_refine_sum(const ard::RefParams& P, int grid, cudaStream_t s);
 ar_status launch_sum(const ard::SumParams& P, int grid, cudaStream_t s);
 ar_status launch_decompose_max(const uint32_t* col, int64_t n, uint32_t base, uint32_t* out_max, cudaStream_t s);
-ar_status launch_pack_sliced(const uint32_t* col, int64_t n, int k, uint32_t base, int w, uint32_t* out,
-                             cudaStream_t s);
+ar_status launch_pack_sliced(const uint32_t* col, int64_t n, int shift, uint32_t mask, uint32_t base, int w,
+                             uint32_t* out, cudaStream_t s);
 ar_status launch_pack_packed(const uint32_t* col, int64_t n, int shift, uint32_t mask, uint32_t base, int w,
                              uint64_t out_words, uint32_t* out, cudaStream_t s);
 ar_status launch_exclusive_offset(const long long* all_counts, int world, int rank, long long* out,

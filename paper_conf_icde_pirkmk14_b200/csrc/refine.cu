@@ -23,7 +23,7 @@ __device__ __forceinline__ bool refine_keep(const RefParams& P, uint32_t pos, ui
         if (!p.check) continue;
         const uint32_t m = p.carried ? ((aux >> p.ashift) & (p.w == 32 ? 0xffffffffu : ((1u << p.w) - 1u)))
                                      : major_get(p.major, pos, p.w, p.layout);
-        const uint32_t r = packed_get_any(p.residual, pos, p.k);
+        const uint32_t r = residual_get(p.residual, pos, p.k, p.rlayout);
         const uint32_t v = ((m << p.k) | r) + p.base;
         ok = ok && (v >= p.lo) && (v <= p.hi);
     }
@@ -34,7 +34,7 @@ __device__ __forceinline__ uint32_t agg_value_at(const RefParams& P, const AggCo
     if (a.pred >= 0 && P.p[a.pred].carried) {
         const RefPred& p = P.p[a.pred];
         const uint32_t m = (aux >> p.ashift) & (p.w == 32 ? 0xffffffffu : ((1u << p.w) - 1u));
-        const uint32_t r = a.k ? packed_get_any(a.residual, pos, a.k) : 0u;
+        const uint32_t r = a.k ? residual_get(a.residual, pos, a.k, a.rlayout) : 0u;
         return ((m << a.k) | r) + a.base;
     }
     return agg_gather(a, pos);

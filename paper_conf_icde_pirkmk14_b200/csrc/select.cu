@@ -162,6 +162,65 @@ struct FixedPlanes {
         eval_c<0>(P, cm, dm);
     }
 
+    // Exact predicate (Alg. 2 on the planes): for each decomposed predicate whose
+    // residual planes are in the stage, one borrow chain over the k residual
+    // planes then the w major planes -- the bitwise concatenation "+bw" of the
+    // approximation and the residual -- against the exact bounds.  xm &= result.
+    template <int C, int K>
+    __device__ __forceinline__ void exact_k(const SelParams& P, const uint32_t* stg, uint32_t (&xm)[BPT]) const {
+        constexpr int w = wid<Ws...>(C), o = woff<Ws...>(C);
+        const SelPred& p = P.p[C];
+#pragma unroll
+        for (int b = 0; b < BPT; ++b) {
+            const uint32_t* rp = stg + p.res_soff + (threadIdx.x * BPT + b) * K;
+            uint32_t r[K];
+            if constexpr (K % 4 == 0) {   // 16-B aligned: k = 4, 8
+#pragma unroll
+                for (int q = 0; q < K / 4; ++q) {
+                    const uint4 v = reinterpret_cast<const uint4*>(rp)[q];
+                    r[4 * q] = v.x; r[4 * q + 1] = v.y; r[4 * q + 2] = v.z; r[4 * q + 3] = v.w;
+                }
+            } else {
+#pragma unroll
+                for (int j = 0; j < K; ++j) r[j] = rp[j];
+            }
+            uint32_t bl = 0, bh = 0;
+#pragma unroll
+            for (int j = 0; j < K; ++j) {
+                bl = borrow_sub(r[j], P.pmx[C][j][0], bl);
+                bh = borrow_rsub(r[j], P.pmx[C][j][1], bh);
+            }
+#pragma unroll
+            for (int j = 0; j < w; ++j) {
+                bl = borrow_sub(x[b][o + j], P.pmx[C][K + j][0], bl);
+                bh = borrow_rsub(x[b][o + j], P.pmx[C][K + j][1], bh);
+            }
+            xm[b] &= ~(bl | bh);
+        }
+    }
+    // Exact predicate (Alg. 2 on the planes): for each decomposed predicate whose
+    // residual planes are in the stage, one borrow chain over the k residual
+    // planes then the w major planes -- the bitwise concatenation "+bw" of the
+    // approximation and the residual -- against the exact bounds.  xm &= result.
+    template <int C = 0>
+    __device__ __forceinline__ void exact(const SelParams& P, const uint32_t* stg, uint32_t (&xm)[BPT]) const {
+        if constexpr (C < N) {
+            if (P.p[C].res_stream) {
+                switch (P.p[C].k) {   // residual planes are only streamed for k <= 8
+                    case 1: exact_k<C, 1>(P, stg, xm); break;
+                    case 2: exact_k<C, 2>(P, stg, xm); break;
+                    case 3: exact_k<C, 3>(P, stg, xm); break;
+                    case 4: exact_k<C, 4>(P, stg, xm); break;
+                    case 5: exact_k<C, 5>(P, stg, xm); break;
+                    case 6: exact_k<C, 6>(P, stg, xm); break;
+                    case 7: exact_k<C, 7>(P, stg, xm); break;
+                    default: exact_k<C, 8>(P, stg, xm); break;
+                }
+            }
+            exact<C + 1>(P, stg, xm);
+        }
+    }
+
     // major of predicate C at row l of block B
     template <int B, int C>
     __device__ __forceinline__ uint32_t value(uint32_t l) const {
@@ -242,6 +301,25 @@ struct DynPlanes {
                 const uint32_t c0 = ~(cl[b] | ch[b]);
                 cm[b] &= c0;
                 dm[b] = p.mode == 0 ? (dm[b] & c0) : (p.mode == 1 ? (dm[b] & ~(dl[b] | dh[b])) : 0u);
+            }
+        }
+    }
+    __device__ __forceinline__ void exact(const SelParams& P, const uint32_t* s, uint32_t (&xm)[BPT]) const {
+        for (int c = 0; c < P.npred; ++c) {
+            const SelPred& p = P.p[c];
+            if (!p.res_stream) continue;
+            const uint32_t k = p.k, w = p.w;
+#pragma unroll
+            for (int b = 0; b < BPT; ++b) {
+                const uint32_t* rp = s + p.res_soff + (threadIdx.x * BPT + b) * k;
+                const uint32_t* mp = s + p.soff + (threadIdx.x * BPT + b) * w;
+                uint32_t bl = 0, bh = 0;
+                for (uint32_t j = 0; j < k + w; ++j) {
+                    const uint32_t x = j < k ? rp[j] : mp[j - k];
+                    bl = borrow_sub(x, P.pmx[c][j][0], bl);
+                    bh = borrow_rsub(x, P.pmx[c][j][1], bh);
+                }
+                xm[b] &= ~(bl | bh);
             }
         }
     }
@@ -333,7 +411,7 @@ __device__ __forceinline__ void produce(const SelParams& P, const SmemLayout& L)
         uint32_t bytes = 0;
         for (int c = 0; c < P.npred; ++c) {
             bytes += groups * 16u * P.p[c].w;
-            if (P.p[c].res_stream) bytes += (uint32_t)(((rows * P.p[c].k + 7) / 8 + 15) / 16 * 16);
+            if (P.p[c].res_stream) bytes += groups * 16u * P.p[c].k;
         }
         mbar_arrive_expect_tx(L.full + s, bytes);
         uint32_t* stg = L.stages + (size_t)s * P.stage_words;
@@ -343,10 +421,10 @@ __device__ __forceinline__ void produce(const SelParams& P, const SmemLayout& L)
                 const uint32_t* src = P.p[c].planes + (size_t)t * blocks_per_tile * w;
                 bulk_g2s(stg + P.p[c].soff, src, groups * 16u * w, L.full + s, pol);
             }
-            if (P.p[c].res_stream) {   // the tile's residual bits, a contiguous 16-B aligned byte range
+            if (P.p[c].res_stream) {   // the tile's SLICED residual planes
                 const uint32_t k = P.p[c].k;
                 const uint32_t* src = P.p[c].residual + (size_t)t * (P.tile_rows / 32) * k;
-                bulk_g2s(stg + P.p[c].res_soff, src, (uint32_t)(((rows * k + 7) / 8 + 15) / 16 * 16), L.full + s, pol);
+                bulk_g2s(stg + P.p[c].res_soff, src, groups * 16u * k, L.full + s, pol);
             }
         }
         if (++s == P.nstages) {
@@ -588,6 +666,22 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_kernel(const __grid_co
             ndef += __popc(dm[b]);
         }
         ncand += cnt;
+        const bool exact_mode = P.exact_mode != 0;
+        if (exact_mode) {
+            // a5 in place: exact predicate on major + residual planes of the candidate rows;
+            // the list below then holds result rows only (no per-candidate refine pass)
+            uint32_t xm[BPT];
+#pragma unroll
+            for (int b = 0; b < BPT; ++b) xm[b] = cm[b];
+            ps.exact(P, stg, xm);
+            cnt = 0;
+#pragma unroll
+            for (int b = 0; b < BPT; ++b) {
+                cm[b] = xm[b];
+                dm[b] = xm[b];        // every listed row is a result: marked definite, skips the refine pass
+                cnt += __popc(xm[b]);
+            }
+        }
 
         // compact the warp's candidates into its list (ascending row order)
         uint32_t incl = cnt;
@@ -633,9 +727,11 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_kernel(const __grid_co
                 for (int q = 0; q < kPer; ++q) {
                     const bool need = ok[q] && !dfn[q];
                     if (p.res_stream)
-                        r[q] = need ? packed_get_smem(stg + p.res_soff, (row_in_tile0 + off[q]) * p.k, p.k) : 0u;
+                        r[q] = need ? plane_value(stg + p.res_soff + ((row_in_tile0 + off[q]) >> 5) * p.k, p.k,
+                                                  off[q] & 31u)
+                                    : 0u;
                     else
-                        r[q] = need ? packed_get_any(p.residual, row_base + off[q], p.k) : 0u;
+                        r[q] = need ? residual_get(p.residual, row_base + off[q], p.k, p.rlayout) : 0u;
                 }
 #pragma unroll
                 for (int q = 0; q < kPer; ++q) {
@@ -673,8 +769,9 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_kernel(const __grid_co
                             for (uint32_t j = 0; j < w; ++j) m |= ((pl[j] >> l) & 1u) << j;
                             uint32_t r = 0u;
                             if (p.k)
-                                r = p.res_stream ? packed_get_smem(stg + p.res_soff, (row_in_tile0 + off[q]) * p.k, p.k)
-                                                 : packed_get_any(p.residual, row_base + off[q], p.k);
+                                r = p.res_stream ? plane_value(stg + p.res_soff + ((row_in_tile0 + off[q]) >> 5) * p.k,
+                                                               p.k, off[q] & 31u)
+                                                 : residual_get(p.residual, row_base + off[q], p.k, p.rlayout);
                             mult = ((m << p.k) | r) + p.base;
                         });
                     }
@@ -720,8 +817,10 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_kernel(const __grid_co
                                 for (uint32_t j = 0; j < w; ++j) m |= ((pl[j] >> l) & 1u) << j;
                                 uint32_t r = 0u;
                                 if (p.k)
-                                    r = p.res_stream ? packed_get_smem(stg + p.res_soff, (row_in_tile0 + off[q]) * p.k, p.k)
-                                                     : packed_get_any(p.residual, row_base + off[q], p.k);
+                                    r = p.res_stream
+                                            ? plane_value(stg + p.res_soff + ((row_in_tile0 + off[q]) >> 5) * p.k, p.k,
+                                                          off[q] & 31u)
+                                            : residual_get(p.residual, row_base + off[q], p.k, p.rlayout);
                                 v[q] = ((m << p.k) | r) + p.base;
                             }
                         });

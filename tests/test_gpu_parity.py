@@ -29,6 +29,12 @@ def _bytes(t):
     return t.cpu().numpy().tobytes()
 
 
+def _residual(c, n):
+    """Decode a column's residual part per its layout (ar.h: SLICED for k <= 8, else PACKED)."""
+    dec = unpack_sliced if c.desc.residual_layout == 0 else unpack_packed
+    return dec(_bytes(c.residual), n, c.k)
+
+
 # ----------------------------------------------------------------- a1 decompose
 
 def test_gpu_decompose_fig2(cu, golden):
@@ -38,7 +44,8 @@ def test_gpu_decompose_fig2(cu, golden):
     c = _col(cu, v, 32 - k)
     assert c.w_major == int(g["gpu_bits"]) and c.k == k
     assert int(unpack_sliced(_bytes(c.major), 1, c.w_major)[0]) == int(g["major_bits_string"], 2)
-    assert int(unpack_packed(_bytes(c.residual), 1, k)[0]) == int(g["residual_bits_string"], 2)
+    assert c.desc.residual_layout == 0                 # k = 7 <= 8: bit-sliced residual planes
+    assert int(_residual(c, 1)[0]) == int(g["residual_bits_string"], 2)
 
 
 @pytest.mark.parametrize("n", [0, 1, 31, 32, 33, 127, 128, 129, 4095, 4096, 4097, 2**20 - 1, 2**20 + 1])
@@ -53,7 +60,8 @@ def test_gpu_decompose_matches_oracle(cu, n, major_bits, layout):
     got_major = dec(_bytes(c.major), n, w)
     assert np.array_equal(got_major, major.astype(np.uint64))
     if c.k:
-        assert np.array_equal(unpack_packed(_bytes(c.residual), n, c.k), residual.astype(np.uint64))
+        assert c.desc.residual_layout == (0 if c.k <= 8 else 1)
+        assert np.array_equal(_residual(c, n), residual.astype(np.uint64))
     if layout == 0 and n % 128:
         # padding rows of the last 128-row group are zero planes
         words = np.frombuffer(_bytes(c.major), dtype="<u4")
@@ -67,7 +75,7 @@ def test_gpu_decompose_base(cu):
     major, residual, w = oracle.decompose(v, 8, base=1000)
     assert c.w_major == w
     assert np.array_equal(unpack_sliced(_bytes(c.major), 5, w), major.astype(np.uint64))
-    assert np.array_equal(unpack_packed(_bytes(c.residual), 5, 8), residual.astype(np.uint64))
+    assert np.array_equal(_residual(c, 5), residual.astype(np.uint64))
 
 
 # ------------------------------------------------------------ a2+a3 approx select
