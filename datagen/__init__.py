@@ -12,6 +12,7 @@ Workload configs (BASELINE.json `configs`):
   C3  1 G-row u32 column (uniform, or a keyed bijection of [0, N))
   C4  SF100 Q6 row-sharded over G GPUs
   C5  SF1000 Q6, residuals in pinned host memory
+  C6  spatial range count of Table I on GPS-fix-shaped int32 lon/lat
 """
 from __future__ import annotations
 
@@ -36,6 +37,12 @@ PARTS_PER_SF = 200_000           # TPC-H part table cardinality [ext]
 Q6_SHIPDATE = (731, 1095)        # [1994-01-01, 1995-01-01)
 Q6_DISCOUNT = (5, 7)             # BETWEEN 0.05 AND 0.07, hundredths
 Q6_QUANTITY = (0, 23)            # < 24
+
+# config C6: Table I, degrees scaled 1e5 (decimal(8,5) / decimal(7,5))
+SPATIAL_ROWS = 250_000_000        # "around 250 million tuples"
+SPATIAL_LON = (268288, 270228)    # lon BETWEEN 2.68288 AND 2.70228
+SPATIAL_LAT = (5042220, 5044850)  # lat BETWEEN 50.4222 AND 50.4485
+SPATIAL_BOX = ((-1262427, 2964975), (2709371, 7013643))   # data range
 
 # config C1
 C1_N = 1_000_000
@@ -64,6 +71,7 @@ def _load():
         lib.dg_uniform_u32.argtypes = [u64, u32, u64, i64, u32, u32, p, i32]
         lib.dg_bijection_u32.argtypes = [u64, u32, u64, u64, i64, p, i32]
         lib.dg_q6.argtypes = [u64, u64, u64, i64, p, p, p, p, i32]
+        lib.dg_spatial.argtypes = [u64, u64, i64, p, p, i32]
         lib.dg_threads_default.restype = i32
         _lib = lib
     return _lib
@@ -103,6 +111,14 @@ def q6_columns(seed, sf, n=None, row0=0, threads=0, which=("shipdate", "discount
     _load().dg_q6(seed, n_parts, row0, n, _ptr(cols["shipdate"]), _ptr(cols["discount"]),
                   _ptr(cols["quantity"]), _ptr(cols["extprice"]), threads)
     return {k: v for k, v in cols.items() if v is not None}
+
+
+def spatial_columns(seed, n, row0=0, threads=0):
+    """GPS-fix (lon, lat) int32 columns in 1e-5 degrees for rows [row0, row0+n) (config C6)."""
+    lon = np.empty(n, dtype=np.int32)
+    lat = np.empty(n, dtype=np.int32)
+    _load().dg_spatial(seed, row0, n, _ptr(lon), _ptr(lat), threads)
+    return {"lon": lon, "lat": lat}
 
 
 def default_threads() -> int:
@@ -157,3 +173,23 @@ def q6_columns_np(seed, sf, n, row0=0):
               + np.uint64(100) * (pk % np.uint64(1000)))
     return {"shipdate": (od + sd).astype(np.uint32), "discount": d.astype(np.uint32),
             "quantity": q.astype(np.uint32), "extprice": (q * retail).astype(np.uint32)}
+
+
+def spatial_columns_np(seed, n, row0=0):
+    rows = np.arange(row0, row0 + n, dtype=np.uint64)
+    trip, j = rows // np.uint64(128), (rows % np.uint64(128)).astype(np.int64)
+
+    def uni(stream, r, lo, hi):
+        return lo + _span_np(_draw_np(key_np(seed, stream), r), hi - lo + 1).astype(np.int64)
+
+    u = _span_np(_draw_np(key_np(seed, 12), trip), 1 << 16)
+    with np.errstate(over="ignore"):
+        city = (np.uint64(32) * u * u) >> np.uint64(32)
+    (lon_lo, lon_hi), (lat_lo, lat_hi) = SPATIAL_BOX
+    clon = np.where(city == 0, 269258, uni(10, city, lon_lo, lon_hi))
+    clat = np.where(city == 0, 5043535, uni(11, city, lat_lo, lat_hi))
+    slon = clon + uni(13, trip, -10000, 10000) + uni(19, trip, -10000, 10000)
+    slat = clat + uni(14, trip, -10000, 10000) + uni(20, trip, -10000, 10000)
+    lon = slon + j * uni(15, trip, -30, 30) + uni(17, rows, -3, 3)
+    lat = slat + j * uni(16, trip, -30, 30) + uni(18, rows, -3, 3)
+    return {"lon": np.clip(lon, lon_lo, lon_hi).astype(np.int32), "lat": np.clip(lat, lat_lo, lat_hi).astype(np.int32)}

@@ -24,6 +24,10 @@
  *  - TPC-H-lineitem-shaped Q6 columns                   (configs C2, C4, C5;
  *    value domains from PAPER.md:1294-1299, s VI-D-1: l_quantity 50 values /
  *    6 bits, l_discount 4 bits, l_shipdate 2526 values / 12 bits)
+ *  - GPS-fix-shaped (lon, lat) pairs                     (config C6, the
+ *    spatial range query of Table I, s VI-C: ~250 M
+ *    fixes from navigation devices, decimal(8,5)/(7,5) degrees, lat
+ *    27.09371..70.13643, lon -12.62427..29.64975)
  */
 #include <stdint.h>
 #include <stdlib.h>
@@ -172,4 +176,65 @@ void dg_q6(uint64_t seed, uint64_t n_parts, uint64_t row0, int64_t n,
                 dg_key(seed, S_DISCOUNT), dg_key(seed, S_PARTKEY), row0, n_parts,
                 shipdate, discount, quantity, extprice};
     parallel_for(n, threads, q6_chunk, &c);
+}
+
+/* ------------------------------------------------------------ spatial C6 */
+
+/*
+ * GPS fixes as int32 in 1e-5 degree units (decimal(8,5) / decimal(7,5) scaled),
+ * inside the paper's bounding box.  Fixes come in trips of
+ * SP_TRIP consecutive rows: trip t starts near one of SP_CITIES city centres
+ * (city = floor(SP_CITIES * u^2): a skewed, Zipf-like popularity; city 0 sits
+ * at the centre of Table I's query box), offset by a
+ * triangular U[-R,R] + U[-R,R] displacement, and moves by a constant per-fix
+ * step (dx, dy) in U[-SP_STEP, SP_STEP]^2 with U[-SP_JIT, SP_JIT] jitter on
+ * every fix.  Coordinates are clamped to the bounding box.  Row-addressable
+ * (counter-based), so every shard regenerates its own rows.
+ */
+#define SP_LON_MIN (-1262427)
+#define SP_LON_MAX 2964975
+#define SP_LAT_MIN 2709371
+#define SP_LAT_MAX 7013643
+#define SP_TRIP 128
+#define SP_CITIES 32
+#define SP_R 10000
+#define SP_STEP 30
+#define SP_JIT 3
+#define SP_BOX_LON 269258   /* centre of lon BETWEEN 2.68288 AND 2.70228 */
+#define SP_BOX_LAT 5043535  /* centre of lat BETWEEN 50.4222 AND 50.4485  */
+
+enum { S_CITY_LON = 10, S_CITY_LAT = 11, S_TRIP_CITY = 12, S_TRIP_DLON = 13, S_TRIP_DLAT = 14,
+       S_TRIP_SLON = 15, S_TRIP_SLAT = 16, S_FIX_JLON = 17, S_FIX_JLAT = 18, S_TRIP_DLON2 = 19, S_TRIP_DLAT2 = 20 };
+
+typedef struct { uint64_t seed, row0; int32_t *lon, *lat; } sp_ctx;
+
+static inline int64_t sp_uni(uint64_t seed, uint32_t stream, uint64_t row, int64_t lo, int64_t hi) {
+    return lo + (int64_t)uniform_span(draw(dg_key(seed, stream), row), (uint64_t)(hi - lo + 1));
+}
+
+static inline int64_t sp_clamp(int64_t x, int64_t lo, int64_t hi) { return x < lo ? lo : (x > hi ? hi : x); }
+
+static void sp_chunk(void* p, int64_t b, int64_t e) {
+    sp_ctx* c = (sp_ctx*)p;
+    for (int64_t i = b; i < e; ++i) {
+        uint64_t row = c->row0 + (uint64_t)i, trip = row / SP_TRIP, j = row % SP_TRIP;
+        uint64_t u = (uint64_t)uniform_span(draw(dg_key(c->seed, S_TRIP_CITY), trip), 1ull << 16);
+        uint64_t city = (SP_CITIES * u * u) >> 32;                       /* floor(C * (u/2^16)^2) */
+        int64_t clon = city == 0 ? SP_BOX_LON : sp_uni(c->seed, S_CITY_LON, city, SP_LON_MIN, SP_LON_MAX);
+        int64_t clat = city == 0 ? SP_BOX_LAT : sp_uni(c->seed, S_CITY_LAT, city, SP_LAT_MIN, SP_LAT_MAX);
+        int64_t slon = clon + sp_uni(c->seed, S_TRIP_DLON, trip, -SP_R, SP_R) + sp_uni(c->seed, S_TRIP_DLON2, trip, -SP_R, SP_R);
+        int64_t slat = clat + sp_uni(c->seed, S_TRIP_DLAT, trip, -SP_R, SP_R) + sp_uni(c->seed, S_TRIP_DLAT2, trip, -SP_R, SP_R);
+        int64_t dx = sp_uni(c->seed, S_TRIP_SLON, trip, -SP_STEP, SP_STEP);
+        int64_t dy = sp_uni(c->seed, S_TRIP_SLAT, trip, -SP_STEP, SP_STEP);
+        int64_t lon = slon + (int64_t)j * dx + sp_uni(c->seed, S_FIX_JLON, row, -SP_JIT, SP_JIT);
+        int64_t lat = slat + (int64_t)j * dy + sp_uni(c->seed, S_FIX_JLAT, row, -SP_JIT, SP_JIT);
+        if (c->lon) c->lon[i] = (int32_t)sp_clamp(lon, SP_LON_MIN, SP_LON_MAX);
+        if (c->lat) c->lat[i] = (int32_t)sp_clamp(lat, SP_LAT_MIN, SP_LAT_MAX);
+    }
+}
+
+/* GPS-fix columns (int32, 1e-5 degrees) for rows row0 .. row0+n-1; either output may be NULL. */
+void dg_spatial(uint64_t seed, uint64_t row0, int64_t n, int32_t* lon, int32_t* lat, int threads) {
+    sp_ctx c = {seed, row0, lon, lat};
+    parallel_for(n, threads, sp_chunk, &c);
 }

@@ -96,13 +96,20 @@ typedef struct {
                                   aggregate column): kernels then read it over the host link.
                                   Predicate columns must keep their majors on the device.  */
     int32_t residual_layout;   /* ar_layout of the residual part (set by the plan, see above) */
+    int32_t value_signed;      /* 1: values are int32 (two's complement).  The column is
+                                  decomposed in the order-preserving key domain
+                                  d = v ^ 0x80000000: u = d - base, and
+                                  predicate bounds of ar_pred are int32 bit patterns that
+                                  the library maps the same way.  0: uint32 values, d = v. */
+    int32_t reserved;          /* 0 */
 } ar_column_desc;
 
 typedef struct ar_column ar_column;   /* opaque: desc + part pointers (host object) */
 
 /* One conjunct lo <= value <= hi (inclusive, exact bounds; lo > hi selects nothing).
  * Operators normalise to this form: <x -> [0,x-1], >x -> [x+1,2^32-1],
- * ==x -> [x,x], between a and b -> [a,b]. */
+ * ==x -> [x,x], between a and b -> [a,b].  On a signed column lo and hi are
+ * int32 bit patterns compared in signed order. */
 typedef struct {
     const ar_column* col;
     uint32_t lo;
@@ -156,14 +163,21 @@ size_t ar_decompose_ws_bytes(void);
  * Plan a BWD decomposition of column `col` (n uint32 values, device pointer or
  * host-pinned pointer) into `major_bits` major bits and k = 32 - major_bits
  * residual bits, the split of bwdecompose(A, bits) (s V-A).
- * Computes w_major = bit length of max((v - base) >> k) (leading zeros are
- * removed) with a max-reduction kernel, then the byte sizes of
- * both parts.  SYNCHRONISES `stream` once (the sizing pass).
+ * Computes w_major = bit length of max((d - base) >> k) (leading zeros are
+ * removed) with a min/max-reduction kernel, then the byte sizes
+ * of both parts.  SYNCHRONISES `stream` once (the sizing pass).
+ * flags: AR_DECOMPOSE_SIGNED   -- int32 values (desc->value_signed);
+ *        AR_DECOMPOSE_BASE_MIN -- prefix compression with base = min(d) (the
+ *          frame of reference; `base` is ignored).
+ * `base` is in the key domain d (d = v ^ 0x80000000 for signed columns).
  * Errors: AR_ERR_INVALID if col == NULL && n > 0, n < 0, n >= 2^32,
- * major_bits outside [1,32], bad layout / location, ws too small or desc NULL.
+ * major_bits outside [1,32], bad layout / location / flags, ws too small or
+ * desc NULL; AR_ERR_RANGE if base > min(d) (a value below the base).
  */
+#define AR_DECOMPOSE_SIGNED 1
+#define AR_DECOMPOSE_BASE_MIN 2
 ar_status ar_decompose_plan(const uint32_t* col, int64_t n, int32_t major_bits,
-                            int32_t major_layout, int32_t residual_loc, uint32_t base,
+                            int32_t major_layout, int32_t residual_loc, uint32_t base, int32_t flags,
                             void* ws, size_t ws_bytes, ar_column_desc* desc, void* stream);
 
 /*
@@ -247,6 +261,41 @@ ar_status ar_refine(const ar_cands* in, const ar_pred* preds, int32_t npred, ar_
  */
 ar_status ar_sum(const ar_positions* pos, const ar_column* const* cols, int32_t ncols,
                  int64_t* out_sum_dev, void* stream);
+
+/*
+ * Approximate SUM (bwd.sumapproximate of Fig. 7): the
+ * approximate query answer from the approximation subplan alone, before any
+ * residual is read, as strict error bounds
+ * (PAPER.md:375-382).  `in` is the output of ar_approx_select; the exact
+ * result R satisfies definite <= R <= candidates, and a value with major m
+ * lies in its bucket [b + m 2^k, b + m 2^k + 2^k - 1] (clamped to 2^32 - 1).
+ * Reads only the major parts of `cols`.  Writes device int64[4]:
+ *   out4[0] = sum over definite candidates of prod_c bucket_min_c  (<= SUM(R))
+ *   out4[1] = sum over all candidates of prod_c bucket_max_c       (>= SUM(R))
+ *   out4[2] = |definite| (<= |R|),  out4[3] = |candidates| (>= |R|)
+ * ncols in [0, 2] (0: COUNT bounds only, out4[0..1] = 0).
+ * Errors: AR_ERR_INVALID (null pointers, ncols > 2), AR_ERR_RANGE as ar_sum.
+ */
+ar_status ar_sum_approximate(const ar_cands* in, const ar_column* const* cols, int32_t ncols,
+                             int64_t* out4_dev, void* stream);
+
+/*
+ * Positional projection of one column at the rows of `pos` (the invisible /
+ * positional join of the A&R plan: bwd.leftjoinapproximate and
+ * bwd.leftjoinrefine of Fig. 7; positional joins
+ * PAPER.md:537-549).  out_values[j] (device, capacity >= pos->capacity) =
+ *   AR_PROJECT_EXACT : the exact value ((major << k) | residual) + base
+ *                      (reads the residual, device or host-pinned)
+ *   AR_PROJECT_APPROX: the approximation base + (major << k), the bucket
+ *                      minimum; the exact value lies in [out, out + 2^k - 1].
+ * for j < *pos->count.  Candidate positions are projected by passing an
+ * ar_positions {cands.pos, cands.count, cands.capacity}.
+ * Errors: AR_ERR_INVALID (null pointers, bad mode).
+ */
+#define AR_PROJECT_APPROX 0
+#define AR_PROJECT_EXACT 1
+ar_status ar_project(const ar_positions* pos, const ar_column* col, int32_t mode, uint32_t* out_values,
+                     void* stream);
 
 /*
  * Fused refine + SUM (a5 + a6): the refinement of ar_refine without

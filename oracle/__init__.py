@@ -16,6 +16,8 @@ Pins (tests/test_oracle_*.py):
                   exists/forall over residuals, printed f(x) superset
   select_sum      brute force on tiny tables, closed-form sums, thread-count invariance
   sum_at          closed forms
+  sum_bounds      brute force over every residual of tiny tables, k = 0 collapse to the
+                  exact answer, closed forms, containment of the exact answer
 No function is "parity unpinned".
 """
 from __future__ import annotations
@@ -55,10 +57,12 @@ def _load():
         lib.or_decompose.restype = i32
         lib.or_bucket_flags.argtypes = [p, i64, i32, u32, u32, u32, p, p]
         lib.or_paper_f_flags.argtypes = [p, i64, i32, i32, u32, p]
-        lib.or_select_sum.argtypes = [i64, i32, p, p, p, i32, p, p, p, p, i32]
+        lib.or_select_sum.argtypes = [i64, i32, p, p, p, p, i32, p, p, p, p, i32]
         lib.or_select_sum.restype = i32
         lib.or_sum_at.argtypes = [p, i64, i32, p, p]
         lib.or_sum_at.restype = i32
+        lib.or_sum_bounds.argtypes = [i64, i32, p, p, p, p, p, i32, p, p, p, p]
+        lib.or_sum_bounds.restype = i32
         lib.or_threads_default.restype = i32
         _lib = lib
     return _lib
@@ -125,8 +129,16 @@ def approx_select(values, ks, los, his, base=None):
     return pos, dfn[pos]
 
 
-def select_sum(pred_cols, los, his, agg_cols=(), threads: int = 1, positions: bool = True):
-    """Exact select + product SUM (the plain definition): returns (positions|None, count, sum)."""
+def select_sum(pred_cols, los, his, agg_cols=(), threads: int = 1, positions: bool = True, signed=None):
+    """Exact select + product SUM (the plain definition): returns (positions|None, count, sum).
+    signed[p] true: predicate p's column (int32 array) and bounds compare as int32."""
+    sg = None
+    if signed is not None:
+        sg = np.asarray([1 if x else 0 for x in signed], dtype=np.int32)
+        pred_cols = [np.ascontiguousarray(c).view(np.uint32) if np.asarray(c).dtype == np.int32 else c
+                     for c in pred_cols]
+        los = [int(x) & 0xFFFFFFFF for x in los]
+        his = [int(x) & 0xFFFFFFFF for x in his]
     pred_cols = [_u32(c) for c in pred_cols]
     agg_cols = [_u32(c) for c in agg_cols]
     n = pred_cols[0].size if pred_cols else (agg_cols[0].size if agg_cols else 0)
@@ -137,7 +149,7 @@ def select_sum(pred_cols, los, his, agg_cols=(), threads: int = 1, positions: bo
     s = ctypes.c_int64(0)
     pc, ac = _ptr_array(pred_cols), _ptr_array(agg_cols)
     ovf = _load().or_select_sum(n, len(pred_cols), ctypes.cast(pc, ctypes.c_void_p), _ptr(lo), _ptr(hi),
-                                len(agg_cols), ctypes.cast(ac, ctypes.c_void_p),
+                                _ptr(sg) if sg is not None else None, len(agg_cols), ctypes.cast(ac, ctypes.c_void_p),
                                 _ptr(out) if positions else None, ctypes.byref(cnt), ctypes.byref(s),
                                 threads)
     if ovf:
@@ -154,3 +166,24 @@ def sum_at(pos, agg_cols):
     if _load().or_sum_at(_ptr(pos), pos.size, len(agg_cols), ctypes.cast(ac, ctypes.c_void_p), ctypes.byref(s)):
         raise OverflowError("exact SUM does not fit in int64")
     return int(s.value)
+
+
+def sum_bounds(pred_cols, pred_ks, los, his, agg_cols=(), agg_ks=(), pred_bases=None, agg_bases=None):
+    """bwd.sumapproximate (Fig. 7; bounds PAPER.md:375-382):
+    (sum_lo, sum_hi, count_lo, count_hi) from the approximation alone."""
+    pred_cols = [_u32(c) for c in pred_cols]
+    agg_cols = [_u32(c) for c in agg_cols]
+    n = pred_cols[0].size
+    npred, nagg = len(pred_cols), len(agg_cols)
+    pks = np.asarray(pred_ks, dtype=np.int32)
+    aks = np.asarray(list(agg_ks) or [0], dtype=np.int32)
+    pb = np.asarray(pred_bases if pred_bases is not None else [0] * npred, dtype=np.uint32)
+    ab = np.asarray(agg_bases if agg_bases is not None else [0] * max(nagg, 1), dtype=np.uint32)
+    lo = np.asarray(los, dtype=np.uint32)
+    hi = np.asarray(his, dtype=np.uint32)
+    out = np.zeros(4, dtype=np.int64)
+    pc, ac = _ptr_array(pred_cols), _ptr_array(agg_cols)
+    if _load().or_sum_bounds(n, npred, ctypes.cast(pc, ctypes.c_void_p), _ptr(pks), _ptr(pb), _ptr(lo), _ptr(hi),
+                             nagg, ctypes.cast(ac, ctypes.c_void_p), _ptr(aks), _ptr(ab), _ptr(out)):
+        raise OverflowError("SUM bound does not fit in int64")
+    return tuple(int(x) for x in out)

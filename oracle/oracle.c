@@ -160,6 +160,7 @@ typedef struct {
     const uint32_t* const* pcols;
     const uint32_t* lo;
     const uint32_t* hi;
+    const int* sgn;              /* per predicate: 1 = int32 column (NULL: all uint32) */
     int nagg;
     const uint32_t* const* acols;
     int64_t* out_pos;            /* may be NULL                      */
@@ -172,8 +173,13 @@ typedef struct {
 
 static int row_qualifies(const sel_ctx* c, int64_t i) {
     for (int p = 0; p < c->npred; ++p) {
-        uint32_t v = c->pcols[p][i];
-        if (!(c->lo[p] <= v && v <= c->hi[p])) return 0;
+        if (c->sgn && c->sgn[p]) {          /* signed column: compare as int32 */
+            int32_t v = (int32_t)c->pcols[p][i], lo = (int32_t)c->lo[p], hi = (int32_t)c->hi[p];
+            if (!(lo <= v && v <= hi)) return 0;
+        } else {
+            uint32_t v = c->pcols[p][i];
+            if (!(c->lo[p] <= v && v <= c->hi[p])) return 0;
+        }
     }
     return 1;
 }
@@ -208,17 +214,19 @@ static void sel_chunk(void* p, int t, int64_t b, int64_t e) {
  *   out_pos (optional): ascending positions of qualifying rows
  *   *out_count       : |R|
  *   *out_sum         : sum over R of prod_a acols[a][i]  (0 if nagg == 0)
+ * sgn (optional): sgn[p] = 1 compares predicate p's column and bounds as int32
+ * (the spatial query of Table I has signed longitudes).
  * Rows are split over `threads` contiguous chunks and chunk results are
  * concatenated / added in chunk order, so the result does not depend on T.
  * Returns 0, or 1 if the exact sum does not fit in int64.
  */
 int or_select_sum(int64_t n, int npred, const uint32_t* const* pcols,
-                  const uint32_t* lo, const uint32_t* hi,
+                  const uint32_t* lo, const uint32_t* hi, const int* sgn,
                   int nagg, const uint32_t* const* acols,
                   int64_t* out_pos, int64_t* out_count, int64_t* out_sum, int threads) {
     sel_ctx* c = (sel_ctx*)calloc(1, sizeof(sel_ctx));
     int64_t bounds[2 * OR_MAX_THREADS];
-    c->npred = npred; c->pcols = pcols; c->lo = lo; c->hi = hi;
+    c->npred = npred; c->pcols = pcols; c->lo = lo; c->hi = hi; c->sgn = sgn;
     c->nagg = nagg; c->acols = acols; c->out_pos = out_pos; c->bounds = bounds;
     c->pass = 0;
     int T = or_parallel(n, threads, sel_chunk, c, bounds);
@@ -243,4 +251,59 @@ int or_sum_at(const int64_t* pos, int64_t npos, int nagg, const uint32_t* const*
     }
     *out_sum = (int64_t)s;
     return (s > (__int128)INT64_MAX) || (s < (__int128)INT64_MIN);
+}
+
+/* ------------------------------------------- approximate answer (bounds) */
+
+/*
+ * bwd.sumapproximate (Fig. 7): the answer of the
+ * approximation subplan alone, available before any residual is read
+ * (PAPER.md:360-362, 894-897), given as strict error bounds.
+ * Each value v of a column decomposed with k residual bits and base b is only
+ * known to lie in its bucket  [b + m 2^k, b + m 2^k + 2^k - 1],  m = (v - b) >> k
+ * (the upper end clamped to 2^32 - 1).  From the candidate / definite rows of
+ * the conjunction (or_bucket_flags), since definite <= R <= cand:
+ *   out[0] = sum over definite rows of prod_a min(bucket_a)     (<= SUM over R)
+ *   out[1] = sum over candidate rows of prod_a max(bucket_a)    (>= SUM over R)
+ *   out[2] = |definite|,  out[3] = |candidates|
+ * pks/pbase: k and base of each predicate column; aks/abase: of each aggregate.
+ * Returns 1 if a bound does not fit in int64.
+ */
+int or_sum_bounds(int64_t n, int npred, const uint32_t* const* pcols, const int* pks, const uint32_t* pbase,
+                  const uint32_t* lo, const uint32_t* hi, int nagg, const uint32_t* const* acols,
+                  const int* aks, const uint32_t* abase, int64_t* out) {
+    __int128 slo = 0, shi = 0;
+    int64_t ndef = 0, ncand = 0;
+    for (int64_t i = 0; i < n; ++i) {
+        int cand = 1, def = 1;
+        for (int p = 0; p < npred; ++p) {
+            uint64_t two_k = (uint64_t)1 << pks[p];
+            uint64_t m = (uint64_t)(uint32_t)(pcols[p][i] - pbase[p]) / two_k;
+            uint64_t first = (uint64_t)pbase[p] + m * two_k;
+            uint64_t last = first + two_k - 1;
+            if (!(lo[p] <= hi[p] && first <= hi[p] && last >= lo[p])) cand = 0;
+            if (!(first >= lo[p] && last <= hi[p])) def = 0;
+        }
+        if (!cand) continue;
+        ++ncand;
+        if (def) ++ndef;
+        if (nagg == 0) continue;
+        __int128 plo = 1, phi = 1;
+        for (int a = 0; a < nagg; ++a) {
+            uint64_t two_k = (uint64_t)1 << aks[a];
+            uint64_t m = (uint64_t)(uint32_t)(acols[a][i] - abase[a]) / two_k;
+            uint64_t first = (uint64_t)abase[a] + m * two_k;
+            uint64_t last = first + two_k - 1;
+            if (last > 0xffffffffull) last = 0xffffffffull;
+            plo *= first;
+            phi *= last;
+        }
+        shi += phi;
+        if (def) slo += plo;
+    }
+    out[0] = (int64_t)slo;
+    out[1] = (int64_t)shi;
+    out[2] = ndef;
+    out[3] = ncand;
+    return shi > (__int128)INT64_MAX;
 }

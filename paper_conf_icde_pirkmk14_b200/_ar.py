@@ -17,7 +17,9 @@ AR_LOC_DEVICE, AR_LOC_HOST_PINNED = 0, 1
 AR_LAYOUT_SLICED, AR_LAYOUT_PACKED = 0, 1
 AR_MAX_PRED, AR_MAX_AGG, AR_MAX_PLANES = 8, 2, 64
 AR_SELECT_CARRY_APPR = 1
+AR_DECOMPOSE_SIGNED, AR_DECOMPOSE_BASE_MIN = 1, 2
 AR_AUX_DEFINITE = 0x80000000
+AR_PROJECT_APPROX, AR_PROJECT_EXACT = 0, 1
 
 
 class ARError(RuntimeError):
@@ -34,7 +36,8 @@ class ColumnDesc(ctypes.Structure):
     _fields_ = [("n", ctypes.c_int64), ("major_bits", ctypes.c_int32), ("k", ctypes.c_int32),
                 ("w_major", ctypes.c_int32), ("major_layout", ctypes.c_int32), ("residual_loc", ctypes.c_int32),
                 ("base", ctypes.c_uint32), ("major_bytes", ctypes.c_uint64), ("residual_bytes", ctypes.c_uint64),
-                ("major_loc", ctypes.c_int32), ("residual_layout", ctypes.c_int32)]
+                ("major_loc", ctypes.c_int32), ("residual_layout", ctypes.c_int32),
+                ("value_signed", ctypes.c_int32), ("reserved", ctypes.c_int32)]
 
 
 class Pred(ctypes.Structure):
@@ -58,7 +61,8 @@ SIGNATURES = {
     "ar_last_error": (ctypes.c_char_p, []),
     "ar_version": (ctypes.c_char_p, []),
     "ar_decompose_ws_bytes": (_SZ, []),
-    "ar_decompose_plan": (ctypes.c_int, [_P, _I64, _I32, _I32, _I32, _U32, _P, _SZ, ctypes.POINTER(ColumnDesc), _P]),
+    "ar_decompose_plan": (ctypes.c_int, [_P, _I64, _I32, _I32, _I32, _U32, _I32, _P, _SZ, ctypes.POINTER(ColumnDesc),
+                                         _P]),
     "ar_decompose": (ctypes.c_int, [_P, ctypes.POINTER(ColumnDesc), _P, _U64, _P, _U64, _P, ctypes.POINTER(_P)]),
     "ar_column_wrap": (ctypes.c_int, [ctypes.POINTER(ColumnDesc), _P, _P, ctypes.POINTER(_P)]),
     "ar_column_get_desc": (ctypes.c_int, [_P, ctypes.POINTER(ColumnDesc)]),
@@ -69,6 +73,8 @@ SIGNATURES = {
     "ar_refine": (ctypes.c_int, [ctypes.POINTER(Cands), ctypes.POINTER(Pred), _I32, ctypes.POINTER(Positions), _P,
                                  _SZ, _P]),
     "ar_sum": (ctypes.c_int, [ctypes.POINTER(Positions), ctypes.POINTER(_P), _I32, _P, _P]),
+    "ar_sum_approximate": (ctypes.c_int, [ctypes.POINTER(Cands), ctypes.POINTER(_P), _I32, _P, _P]),
+    "ar_project": (ctypes.c_int, [ctypes.POINTER(Positions), _P, _I32, _P, _P]),
     "ar_refine_sum": (ctypes.c_int, [ctypes.POINTER(Cands), ctypes.POINTER(Pred), _I32, ctypes.POINTER(_P), _I32,
                                      _P, _P, _P]),
     "ar_select_refine_sum": (ctypes.c_int, [ctypes.POINTER(Pred), _I32, ctypes.POINTER(_P), _I32, _P, _P]),
@@ -123,9 +129,10 @@ def ar_decompose_ws_bytes() -> int:
     return int(load().ar_decompose_ws_bytes())
 
 
-def ar_decompose_plan(col, n, major_bits, major_layout, residual_loc, base, ws, ws_bytes, stream) -> ColumnDesc:
+def ar_decompose_plan(col, n, major_bits, major_layout, residual_loc, base, flags, ws, ws_bytes,
+                      stream) -> ColumnDesc:
     desc = ColumnDesc()
-    _call("ar_decompose_plan", col, n, major_bits, major_layout, residual_loc, base, ws, ws_bytes,
+    _call("ar_decompose_plan", col, n, major_bits, major_layout, residual_loc, base, flags, ws, ws_bytes,
           ctypes.byref(desc), stream)
     return desc
 
@@ -183,6 +190,14 @@ def ar_refine(cands: Cands, preds, out: Positions, ws, ws_bytes, stream):
 
 def ar_sum(pos: Positions, cols, out_sum_dev, stream):
     _call("ar_sum", ctypes.byref(pos), _handles(cols), len(cols), out_sum_dev, stream)
+
+
+def ar_sum_approximate(cands: Cands, cols, out4_dev, stream):
+    _call("ar_sum_approximate", ctypes.byref(cands), _handles(cols), len(cols), out4_dev, stream)
+
+
+def ar_project(pos: Positions, col, mode, out_values_dev, stream):
+    _call("ar_project", ctypes.byref(pos), col, mode, out_values_dev, stream)
 
 
 def ar_refine_sum(cands: Cands, preds, cols, out_sum_dev, out_count_dev, stream):

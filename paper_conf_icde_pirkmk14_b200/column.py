@@ -30,17 +30,22 @@ def _nbytes_tensor(nbytes: int, device, pinned: bool = False) -> torch.Tensor:
 
 
 def as_u32_device(values, device="cuda") -> torch.Tensor:
-    """uint32 numpy array / int32 tensor -> contiguous int32 CUDA tensor holding the same bits."""
+    """uint32 / int32 numpy array or int32 tensor -> contiguous int32 CUDA tensor holding the same bits."""
     if isinstance(values, np.ndarray):
+        if values.dtype == np.int32:
+            values = values.view(np.uint32)
         values = torch.from_numpy(np.ascontiguousarray(values, dtype=np.uint32).view(np.int32))
     return values.to(device=device, dtype=torch.int32).contiguous()
 
 
 class BWDColumn:
-    """A bitwise-decomposed column (major part in HBM, residual in HBM or pinned host memory)."""
+    """A bitwise-decomposed column (major part in HBM, residual in HBM or pinned host memory).
+
+    signed=True decomposes int32 values in the order-preserving key domain v ^ 0x80000000 (predicate
+    bounds are then int32 values); base="min" is the frame-of-reference prefix base min(key)."""
 
     def __init__(self, values, major_bits: int, layout: int = AR_LAYOUT_SLICED,
-                 residual_loc: int = AR_LOC_DEVICE, base: int = 0, device="cuda", stream=None,
+                 residual_loc: int = AR_LOC_DEVICE, base=0, signed: bool = False, device="cuda", stream=None,
                  _wrap=None):
         self.device = torch.device(device)
         if _wrap is not None:
@@ -52,8 +57,9 @@ class BWDColumn:
         s = _stream(stream)
         ws = torch.empty(_ar.ar_decompose_ws_bytes(), dtype=torch.uint8, device=self.device)
         n = col.numel()
-        self.desc = _ar.ar_decompose_plan(col.data_ptr() if n else None, n, major_bits, layout, residual_loc, base,
-                                          ws.data_ptr(), ws.numel(), s)
+        flags = (_ar.AR_DECOMPOSE_SIGNED if signed else 0) | (_ar.AR_DECOMPOSE_BASE_MIN if base == "min" else 0)
+        self.desc = _ar.ar_decompose_plan(col.data_ptr() if n else None, n, major_bits, layout, residual_loc,
+                                          0 if base == "min" else int(base), flags, ws.data_ptr(), ws.numel(), s)
         self.major = _nbytes_tensor(self.desc.major_bytes, self.device)
         self.residual = _nbytes_tensor(self.desc.residual_bytes, self.device,
                                        pinned=(residual_loc == AR_LOC_HOST_PINNED))
@@ -176,6 +182,25 @@ def refine(cands: CandidateList, preds, out: PositionList, ws: Workspace, stream
 def sum_at(pos: PositionList, cols, out: torch.Tensor, stream=None):
     """Step a6: out[0] = SUM over pos of prod(cols)."""
     _ar.ar_sum(pos.p, [c.handle for c in cols], out.data_ptr(), _stream(stream))
+
+
+def sum_approximate(cands: CandidateList, cols, out4: torch.Tensor, stream=None):
+    """bwd.sumapproximate (Fig. 7): out4 = [SUM lower bound, SUM upper bound, |definite|, |candidates|]
+    from the candidate relation and the majors of `cols` only (no residual is read)."""
+    _ar.ar_sum_approximate(cands.c, [c.handle for c in cols], out4.data_ptr(), _stream(stream))
+
+
+def project(pos, col: BWDColumn, exact: bool = True, stream=None) -> torch.Tensor:
+    """bwd.leftjoinrefine (exact values) / bwd.leftjoinapproximate (bucket minima) of `col` at the rows of
+    a PositionList or CandidateList; returns a device int32 tensor (uint32 bits) of its capacity."""
+    if isinstance(pos, CandidateList):
+        p = Positions(pos.pos.data_ptr(), pos.count_t.data_ptr(), pos.c.capacity)
+    else:
+        p = pos.p
+    out = torch.empty(max(int(p.capacity), 1), dtype=torch.int32, device=col.device)
+    _ar.ar_project(p, col.handle, _ar.AR_PROJECT_EXACT if exact else _ar.AR_PROJECT_APPROX, out.data_ptr(),
+                   _stream(stream))
+    return out
 
 
 def refine_sum(cands: CandidateList, preds, cols, out_sum: torch.Tensor, out_count: torch.Tensor = None,

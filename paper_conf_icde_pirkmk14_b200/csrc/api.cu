@@ -1,6 +1,7 @@
 // api.cu -- the C ABI (include/ar.h): argument validation, relaxation of the
 // predicates (step a2, host scalars), workspace sizing and kernel launches.
 #include <algorithm>
+#include <cmath>
 #include <cstring>
 #include <new>
 
@@ -143,8 +144,8 @@ const char* ar_version(void) { return "ar-b200 0.1 (sm_100a)"; }
 size_t ar_decompose_ws_bytes(void) { return 256; }
 
 ar_status ar_decompose_plan(const uint32_t* col, int64_t n, int32_t major_bits, int32_t major_layout,
-                            int32_t residual_loc, uint32_t base, void* ws, size_t ws_bytes, ar_column_desc* desc,
-                            void* stream) {
+                            int32_t residual_loc, uint32_t base, int32_t flags, void* ws, size_t ws_bytes,
+                            ar_column_desc* desc, void* stream) {
     if (!desc || n < 0 || n >= (int64_t)1 << 32 || (n > 0 && !col)) {
         set_error("ar_decompose_plan: bad column pointer / size (n=%lld)", (long long)n);
         return AR_ERR_INVALID;
@@ -154,8 +155,10 @@ ar_status ar_decompose_plan(const uint32_t* col, int64_t n, int32_t major_bits, 
         return AR_ERR_INVALID;
     }
     if ((major_layout != AR_LAYOUT_SLICED && major_layout != AR_LAYOUT_PACKED) ||
-        (residual_loc != AR_LOC_DEVICE && residual_loc != AR_LOC_HOST_PINNED)) {
-        set_error("ar_decompose_plan: bad layout (%d) or residual location (%d)", major_layout, residual_loc);
+        (residual_loc != AR_LOC_DEVICE && residual_loc != AR_LOC_HOST_PINNED) ||
+        (flags & ~(AR_DECOMPOSE_SIGNED | AR_DECOMPOSE_BASE_MIN)) != 0) {
+        set_error("ar_decompose_plan: bad layout (%d), residual location (%d) or flags (%d)", major_layout,
+                  residual_loc, flags);
         return AR_ERR_INVALID;
     }
     if (!ws || ws_bytes < ar_decompose_ws_bytes()) {
@@ -164,14 +167,21 @@ ar_status ar_decompose_plan(const uint32_t* col, int64_t n, int32_t major_bits, 
     }
     cudaStream_t s = (cudaStream_t)stream;
     const int k = 32 - major_bits;
-    uint32_t maxu = 0;
+    const uint32_t flip = (flags & AR_DECOMPOSE_SIGNED) ? 0x80000000u : 0u;
+    uint32_t mm[2] = {0u, 0xffffffffu};   // max(d), min(d)
     if (n > 0) {
-        AR_TRY_CUDA(cudaMemsetAsync(ws, 0, 4, s));
-        ar_status st = launch_decompose_max(col, n, base, (uint32_t*)ws, s);
+        AR_TRY_CUDA(cudaMemcpyAsync(ws, mm, 8, cudaMemcpyHostToDevice, s));
+        ar_status st = launch_decompose_minmax(col, n, flip, (uint32_t*)ws, s);
         if (st != AR_OK) return st;
-        AR_TRY_CUDA(cudaMemcpyAsync(&maxu, ws, 4, cudaMemcpyDeviceToHost, s));
+        AR_TRY_CUDA(cudaMemcpyAsync(mm, ws, 8, cudaMemcpyDeviceToHost, s));
         AR_TRY_CUDA(cudaStreamSynchronize(s));
     }
+    if (flags & AR_DECOMPOSE_BASE_MIN) base = n > 0 ? mm[1] : 0u;
+    if (n > 0 && mm[1] < base) {
+        set_error("ar_decompose_plan: base %u exceeds the column minimum %u (key domain)", base, mm[1]);
+        return AR_ERR_RANGE;
+    }
+    const uint32_t maxu = n > 0 ? mm[0] - base : 0u;
     const uint32_t maxm = k >= 32 ? 0 : (maxu >> k);
     int w = 0;
     while (w < 32 && (maxm >> w) != 0) ++w;
@@ -186,6 +196,7 @@ ar_status ar_decompose_plan(const uint32_t* col, int64_t n, int32_t major_bits, 
     desc->major_bytes = major_layout == AR_LAYOUT_SLICED ? sliced_bytes(n, w) : packed_bytes(n, w);
     desc->residual_layout = (k >= 1 && k <= 8) ? AR_LAYOUT_SLICED : AR_LAYOUT_PACKED;
     desc->residual_bytes = desc->residual_layout == AR_LAYOUT_SLICED ? sliced_bytes(n, k) : packed_bytes(n, k);
+    desc->value_signed = flip ? 1 : 0;
     return AR_OK;
 }
 
@@ -195,7 +206,8 @@ static ar_status check_desc(const ar_column_desc* d) {
         (d->major_layout != AR_LAYOUT_SLICED && d->major_layout != AR_LAYOUT_PACKED) ||
         (d->residual_loc != AR_LOC_DEVICE && d->residual_loc != AR_LOC_HOST_PINNED) ||
         (d->major_loc != AR_LOC_DEVICE && d->major_loc != AR_LOC_HOST_PINNED) ||
-        (d->residual_layout != AR_LAYOUT_SLICED && d->residual_layout != AR_LAYOUT_PACKED)) {
+        (d->residual_layout != AR_LAYOUT_SLICED && d->residual_layout != AR_LAYOUT_PACKED) ||
+        (d->value_signed != 0 && d->value_signed != 1) || d->reserved != 0) {
         set_error("invalid ar_column_desc");
         return AR_ERR_INVALID;
     }
@@ -264,19 +276,21 @@ ar_status ar_decompose(const uint32_t* col, const ar_column_desc* desc, void* ma
     cudaStream_t s = (cudaStream_t)stream;
     const int64_t n = desc->n;
     const int w = desc->w_major, k = desc->k;
+    const uint32_t flip = desc->value_signed ? 0x80000000u : 0u;
     if (w > 0) {
         uint32_t* mdst = const_cast<uint32_t*>(c->major);   // device alias (mapped when host-resident)
         if (desc->major_layout == AR_LAYOUT_SLICED)
-            st = launch_pack_sliced(col, n, k, 0xffffffffu, desc->base, w, mdst, s);
+            st = launch_pack_sliced(col, n, k, 0xffffffffu, flip, desc->base, w, mdst, s);
         else
-            st = launch_pack_packed(col, n, k, 0xffffffffu, desc->base, w, desc->major_bytes / 4, mdst, s);
+            st = launch_pack_packed(col, n, k, 0xffffffffu, flip, desc->base, w, desc->major_bytes / 4, mdst, s);
     }
     if (st == AR_OK && k > 0) {
         uint32_t* rdst = const_cast<uint32_t*>(c->residual);
         if (desc->residual_layout == AR_LAYOUT_SLICED)
-            st = launch_pack_sliced(col, n, 0, (1u << k) - 1u, desc->base, k, rdst, s);
+            st = launch_pack_sliced(col, n, 0, (1u << k) - 1u, flip, desc->base, k, rdst, s);
         else
-            st = launch_pack_packed(col, n, 0, (1u << k) - 1u, desc->base, k, desc->residual_bytes / 4, rdst, s);
+            st = launch_pack_packed(col, n, 0, (1u << k) - 1u, flip, desc->base, k, desc->residual_bytes / 4, rdst,
+                                    s);
     }
     if (st != AR_OK) {
         delete c;
@@ -339,7 +353,9 @@ static ar_status setup_scan(const ar_pred* preds, int32_t npred, ard::SelParams&
             return AR_ERR_INVALID;
         }
         const int w = col->d.w_major, k = col->d.k;
-        const Relaxed R = relax(preds[c].lo, preds[c].hi, col->d.base, k, w);
+        const uint32_t flip = col->d.value_signed ? 0x80000000u : 0u;
+        const uint32_t plo = preds[c].lo ^ flip, phi = preds[c].hi ^ flip;   // key domain
+        const Relaxed R = relax(plo, phi, col->d.base, k, w);
         if (R.empty) empty = true;
         ard::SelPred& p = P.p[c];
         p.planes = col->major;
@@ -354,15 +370,28 @@ static ar_status setup_scan(const ar_pred* preds, int32_t npred, ard::SelParams&
         p.residual = col->residual;
         p.k = (uint32_t)k;
         p.base = col->d.base;
-        p.lo = preds[c].lo;
-        p.hi = preds[c].hi;
+        p.lo = plo;
+        p.hi = phi;
         p.rlayout = (uint32_t)col->d.residual_layout;
         words += (P.tile_rows / 32) * (uint32_t)w;
         ashift += (uint32_t)w;
         // the one-pass kernel streams device-resident SLICED residual tiles (k <= 8) with the
-        // majors and evaluates the exact predicate on major + residual planes in place
+        // majors and evaluates the exact predicate on major + residual planes in place -- when
+        // most 32-row blocks would need a residual gather anyway (a block's k planes are one
+        // sector).  Estimate with majors uniform over [0, 2^w): the non-definite candidate
+        // buckets (at most the two boundary ones) hold f of the rows and a block is touched with
+        // probability 1 - (1 - f)^32; stream iff that is >= 1/2 (f >= 2.14 %).
+        // AR_RES_STREAM=0/1 forces the choice.
+        bool stream_res = false;
         if (fused && k > 0 && col->d.residual_loc == AR_LOC_DEVICE && col->residual &&
-            col->d.residual_layout == AR_LAYOUT_SLICED) {
+            col->d.residual_layout == AR_LAYOUT_SLICED && !R.empty) {
+            static const int force = env_int("AR_RES_STREAM", -1);
+            const double buckets = std::ldexp(1.0, w);
+            const double nondef = (double)(R.chi - R.clo + 1) - (R.def_any ? (double)(R.dhi - R.dlo + 1) : 0.0);
+            const double f = std::min(1.0, nondef / buckets);
+            stream_res = force >= 0 ? force != 0 : (1.0 - std::pow(1.0 - f, 32.0)) >= 0.5;
+        }
+        if (stream_res) {
             p.res_stream = 1;
             p.res_soff = words;
             words += (P.tile_rows / 32) * (uint32_t)k;
@@ -486,8 +515,9 @@ static ar_status setup_refine(const ar_cands* in, const ar_pred* preds, int32_t 
         p.k = (uint32_t)col->d.k;
         p.layout = (uint32_t)col->d.major_layout;
         p.base = col->d.base;
-        p.lo = preds[c].lo;
-        p.hi = preds[c].hi;
+        const uint32_t flip = col->d.value_signed ? 0x80000000u : 0u;
+        p.lo = preds[c].lo ^ flip;   // key domain
+        p.hi = preds[c].hi ^ flip;
         p.rlayout = (uint32_t)col->d.residual_layout;
         p.ashift = ashift;
         p.carried = in->appr_bits > 0 ? 1u : 0u;
@@ -541,7 +571,7 @@ ar_status ar_refine(const ar_cands* in, const ar_pred* preds, int32_t npred, ar_
 // ------------------------------------------------------------------ a6
 
 static ar_status setup_aggs(const ar_column* const* cols, int32_t ncols, const ar_pred* preds, int32_t npred,
-                            int64_t n, ard::AggCol* a, int32_t min_cols) {
+                            int64_t n, ard::AggCol* a, int32_t min_cols, bool allow_signed = false) {
     if (ncols < min_cols || ncols > AR_MAX_AGG || (ncols > 0 && !cols)) {
         set_error("sum: ncols=%d outside [%d,%d]", ncols, min_cols, AR_MAX_AGG);
         return AR_ERR_INVALID;
@@ -560,6 +590,11 @@ static ar_status setup_aggs(const ar_column* const* cols, int32_t ncols, const a
         a[i].layout = (uint32_t)c->d.major_layout;
         a[i].base = c->d.base;
         a[i].rlayout = (uint32_t)c->d.residual_layout;
+        a[i].flip = c->d.value_signed ? 0x80000000u : 0u;
+        if (c->d.value_signed && !allow_signed) {
+            set_error("sum: aggregate column %d is signed; the unsigned product SUM does not apply", i);
+            return AR_ERR_UNSUPPORTED;
+        }
         a[i].pred = -1;
         for (int p = 0; p < npred; ++p)
             if (preds[p].col == c) { a[i].pred = p; break; }
@@ -597,6 +632,49 @@ ar_status ar_sum(const ar_positions* pos, const ar_column* const* cols, int32_t 
     if (pos->capacity <= 0) return AR_OK;
     const int grid = (int)std::min<int64_t>((pos->capacity + 255) / 256, (int64_t)num_sms() * 8);
     return launch_sum(P, grid, s);
+}
+
+ar_status ar_sum_approximate(const ar_cands* in, const ar_column* const* cols, int32_t ncols, int64_t* out4_dev,
+                             void* stream) {
+    if (!in || !in->pos || !in->aux || !in->count || !out4_dev) {
+        set_error("ar_sum_approximate: null argument");
+        return AR_ERR_INVALID;
+    }
+    ard::ApproxSumParams P;
+    memset(&P, 0, sizeof(P));
+    const int64_t n = (cols && ncols > 0 && cols[0]) ? cols[0]->d.n : -1;
+    ar_status st = setup_aggs(cols, ncols, nullptr, 0, n, P.a, 0);
+    if (st != AR_OK) return st;
+    P.pos = in->pos;
+    P.aux = in->aux;
+    P.count = (const long long*)in->count;
+    P.nagg = ncols;
+    P.out4 = (unsigned long long*)out4_dev;
+    cudaStream_t s = (cudaStream_t)stream;
+    AR_TRY_CUDA(cudaMemsetAsync(out4_dev, 0, 4 * sizeof(int64_t), s));
+    const int grid = (int)std::max<int64_t>(1, std::min<int64_t>((std::max<int64_t>(in->capacity, 0) + 255) / 256,
+                                                                 (int64_t)num_sms() * 8));
+    return launch_approx_sum(P, grid, s);
+}
+
+ar_status ar_project(const ar_positions* pos, const ar_column* col, int32_t mode, uint32_t* out_values,
+                     void* stream) {
+    if (!pos || !pos->pos || !pos->count || !out_values || !valid_col(col) ||
+        (mode != AR_PROJECT_APPROX && mode != AR_PROJECT_EXACT)) {
+        set_error("ar_project: null argument or mode %d not AR_PROJECT_APPROX/EXACT", mode);
+        return AR_ERR_INVALID;
+    }
+    ard::ProjectParams P;
+    memset(&P, 0, sizeof(P));
+    ar_status st = setup_aggs(&col, 1, nullptr, 0, -1, &P.a, 1, true);
+    if (st != AR_OK) return st;
+    P.pos = pos->pos;
+    P.count = (const long long*)pos->count;
+    P.exact = mode == AR_PROJECT_EXACT ? 1 : 0;
+    P.out = out_values;
+    if (pos->capacity <= 0) return AR_OK;
+    const int grid = (int)std::min<int64_t>((pos->capacity + 255) / 256, (int64_t)num_sms() * 8);
+    return launch_project(P, grid, (cudaStream_t)stream);
 }
 
 ar_status ar_refine_sum(const ar_cands* in, const ar_pred* preds, int32_t npred, const ar_column* const* cols,

@@ -26,6 +26,7 @@ struct AggCol {
     const uint32_t* major;
     const uint32_t* residual;
     uint32_t w, k, layout, base, rlayout;
+    uint32_t flip;            // 0x80000000 for a signed column (key domain d = v ^ flip)
     int32_t pred;             // index of the predicate over the same column, or -1
 };
 
@@ -113,6 +114,25 @@ struct SumParams {
     unsigned long long* out_sum;
 };
 
+// sumapproximate over a candidate relation (bounds from the majors only)
+struct ApproxSumParams {
+    const uint32_t* pos;
+    const uint32_t* aux;
+    const long long* count;
+    AggCol a[AR_MAX_AGG];
+    int32_t nagg;
+    unsigned long long* out4;   // [sum_lo, sum_hi, count_lo, count_hi]
+};
+
+// leftjoinapproximate / leftjoinrefine (positional projection)
+struct ProjectParams {
+    const uint32_t* pos;
+    const long long* count;
+    AggCol a;
+    int32_t exact;
+    uint32_t* out;
+};
+
 }  // namespace ard
 
 namespace ar {
@@ -127,11 +147,13 @@ ar_status launch_select_rest(const ard::SelParams& P, cudaStream_t s);
 ar_status launch_refine(const ard::RefParams& P, int grid, cudaStream_t s);
 ar_status launch_refine_sum(const ard::RefParams& P, int grid, cudaStream_t s);
 ar_status launch_sum(const ard::SumParams& P, int grid, cudaStream_t s);
-ar_status launch_decompose_max(const uint32_t* col, int64_t n, uint32_t base, uint32_t* out_max, cudaStream_t s);
-ar_status launch_pack_sliced(const uint32_t* col, int64_t n, int shift, uint32_t mask, uint32_t base, int w,
-                             uint32_t* out, cudaStream_t s);
-ar_status launch_pack_packed(const uint32_t* col, int64_t n, int shift, uint32_t mask, uint32_t base, int w,
-                             uint64_t out_words, uint32_t* out, cudaStream_t s);
+ar_status launch_approx_sum(const ard::ApproxSumParams& P, int grid, cudaStream_t s);
+ar_status launch_project(const ard::ProjectParams& P, int grid, cudaStream_t s);
+ar_status launch_decompose_minmax(const uint32_t* col, int64_t n, uint32_t flip, uint32_t* out2, cudaStream_t s);
+ar_status launch_pack_sliced(const uint32_t* col, int64_t n, int shift, uint32_t mask, uint32_t flip, uint32_t base,
+                             int w, uint32_t* out, cudaStream_t s);
+ar_status launch_pack_packed(const uint32_t* col, int64_t n, int shift, uint32_t mask, uint32_t flip, uint32_t base,
+                             int w, uint64_t out_words, uint32_t* out, cudaStream_t s);
 ar_status launch_exclusive_offset(const long long* all_counts, int world, int rank, long long* out,
                                   cudaStream_t s);
 }  // namespace ar

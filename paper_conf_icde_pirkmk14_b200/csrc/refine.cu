@@ -161,6 +161,67 @@ __global__ void __launch_bounds__(kRefThreads) sum_kernel(const __grid_constant_
     block_add(sum, P.out_sum);
 }
 
+// sumapproximate (Fig. 7 bwd.sumapproximate): the approximate
+// answer from the approximation subplan alone, before any residual is read
+// (PAPER.md:360-362, 894-897), as strict error bounds.  With
+// definite <= R <= candidates and each value in its bucket
+// [b + m 2^k, b + m 2^k + 2^k - 1]:
+//   sum_lo = sum_{definite} prod_c bucket_min_c  <=  SUM(R)  <=  sum_hi = sum_{cand} prod_c bucket_max_c
+//   count_lo = |definite| <= |R| <= count_hi = |candidates|
+__device__ __forceinline__ void bucket_bounds(const AggCol& a, uint32_t p, unsigned long long& lo,
+                                              unsigned long long& hi) {
+    const uint32_t m = a.w ? major_get(a.major, p, (int)a.w, (int)a.layout) : 0u;
+    lo = ((unsigned long long)m << a.k) + a.base;
+    hi = lo + ((1ull << a.k) - 1ull);
+    if (hi > 0xffffffffull) hi = 0xffffffffull;
+}
+
+__global__ void __launch_bounds__(kRefThreads) approx_sum_kernel(const __grid_constant__ ApproxSumParams P) {
+    const long long count = *P.count;
+    unsigned long long slo = 0, shi = 0, ndef = 0;
+    const long long stride = (long long)gridDim.x * kRefThreads;
+    for (long long j = (long long)blockIdx.x * kRefThreads + threadIdx.x; j < count; j += stride) {
+        const uint32_t pos = P.pos[j];
+        const bool def = (P.aux[j] & AR_AUX_DEFINITE) != 0;
+        ndef += def;
+        if (P.nagg > 0) {
+            unsigned long long plo = 1, phi = 1;
+            for (int c = 0; c < P.nagg; ++c) {
+                unsigned long long lo, hi;
+                bucket_bounds(P.a[c], pos, lo, hi);
+                plo *= lo;
+                phi *= hi;
+            }
+            shi += phi;
+            if (def) slo += plo;
+        }
+    }
+    block_add(slo, &P.out4[0]);
+    block_add(shi, &P.out4[1]);
+    block_add(ndef, &P.out4[2]);
+    if (blockIdx.x == 0 && threadIdx.x == 0) P.out4[3] = (unsigned long long)count;
+}
+
+// Positional projection (Fig. 7 bwd.leftjoinapproximate / bwd.leftjoinrefine,
+// PAPER.md:884-889; invisible join on positions):
+// out[j] = value of column a at row pos[j] -- exact ((major << k) | residual) + b,
+// or its approximation b + (major << k) (the bucket minimum; error in [0, 2^k - 1]).
+__global__ void __launch_bounds__(kRefThreads) project_kernel(const __grid_constant__ ProjectParams P) {
+    const long long count = *P.count;
+    const long long stride = (long long)gridDim.x * kRefThreads;
+    for (long long j = (long long)blockIdx.x * kRefThreads + threadIdx.x; j < count; j += stride) {
+        const uint32_t p = P.pos[j];
+        uint32_t v;
+        if (P.exact) {
+            v = agg_gather(P.a, p);
+        } else {
+            const uint32_t m = P.a.w ? major_get(P.a.major, p, (int)P.a.w, (int)P.a.layout) : 0u;
+            v = (m << P.a.k) + P.a.base;
+        }
+        P.out[j] = v ^ P.a.flip;   // back from the key domain of a signed column
+    }
+}
+
 __global__ void exclusive_offset_kernel(const long long* all, int world, int rank, long long* out) {
     long long s = 0;
     for (int r = 0; r < rank && r < world; ++r) s += all[r];
@@ -184,6 +245,16 @@ ar_status launch_refine_sum(const ard::RefParams& P, int grid, cudaStream_t s) {
 ar_status launch_sum(const ard::SumParams& P, int grid, cudaStream_t s) {
     ard::sum_kernel<<<grid, ard::kRefThreads, 0, s>>>(P);
     AR_CHECK_LAUNCH("sum_kernel");
+    return AR_OK;
+}
+ar_status launch_approx_sum(const ard::ApproxSumParams& P, int grid, cudaStream_t s) {
+    ard::approx_sum_kernel<<<grid, ard::kRefThreads, 0, s>>>(P);
+    AR_CHECK_LAUNCH("approx_sum_kernel");
+    return AR_OK;
+}
+ar_status launch_project(const ard::ProjectParams& P, int grid, cudaStream_t s) {
+    ard::project_kernel<<<grid, ard::kRefThreads, 0, s>>>(P);
+    AR_CHECK_LAUNCH("project_kernel");
     return AR_OK;
 }
 ar_status launch_exclusive_offset(const long long* all_counts, int world, int rank, long long* out,

@@ -58,17 +58,17 @@ def test_host_only_entry_points():
     assert _ar.ar_select_ws_bytes(4096) >= 8 * 4096 and _ar.ar_select_ws_bytes(4097) >= 8 * 4097
     assert _ar.ar_refine_ws_bytes(2048) == 16 + 8
     assert _ar.ar_dist_unique_id_bytes() == 128
-    assert ctypes.sizeof(_ar.ColumnDesc) == 56
+    assert ctypes.sizeof(_ar.ColumnDesc) == 64
 
 
 def test_host_validation_without_gpu():
     from paper_conf_icde_pirkmk14_b200 import _ar
     import pytest
     with pytest.raises(_ar.ARError) as e:
-        _ar.ar_decompose_plan(None, 10, 24, 0, 0, 0, None, 0, None)
+        _ar.ar_decompose_plan(None, 10, 24, 0, 0, 0, 0, None, 0, None)
     assert e.value.status == _ar.AR_ERR_INVALID
     with pytest.raises(_ar.ARError) as e:
-        _ar.ar_decompose_plan(None, 0, 33, 0, 0, 0, None, 0, None)
+        _ar.ar_decompose_plan(None, 0, 33, 0, 0, 0, 0, None, 0, None)
     assert e.value.status == _ar.AR_ERR_INVALID
     with pytest.raises(_ar.ARError) as e:
         _ar.ar_approx_select([], 0, _ar.Cands(), None, 0, None)

@@ -74,3 +74,25 @@ def test_q6_selectivity_closed_form():
     cpos, cdef = oracle.approx_select(cols, [8, 0, 0], los, his)
     assert _within_5sigma(cpos.size, n, 768 / 2406 * 3 / 11 * 23 / 50)   # 4.00 %
     assert _within_5sigma(int(cdef.sum()), n, 256 / 2406 * 3 / 11 * 23 / 50)  # 1.33 %
+
+
+def test_spatial_c_matches_numpy():
+    for row0 in (0, 1_000_003):
+        c = datagen.spatial_columns(6, 50_000, row0=row0)
+        m = datagen.spatial_columns_np(6, 50_000, row0=row0)
+        assert np.array_equal(c["lon"], m["lon"]) and np.array_equal(c["lat"], m["lat"])
+
+
+def test_spatial_shape():
+    # inside the paper's bounding box; trips of 128 fixes; the Table I query
+    # box holds a small, non-empty fraction of the fixes
+    c = datagen.spatial_columns(6, 2_000_000)
+    (lon_lo, lon_hi), (lat_lo, lat_hi) = datagen.SPATIAL_BOX
+    assert c["lon"].min() >= lon_lo and c["lon"].max() <= lon_hi and c["lon"].min() < 0 < c["lon"].max()
+    assert c["lat"].min() >= lat_lo and c["lat"].max() <= lat_hi
+    hit = ((c["lon"] >= datagen.SPATIAL_LON[0]) & (c["lon"] <= datagen.SPATIAL_LON[1])
+           & (c["lat"] >= datagen.SPATIAL_LAT[0]) & (c["lat"] <= datagen.SPATIAL_LAT[1]))
+    assert 1e-4 < hit.mean() < 1e-2
+    # consecutive fixes of one trip move by at most step + jitter
+    d = np.abs(np.diff(c["lon"][:128].astype(np.int64)))
+    assert d.max() <= 30 + 6

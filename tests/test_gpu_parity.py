@@ -168,7 +168,8 @@ def test_gpu_select_base(cu):
 
 # ------------------------------------------------------------------- a5 refine
 
-def check_refine_and_sums(cu, values, ks, los, his, agg_values, agg_layouts, carry=True, loc=0):
+def check_refine_and_sums(cu, values, ks, los, his, agg_values, agg_layouts, carry=True, loc=0, agg_ks=None,
+                          agg_loc=0):
     from paper_conf_icde_pirkmk14_b200 import _ar
     cols = [_col(cu, v, 32 - k, loc=loc) for v, k in zip(values, ks)]
     n = cols[0].n
@@ -182,10 +183,12 @@ def check_refine_and_sums(cu, values, ks, los, his, agg_values, agg_layouts, car
     assert out.count() == ref_cnt
     assert np.array_equal(out.positions(), ref_pos)
     # aggregate columns: reuse a predicate column object when it is the same data
-    aggs = []
-    for av, lay in zip(agg_values, agg_layouts):
-        same = [c for c, v in zip(cols, values) if v is av]
-        aggs.append(same[0] if same else _col(cu, av, 32, layout=lay))
+    aggs, aks = [], []
+    agg_ks = agg_ks or [0] * len(agg_values)
+    for av, lay, ak in zip(agg_values, agg_layouts, agg_ks):
+        same = [(c, k) for c, v, k in zip(cols, values, ks) if v is av]
+        aggs.append(same[0][0] if same else _col(cu, av, 32 - ak, layout=lay, loc=agg_loc))
+        aks.append(same[0][1] if same else ak)
     ref_sum = oracle.sum_at(ref_pos, agg_values)
     s = torch.zeros(1, dtype=torch.int64, device="cuda")
     cu.sum_at(out, aggs, s)
@@ -199,6 +202,13 @@ def check_refine_and_sums(cu, values, ks, los, his, agg_values, agg_layouts, car
     assert int(s2.item()) == ref_sum and int(c2.item()) == ref_cnt
     cpos, cdef = oracle.approx_select(values, ks, los, his)
     assert o4.cpu().tolist() == [ref_sum, ref_cnt, cpos.size, int(cdef.sum())]
+    # bwd.sumapproximate: bounds from the candidates and the majors only
+    b4 = torch.zeros(4, dtype=torch.int64, device="cuda")
+    cu.sum_approximate(cands, aggs, b4)
+    torch.cuda.synchronize()
+    ref_b = oracle.sum_bounds(values, ks, los, his, agg_values, aks)
+    assert tuple(b4.cpu().tolist()) == ref_b
+    assert ref_b[0] <= ref_sum <= ref_b[1] and ref_b[2] <= ref_cnt <= ref_b[3]
     return ref_cnt, ref_sum
 
 
@@ -232,6 +242,69 @@ def test_gpu_q6_host_pinned_residual(cu):
     los = [datagen.Q6_SHIPDATE[0], datagen.Q6_DISCOUNT[0], datagen.Q6_QUANTITY[0]]
     his = [datagen.Q6_SHIPDATE[1], datagen.Q6_DISCOUNT[1], datagen.Q6_QUANTITY[1]]
     check_refine_and_sums(cu, values, [8, 0, 0], los, his, [c["extprice"], c["discount"]], [1, 0], loc=1)
+
+
+@pytest.mark.parametrize("agg_loc", [0, 1])
+@pytest.mark.parametrize("ep_k", [4, 8, 12])
+def test_gpu_q6_decomposed_extprice(cu, ep_k, agg_loc):
+    # the aggregate column itself is decomposed (residual in HBM or pinned host
+    # memory); SUM(refine) rebuilds ((major << k) | residual) before multiplying
+    c = datagen.q6_columns(12, 0.3)
+    values = [c["shipdate"], c["discount"], c["quantity"]]
+    los = [datagen.Q6_SHIPDATE[0], datagen.Q6_DISCOUNT[0], datagen.Q6_QUANTITY[0]]
+    his = [datagen.Q6_SHIPDATE[1], datagen.Q6_DISCOUNT[1], datagen.Q6_QUANTITY[1]]
+    for lay in (0, 1):
+        check_refine_and_sums(cu, values, [8, 0, 0], los, his, [c["extprice"], c["discount"]], [lay, 0],
+                              agg_ks=[ep_k, 0], agg_loc=agg_loc)
+
+
+def test_gpu_sum_approximate_edges(cu):
+    from paper_conf_icde_pirkmk14_b200 import _ar
+    v = datagen.uniform_u32(21, 50_001)
+    col = _col(cu, v, 24)
+    # empty candidate relation: all bounds 0
+    cands = run_select(cu, [col], [10], [5])
+    b4 = torch.full((4,), -1, dtype=torch.int64, device="cuda")
+    cu.sum_approximate(cands, [col], b4)
+    torch.cuda.synchronize()
+    assert b4.cpu().tolist() == [0, 0, 0, 0]
+    # COUNT only (ncols = 0)
+    cands = run_select(cu, [col], [datagen.C1_LO], [datagen.C1_HI])
+    cu.sum_approximate(cands, [], b4)
+    torch.cuda.synchronize()
+    pos, dfn = oracle.approx_select([v], [8], [datagen.C1_LO], [datagen.C1_HI])
+    assert b4.cpu().tolist() == [0, 0, int(dfn.sum()), pos.size]
+    with pytest.raises(_ar.ARError):
+        cu.sum_approximate(cands, [col, col, col], b4)
+
+
+@pytest.mark.parametrize("k,loc,lay", [(0, 0, 1), (8, 0, 0), (8, 1, 1), (12, 0, 1), (20, 1, 0)])
+def test_gpu_project(cu, k, loc, lay):
+    # positional projection of the exact value (leftjoinrefine) and of the approximation
+    # (leftjoinapproximate) at candidate and at refined positions
+    v = datagen.uniform_u32(30 + k, 200_003, 1_000, 2**31)
+    base = 1_000 if k == 12 else 0
+    col = cu.BWDColumn(v, 32 - k, layout=lay, residual_loc=loc, base=base)
+    sel = _col(cu, v, 24)
+    lo, hi = 2**30, 2**30 + 2**27
+    cands = run_select(cu, [sel], [lo], [hi])
+    n = cands.count()
+    ex = cu.project(cands, col, exact=True)
+    ap = cu.project(cands, col, exact=False)
+    torch.cuda.synchronize()
+    pos = cands.positions()
+    assert n > 1000
+    assert np.array_equal(ex[:n].cpu().numpy().view(np.uint32), v[pos])
+    major, _, _ = oracle.decompose(v, k, base)
+    want = ((major[pos].astype(np.uint64) << k) + base).astype(np.uint32)
+    assert np.array_equal(ap[:n].cpu().numpy().view(np.uint32), want)
+    out = cu.PositionList(sel.n)
+    from paper_conf_icde_pirkmk14_b200 import _ar
+    cu.refine(cands, [(sel, lo, hi)], out, cu.Workspace(_ar.ar_refine_ws_bytes(sel.n)))
+    ex2 = cu.project(out, col, exact=True)
+    torch.cuda.synchronize()
+    m = out.count()
+    assert np.array_equal(ex2[:m].cpu().numpy().view(np.uint32), v[out.positions()])
 
 
 def test_gpu_sum_closed_form(cu):

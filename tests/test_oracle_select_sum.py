@@ -95,3 +95,24 @@ def test_sum_overflow_detected():
     a = np.full(4, 2**32 - 1, dtype=np.uint32)
     with pytest.raises(OverflowError):
         oracle.select_sum([a], [0], [2**32 - 1], [a, a])
+
+
+@pytest.mark.parametrize("seed", range(6))
+def test_select_signed_bruteforce_tiny(seed):
+    # int32 columns with int32 bounds (Table I longitudes are negative)
+    rng = np.random.default_rng(50 + seed)
+    n = int(rng.integers(0, 80))
+    a = rng.integers(-2**31, 2**31, n, dtype=np.int64).astype(np.int32)
+    b = rng.integers(-300, 300, n).astype(np.int32)
+    lo_a, hi_a = sorted(rng.integers(-2**31, 2**31, 2, dtype=np.int64).tolist())
+    lo_b, hi_b = sorted(rng.integers(-300, 300, 2).tolist())
+    pos, cnt, _ = oracle.select_sum([a, b], [lo_a, lo_b], [hi_a, hi_b], signed=[True, True])
+    want = [i for i in range(n) if lo_a <= int(a[i]) <= hi_a and lo_b <= int(b[i]) <= hi_b]
+    assert pos.tolist() == want and cnt == len(want)
+
+
+def test_select_signed_spans_zero():
+    # [-5, 5] on int32: unsigned order would select nothing of the negatives
+    v = np.array([-7, -5, -1, 0, 4, 5, 6, -2**31, 2**31 - 1], dtype=np.int32)
+    pos, cnt, _ = oracle.select_sum([v], [-5], [5], signed=[True])
+    assert pos.tolist() == [1, 2, 3, 4, 5]
