@@ -153,6 +153,11 @@ typedef struct {
 const char* ar_status_str(ar_status s);
 const char* ar_last_error(void);     /* thread-local detail of the last failure */
 const char* ar_version(void);
+/* Name of the kernel the calling thread's last ar_select_refine_sum launched
+ * ("fused_rl_kernel" = the result-ring one-pass kernel, "fused_kernel" = the
+ * general one-pass kernel, "" = none: empty input or an error).  Static
+ * storage; for tests and benchmarks that must know which path ran. */
+const char* ar_last_scan_kernel(void);
 
 /* --------------------------------------------------- a1: decomposition */
 

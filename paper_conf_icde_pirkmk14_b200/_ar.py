@@ -60,6 +60,7 @@ SIGNATURES = {
     "ar_status_str": (ctypes.c_char_p, [ctypes.c_int]),
     "ar_last_error": (ctypes.c_char_p, []),
     "ar_version": (ctypes.c_char_p, []),
+    "ar_last_scan_kernel": (ctypes.c_char_p, []),
     "ar_decompose_ws_bytes": (_SZ, []),
     "ar_decompose_plan": (ctypes.c_int, [_P, _I64, _I32, _I32, _I32, _U32, _I32, _P, _SZ, ctypes.POINTER(ColumnDesc),
                                          _P]),
@@ -123,6 +124,10 @@ def _call(name, *args):
 
 def ar_version() -> str:
     return load().ar_version().decode()
+
+
+def ar_last_scan_kernel() -> str:
+    return load().ar_last_scan_kernel().decode()
 
 
 def ar_decompose_ws_bytes() -> int:

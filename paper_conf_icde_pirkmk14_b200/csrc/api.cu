@@ -138,6 +138,8 @@ const char* ar_status_str(ar_status s) {
 
 const char* ar_last_error(void) { return g_err.c_str(); }
 const char* ar_version(void) { return "ar-b200 0.1 (sm_100a)"; }
+static thread_local const char* g_last_scan = "";
+const char* ar_last_scan_kernel(void) { return g_last_scan; }
 
 // ------------------------------------------------------------------ a1
 
@@ -424,8 +426,9 @@ static ar_status setup_scan(const ar_pred* preds, int32_t npred, ard::SelParams&
             uint32_t* m = P.pm[p.ashift + j];
             m[0] = 0u - ((p.clo >> j) & 1u);
             m[1] = 0u - ((p.chi >> j) & 1u);
-            m[2] = 0u - ((p.dlo >> j) & 1u);
-            m[3] = 0u - ((p.dhi >> j) & 1u);
+            // mode 2 (no definite bucket): an empty definite range, lo = 2^w - 1 > hi = 0
+            m[2] = p.mode == 2 ? ~0u : 0u - ((p.dlo >> j) & 1u);
+            m[3] = p.mode == 2 ? 0u : 0u - ((p.dhi >> j) & 1u);
         }
     }
     P.npred = npred;
@@ -734,7 +737,16 @@ ar_status ar_select_refine_sum(const ar_pred* preds, int32_t npred, const ar_col
     }
     cudaStream_t s = (cudaStream_t)stream;
     AR_TRY_CUDA(cudaMemsetAsync(out_dev, 0, 4 * sizeof(int64_t), s));
+    g_last_scan = "";
     if (empty || n == 0) return AR_OK;
+    bool launched = false;   // the result-ring kernel (fused.cu) where it applies
+    st = launch_fused_rl(P, cols, &launched, s);
+    if (st != AR_OK) return st;
+    if (launched) {
+        g_last_scan = "fused_rl_kernel";
+        return AR_OK;
+    }
+    g_last_scan = "fused_kernel";
     int occ = 1;
     const void* fn = select_kernel_fn(P, true);
     P.nstages = pick_stages(fn, P.stage_words, true, &occ);

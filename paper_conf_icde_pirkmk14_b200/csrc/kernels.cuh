@@ -75,7 +75,58 @@ struct SelParams {
     int32_t async_agg;            // fused: the one gathered aggregate column uses asynchronous gathers
     int32_t gidx;                 // index of that column in a[]
     unsigned long long* out4;     // sum, |result|, |cand|, |def|
+    // result-ring kernel (fused.cu) only
+    int32_t rl_list;              // 1: one gathered SUM factor, rows queued in the warp result ring
+    int32_t rl_mpred;             // predicate whose exact value is the other SUM factor, or -1
+    uint32_t rl_ring;             // result-ring entries per warp (power of two)
 };
+
+// Producer of the persistent scan kernels: one lane streams tiles (tile =
+// blockIdx + i * gridDim) of every predicate's bit planes -- and, for streamed
+// predicates, the tile's SLICED residual planes -- into a ring of nstages
+// shared-memory stages with 1-D TMA bulk copies completing on full[s].  A tile
+// index past the end is passed on as -1 and ends the stream.
+__device__ __forceinline__ void produce_ring(const SelParams& P, uint64_t* full, uint64_t* empty, long long* slot,
+                                             uint32_t* stages) {
+    const uint64_t pol = policy_evict_first();
+    const uint32_t blocks_per_tile = P.tile_rows / 32;
+    uint32_t s = 0, ph = 0;   // ring slot and its phase parity (no integer division in the loop)
+    for (uint32_t i = 0;; ++i) {
+        if (i >= P.nstages) mbar_wait_sleep(empty + s, ph ^ 1u);   // producer backs off instead of spinning
+        const long long t = (long long)blockIdx.x + (long long)i * gridDim.x;
+        if (t >= P.num_tiles) {
+            slot[s] = -1;
+            mbar_arrive(full + s);
+            return;
+        }
+        slot[s] = t;
+        const int64_t r0 = t * (int64_t)P.tile_rows;
+        const int64_t rows = min((int64_t)P.tile_rows, P.n - r0);
+        const uint32_t groups = (uint32_t)((rows + 127) / 128);   // 128-row groups, 16 B per plane
+        uint32_t bytes = 0;
+        for (int c = 0; c < P.npred; ++c) {
+            bytes += groups * 16u * P.p[c].w;
+            if (P.p[c].res_stream) bytes += groups * 16u * P.p[c].k;
+        }
+        mbar_arrive_expect_tx(full + s, bytes);
+        uint32_t* stg = stages + (size_t)s * P.stage_words;
+        for (int c = 0; c < P.npred; ++c) {
+            const uint32_t w = P.p[c].w;
+            if (w > 0)
+                bulk_g2s(stg + P.p[c].soff, P.p[c].planes + (size_t)t * blocks_per_tile * w, groups * 16u * w,
+                         full + s, pol);
+            if (P.p[c].res_stream) {   // the tile's SLICED residual planes
+                const uint32_t k = P.p[c].k;
+                bulk_g2s(stg + P.p[c].res_soff, P.p[c].residual + (size_t)t * blocks_per_tile * k,
+                         groups * 16u * k, full + s, pol);
+            }
+        }
+        if (++s == P.nstages) {
+            s = 0;
+            ph ^= 1u;
+        }
+    }
+}
 
 struct RefPred {
     const uint32_t* major;
@@ -144,6 +195,7 @@ const void* select_kernel_fn(const ard::SelParams& P, bool fused);
 int select_occupancy(const void* fn, size_t smem, bool fused);
 ar_status launch_scan(const void* fn, const ard::SelParams& P, int grid, size_t smem, bool fused, cudaStream_t s);
 ar_status launch_select_rest(const ard::SelParams& P, cudaStream_t s);
+ar_status launch_fused_rl(const ard::SelParams& P, const ar_column* const* cols, bool* launched, cudaStream_t s);
 ar_status launch_refine(const ard::RefParams& P, int grid, cudaStream_t s);
 ar_status launch_refine_sum(const ard::RefParams& P, int grid, cudaStream_t s);
 ar_status launch_sum(const ard::SumParams& P, int grid, cudaStream_t s);

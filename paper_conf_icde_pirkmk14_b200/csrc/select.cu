@@ -390,48 +390,9 @@ __device__ __forceinline__ SmemLayout carve(unsigned char* smem, uint32_t nstage
     return L;
 }
 
-// Producer: one lane streams tiles (tile = blockIdx + i * gridDim) into the
-// stage ring; a tile index past the end is passed on as -1 and ends the stream.
+// Producer: produce_ring (kernels.cuh) over this kernel's shared-memory carve-up.
 __device__ __forceinline__ void produce(const SelParams& P, const SmemLayout& L) {
-    const uint64_t pol = policy_evict_first();
-    const uint32_t blocks_per_tile = P.tile_rows / 32;
-    uint32_t s = 0, ph = 0;   // ring slot and its phase parity (no integer division in the loop)
-    for (uint32_t i = 0;; ++i) {
-        if (i >= P.nstages) mbar_wait_sleep(L.empty + s, ph ^ 1u);   // producer backs off instead of spinning
-        const long long t = (long long)blockIdx.x + (long long)i * gridDim.x;
-        if (t >= P.num_tiles) {
-            L.slot[s] = -1;
-            mbar_arrive(L.full + s);
-            return;
-        }
-        L.slot[s] = t;
-        const int64_t r0 = t * (int64_t)P.tile_rows;
-        const int64_t rows = min((int64_t)P.tile_rows, P.n - r0);
-        const uint32_t groups = (uint32_t)((rows + 127) / 128);   // 128-row groups, 16 B per plane
-        uint32_t bytes = 0;
-        for (int c = 0; c < P.npred; ++c) {
-            bytes += groups * 16u * P.p[c].w;
-            if (P.p[c].res_stream) bytes += groups * 16u * P.p[c].k;
-        }
-        mbar_arrive_expect_tx(L.full + s, bytes);
-        uint32_t* stg = L.stages + (size_t)s * P.stage_words;
-        for (int c = 0; c < P.npred; ++c) {
-            const uint32_t w = P.p[c].w;
-            if (w > 0) {
-                const uint32_t* src = P.p[c].planes + (size_t)t * blocks_per_tile * w;
-                bulk_g2s(stg + P.p[c].soff, src, groups * 16u * w, L.full + s, pol);
-            }
-            if (P.p[c].res_stream) {   // the tile's SLICED residual planes
-                const uint32_t k = P.p[c].k;
-                const uint32_t* src = P.p[c].residual + (size_t)t * (P.tile_rows / 32) * k;
-                bulk_g2s(stg + P.p[c].res_soff, src, groups * 16u * k, L.full + s, pol);
-            }
-        }
-        if (++s == P.nstages) {
-            s = 0;
-            ph ^= 1u;
-        }
-    }
+    produce_ring(P, L.full, L.empty, L.slot, L.stages);
 }
 
 template <int NW>

@@ -1,0 +1,140 @@
+"""GPU parity of the one-pass result-ring kernel (fused.cu, ar_select_refine_sum
+with the exact predicate on streamed residual planes) against the CPU oracle:
+ragged tails, every SUM-factor mode (COUNT only, predicate-column factors,
+one gathered column with and without a second factor), ring overflow at high
+selectivity, and every (warps, blocks-per-thread) configuration plus the
+general kernel in subprocesses (the kernel choice is read from the
+environment once per process)."""
+import os
+import subprocess
+import sys
+
+import numpy as np
+import pytest
+
+import datagen
+import oracle
+
+pytestmark = pytest.mark.gpu
+torch = pytest.importorskip("torch")
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+
+
+@pytest.fixture(scope="module")
+def cu():
+    if not torch.cuda.is_available():
+        pytest.skip("no CUDA device")
+    from paper_conf_icde_pirkmk14_b200 import column
+    return column
+
+
+def q6(cu, seed, n, bounds=None):
+    from paper_conf_icde_pirkmk14_b200 import _ar
+    c = datagen.q6_columns(seed, 1.0, n=n)
+    los = [datagen.Q6_SHIPDATE[0], datagen.Q6_DISCOUNT[0], datagen.Q6_QUANTITY[0]]
+    his = [datagen.Q6_SHIPDATE[1], datagen.Q6_DISCOUNT[1], datagen.Q6_QUANTITY[1]]
+    if bounds:
+        los, his = [b[0] for b in bounds], [b[1] for b in bounds]
+    cols = {"shipdate": cu.BWDColumn(c["shipdate"], 24), "discount": cu.BWDColumn(c["discount"], 32),
+            "quantity": cu.BWDColumn(c["quantity"], 32),
+            "extprice": cu.BWDColumn(c["extprice"], 32, layout=_ar.AR_LAYOUT_PACKED)}
+    return c, cols, los, his
+
+
+def run(cu, c, cols, los, his, aggs):
+    from paper_conf_icde_pirkmk14_b200 import _ar
+    preds = [(cols["shipdate"], los[0], his[0]), (cols["discount"], los[1], his[1]),
+             (cols["quantity"], los[2], his[2])]
+    o4 = torch.zeros(4, dtype=torch.int64, device="cuda")
+    cu.select_refine_sum(preds, [cols[a] for a in aggs], o4)
+    torch.cuda.synchronize()
+    kernel = _ar.ar_last_scan_kernel()
+    values = [c["shipdate"], c["discount"], c["quantity"]]
+    _, ref_cnt, ref_sum = oracle.select_sum(values, los, his, [c[a] for a in aggs], positions=False)
+    cpos, cdef = oracle.approx_select(values, [8, 0, 0], los, his)
+    assert o4.cpu().tolist() == [ref_sum if aggs else 0, ref_cnt, cpos.size, int(cdef.sum())]
+    return kernel, ref_cnt
+
+
+@pytest.mark.parametrize("n", [1, 31, 8191, 8192, 8193, 3 * 8192 + 127, 300_001])
+@pytest.mark.parametrize("aggs", [("extprice", "discount"), ("extprice",), (), ("discount",),
+                                  ("discount", "quantity")])
+def test_rl_q6_modes_and_tails(cu, n, aggs):
+    c, cols, los, his = q6(cu, 40 + n % 97, n)
+    kernel, _ = run(cu, c, cols, los, his, list(aggs))
+    if n >= 8192:
+        assert kernel == "fused_rl_kernel"
+
+
+@pytest.mark.parametrize("aggs", [("extprice", "discount"), ("extprice", "quantity")])
+def test_rl_ring_overflow(cu, aggs):
+    # unaligned shipdate bounds keep both boundary buckets (12.5 % of the 16 majors) non-definite,
+    # so the residual planes stream; nearly every row qualifies, so each warp's share of a tile
+    # overflows the 256-entry result ring many times over
+    c, cols, los, his = q6(cu, 7, 200_000, bounds=[(3, 2523), (0, 10), (1, 50)])
+    kernel, cnt = run(cu, c, cols, los, his, list(aggs))
+    assert kernel == "fused_rl_kernel" and cnt > 190_000
+
+
+def test_rl_single_column_c1(cu):
+    v = datagen.uniform_u32(1, datagen.C1_N)
+    col = cu.BWDColumn(v, 24)
+    # a 25 %-wide range: the two boundary buckets are non-definite, residual planes stream (AR_RES_STREAM
+    # heuristics: forced on by the subprocess sweep below for the narrow C1 range)
+    lo, hi = 0x12345678, 0x12345678 + (1 << 30)
+    o4 = torch.zeros(4, dtype=torch.int64, device="cuda")
+    cu.select_refine_sum([(col, lo, hi)], [col], o4)
+    torch.cuda.synchronize()
+    _, cnt, s = oracle.select_sum([v], [lo], [hi], [v], positions=False)
+    cpos, cdef = oracle.approx_select([v], [8], [lo], [hi])
+    assert o4.cpu().tolist() == [s, cnt, cpos.size, int(cdef.sum())]
+
+
+SWEEP = r"""
+import sys, numpy as np, torch
+sys.path.insert(0, {root!r})
+import datagen, oracle
+from paper_conf_icde_pirkmk14_b200 import _ar, column as cu
+want = sys.argv[1]
+for seed, n, bounds in [(3, 100_003, None), (4, 70_001, [(3, 2523), (0, 10), (1, 50)])]:
+    c = datagen.q6_columns(seed, 1.0, n=n)
+    los = [datagen.Q6_SHIPDATE[0], datagen.Q6_DISCOUNT[0], datagen.Q6_QUANTITY[0]]
+    his = [datagen.Q6_SHIPDATE[1], datagen.Q6_DISCOUNT[1], datagen.Q6_QUANTITY[1]]
+    if bounds:
+        los, his = [b[0] for b in bounds], [b[1] for b in bounds]
+    sd, dc, qt = cu.BWDColumn(c["shipdate"], 24), cu.BWDColumn(c["discount"], 32), cu.BWDColumn(c["quantity"], 32)
+    ep = cu.BWDColumn(c["extprice"], 32, layout=_ar.AR_LAYOUT_PACKED)
+    preds = [(sd, los[0], his[0]), (dc, los[1], his[1]), (qt, los[2], his[2])]
+    vals = [c["shipdate"], c["discount"], c["quantity"]]
+    cpos, cdef = oracle.approx_select(vals, [8, 0, 0], los, his)
+    for aggs in ([ep, dc], [ep], []):
+        o4 = torch.zeros(4, dtype=torch.int64, device="cuda")
+        cu.select_refine_sum(preds, aggs, o4)
+        torch.cuda.synchronize()
+        assert _ar.ar_last_scan_kernel() == want, (_ar.ar_last_scan_kernel(), want)
+        av = [c["extprice"], c["discount"]][:len(aggs)]
+        _, cnt, s = oracle.select_sum(vals, los, his, av, positions=False)
+        assert o4.cpu().tolist() == [s if aggs else 0, cnt, cpos.size, int(cdef.sum())], (o4.tolist(), s, cnt)
+# C1: narrow range, residual streaming forced on
+v = datagen.uniform_u32(1, datagen.C1_N)
+col = cu.BWDColumn(v, 24)
+o4 = torch.zeros(4, dtype=torch.int64, device="cuda")
+cu.select_refine_sum([(col, datagen.C1_LO, datagen.C1_HI)], [col], o4)
+torch.cuda.synchronize()
+assert _ar.ar_last_scan_kernel() == want
+_, cnt, s = oracle.select_sum([v], [datagen.C1_LO], [datagen.C1_HI], [v], positions=False)
+cpos, cdef = oracle.approx_select([v], [8], [datagen.C1_LO], [datagen.C1_HI])
+assert o4.cpu().tolist() == [s, cnt, cpos.size, int(cdef.sum())]
+print("ok")
+"""
+
+
+@pytest.mark.parametrize("env,want", [({"AR_RL_CFG": "0"}, "fused_rl_kernel"),
+                                      ({"AR_RL_CFG": "1"}, "fused_rl_kernel"),
+                                      ({"AR_RL_CFG": "2"}, "fused_rl_kernel"),
+                                      ({"AR_FUSED_LEGACY": "1"}, "fused_kernel")])
+def test_rl_config_sweep_subprocess(cu, env, want):
+    e = dict(os.environ, AR_RES_STREAM="1", **env)
+    r = subprocess.run([sys.executable, "-c", SWEEP.format(root=ROOT), want], env=e, capture_output=True,
+                       text=True, timeout=600)
+    assert r.returncode == 0 and "ok" in r.stdout, r.stdout + r.stderr
