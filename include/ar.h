@@ -153,10 +153,12 @@ typedef struct {
 const char* ar_status_str(ar_status s);
 const char* ar_last_error(void);     /* thread-local detail of the last failure */
 const char* ar_version(void);
-/* Name of the kernel the calling thread's last ar_select_refine_sum launched
- * ("fused_rl_kernel" = the result-ring one-pass kernel, "fused_kernel" = the
- * general one-pass kernel, "" = none: empty input or an error).  Static
- * storage; for tests and benchmarks that must know which path ran. */
+/* Name of the scan kernel the calling thread's last ar_select_refine_sum or
+ * ar_approx_select launched: "fused_rl_kernel" (result-ring one-pass kernel),
+ * "fused_kernel" (general one-pass kernel), "select_pipe_kernel" (pipelined
+ * ordered select), "select_tile_kernel" (general ordered select), "" (none:
+ * empty input or an error).  Static storage; for tests and benchmarks that
+ * must know which path ran. */
 const char* ar_last_scan_kernel(void);
 
 /* --------------------------------------------------- a1: decomposition */
@@ -328,6 +330,35 @@ ar_status ar_refine_sum(const ar_cands* in, const ar_pred* preds, int32_t npred,
 ar_status ar_select_refine_sum(const ar_pred* preds, int32_t npred,
                                const ar_column* const* cols, int32_t ncols,
                                int64_t* out_dev, void* stream);
+
+/*
+ * The same one-pass query for back-to-back query streams (and CUDA graphs):
+ * with a workspace the call is a single kernel launch -- out_dev is written,
+ * not accumulated, so no memset precedes it -- and may use programmatic
+ * dependent launch so that its prologue and first tile loads overlap the tail
+ * of the preceding kernel in the stream.
+ *   ws        device memory of >= ar_select_refine_sum_ws_bytes() bytes whose
+ *             first 4 bytes are zero before the first call (e.g. cudaMemset
+ *             once); every call leaves them zero.  One workspace per stream:
+ *             calls sharing it must be stream-ordered.  NULL = as
+ *             ar_select_refine_sum (flags must be 0).
+ *   flags     AR_SRS_PDL: launch as a programmatic dependent of the previous
+ *             kernel; inputs are read after it completes, out_dev is written
+ *             after it completes.
+ *             AR_SRS_PDL_EARLY_READ: as AR_SRS_PDL, but the column parts are
+ *             read while the previous kernel may still run -- the caller
+ *             guarantees that kernel does not write them (e.g. the previous
+ *             call of a query stream over immutable, already-decomposed columns).
+ * Results are identical to ar_select_refine_sum.
+ * Errors: as ar_select_refine_sum; AR_ERR_RANGE (ws_bytes too small);
+ * AR_ERR_INVALID (unknown flags, or flags without a workspace).
+ */
+#define AR_SRS_PDL 1
+#define AR_SRS_PDL_EARLY_READ 2
+size_t ar_select_refine_sum_ws_bytes(void);
+ar_status ar_select_refine_sum_ws(const ar_pred* preds, int32_t npred,
+                                  const ar_column* const* cols, int32_t ncols, int32_t flags,
+                                  int64_t* out_dev, void* ws, size_t ws_bytes, void* stream);
 
 /* -------------------------------- a4: row-sharded multi-GPU exchange */
 

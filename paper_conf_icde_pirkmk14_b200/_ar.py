@@ -20,6 +20,7 @@ AR_SELECT_CARRY_APPR = 1
 AR_DECOMPOSE_SIGNED, AR_DECOMPOSE_BASE_MIN = 1, 2
 AR_AUX_DEFINITE = 0x80000000
 AR_PROJECT_APPROX, AR_PROJECT_EXACT = 0, 1
+AR_SRS_PDL, AR_SRS_PDL_EARLY_READ = 1, 2
 
 
 class ARError(RuntimeError):
@@ -79,6 +80,9 @@ SIGNATURES = {
     "ar_refine_sum": (ctypes.c_int, [ctypes.POINTER(Cands), ctypes.POINTER(Pred), _I32, ctypes.POINTER(_P), _I32,
                                      _P, _P, _P]),
     "ar_select_refine_sum": (ctypes.c_int, [ctypes.POINTER(Pred), _I32, ctypes.POINTER(_P), _I32, _P, _P]),
+    "ar_select_refine_sum_ws_bytes": (_SZ, []),
+    "ar_select_refine_sum_ws": (ctypes.c_int, [ctypes.POINTER(Pred), _I32, ctypes.POINTER(_P), _I32, _I32, _P, _P,
+                                               _SZ, _P]),
     "ar_dist_unique_id_bytes": (_SZ, []),
     "ar_dist_get_unique_id": (ctypes.c_int, [_P]),
     "ar_dist_init": (ctypes.c_int, [ctypes.POINTER(_P), _P, _I32, _I32]),
@@ -212,6 +216,15 @@ def ar_refine_sum(cands: Cands, preds, cols, out_sum_dev, out_count_dev, stream)
 
 def ar_select_refine_sum(preds, cols, out_dev, stream):
     _call("ar_select_refine_sum", _preds(preds), len(preds), _handles(cols), len(cols), out_dev, stream)
+
+
+def ar_select_refine_sum_ws_bytes() -> int:
+    return int(load().ar_select_refine_sum_ws_bytes())
+
+
+def ar_select_refine_sum_ws(preds, cols, flags, out_dev, ws, ws_bytes, stream):
+    _call("ar_select_refine_sum_ws", _preds(preds), len(preds), _handles(cols), len(cols), flags, out_dev, ws,
+          ws_bytes, stream)
 
 
 def ar_dist_unique_id_bytes() -> int:

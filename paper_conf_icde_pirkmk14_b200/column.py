@@ -210,6 +210,18 @@ def refine_sum(cands: CandidateList, preds, cols, out_sum: torch.Tensor, out_cou
                       out_count.data_ptr() if out_count is not None else None, _stream(stream))
 
 
-def select_refine_sum(preds, cols, out4: torch.Tensor, stream=None):
-    """Steps a3+a5+a6 in one pass: out4 = [SUM, |result|, |candidates|, |definite|]."""
-    _ar.ar_select_refine_sum(_pred_tuples(preds), [c.handle for c in cols], out4.data_ptr(), _stream(stream))
+def select_refine_sum(preds, cols, out4: torch.Tensor, stream=None, ws: "Workspace" = None, flags: int = 0):
+    """Steps a3+a5+a6 in one pass: out4 = [SUM, |result|, |candidates|, |definite|].  With a workspace
+    (SrsWorkspace) the call is one kernel launch, optionally a programmatic dependent one (flags)."""
+    if ws is None:
+        _ar.ar_select_refine_sum(_pred_tuples(preds), [c.handle for c in cols], out4.data_ptr(), _stream(stream))
+    else:
+        _ar.ar_select_refine_sum_ws(_pred_tuples(preds), [c.handle for c in cols], flags, out4.data_ptr(), ws.ptr,
+                                    ws.nbytes, _stream(stream))
+
+
+def SrsWorkspace(device="cuda") -> "Workspace":
+    """Workspace of ar_select_refine_sum_ws: zeroed once here (the ticket word), left zero by every call."""
+    w = Workspace(_ar.ar_select_refine_sum_ws_bytes(), device)
+    w.t.zero_()
+    return w

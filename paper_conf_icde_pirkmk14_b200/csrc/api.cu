@@ -340,6 +340,8 @@ static ar_status setup_scan(const ar_pred* preds, int32_t npred, ard::SelParams&
     P.bpt = (uint32_t)kernel_bpt(fused);
     static const int suspend_ns = env_int("AR_SUSPEND_NS", 0);
     P.suspend_ns = (uint32_t)suspend_ns;
+    static const int prod_wait = env_int("AR_PROD_WAIT", 0);
+    P.prod_wait = (uint32_t)prod_wait;
     static const int debug = env_int("AR_DEBUG", 0);
     P.debug = (uint32_t)debug;
     P.tile_rows = (uint32_t)kernel_warps(fused) * 32u * 32u * P.bpt;
@@ -467,6 +469,7 @@ ar_status ar_approx_select(const ar_pred* preds, int32_t npred, int32_t flags, a
     out->appr_bits = carry ? (int32_t)std::max<uint32_t>(abits, 1) : 0;
     cudaStream_t s = (cudaStream_t)stream;
     AR_TRY_CUDA(cudaMemsetAsync(out->count, 0, sizeof(int64_t), s));
+    g_last_scan = "";
     if (empty || n == 0) return AR_OK;
     P.carry = carry ? 1 : 0;
     P.out_pos = out->pos;
@@ -484,6 +487,11 @@ ar_status ar_approx_select(const ar_pred* preds, int32_t npred, int32_t flags, a
     P.tmp_pos = (uint32_t*)tmp;
     P.tmp_aux = P.tmp_pos + slice_rows;
     (void)T;
+    bool launched = false;   // the pipelined scan (select_pipe.cu) where the shape has one
+    st = launch_select_pipe(P, &launched, s);
+    if (st != AR_OK) return st;
+    g_last_scan = launched ? "select_pipe_kernel" : "select_tile_kernel";
+    if (launched) return launch_select_rest(P, s);
     const void* fn = select_kernel_fn(P, false);
     P.nstages = 1;
     const size_t smem = select_smem_bytes(P.stage_words, 1, true);
@@ -701,8 +709,23 @@ ar_status ar_refine_sum(const ar_cands* in, const ar_pred* preds, int32_t npred,
 
 // ----------------------------------------------------------- fused a3+a5+a6
 
+size_t ar_select_refine_sum_ws_bytes(void) { return kSrsTicketBytes + (size_t)kSrsMaxGrid * 32; }
+
 ar_status ar_select_refine_sum(const ar_pred* preds, int32_t npred, const ar_column* const* cols, int32_t ncols,
                                int64_t* out_dev, void* stream) {
+    return ar_select_refine_sum_ws(preds, npred, cols, ncols, 0, out_dev, nullptr, 0, stream);
+}
+
+ar_status ar_select_refine_sum_ws(const ar_pred* preds, int32_t npred, const ar_column* const* cols, int32_t ncols,
+                                  int32_t flags, int64_t* out_dev, void* ws, size_t ws_bytes, void* stream) {
+    if (ws && ws_bytes < ar_select_refine_sum_ws_bytes()) {
+        set_error("ar_select_refine_sum_ws: ws_bytes %zu < %zu", ws_bytes, ar_select_refine_sum_ws_bytes());
+        return AR_ERR_RANGE;
+    }
+    if ((flags & ~(AR_SRS_PDL | AR_SRS_PDL_EARLY_READ)) || (flags && !ws)) {
+        set_error("ar_select_refine_sum_ws: flags 0x%x invalid (the PDL flags need a workspace)", flags);
+        return AR_ERR_INVALID;
+    }
     ard::SelParams P;
     bool empty = false;
     int64_t n = 0;
@@ -736,17 +759,19 @@ ar_status ar_select_refine_sum(const ar_pred* preds, int32_t npred, const ar_col
         P.gidx = g < 0 ? 0 : g;
     }
     cudaStream_t s = (cudaStream_t)stream;
-    AR_TRY_CUDA(cudaMemsetAsync(out_dev, 0, 4 * sizeof(int64_t), s));
     g_last_scan = "";
+    if (!ws || empty || n == 0) AR_TRY_CUDA(cudaMemsetAsync(out_dev, 0, 4 * sizeof(int64_t), s));
     if (empty || n == 0) return AR_OK;
     bool launched = false;   // the result-ring kernel (fused.cu) where it applies
-    st = launch_fused_rl(P, cols, &launched, s);
+    const int pdl = (flags & AR_SRS_PDL_EARLY_READ) ? 2 : ((flags & AR_SRS_PDL) ? 1 : 0);
+    st = launch_fused_rl(P, cols, ws, pdl, &launched, s);
     if (st != AR_OK) return st;
     if (launched) {
         g_last_scan = "fused_rl_kernel";
         return AR_OK;
     }
     g_last_scan = "fused_kernel";
+    if (ws) AR_TRY_CUDA(cudaMemsetAsync(out_dev, 0, 4 * sizeof(int64_t), s));   // fused_kernel accumulates
     int occ = 1;
     const void* fn = select_kernel_fn(P, true);
     P.nstages = pick_stages(fn, P.stage_words, true, &occ);

@@ -23,86 +23,14 @@
 // per BPT blocks, the list holds results only, and its passes are always full.
 #include <type_traits>
 
-#include "kernels.cuh"
+#include "rl_common.cuh"
 
 namespace ard {
 namespace rl {
 
-constexpr int kRingDefault = 256;         // result entries (row, factor) per warp (power of two)
+constexpr int kRingDefault = 128;         // result entries (row, factor) per warp (power of two)
 constexpr int kDepth = 4;                 // gather passes in flight per warp
 constexpr int kSlotWords = 4 * 32;        // per pass: lo[32], hi[32], info[32], factor[32]
-
-template <int I>
-using ic = std::integral_constant<int, I>;
-template <int N, int I = 0, class F>
-__device__ __forceinline__ void static_for(F&& f) {
-    if constexpr (I < N) {
-        f(ic<I>{});
-        static_for<N, I + 1>(f);
-    }
-}
-
-// Decomposition shape: per predicate (w_major << 6) | streamed residual width k.
-template <int... WK>
-struct Shape {
-    static constexpr int N = sizeof...(WK);
-    static constexpr int w(int c) {
-        constexpr int a[] = {(WK >> 6)..., 0};
-        return a[c];
-    }
-    static constexpr int k(int c) {
-        constexpr int a[] = {(WK & 63)..., 0};
-        return a[c];
-    }
-    static constexpr int off(int c) {   // global plane index of predicate c (its ashift)
-        int o = 0;
-        for (int i = 0; i < c; ++i) o += w(i);
-        return o;
-    }
-};
-
-// W consecutive 32-bit words from shared memory, vectorised as far as the
-// width allows (a block's planes start at a multiple of W words).
-template <int W>
-__device__ __forceinline__ void lds_words(uint32_t (&x)[W], const uint32_t* p) {
-    if constexpr (W % 4 == 0) {
-#pragma unroll
-        for (int q = 0; q < W / 4; ++q) {
-            const uint4 v = reinterpret_cast<const uint4*>(p)[q];
-            x[4 * q] = v.x; x[4 * q + 1] = v.y; x[4 * q + 2] = v.z; x[4 * q + 3] = v.w;
-        }
-    } else if constexpr (W % 2 == 0) {
-#pragma unroll
-        for (int q = 0; q < W / 2; ++q) {
-            const uint2 v = reinterpret_cast<const uint2*>(p)[q];
-            x[2 * q] = v.x; x[2 * q + 1] = v.y;
-        }
-    } else {
-#pragma unroll
-        for (int j = 0; j < W; ++j) x[j] = p[j];
-    }
-}
-
-// Borrow steps (see select.cu): v < lo iff v - lo borrows out of the top plane.
-__device__ __forceinline__ uint32_t bsub(uint32_t x, uint32_t cbit, uint32_t b) {
-    uint32_t d;
-    asm("lop3.b32 %0, %1, %2, %3, 0x8E;" : "=r"(d) : "r"(x), "r"(cbit), "r"(b));
-    return d;
-}
-__device__ __forceinline__ uint32_t brsub(uint32_t x, uint32_t cbit, uint32_t b) {
-    uint32_t d;
-    asm("lop3.b32 %0, %1, %2, %3, 0xB2;" : "=r"(d) : "r"(x), "r"(cbit), "r"(b));
-    return d;
-}
-
-// Value of row l from W planes held in registers.
-template <int W>
-__device__ __forceinline__ uint32_t row_of(const uint32_t (&x)[W], uint32_t l) {
-    uint32_t v = 0;
-#pragma unroll
-    for (int j = 0; j < W; ++j) v |= ((x[j] >> l) & 1u) << j;
-    return v;
-}
 
 // Exact value of predicate C's column at row l of block blk, from the stage.
 template <class S, int C>
@@ -161,7 +89,12 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
     }
     __syncthreads();
     if (warp == NW) {
-        if (lane == 0) produce_ring(P, full, empty, slot, stages);
+        if (lane == 0) {
+            if (P.rl_pdl == 1) asm volatile("griddepcontrol.wait;" ::: "memory");   // inputs may be in flight
+            produce_ring(P, full, empty, slot, stages);
+            // every tile of this CTA is loading: the next call in the stream may start its prologue
+            if (P.rl_pdl) asm volatile("griddepcontrol.launch_dependents;" ::: "memory");
+        }
         return;
     }
 
@@ -205,6 +138,11 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
         const long long t = slot[s];
         if (t < 0) break;
         const uint32_t* stg = stages + (size_t)s * P.stage_words;
+        if (P.debug == 7) {   // experiment: the TMA stream alone (no evaluation)
+            __syncwarp();
+            if (lane == 0) mbar_arrive(empty + s);
+            continue;
+        }
         const int64_t tile_r0 = t * (int64_t)P.tile_rows;
         const bool full_tile = tile_r0 + (int64_t)P.tile_rows <= P.n;
 
@@ -214,47 +152,8 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
         for (int b = 0; b < BPT; ++b) {
             const uint32_t blk = b * NT + threadIdx.x;
             const uint32_t vm = full_tile ? 0xffffffffu : valid_mask(tile_r0 + 32 * (int64_t)blk, P.n);
-            uint32_t cm = vm, dm = vm, em = vm;
-            static_for<S::N>([&](auto cc) {
-                constexpr int C = decltype(cc)::value;
-                constexpr int W = S::w(C), K = S::k(C), O = S::off(C);
-                uint32_t x[W];
-                lds_words<W>(x, stg + P.p[C].soff + blk * W);
-                uint32_t cl = 0, ch = 0;
-#pragma unroll
-                for (int j = 0; j < W; ++j) {
-                    cl = bsub(x[j], P.pm[O + j][0], cl);
-                    ch = brsub(x[j], P.pm[O + j][1], ch);
-                }
-                const uint32_t c = ~(cl | ch);
-                cm &= c;
-                if constexpr (K == 0) {   // k = 0: candidate = definite = exact
-                    dm &= c;
-                    em &= c;
-                } else {
-                    uint32_t dl = 0, dh = 0;
-#pragma unroll
-                    for (int j = 0; j < W; ++j) {
-                        dl = bsub(x[j], P.pm[O + j][2], dl);
-                        dh = brsub(x[j], P.pm[O + j][3], dh);
-                    }
-                    dm &= ~(dl | dh);
-                    uint32_t r[K];
-                    lds_words<K>(r, stg + P.p[C].res_soff + blk * K);
-                    uint32_t el = 0, eh = 0;
-#pragma unroll
-                    for (int j = 0; j < K; ++j) {
-                        el = bsub(r[j], P.pmx[C][j][0], el);
-                        eh = brsub(r[j], P.pmx[C][j][1], eh);
-                    }
-#pragma unroll
-                    for (int j = 0; j < W; ++j) {
-                        el = bsub(x[j], P.pmx[C][K + j][0], el);
-                        eh = brsub(x[j], P.pmx[C][K + j][1], eh);
-                    }
-                    em &= ~(el | eh);
-                }
-            });
+            uint32_t cm, dm, em;
+            eval_block<S, true>(P, stg, blk, vm, cm, dm, em);
             ncand += __popc(cm);
             ndef += __popc(dm);
             nres += __popc(em);
@@ -363,11 +262,56 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
         c1 += __shfl_xor_sync(0xffffffffu, c1, o);
         c2 += __shfl_xor_sync(0xffffffffu, c2, o);
     }
+    if (!P.rl_fin) {   // out4 zeroed by the caller: one atomic per counter and warp
+        if (lane == 0) {
+            atomicAdd(P.out4 + 0, sum);
+            atomicAdd(P.out4 + 1, c2);
+            atomicAdd(P.out4 + 2, c0);
+            atomicAdd(P.out4 + 3, c1);
+        }
+        return;
+    }
+    // Workspace finalize (no memset before the launch): CTA partial -> rl_part[blockIdx]; the last
+    // CTA to arrive (ticket) sums all partials into out4 and re-arms the ticket.  Consumer warps
+    // only: the producer warp has exited, so they meet at named barrier 1.
+    __shared__ unsigned long long red[NW][4];
+    __shared__ uint32_t last;
     if (lane == 0) {
-        atomicAdd(P.out4 + 0, sum);
-        atomicAdd(P.out4 + 1, c2);
-        atomicAdd(P.out4 + 2, c0);
-        atomicAdd(P.out4 + 3, c1);
+        red[warp][0] = sum;
+        red[warp][1] = c2;
+        red[warp][2] = c0;
+        red[warp][3] = c1;
+    }
+    bar_sync(1, NT);
+    if (threadIdx.x == 0) {
+        unsigned long long t4[4] = {0, 0, 0, 0};
+        for (int w = 0; w < NW; ++w)
+            for (int i = 0; i < 4; ++i) t4[i] += red[w][i];
+        if (P.rl_pdl) asm volatile("griddepcontrol.wait;" ::: "memory");   // the previous call is done with out4
+        unsigned long long* part = P.rl_part + 4ull * blockIdx.x;
+        for (int i = 0; i < 4; ++i) __stcg(part + i, t4[i]);
+        __threadfence();
+        last = atomicAdd(P.rl_ticket, 1u) == gridDim.x - 1 ? 1u : 0u;
+    }
+    bar_sync(1, NT);
+    if (!last) return;
+    __threadfence();
+    unsigned long long t4[4] = {0, 0, 0, 0};
+    for (uint32_t b = threadIdx.x; b < gridDim.x; b += NT)
+        for (int i = 0; i < 4; ++i) t4[i] += __ldcg(P.rl_part + 4ull * b + i);
+#pragma unroll
+    for (int o = 16; o > 0; o >>= 1)
+        for (int i = 0; i < 4; ++i) t4[i] += __shfl_xor_sync(0xffffffffu, t4[i], o);
+    bar_sync(1, NT);
+    if (lane == 0)
+        for (int i = 0; i < 4; ++i) red[warp][i] = t4[i];
+    bar_sync(1, NT);
+    if (threadIdx.x == 0) {
+        unsigned long long o4[4] = {0, 0, 0, 0};
+        for (int w = 0; w < NW; ++w)
+            for (int i = 0; i < 4; ++i) o4[i] += red[w][i];
+        for (int i = 0; i < 4; ++i) P.out4[i] = o4[i];
+        *P.rl_ticket = 0u;
     }
 }
 
@@ -407,8 +351,8 @@ void retile(ard::SelParams& P, uint32_t tile_rows) {
     P.num_tiles = (int64_t)ceil_div_u64((uint64_t)P.n, tile_rows);
 }
 
-// (consumer warps, blocks per thread): AR_RL_CFG = 0/1/2/3/4 picks (8,1), (4,2),
-// (2,4), (16,1), (4,1); tile rows = NW * BPT * 1024.
+// (consumer warps, blocks per thread): AR_RL_CFG = 0/1/2/3/4/5 picks (8,1), (4,2),
+// (2,4), (16,1), (4,1), (8,2); tile rows = NW * BPT * 1024.
 template <int... Ws>
 RlFn rl_pick(int cfg) {
     switch (cfg) {
@@ -416,6 +360,7 @@ RlFn rl_pick(int cfg) {
         case 2: return {(const void*)ard::rl::fused_rl_kernel<2, 4, Ws...>, 2, 8192};
         case 3: return {(const void*)ard::rl::fused_rl_kernel<16, 1, Ws...>, 16, 16384};
         case 4: return {(const void*)ard::rl::fused_rl_kernel<4, 1, Ws...>, 4, 4096};
+        case 5: return {(const void*)ard::rl::fused_rl_kernel<8, 2, Ws...>, 8, 16384};
         default: return {(const void*)ard::rl::fused_rl_kernel<8, 1, Ws...>, 8, 8192};
     }
 }
@@ -478,9 +423,14 @@ size_t rl_smem_bytes(const ard::SelParams& P, uint32_t nstages, int nw) {
 
 // Launch the result-ring kernel if it applies (returns AR_OK and *launched);
 // otherwise *launched = false and the caller takes fused_kernel.
-ar_status launch_fused_rl(const ard::SelParams& P0, const ar_column* const* cols, bool* launched, cudaStream_t s) {
+ar_status launch_fused_rl(const ard::SelParams& P0, const ar_column* const* cols, void* ws, int pdl, bool* launched,
+                          cudaStream_t s) {
     *launched = false;
     ard::SelParams P = P0;   // the caller's copy stays valid for fused_kernel
+    P.rl_fin = ws ? 1 : 0;
+    P.rl_pdl = ws ? pdl : 0;
+    P.rl_ticket = ws ? (unsigned int*)ws : nullptr;
+    P.rl_part = ws ? (unsigned long long*)((char*)ws + kSrsTicketBytes) : nullptr;
     static const bool off = getenv("AR_FUSED_LEGACY") && atoi(getenv("AR_FUSED_LEGACY"));
     if (off || !P.exact_mode || P.n >= (int64_t)1 << 32) return AR_OK;
     // factors: none (COUNT), all predicate columns (direct), or one gathered bit-packed column
@@ -519,6 +469,8 @@ ar_status launch_fused_rl(const ard::SelParams& P0, const ar_column* const* cols
         int dev = 0, max_optin = 227 * 1024;
         if (cudaGetDevice(&dev) == cudaSuccess)
             cudaDeviceGetAttribute(&max_optin, cudaDevAttrMaxSharedMemoryPerBlockOptin, dev);
+        cudaFuncAttributes fa{};   // dynamic + static shared memory <= the opt-in maximum
+        if (cudaFuncGetAttributes(&fa, k.fn) == cudaSuccess) max_optin -= (int)fa.sharedSizeBytes;
         cudaFuncSetAttribute(k.fn, cudaFuncAttributeMaxDynamicSharedMemorySize, max_optin);
         cudaGetLastError();
         if (nopted < 64) opted[nopted++] = k.fn;
@@ -544,8 +496,19 @@ ar_status launch_fused_rl(const ard::SelParams& P0, const ar_column* const* cols
     if (!stages) return AR_OK;
     P.nstages = stages;
     const int grid = (int)std::min<int64_t>(P.num_tiles, (int64_t)num_sms() * std::min(occ, std::max(want_ctas, 1)));
+    if (ws && grid > kSrsMaxGrid) return AR_OK;
     void* args[] = {&P};
-    AR_TRY_CUDA(cudaLaunchKernel(k.fn, dim3(grid), dim3(threads), args, rl_smem_bytes(P, stages, k.nw), s));
+    cudaLaunchConfig_t cfg = {};
+    cfg.gridDim = dim3(grid);
+    cfg.blockDim = dim3(threads);
+    cfg.dynamicSmemBytes = rl_smem_bytes(P, stages, k.nw);
+    cfg.stream = s;
+    cudaLaunchAttribute attr[1];
+    attr[0].id = cudaLaunchAttributeProgrammaticStreamSerialization;
+    attr[0].val.programmaticStreamSerializationAllowed = P.rl_pdl ? 1 : 0;
+    cfg.attrs = attr;
+    cfg.numAttrs = 1;
+    AR_TRY_CUDA(cudaLaunchKernelExC(&cfg, k.fn, args));
     *launched = true;
     return AR_OK;
 }

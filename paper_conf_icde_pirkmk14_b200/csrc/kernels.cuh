@@ -55,6 +55,8 @@ struct SelParams {
     uint32_t nstages;
     uint32_t bpt;             // 32-row blocks per consumer thread (template parameter of the launch)
     uint32_t suspend_ns;      // mbarrier wait suspend hint (0 = spin)
+    uint32_t prod_wait;       // producer's wait for a free stage: 0 = nanosleep back-off, 1 = try_wait,
+                              // > 1 = try_wait with that suspend hint (ns)
     uint32_t debug;           // experiments only (AR_DEBUG): 1 = no look-back (provisional offsets), 2 = no copy-out
     uint32_t tile_rows;       // kSelMinTileRows * bpt
     uint32_t* out_pos;
@@ -79,6 +81,11 @@ struct SelParams {
     int32_t rl_list;              // 1: one gathered SUM factor, rows queued in the warp result ring
     int32_t rl_mpred;             // predicate whose exact value is the other SUM factor, or -1
     uint32_t rl_ring;             // result-ring entries per warp (power of two)
+    int32_t rl_fin;               // 1: finalize out4 through rl_part / rl_ticket (no memset before the launch)
+    int32_t rl_pdl;               // programmatic dependent launch: 1 = wait before reading inputs, 2 = read
+                                  // inputs at once (caller: the previous kernel does not write them)
+    unsigned long long* rl_part;  // [gridDim][4] CTA partials
+    unsigned int* rl_ticket;      // CTAs done (zero between calls)
 };
 
 // Producer of the persistent scan kernels: one lane streams tiles (tile =
@@ -92,7 +99,12 @@ __device__ __forceinline__ void produce_ring(const SelParams& P, uint64_t* full,
     const uint32_t blocks_per_tile = P.tile_rows / 32;
     uint32_t s = 0, ph = 0;   // ring slot and its phase parity (no integer division in the loop)
     for (uint32_t i = 0;; ++i) {
-        if (i >= P.nstages) mbar_wait_sleep(empty + s, ph ^ 1u);   // producer backs off instead of spinning
+        if (i >= P.nstages) {
+            if (P.prod_wait == 0)
+                mbar_wait_sleep(empty + s, ph ^ 1u);   // back off with __nanosleep instead of spinning
+            else
+                mbar_wait(empty + s, ph ^ 1u, P.prod_wait == 1 ? 0u : P.prod_wait);   // hardware-suspended try_wait
+        }
         const long long t = (long long)blockIdx.x + (long long)i * gridDim.x;
         if (t >= P.num_tiles) {
             slot[s] = -1;
@@ -195,7 +207,12 @@ const void* select_kernel_fn(const ard::SelParams& P, bool fused);
 int select_occupancy(const void* fn, size_t smem, bool fused);
 ar_status launch_scan(const void* fn, const ard::SelParams& P, int grid, size_t smem, bool fused, cudaStream_t s);
 ar_status launch_select_rest(const ard::SelParams& P, cudaStream_t s);
-ar_status launch_fused_rl(const ard::SelParams& P, const ar_column* const* cols, bool* launched, cudaStream_t s);
+// ar_select_refine_sum_ws workspace: a ticket word (padded), then kSrsMaxGrid CTA partials of 4 x u64
+constexpr size_t kSrsTicketBytes = 128;
+constexpr int kSrsMaxGrid = 2048;
+ar_status launch_select_pipe(const ard::SelParams& P, bool* launched, cudaStream_t s);
+ar_status launch_fused_rl(const ard::SelParams& P, const ar_column* const* cols, void* ws, int pdl, bool* launched,
+                          cudaStream_t s);
 ar_status launch_refine(const ard::RefParams& P, int grid, cudaStream_t s);
 ar_status launch_refine_sum(const ard::RefParams& P, int grid, cudaStream_t s);
 ar_status launch_sum(const ard::SumParams& P, int grid, cudaStream_t s);

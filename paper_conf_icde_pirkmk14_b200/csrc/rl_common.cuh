@@ -1,0 +1,142 @@
+// rl_common.cuh -- device helpers shared by the persistent TMA-pipelined scan
+// kernels (fused.cu: one-pass select + refine + SUM; select_pipe.cu: ordered
+// approximate select): compile-time decomposition shapes, shared-memory plane
+// loads and the bit-plane range tests of step a3.
+#pragma once
+#include <type_traits>
+
+#include "kernels.cuh"
+
+namespace ard {
+namespace rl {
+
+template <int I>
+using ic = std::integral_constant<int, I>;
+template <int N, int I = 0, class F>
+__device__ __forceinline__ void static_for(F&& f) {
+    if constexpr (I < N) {
+        f(ic<I>{});
+        static_for<N, I + 1>(f);
+    }
+}
+
+// Decomposition shape: per predicate (w_major << 6) | streamed residual width k.
+template <int... WK>
+struct Shape {
+    static constexpr int N = sizeof...(WK);
+    static constexpr int w(int c) {
+        constexpr int a[] = {(WK >> 6)..., 0};
+        return a[c];
+    }
+    static constexpr int k(int c) {
+        constexpr int a[] = {(WK & 63)..., 0};
+        return a[c];
+    }
+    static constexpr int off(int c) {   // global plane index of predicate c (its ashift)
+        int o = 0;
+        for (int i = 0; i < c; ++i) o += w(i);
+        return o;
+    }
+};
+
+// W consecutive 32-bit words from shared memory, vectorised as far as the
+// width allows (a block's planes start at a multiple of W words).
+template <int W>
+__device__ __forceinline__ void lds_words(uint32_t (&x)[W], const uint32_t* p) {
+    if constexpr (W % 4 == 0) {
+#pragma unroll
+        for (int q = 0; q < W / 4; ++q) {
+            const uint4 v = reinterpret_cast<const uint4*>(p)[q];
+            x[4 * q] = v.x; x[4 * q + 1] = v.y; x[4 * q + 2] = v.z; x[4 * q + 3] = v.w;
+        }
+    } else if constexpr (W % 2 == 0) {
+#pragma unroll
+        for (int q = 0; q < W / 2; ++q) {
+            const uint2 v = reinterpret_cast<const uint2*>(p)[q];
+            x[2 * q] = v.x; x[2 * q + 1] = v.y;
+        }
+    } else {
+#pragma unroll
+        for (int j = 0; j < W; ++j) x[j] = p[j];
+    }
+}
+
+// Borrow steps (see select.cu): v < lo iff v - lo borrows out of the top plane.
+__device__ __forceinline__ uint32_t bsub(uint32_t x, uint32_t cbit, uint32_t b) {
+    uint32_t d;
+    asm("lop3.b32 %0, %1, %2, %3, 0x8E;" : "=r"(d) : "r"(x), "r"(cbit), "r"(b));
+    return d;
+}
+__device__ __forceinline__ uint32_t brsub(uint32_t x, uint32_t cbit, uint32_t b) {
+    uint32_t d;
+    asm("lop3.b32 %0, %1, %2, %3, 0xB2;" : "=r"(d) : "r"(x), "r"(cbit), "r"(b));
+    return d;
+}
+
+// Value of row l from W planes held in registers.
+template <int W>
+__device__ __forceinline__ uint32_t row_of(const uint32_t (&x)[W], uint32_t l) {
+    uint32_t v = 0;
+#pragma unroll
+    for (int j = 0; j < W; ++j) v |= ((x[j] >> l) & 1u) << j;
+    return v;
+}
+
+// Per-block evaluation of every predicate on the 32 rows of block `blk` of a
+// stage (vm = valid rows): candidate mask cm (major in the candidate range of
+// every predicate), definite mask dm (major in the definite range of every
+// decomposed predicate, candidate range otherwise) and -- with kExact, for
+// shapes whose residual planes are streamed (K = residual width) -- the exact
+// mask em: one borrow chain over the residual then the major planes (the
+// bitwise concatenation "+bw") against the exact bounds.
+// Without kExact, K > 0 only marks a decomposed predicate.
+template <class S, bool kExact>
+__device__ __forceinline__ void eval_block(const SelParams& P, const uint32_t* stg, uint32_t blk, uint32_t vm,
+                                           uint32_t& cm, uint32_t& dm, uint32_t& em) {
+    cm = dm = em = vm;
+    static_for<S::N>([&](auto cc) {
+        constexpr int C = decltype(cc)::value;
+        constexpr int W = S::w(C), K = S::k(C), O = S::off(C);
+        uint32_t x[W];
+        lds_words<W>(x, stg + P.p[C].soff + blk * W);
+        uint32_t cl = 0, ch = 0;
+#pragma unroll
+        for (int j = 0; j < W; ++j) {
+            cl = bsub(x[j], P.pm[O + j][0], cl);
+            ch = brsub(x[j], P.pm[O + j][1], ch);
+        }
+        const uint32_t c = ~(cl | ch);
+        cm &= c;
+        if constexpr (K == 0) {   // k = 0: candidate = definite = exact
+            dm &= c;
+            em &= c;
+        } else {
+            uint32_t dl = 0, dh = 0;   // mode 2 (no definite bucket) has empty bounds in pm
+#pragma unroll
+            for (int j = 0; j < W; ++j) {
+                dl = bsub(x[j], P.pm[O + j][2], dl);
+                dh = brsub(x[j], P.pm[O + j][3], dh);
+            }
+            dm &= ~(dl | dh);
+            if constexpr (kExact) {
+                uint32_t r[K];
+                lds_words<K>(r, stg + P.p[C].res_soff + blk * K);
+                uint32_t el = 0, eh = 0;
+#pragma unroll
+                for (int j = 0; j < K; ++j) {
+                    el = bsub(r[j], P.pmx[C][j][0], el);
+                    eh = brsub(r[j], P.pmx[C][j][1], eh);
+                }
+#pragma unroll
+                for (int j = 0; j < W; ++j) {
+                    el = bsub(x[j], P.pmx[C][K + j][0], el);
+                    eh = brsub(x[j], P.pmx[C][K + j][1], eh);
+                }
+                em &= ~(el | eh);
+            }
+        }
+    });
+}
+
+}  // namespace rl
+}  // namespace ard

@@ -73,6 +73,14 @@ def test_host_validation_without_gpu():
     with pytest.raises(_ar.ARError) as e:
         _ar.ar_approx_select([], 0, _ar.Cands(), None, 0, None)
     assert e.value.status == _ar.AR_ERR_INVALID
+    # the PDL flags need a workspace; a short workspace is a range error (checked before any CUDA call)
+    with pytest.raises(_ar.ARError) as e:
+        _ar.ar_select_refine_sum_ws([], [], _ar.AR_SRS_PDL, None, None, 0, None)
+    assert e.value.status == _ar.AR_ERR_INVALID
+    with pytest.raises(_ar.ARError) as e:
+        _ar.ar_select_refine_sum_ws([], [], 0, None, 16, 8, None)
+    assert e.value.status == _ar.AR_ERR_RANGE
+    assert _ar.ar_select_refine_sum_ws_bytes() >= 128 + 296 * 32
 
 
 def test_layout_decoders_by_hand():

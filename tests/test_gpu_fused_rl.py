@@ -138,3 +138,51 @@ def test_rl_config_sweep_subprocess(cu, env, want):
     r = subprocess.run([sys.executable, "-c", SWEEP.format(root=ROOT), want], env=e, capture_output=True,
                        text=True, timeout=600)
     assert r.returncode == 0 and "ok" in r.stdout, r.stdout + r.stderr
+
+
+@pytest.mark.parametrize("flags", [0, 1, 2])
+def test_rl_workspace_and_pdl_back_to_back(cu, flags):
+    # ar_select_refine_sum_ws: one launch per query, out4 written (not accumulated), ticket re-armed;
+    # alternate two different queries on the same workspace and output, 6 calls without a sync
+    from paper_conf_icde_pirkmk14_b200 import _ar
+    c, cols, los, his = q6(cu, 91, 250_001)
+    _, _, los2, his2 = q6(cu, 91, 8, bounds=[(3, 2523), (0, 10), (1, 50)])
+    values = [c["shipdate"], c["discount"], c["quantity"]]
+    ws = cu.SrsWorkspace()
+    outs = [torch.full((4,), -7, dtype=torch.int64, device="cuda") for _ in range(6)]
+    shared = torch.full((4,), -7, dtype=torch.int64, device="cuda")
+    aggs = [cols["extprice"], cols["discount"]]
+    for i in range(6):
+        lo, hi = (los, his) if i % 2 == 0 else (los2, his2)
+        preds = [(cols["shipdate"], lo[0], hi[0]), (cols["discount"], lo[1], hi[1]),
+                 (cols["quantity"], lo[2], hi[2])]
+        cu.select_refine_sum(preds, aggs, shared, ws=ws, flags=flags)
+        outs[i].copy_(shared)
+        assert _ar.ar_last_scan_kernel() == "fused_rl_kernel"
+    torch.cuda.synchronize()
+    for i in range(6):
+        lo, hi = (los, his) if i % 2 == 0 else (los2, his2)
+        _, cnt, s = oracle.select_sum(values, lo, hi, [c["extprice"], c["discount"]], positions=False)
+        cpos, cdef = oracle.approx_select(values, [8, 0, 0], lo, hi)
+        assert outs[i].cpu().tolist() == [s, cnt, cpos.size, int(cdef.sum())]
+    assert int(ws.t[:4].view(torch.int32).item()) == 0        # ticket left zero
+
+
+def test_rl_workspace_general_kernel_and_empty(cu):
+    # the workspace call on a shape without a result-ring kernel (general fused_kernel) and on an
+    # empty predicate still writes out4 (the output is not accumulated)
+    from paper_conf_icde_pirkmk14_b200 import _ar
+    v = datagen.uniform_u32(5, 100_000, 0, (1 << 11) - 1)      # w_major = 3: no result-ring shape
+    col = cu.BWDColumn(v, 24)
+    ws = cu.SrsWorkspace()
+    o4 = torch.full((4,), -7, dtype=torch.int64, device="cuda")
+    cu.select_refine_sum([(col, 300, 1500)], [col], o4, ws=ws)
+    torch.cuda.synchronize()
+    assert _ar.ar_last_scan_kernel() == "fused_kernel"
+    _, cnt, s = oracle.select_sum([v], [300], [1500], [v], positions=False)
+    cpos, cdef = oracle.approx_select([v], [8], [300], [1500])
+    assert o4.cpu().tolist() == [s, cnt, cpos.size, int(cdef.sum())]
+    o4.fill_(-7)
+    cu.select_refine_sum([(col, 1500, 300)], [col], o4, ws=ws, flags=_ar.AR_SRS_PDL)
+    torch.cuda.synchronize()
+    assert o4.cpu().tolist() == [0, 0, 0, 0]
