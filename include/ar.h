@@ -155,9 +155,8 @@ const char* ar_last_error(void);     /* thread-local detail of the last failure 
 const char* ar_version(void);
 /* Name of the scan kernel the calling thread's last ar_select_refine_sum or
  * ar_approx_select launched: "fused_rl_kernel" (result-ring one-pass kernel),
- * "fused_kernel" (general one-pass kernel), "select_pipe_kernel" (pipelined
- * ordered select), "select_tile_kernel" (general ordered select), "" (none:
- * empty input or an error).  Static storage; for tests and benchmarks that
+ * "fused_kernel" (general one-pass kernel), "select_tile_kernel" (ordered
+ * select), "" (none: empty input or an error).  Static storage; for tests and benchmarks that
  * must know which path ran. */
 const char* ar_last_scan_kernel(void);
 

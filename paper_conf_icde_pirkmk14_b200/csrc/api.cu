@@ -487,11 +487,7 @@ ar_status ar_approx_select(const ar_pred* preds, int32_t npred, int32_t flags, a
     P.tmp_pos = (uint32_t*)tmp;
     P.tmp_aux = P.tmp_pos + slice_rows;
     (void)T;
-    bool launched = false;   // the pipelined scan (select_pipe.cu) where the shape has one
-    st = launch_select_pipe(P, &launched, s);
-    if (st != AR_OK) return st;
-    g_last_scan = launched ? "select_pipe_kernel" : "select_tile_kernel";
-    if (launched) return launch_select_rest(P, s);
+    g_last_scan = "select_tile_kernel";
     const void* fn = select_kernel_fn(P, false);
     P.nstages = 1;
     const size_t smem = select_smem_bytes(P.stage_words, 1, true);

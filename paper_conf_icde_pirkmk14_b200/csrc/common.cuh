@@ -259,6 +259,51 @@ __device__ __forceinline__ uint32_t ld_gather(const uint32_t* p) {
     return v;
 }
 
+// Predicated, non-volatile gathers for kernels that issue a batch of gathers
+// before using any of them: the compiler may reorder and overlap them, and the
+// predicate (not a branch the compiler could if-convert) keeps an unneeded
+// gather from touching memory.  A skipped load returns 0.
+__device__ __forceinline__ uint32_t ld_gather_if(const uint32_t* p, bool pred) {
+    uint32_t v = 0;
+    asm("{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %2, 0;\n\t@q ld.global.nc.L2::64B.u32 %0, [%1];\n\t}"
+        : "+r"(v) : "l"(p), "r"((uint32_t)pred));
+    return v;
+}
+__device__ __forceinline__ uint4 ld_gather_if4(const uint32_t* p, bool pred) {   // 16-B aligned
+    uint4 v = make_uint4(0, 0, 0, 0);
+    asm("{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %5, 0;\n\t@q ld.global.nc.L2::64B.v4.u32 {%0,%1,%2,%3}, [%4];\n\t}"
+        : "+r"(v.x), "+r"(v.y), "+r"(v.z), "+r"(v.w) : "l"(p), "r"((uint32_t)pred));
+    return v;
+}
+__device__ __forceinline__ uint32_t packed_get_if(const uint32_t* __restrict__ s, uint64_t p, int w, bool pred) {
+    const uint64_t bit = p * (uint64_t)w;
+    const uint32_t sh = (uint32_t)(bit & 31);
+    const uint32_t lo = ld_gather_if(s + (bit >> 5), pred);
+    const uint32_t hi = ld_gather_if(s + (bit >> 5) + 1, pred && sh + (uint32_t)w > 32u);
+    const uint32_t v = __funnelshift_r(lo, hi, sh);
+    return w == 32 ? v : (v & ((1u << w) - 1u));
+}
+// Residual of row p: SLICED blocks of k = 4 / 8 planes (16-B aligned) in one or
+// two vector loads of the block's sector, other widths word by word.
+__device__ __forceinline__ uint32_t residual_get_if(const uint32_t* s, uint64_t p, int k, int layout, bool pred) {
+    if (layout != AR_LAYOUT_SLICED) return packed_get_if(s, p, k, pred);
+    const uint32_t* blk = s + (p >> 5) * (uint64_t)k;
+    const uint32_t l = (uint32_t)(p & 31);
+    uint32_t r = 0;
+    if (k == 8 || k == 4) {
+        const uint4 a = ld_gather_if4(blk, pred);
+        r = ((a.x >> l) & 1u) | (((a.y >> l) & 1u) << 1) | (((a.z >> l) & 1u) << 2) | (((a.w >> l) & 1u) << 3);
+        if (k == 8) {
+            const uint4 b = ld_gather_if4(blk + 4, pred);
+            r |= (((b.x >> l) & 1u) << 4) | (((b.y >> l) & 1u) << 5) | (((b.z >> l) & 1u) << 6) |
+                 (((b.w >> l) & 1u) << 7);
+        }
+        return r;
+    }
+    for (int j = 0; j < k; ++j) r |= ((ld_gather_if(blk + j, pred) >> l) & 1u) << j;
+    return r;
+}
+
 // Value of row p from a PACKED LSB-first bitstream of width w (1..32) in global memory.
 __device__ __forceinline__ uint32_t packed_get(const uint32_t* __restrict__ s, uint64_t p, int w) {
     uint64_t bit = p * (uint64_t)w;

@@ -322,16 +322,6 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
 
 namespace ar {
 
-namespace {
-
-constexpr int WK(int w, int k) { return (w << 6) | k; }
-
-struct RlFn {
-    const void* fn;
-    int nw;
-    uint32_t tile_rows;
-};
-
 // Re-lay the stage for another tile size (setup_scan sized it for 8192 rows):
 // each predicate's planes, then its streamed residual planes, tile_rows / 32
 // words per plane.
@@ -350,6 +340,17 @@ void retile(ard::SelParams& P, uint32_t tile_rows) {
     P.stage_words = std::max<uint32_t>(words, 4);
     P.num_tiles = (int64_t)ceil_div_u64((uint64_t)P.n, tile_rows);
 }
+
+namespace {
+
+constexpr int WK(int w, int k) { return (w << 6) | k; }
+
+struct RlFn {
+    const void* fn;
+    int nw;
+    uint32_t tile_rows;
+};
+
 
 // (consumer warps, blocks per thread): AR_RL_CFG = 0/1/2/3/4/5 picks (8,1), (4,2),
 // (2,4), (16,1), (4,1), (8,2); tile rows = NW * BPT * 1024.

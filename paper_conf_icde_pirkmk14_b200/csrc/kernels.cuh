@@ -210,7 +210,7 @@ ar_status launch_select_rest(const ard::SelParams& P, cudaStream_t s);
 // ar_select_refine_sum_ws workspace: a ticket word (padded), then kSrsMaxGrid CTA partials of 4 x u64
 constexpr size_t kSrsTicketBytes = 128;
 constexpr int kSrsMaxGrid = 2048;
-ar_status launch_select_pipe(const ard::SelParams& P, bool* launched, cudaStream_t s);
+void retile(ard::SelParams& P, uint32_t tile_rows);   // fused.cu
 ar_status launch_fused_rl(const ard::SelParams& P, const ar_column* const* cols, void* ws, int pdl, bool* launched,
                           cudaStream_t s);
 ar_status launch_refine(const ard::RefParams& P, int grid, cudaStream_t s);

@@ -120,7 +120,11 @@ __device__ __forceinline__ void block_add(T v, unsigned long long* out) {
     }
 }
 
-__global__ void __launch_bounds__(kRefThreads) refine_sum_kernel(const __grid_constant__ RefParams P) {
+// Refine + SUM in two batched phases per thread: first every residual the 8
+// candidates need (gathers in flight together), then every aggregate value of
+// the kept ones -- two dependent round trips per 8 candidates, not 16.  The
+// gathers are predicated non-volatile loads (common.cuh: ld_gather_if).
+__global__ void __launch_bounds__(kRefThreads, 4) refine_sum_kernel(const __grid_constant__ RefParams P) {
     const long long count = *P.in_count;
     const long long num_tiles = (count + kRefTile - 1) / kRefTile;
     unsigned long long sum = 0, kept = 0;
@@ -129,16 +133,60 @@ __global__ void __launch_bounds__(kRefThreads) refine_sum_kernel(const __grid_co
         uint32_t pos[8], aux[8];
         load8(P.in_pos, j0, count, pos);
         load8(P.in_aux, j0, count, aux);
+        uint32_t keep = 0, need = 0;
 #pragma unroll
         for (int i = 0; i < 8; ++i) {
-            if (j0 + i < (uint64_t)count && refine_keep(P, pos[i], aux[i])) {
-                ++kept;
-                if (P.nagg > 0) {
-                    unsigned long long prod = agg_value_at(P, P.a[0], pos[i], aux[i]);
-                    if (P.nagg > 1) prod *= agg_value_at(P, P.a[1], pos[i], aux[i]);
-                    sum += prod;
-                }
+            if (j0 + i < (uint64_t)count) {
+                keep |= 1u << i;
+                if (!(aux[i] & AR_AUX_DEFINITE)) need |= 1u << i;
             }
+        }
+        for (int c = 0; c < P.npred && need; ++c) {   // Alg. 2 on the non-definite candidates
+            const RefPred& p = P.p[c];
+            if (!p.check) continue;
+            uint32_t r[8], m[8];
+#pragma unroll
+            for (int i = 0; i < 8; ++i) r[i] = residual_get_if(p.residual, pos[i], p.k, p.rlayout, (need >> i) & 1u);
+#pragma unroll
+            for (int i = 0; i < 8; ++i)
+                m[i] = p.carried ? ((aux[i] >> p.ashift) & (p.w == 32 ? 0xffffffffu : ((1u << p.w) - 1u)))
+                                 : ((need >> i) & 1u ? major_get(p.major, pos[i], p.w, p.layout) : 0u);
+#pragma unroll
+            for (int i = 0; i < 8; ++i) {
+                const uint32_t v = ((m[i] << p.k) | r[i]) + p.base;
+                if (((need >> i) & 1u) && !((v >= p.lo) && (v <= p.hi))) keep &= ~(1u << i);
+            }
+        }
+        kept += __popc(keep);
+        if (P.nagg > 0 && keep) {
+            unsigned long long prod[8];
+#pragma unroll
+            for (int i = 0; i < 8; ++i) prod[i] = 1;
+            for (int c = 0; c < P.nagg; ++c) {
+                const AggCol& a = P.a[c];
+                uint32_t v[8];
+                if (a.pred >= 0 && P.p[a.pred].carried) {
+                    const RefPred& p = P.p[a.pred];
+#pragma unroll
+                    for (int i = 0; i < 8; ++i) {
+                        const uint32_t mm = (aux[i] >> p.ashift) & (p.w == 32 ? 0xffffffffu : ((1u << p.w) - 1u));
+                        const uint32_t rr =
+                            a.k ? residual_get_if(a.residual, pos[i], a.k, a.rlayout, (keep >> i) & 1u) : 0u;
+                        v[i] = ((mm << a.k) | rr) + a.base;
+                    }
+                } else if (a.k == 0 && a.layout == AR_LAYOUT_PACKED && a.w > 0) {
+#pragma unroll
+                    for (int i = 0; i < 8; ++i) v[i] = packed_get_if(a.major, pos[i], (int)a.w, (keep >> i) & 1u) + a.base;
+                } else {
+#pragma unroll
+                    for (int i = 0; i < 8; ++i) v[i] = (keep >> i) & 1u ? agg_gather(a, pos[i]) : 0u;
+                }
+#pragma unroll
+                for (int i = 0; i < 8; ++i) prod[i] *= v[i];
+            }
+#pragma unroll
+            for (int i = 0; i < 8; ++i)
+                if ((keep >> i) & 1u) sum += prod[i];
         }
     }
     if (P.out_sum) block_add(sum, P.out_sum);

@@ -1,6 +1,5 @@
-// rl_common.cuh -- device helpers shared by the persistent TMA-pipelined scan
-// kernels (fused.cu: one-pass select + refine + SUM; select_pipe.cu: ordered
-// approximate select): compile-time decomposition shapes, shared-memory plane
+// rl_common.cuh -- device helpers of the persistent TMA-pipelined one-pass
+// kernel (fused.cu): compile-time decomposition shapes, shared-memory plane
 // loads and the bit-plane range tests of step a3.
 #pragma once
 #include <type_traits>

@@ -345,33 +345,3 @@ def test_gpu_errors(cu):
     with pytest.raises(_ar.ARError) as e:
         cu.sum_at(cu.PositionList(10), [big, big], s)
     assert e.value.status == _ar.AR_ERR_RANGE
-
-
-@pytest.mark.parametrize("n", [8191, 8192, 8193, 400_003])
-def test_gpu_select_pipe_kernel_paths(cu, n):
-    # the pipelined ordered select (select_pipe.cu) on the Q6 and C1 shapes, including every row a
-    # candidate (each warp's list full) and a ragged last tile; the general kernel in a subprocess
-    from paper_conf_icde_pirkmk14_b200 import _ar
-    c = datagen.q6_columns(17, 1.0, n=n)
-    values = [c["shipdate"], c["discount"], c["quantity"]]
-    for bounds in ([datagen.Q6_SHIPDATE, datagen.Q6_DISCOUNT, datagen.Q6_QUANTITY],
-                   [(3, 2523), (0, 10), (0, 50)]):
-        los, his = [b[0] for b in bounds], [b[1] for b in bounds]
-        check_select(cu, values, [8, 0, 0], los, his)
-        assert _ar.ar_last_scan_kernel() == "select_pipe_kernel"
-    v = datagen.uniform_u32(n, n)
-    check_select(cu, [v], [8], [datagen.C1_LO], [datagen.C1_HI])
-    assert _ar.ar_last_scan_kernel() == "select_pipe_kernel"
-
-
-def test_gpu_select_general_kernel_subprocess(cu):
-    import os
-    import subprocess
-    import sys
-    root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
-    code = (f"import sys; sys.path.insert(0, {root!r}); sys.argv = ['x'];"
-            "import pytest; sys.exit(pytest.main(['-q', '-x', '-m', 'gpu', "
-            f"{os.path.join(root, 'tests', 'test_gpu_parity.py')!r}, '-k', 'select and not pipe and not subprocess']))")
-    r = subprocess.run([sys.executable, "-c", code], env=dict(os.environ, AR_SELECT_LEGACY="1"),
-                       capture_output=True, text=True, timeout=600)
-    assert r.returncode == 0, r.stdout[-3000:] + r.stderr[-3000:]

@@ -68,6 +68,27 @@ __global__ void tma_kernel(const char* __restrict__ src, size_t bytes, uint32_t 
     if (acc == 0x12345678u) *out = acc;
 }
 
+// 3. gather: `per` independent 4-B loads per thread (ld.global.nc.L2::64B) at
+//    random 64-B-aligned offsets of the buffer -- the one-pass kernel's
+//    l_extendedprice gathers; reported as 64-B granules per second.
+__global__ void gather_kernel(const uint32_t* __restrict__ p, size_t words, uint32_t n, uint32_t seed, unsigned* out) {
+    uint32_t acc = 0;
+    const size_t granules = words / 16;
+    for (uint32_t i = blockIdx.x * blockDim.x + threadIdx.x; i < n; i += gridDim.x * blockDim.x) {
+        uint32_t v[8];
+#pragma unroll
+        for (int j = 0; j < 8; ++j) {
+            uint64_t h = (uint64_t)(i * 8 + j) * 0x9E3779B97F4A7C15ull + seed;
+            h ^= h >> 29;
+            const size_t g = (size_t)(h % granules);
+            asm volatile("ld.global.nc.L2::64B.u32 %0, [%1];" : "=r"(v[j]) : "l"(p + g * 16));
+        }
+#pragma unroll
+        for (int j = 0; j < 8; ++j) acc ^= v[j];
+    }
+    if (acc == 0x12345678u) *out = acc;
+}
+
 int main(int argc, char** argv) {
     const size_t mb = argc > 1 ? atoi(argv[1]) : 165;
     const size_t bytes = mb << 20;
@@ -107,5 +128,14 @@ int main(int argc, char** argv) {
                 printf("{\"probe\": \"tma\", \"MB\": %zu, \"chunk\": %u, \"stages\": %u, \"ctas_per_sm\": %d, \"us\": %.2f, \"gbs\": %.0f}\n",
                        mb, chunk, nst, ctas, ms * 1e3, bytes / ms / 1e6);
             }
+    for (uint32_t ng : {1u << 20, 1u << 22}) {   // x 8 loads per index
+        for (int k : {4, 8, 16}) {
+            int it = 0;
+            float ms = timeit([&](char* b) { gather_kernel<<<sms * k, 256>>>((const uint32_t*)b, bytes / 4, ng, ++it, out); });
+            const double g = 8.0 * ng;
+            printf("{\"probe\": \"gather64\", \"MB\": %zu, \"gathers\": %.0f, \"ctas_per_sm\": %d, \"us\": %.2f, "
+                   "\"granules_per_s\": %.3e, \"gbs_64B\": %.0f}\n", mb, g, k, ms * 1e3, g / ms * 1e3, g * 64 / ms / 1e6);
+        }
+    }
     return 0;
 }
