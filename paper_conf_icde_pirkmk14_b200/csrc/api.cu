@@ -316,12 +316,28 @@ void ar_column_free(ar_column* col) { delete col; }
 // ------------------------------------------------------------- a2 + a3
 
 // Select workspace: per-tile counts (u32) + offsets (u64) + tile-local candidate slices (pos, aux).
-size_t ar_select_ws_bytes(int64_t n) {
+// Select workspace, for tiles of >= kSelMinTileRows rows (T_max of them):
+//   [group sums u64 x G][tile counts u32 x T_max][pad to 128 B]
+//   [tmp_pos u32 x S][tmp_aux u32 x S]
+// S = n rounded up to kSelMinTileRows (>= the end of the last tile's slice).
+namespace {
+struct SelWs {
+    uint64_t groups, tiles, slice_rows, counts_bytes, tmp_off, bytes;
+};
+SelWs sel_ws(int64_t n) {
+    SelWs w;
     const uint64_t rows = (uint64_t)std::max<int64_t>(n, 0);
-    const uint64_t tiles = ceil_div_u64(rows, ard::kSelMinTileRows);
-    const uint64_t slice_rows = tiles * ard::kSelMinTileRows;      // >= n, covers the last tile's slice
-    return 16 + 16 * tiles + 8 + 16 + 8 * slice_rows;
+    w.tiles = ceil_div_u64(rows, ard::kSelMinTileRows);
+    w.groups = (w.tiles >> ard::kGroupShift) + 1;
+    w.slice_rows = w.tiles * ard::kSelMinTileRows;
+    w.counts_bytes = 8 * w.groups + 4 * w.tiles;                  // zeroed per call
+    w.tmp_off = (w.counts_bytes + 127) & ~uint64_t(127);
+    w.bytes = 128 + w.tmp_off + 8 * w.slice_rows;                 // + 128: base alignment
+    return w;
 }
+}  // namespace
+
+size_t ar_select_ws_bytes(int64_t n) { return (size_t)sel_ws(n).bytes; }
 
 // Shared predicate setup of ar_approx_select / ar_select_refine_sum.
 static ar_status setup_scan(const ar_pred* preds, int32_t npred, ard::SelParams& P, bool& empty, int64_t& n,
@@ -475,25 +491,21 @@ ar_status ar_approx_select(const ar_pred* preds, int32_t npred, int32_t flags, a
     P.out_pos = out->pos;
     P.out_aux = out->aux;
     P.out_count = (long long*)out->count;
-    // workspace: [16 B pad][counts u32 x T (+pad)][group sums u64][tmp_pos][tmp_aux]
-    const uint64_t T = (uint64_t)P.num_tiles;
-    P.tile_count = (uint32_t*)((char*)ws + 16);
-    P.group_sum = (unsigned long long*)((char*)ws + 16 + 8 * ((T + 1) / 2));
-    const uint64_t ngroups = (T + (1u << ard::kGroupShift) - 1) >> ard::kGroupShift;
-    AR_TRY_CUDA(cudaMemsetAsync(P.group_sum, 0, 8 * ngroups, s));
-    const uint64_t slice_rows = ceil_div_u64((uint64_t)n, ard::kSelMinTileRows) * ard::kSelMinTileRows;
-    char* tmp = (char*)ws + 16 + 16 * ceil_div_u64((uint64_t)n, ard::kSelMinTileRows) + 8;
-    tmp = (char*)(((uintptr_t)tmp + 15) & ~uintptr_t(15));
-    P.tmp_pos = (uint32_t*)tmp;
-    P.tmp_aux = P.tmp_pos + slice_rows;
-    (void)T;
+    // workspace (sel_ws): group sums and tile counts (zeroed), tile slices
+    const SelWs L = sel_ws(n);
+    char* base = (char*)(((uintptr_t)ws + 127) & ~uintptr_t(127));
+    P.group_sum = (unsigned long long*)base;
+    P.tile_count = (uint32_t*)(base + 8 * L.groups);
+    AR_TRY_CUDA(cudaMemsetAsync(base, 0, L.counts_bytes, s));
+    P.tmp_pos = (uint32_t*)(base + L.tmp_off);
+    P.tmp_aux = P.tmp_pos + L.slice_rows;
     g_last_scan = "select_tile_kernel";
     const void* fn = select_kernel_fn(P, false);
     P.nstages = 1;
     const size_t smem = select_smem_bytes(P.stage_words, 1, true);
     ar_status st2 = launch_scan(fn, P, (int)P.num_tiles, smem, false, s);
     if (st2 != AR_OK) return st2;
-    return launch_select_rest(P, s);
+    return launch_select_rest(P, env_int("AR_SEL_PDL", 1) != 0, s);
 }
 
 // ------------------------------------------------------------------ a5

@@ -42,7 +42,7 @@ constexpr int kSelWarps = 4;                      // consumer warps per CTA
 constexpr int kSelThreads = kSelWarps * 32;       // each consumer thread owns BPT consecutive 32-row blocks
 constexpr int kSelMinTileRows = kSelThreads * 32; // tile rows = 4096 * BPT (BPT in {1, 2, 4})
 constexpr int kStageEntries = 2048;
-constexpr int kGroupShift = 8;                    // select: 256 tiles per offset group               // output staging entries (pos + aux) per round
+constexpr int kGroupShift = 8;                    // select: 256 tiles per offset group
 
 struct SelParams {
     SelPred p[AR_MAX_PRED];
@@ -206,7 +206,7 @@ int kernel_bpt(bool fused);
 const void* select_kernel_fn(const ard::SelParams& P, bool fused);
 int select_occupancy(const void* fn, size_t smem, bool fused);
 ar_status launch_scan(const void* fn, const ard::SelParams& P, int grid, size_t smem, bool fused, cudaStream_t s);
-ar_status launch_select_rest(const ard::SelParams& P, cudaStream_t s);
+ar_status launch_select_rest(const ard::SelParams& P, bool pdl, cudaStream_t s);
 // ar_select_refine_sum_ws workspace: a ticket word (padded), then kSrsMaxGrid CTA partials of 4 x u64
 constexpr size_t kSrsTicketBytes = 128;
 constexpr int kSrsMaxGrid = 2048;

@@ -81,6 +81,17 @@ __device__ __forceinline__ uint32_t row_of(const uint32_t (&x)[W], uint32_t l) {
     return v;
 }
 
+// Bits l of planes x[0..W) as a W-bit value (bit j from plane j): two
+// instructions per plane -- shift the plane's bit l down to bit 0, then funnel
+// it into the top of the accumulator -- and one final shift.
+template <int W>
+__device__ __forceinline__ uint32_t row_bits(const uint32_t (&x)[W], uint32_t l) {
+    uint32_t acc = 0;
+#pragma unroll
+    for (int j = 0; j < W; ++j) acc = __funnelshift_r(acc, x[j] >> l, 1);
+    return W >= 32 ? acc : acc >> (32 - W);
+}
+
 // Per-block evaluation of every predicate on the 32 rows of block `blk` of a
 // stage (vm = valid rows): candidate mask cm (major in the candidate range of
 // every predicate), definite mask dm (major in the definite range of every

@@ -27,7 +27,7 @@
 // overlap), then the SUM factors of the exact rows are gathered the same way.
 #include <type_traits>
 
-#include "kernels.cuh"
+#include "rl_common.cuh"
 
 namespace ard {
 
@@ -245,11 +245,9 @@ struct FixedPlanes {
                                                          uint32_t l) {
         if constexpr (C < N) {
             constexpr int w = wid<Ws...>(C), o = woff<Ws...>(C);
-            const uint32_t* pl = stg + P.p[C].soff + blk * w;
-            uint32_t a = 0;
-#pragma unroll
-            for (int j = 0; j < w; ++j) a |= ((pl[j] >> l) & 1u) << (o + j);
-            return a | appr_smem<C + 1>(P, stg, blk, l);
+            uint32_t x[w];   // the block's planes: vector loads (a block starts at a multiple of w words)
+            rl::lds_words<w>(x, stg + P.p[C].soff + blk * w);
+            return (rl::row_bits<w>(x, l) << o) | appr_smem<C + 1>(P, stg, blk, l);
         } else {
             return 0u;
         }
@@ -450,6 +448,8 @@ __global__ void __launch_bounds__(NW * 32) select_tile_kernel(const __grid_const
     }
     __syncthreads();
     mbar_wait(&bar, 0, 0);
+    // compact_kernel (a programmatic dependent) may be scheduled once every tile is loaded
+    asm volatile("griddepcontrol.launch_dependents;" ::: "memory");
 
     const int64_t r0 = t * (int64_t)P.tile_rows + (int64_t)threadIdx.x * (32 * BPT);
     PS ps;
@@ -505,6 +505,7 @@ __global__ void __launch_bounds__(NW * 32) select_tile_kernel(const __grid_const
 // atomic per tile by the select kernel) plus the counts of the earlier tiles of
 // its own group -- two short warp reductions, no separate scan kernel.
 __global__ void __launch_bounds__(256) compact_kernel(const __grid_constant__ SelParams P) {
+    asm volatile("griddepcontrol.wait;" ::: "memory");   // no-op unless launched as a dependent
     const unsigned lane = threadIdx.x & 31;
     const long long nw = (long long)gridDim.x * 8;
     for (long long t = (long long)blockIdx.x * 8 + (threadIdx.x >> 5); t < P.num_tiles; t += nw) {
@@ -534,6 +535,13 @@ __global__ void __launch_bounds__(256) compact_kernel(const __grid_constant__ Se
                     P.out_aux[off + j] = va[k];
                 }
             }
+        }
+        __syncwarp();
+        // the slice is dead: drop its L2 lines without writing them back (slices are
+        // 128-B aligned, 32 entries per line)
+        for (uint32_t L = lane; L < (c + 31) / 32; L += 32) {
+            asm volatile("discard.global.L2 [%0], 128;" ::"l"(sp + 32 * L) : "memory");
+            asm volatile("discard.global.L2 [%0], 128;" ::"l"(sa + 32 * L) : "memory");
         }
     }
 }
@@ -939,10 +947,22 @@ ar_status launch_scan(const void* fn, const ard::SelParams& P, int grid, size_t 
     return AR_OK;
 }
 
-ar_status launch_select_rest(const ard::SelParams& P, cudaStream_t s) {
+// compact_kernel; after the persistent select it is a programmatic dependent
+// launch (the select's producer triggers it once its last tile is loading).
+ar_status launch_select_rest(const ard::SelParams& P, bool pdl, cudaStream_t s) {
     const int grid = (int)std::min<long long>((P.num_tiles + 7) / 8, (long long)num_sms() * 8);
-    ard::compact_kernel<<<grid, 256, 0, s>>>(P);
-    AR_CHECK_LAUNCH("compact_kernel");
+    ard::SelParams Q = P;
+    void* args[] = {&Q};
+    cudaLaunchConfig_t cfg = {};
+    cfg.gridDim = dim3(grid);
+    cfg.blockDim = dim3(256);
+    cfg.stream = s;
+    cudaLaunchAttribute attr[1];
+    attr[0].id = cudaLaunchAttributeProgrammaticStreamSerialization;
+    attr[0].val.programmaticStreamSerializationAllowed = pdl ? 1 : 0;
+    cfg.attrs = attr;
+    cfg.numAttrs = 1;
+    AR_TRY_CUDA(cudaLaunchKernelExC(&cfg, (const void*)ard::compact_kernel, args));
     return AR_OK;
 }
 
