@@ -706,6 +706,34 @@ ar_status ar_refine_sum(const ar_cands* in, const ar_pred* preds, int32_t npred,
     P.nagg = ncols;
     P.out_sum = (unsigned long long*)out_sum_dev;
     P.out_cnt = (unsigned long long*)out_count_dev;
+    // specialised kernel: exactly one checked predicate, SLICED residual of 4 / 8 planes, carried
+    // major; factors = k = 0 carried predicate columns and at most one bit-packed gathered column
+    P.fast_k = 0;
+    P.fast_chk = -1;
+    P.fast_g = -1;
+    {
+        static const int off = env_int("AR_REFINE_GENERIC", 0);
+        bool ok = !off;
+        int nchk = 0;
+        for (int c = 0; c < P.npred; ++c) {
+            const ard::RefPred& p = P.p[c];
+            if (!p.check) continue;
+            ++nchk;
+            P.fast_chk = c;
+            ok = ok && p.carried && p.rlayout == AR_LAYOUT_SLICED && (p.k == 4 || p.k == 8);
+        }
+        ok = ok && nchk == 1;
+        for (int i = 0; i < ncols && ok; ++i) {
+            const ard::AggCol& a = P.a[i];
+            if (a.pred >= 0 && a.k == 0 && P.p[a.pred].carried && a.flip == 0) continue;
+            if (a.pred < 0 && a.k == 0 && a.layout == AR_LAYOUT_PACKED && a.w > 0 && a.flip == 0 && P.fast_g < 0) {
+                P.fast_g = i;
+                continue;
+            }
+            ok = false;
+        }
+        if (ok) P.fast_k = (int32_t)P.p[P.fast_chk].k;
+    }
     cudaStream_t s = (cudaStream_t)stream;
     if (out_sum_dev) AR_TRY_CUDA(cudaMemsetAsync(out_sum_dev, 0, sizeof(int64_t), s));
     if (out_count_dev) AR_TRY_CUDA(cudaMemsetAsync(out_count_dev, 0, sizeof(int64_t), s));

@@ -167,6 +167,8 @@ struct RefParams {
     int32_t nagg;
     unsigned long long* out_sum;
     unsigned long long* out_cnt;
+    // refine_sum_sliced_kernel (fast_k = 4 / 8, else 0): the one checked predicate and the gathered factor
+    int32_t fast_k, fast_chk, fast_g;
 };
 
 struct SumParams {
