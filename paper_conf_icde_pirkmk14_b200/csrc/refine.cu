@@ -9,7 +9,7 @@
 // positions and of aux words), so its residual gathers are independent loads
 // in flight together.  Refine keeps order with the same decoupled look-back
 // as a3; refine+SUM needs no order (integer sums are exact in any order).
-#include "kernels.cuh"
+#include "rl_common.cuh"
 
 namespace ard {
 
@@ -193,6 +193,96 @@ __global__ void __launch_bounds__(kRefThreads, 4) refine_sum_kernel(const __grid
     if (P.out_cnt) block_add(kept, P.out_cnt);
 }
 
+// Refine + SUM specialised for one decomposed predicate with a SLICED
+// residual of K = 4 / 8 planes (a 32-row block's residual is one 16 / 32-B
+// sector) and SUM factors that are k = 0 predicate columns (value in the aux
+// word) or at most one bit-packed gathered column (l_extendedprice in Q6).
+// Straight-line code (no per-candidate branches), so each thread's gathers are
+// in flight together:
+//   phase 1: residual sectors of the non-definite candidates AND the gathered
+//            factor of the definite ones (kept for sure: Alg. 2 never touches
+//            them);
+//   phase 2: the gathered factor of the non-definite candidates that survived.
+template <int K>
+__global__ void __launch_bounds__(kRefThreads, 2) refine_sum_sliced_kernel(const __grid_constant__ RefParams P) {
+    const long long count = *P.in_count;
+    const long long num_tiles = (count + kRefTile - 1) / kRefTile;
+    const RefPred& q = P.p[P.fast_chk];
+    const uint32_t qmask = q.w == 32 ? 0xffffffffu : ((1u << q.w) - 1u);
+    const int g = P.fast_g;   // gathered factor, or -1
+    unsigned long long sum = 0, kept = 0;
+    for (long long t = blockIdx.x; t < num_tiles; t += gridDim.x) {
+        const uint64_t j0 = (uint64_t)t * kRefTile + threadIdx.x * kRefPerThread;
+        uint32_t pos[8], aux[8];
+        load8(P.in_pos, j0, count, pos);
+        load8(P.in_aux, j0, count, aux);
+        uint32_t valid = 0, def = 0;
+#pragma unroll
+        for (int i = 0; i < 8; ++i) {
+            valid |= (j0 + i < (uint64_t)count ? 1u : 0u) << i;
+            def |= (aux[i] >> 31) << i;
+        }
+        def &= valid;
+        const uint32_t need = valid & ~def;
+        // phase 1
+        uint4 ra[8], rb[8];
+#pragma unroll
+        for (int i = 0; i < 8; ++i) {
+            const uint32_t* blk = q.residual + (uint64_t)(pos[i] >> 5) * K;
+            ra[i] = ld_gather_if4(blk, (need >> i) & 1u);
+            if constexpr (K == 8) rb[i] = ld_gather_if4(blk + 4, (need >> i) & 1u);
+        }
+        uint32_t gv[8];
+        if (g >= 0) {
+            const AggCol& a = P.a[g];
+#pragma unroll
+            for (int i = 0; i < 8; ++i) gv[i] = packed_get_if(a.major, pos[i], (int)a.w, (def >> i) & 1u);
+        }
+        uint32_t keep = def;
+#pragma unroll
+        for (int i = 0; i < 8; ++i) {
+            const uint32_t l = pos[i] & 31u;
+            uint32_t x[K];
+            x[0] = ra[i].x; x[1] = ra[i].y; x[2] = ra[i].z; x[3] = ra[i].w;
+            if constexpr (K == 8) {
+                x[4] = rb[i].x; x[5] = rb[i].y; x[6] = rb[i].z; x[7] = rb[i].w;
+            }
+            const uint32_t r = rl::row_bits<K>(x, l);
+            const uint32_t v = ((((aux[i] >> q.ashift) & qmask) << K) | r) + q.base;
+            keep |= (((need >> i) & 1u) && v >= q.lo && v <= q.hi ? 1u : 0u) << i;
+        }
+        kept += __popc(keep);
+        if (P.nagg == 0 || !keep) continue;
+        // phase 2
+        if (g >= 0) {
+            const AggCol& a = P.a[g];
+            const uint32_t late = keep & need;
+#pragma unroll
+            for (int i = 0; i < 8; ++i) {
+                const uint32_t v = packed_get_if(a.major, pos[i], (int)a.w, (late >> i) & 1u);
+                gv[i] = ((late >> i) & 1u ? v : gv[i]) + a.base;
+            }
+        }
+#pragma unroll
+        for (int i = 0; i < 8; ++i) {
+            if (!((keep >> i) & 1u)) continue;
+            unsigned long long prod = 1;
+            for (int c = 0; c < P.nagg; ++c) {
+                const AggCol& a = P.a[c];
+                if (c == g) {
+                    prod *= gv[i];
+                } else {
+                    const RefPred& p = P.p[a.pred];
+                    prod *= ((aux[i] >> p.ashift) & (p.w == 32 ? 0xffffffffu : ((1u << p.w) - 1u))) + a.base;
+                }
+            }
+            sum += prod;
+        }
+    }
+    if (P.out_sum) block_add(sum, P.out_sum);
+    if (P.out_cnt) block_add(kept, P.out_cnt);
+}
+
 __global__ void __launch_bounds__(kRefThreads) sum_kernel(const __grid_constant__ SumParams P) {
     const long long count = *P.count;
     unsigned long long sum = 0;
@@ -286,6 +376,17 @@ ar_status launch_refine(const ard::RefParams& P, int grid, cudaStream_t s) {
     return AR_OK;
 }
 ar_status launch_refine_sum(const ard::RefParams& P, int grid, cudaStream_t s) {
+    if (P.fast_k == 8 || P.fast_k == 4) {
+        const void* fn = P.fast_k == 8 ? (const void*)ard::refine_sum_sliced_kernel<8>
+                                       : (const void*)ard::refine_sum_sliced_kernel<4>;
+        int occ = 0;
+        cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, fn, ard::kRefThreads, 0);
+        const int g2 = std::max(1, std::min(grid, num_sms() * std::max(occ, 1)));
+        ard::RefParams Q = P;
+        void* args[] = {&Q};
+        AR_TRY_CUDA(cudaLaunchKernel(fn, dim3(g2), dim3(ard::kRefThreads), args, 0, s));
+        return AR_OK;
+    }
     ard::refine_sum_kernel<<<grid, ard::kRefThreads, 0, s>>>(P);
     AR_CHECK_LAUNCH("refine_sum_kernel");
     return AR_OK;
