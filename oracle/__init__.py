@@ -18,6 +18,10 @@ Pins (tests/test_oracle_*.py):
   sum_at          closed forms
   sum_bounds      brute force over every residual of tiny tables, k = 0 collapse to the
                   exact answer, closed forms, containment of the exact answer
+  select_minmax   pure-Python brute force on tiny tables, closed forms
+  minmax_ar       Fig. 6 (the false positive holds the single minimal
+                  approximation, the propagated set still holds the true minimum), refined
+                  answer == select_minmax, bounds contain it, k = 0 collapse, brute force
 No function is "parity unpinned".
 """
 from __future__ import annotations
@@ -63,6 +67,8 @@ def _load():
         lib.or_sum_at.restype = i32
         lib.or_sum_bounds.argtypes = [i64, i32, p, p, p, p, p, i32, p, p, p, p]
         lib.or_sum_bounds.restype = i32
+        lib.or_select_minmax.argtypes = [i64, i32, p, p, p, p, p, i32, i32, p]
+        lib.or_minmax_ar.argtypes = [i64, i32, p, p, p, p, p, p, i32, u32, i32, i32, p, p]
         lib.or_threads_default.restype = i32
         _lib = lib
     return _lib
@@ -187,3 +193,51 @@ def sum_bounds(pred_cols, pred_ks, los, his, agg_cols=(), agg_ks=(), pred_bases=
                              nagg, ctypes.cast(ac, ctypes.c_void_p), _ptr(aks), _ptr(ab), _ptr(out)):
         raise OverflowError("SUM bound does not fit in int64")
     return tuple(int(x) for x in out)
+
+
+def select_minmax(pred_cols, los, his, ycol, mode: str = "min", signed=None, y_signed: bool = False):
+    """Exact select min(Y) / max(Y) over the conjunction (the plain definition):
+    (value, |R|); value is 0 when R is empty."""
+    sg = None
+    if signed is not None:
+        sg = np.asarray([1 if x else 0 for x in signed], dtype=np.int32)
+        pred_cols = [np.ascontiguousarray(c).view(np.uint32) if np.asarray(c).dtype == np.int32 else c
+                     for c in pred_cols]
+        los = [int(x) & 0xFFFFFFFF for x in los]
+        his = [int(x) & 0xFFFFFFFF for x in his]
+    pred_cols = [_u32(c) for c in pred_cols]
+    y = np.ascontiguousarray(ycol).view(np.uint32) if np.asarray(ycol).dtype == np.int32 else _u32(ycol)
+    n = y.size
+    lo = np.asarray(los, dtype=np.uint32)
+    hi = np.asarray(his, dtype=np.uint32)
+    out = np.zeros(2, dtype=np.int64)
+    pc = _ptr_array(pred_cols)
+    _load().or_select_minmax(n, len(pred_cols), ctypes.cast(pc, ctypes.c_void_p), _ptr(lo), _ptr(hi),
+                             _ptr(sg) if sg is not None else None, _ptr(y), 1 if y_signed else 0,
+                             0 if mode == "min" else 1, _ptr(out))
+    return int(out[0]), int(out[1])
+
+
+def minmax_ar(pred_cols, pred_ks, los, his, ycol, y_k: int, mode: str = "min", pred_bases=None,
+              y_base: int = 0, y_signed: bool = False, flags: bool = False):
+    """A&R MIN / MAX of s IV-F: dict with the refined answer and survivors,
+    the approximate bounds (lo, hi), |refined|, |D|, |C|, and (flags=True) the refined-row mask."""
+    pred_cols = [_u32(c) for c in pred_cols]
+    y = np.ascontiguousarray(ycol).view(np.uint32) if np.asarray(ycol).dtype == np.int32 else _u32(ycol)
+    n = y.size
+    npred = len(pred_cols)
+    pks = np.asarray(pred_ks, dtype=np.int32)
+    pb = np.asarray(pred_bases if pred_bases is not None else [0] * npred, dtype=np.uint32)
+    lo = np.asarray(los, dtype=np.uint32)
+    hi = np.asarray(his, dtype=np.uint32)
+    out = np.zeros(7, dtype=np.int64)
+    fl = np.zeros(max(n, 1), dtype=np.uint8)
+    pc = _ptr_array(pred_cols)
+    _load().or_minmax_ar(n, npred, ctypes.cast(pc, ctypes.c_void_p), _ptr(pks), _ptr(pb), _ptr(lo), _ptr(hi),
+                         _ptr(y), y_k, y_base & 0xFFFFFFFF, 1 if y_signed else 0, 0 if mode == "min" else 1,
+                         _ptr(out), _ptr(fl) if flags else None)
+    r = {"value": int(out[0]), "survivors": int(out[1]), "lo": int(out[2]), "hi": int(out[3]),
+         "refined": int(out[4]), "definite": int(out[5]), "candidates": int(out[6])}
+    if flags:
+        r["refine_flags"] = fl[:n].astype(bool)
+    return r

@@ -307,3 +307,133 @@ int or_sum_bounds(int64_t n, int npred, const uint32_t* const* pcols, const int*
     out[3] = ncand;
     return shi > (__int128)INT64_MAX;
 }
+
+/* -------------------------------------------------------- MIN / MAX (Fig. 6) */
+
+/*
+ * Exact  select min(Y) / max(Y) from R where <conjunction>: the plain
+ * definition (s IV-F).  mode 0 = MIN, 1 = MAX.  ysgn = 1
+ * compares Y as int32.  out[0] = the aggregate (as int64; 0 when R is empty),
+ * out[1] = |R|.
+ */
+void or_select_minmax(int64_t n, int npred, const uint32_t* const* pcols, const uint32_t* lo, const uint32_t* hi,
+                      const int* sgn, const uint32_t* ycol, int ysgn, int mode, int64_t* out) {
+    sel_ctx c;
+    memset(&c, 0, sizeof(c));
+    c.npred = npred; c.pcols = pcols; c.lo = lo; c.hi = hi; c.sgn = sgn;
+    int64_t count = 0, best = 0;
+    for (int64_t i = 0; i < n; ++i) {
+        if (!row_qualifies(&c, i)) continue;
+        int64_t v = ysgn ? (int64_t)(int32_t)ycol[i] : (int64_t)ycol[i];
+        if (count == 0 || (mode == 0 ? v < best : v > best)) best = v;
+        ++count;
+    }
+    out[0] = count ? best : 0;
+    out[1] = count;
+}
+
+/*
+ * A&R MIN / MAX, step by step as s IV-F describes it:
+ *  1. approximate selection: candidate / definite rows of the conjunction by
+ *     the bucket definition (or_bucket_flags);
+ *  2. "the error bounds of the applied selections are propagated to the
+ *     aggregation": with Y's majors m (key u = v ^ flip - b, m = u >> ky), a
+ *     definite row is certainly in R, so for MIN the true minimum is at most
+ *     the top of the bucket of the smallest definite major mD; every row whose
+ *     major exceeds mD is larger than that definite row and cannot be the
+ *     minimum.  The approximation of the minimum is therefore the set of
+ *     candidates with m <= mD (all candidates when no row is definite), which
+ *     "assuredly include[s] the tuple ID of the actual minimum" -- not merely
+ *     the rows with the minimal approximation, which may be a false positive
+ *     (Fig. 6).  MAX mirrors it (m >= the largest definite major MD).
+ *     Approximate answer before refinement (bucket ends, key domain):
+ *       MIN in [bmin(min_C m), D ? bmax(mD) : bmax(max_C m)]
+ *       MAX in [D ? bmin(MD) : bmin(min_C m), bmax(max_C m)]
+ *  3. refinement: "a join of the candidate set with the input residuals and
+ *     the calculation of the minimum": the exact predicates
+ *     and the exact Y on the set of step 2.
+ * pks / pbase: k and base of each predicate column; ky / ybase: of Y.  Bounds
+ * and the result are values (int32 when ysgn).  out[0] = refined aggregate
+ * (0 if no refined row survives), out[1] = survivors of the refinement (>= 1
+ * iff R is not empty), out[2] / out[3] = approximate lower / upper bound
+ * (0 / 0 when there is no candidate), out[4] = rows refined (|set of step 2|),
+ * out[5] = |D|, out[6] = |C|.  refine_flag (optional, n bytes) marks the rows
+ * of step 2.
+ */
+void or_minmax_ar(int64_t n, int npred, const uint32_t* const* pcols, const int* pks, const uint32_t* pbase,
+                  const uint32_t* lo, const uint32_t* hi, const uint32_t* ycol, int ky, uint32_t ybase, int ysgn,
+                  int mode, int64_t* out, uint8_t* refine_flag) {
+    uint32_t flip = ysgn ? 0x80000000u : 0u;
+    uint64_t two_ky = (uint64_t)1 << ky;
+    uint8_t* cand = (uint8_t*)calloc((size_t)(n > 0 ? n : 1), 1);
+    uint8_t* def = (uint8_t*)calloc((size_t)(n > 0 ? n : 1), 1);
+    /* 1. approximate selection */
+    for (int64_t i = 0; i < n; ++i) {
+        int c = 1, d = 1;
+        for (int p = 0; p < npred; ++p) {
+            uint64_t two_k = (uint64_t)1 << pks[p];
+            uint64_t m = (uint64_t)(uint32_t)(pcols[p][i] - pbase[p]) / two_k;
+            uint64_t first = (uint64_t)pbase[p] + m * two_k;
+            uint64_t last = first + two_k - 1;
+            if (!(lo[p] <= hi[p] && first <= hi[p] && last >= lo[p])) c = 0;
+            if (!(first >= lo[p] && last <= hi[p])) d = 0;
+        }
+        cand[i] = (uint8_t)c;
+        def[i] = (uint8_t)(c && d);
+    }
+    /* 2. propagate the selection's error bounds to the aggregation */
+    int64_t nc = 0, nd = 0;
+    uint64_t minC = 0, maxC = 0, minD = 0, maxD = 0;
+    for (int64_t i = 0; i < n; ++i) {
+        if (!cand[i]) continue;
+        uint64_t m = (uint64_t)((ycol[i] ^ flip) - ybase) / two_ky;
+        if (nc == 0 || m < minC) minC = m;
+        if (nc == 0 || m > maxC) maxC = m;
+        ++nc;
+        if (def[i]) {
+            if (nd == 0 || m < minD) minD = m;
+            if (nd == 0 || m > maxD) maxD = m;
+            ++nd;
+        }
+    }
+    int64_t nref = 0, surv = 0, best = 0;
+    int64_t blo = 0, bhi = 0;
+    if (nc > 0) {
+        uint64_t mlo = mode == 0 ? minC : (nd ? maxD : minC);   /* bucket whose bottom bounds the answer */
+        uint64_t mhi = mode == 0 ? (nd ? minD : maxC) : maxC;   /* bucket whose top bounds the answer */
+        uint64_t klo = (uint64_t)ybase + mlo * two_ky;
+        uint64_t khi = (uint64_t)ybase + mhi * two_ky + two_ky - 1;
+        if (khi > 0xffffffffull) khi = 0xffffffffull;
+        uint32_t vlo = (uint32_t)klo ^ flip, vhi = (uint32_t)khi ^ flip;
+        blo = ysgn ? (int64_t)(int32_t)vlo : (int64_t)vlo;
+        bhi = ysgn ? (int64_t)(int32_t)vhi : (int64_t)vhi;
+        /* 3. refine the rows that can hold the answer */
+        uint64_t thr = mode == 0 ? (nd ? minD : maxC) : (nd ? maxD : minC);
+        for (int64_t i = 0; i < n; ++i) {
+            if (refine_flag) refine_flag[i] = 0;
+            if (!cand[i]) continue;
+            uint64_t m = (uint64_t)((ycol[i] ^ flip) - ybase) / two_ky;
+            if (mode == 0 ? m > thr : m < thr) continue;
+            if (refine_flag) refine_flag[i] = 1;
+            ++nref;
+            int ok = 1;
+            for (int p = 0; p < npred; ++p)
+                if (!(lo[p] <= pcols[p][i] && pcols[p][i] <= hi[p])) ok = 0;
+            if (!ok) continue;
+            int64_t v = ysgn ? (int64_t)(int32_t)ycol[i] : (int64_t)ycol[i];
+            if (surv == 0 || (mode == 0 ? v < best : v > best)) best = v;
+            ++surv;
+        }
+    } else if (refine_flag) {
+        memset(refine_flag, 0, (size_t)n);
+    }
+    out[0] = surv ? best : 0;
+    out[1] = surv;
+    out[2] = blo;
+    out[3] = bhi;
+    out[4] = nref;
+    out[5] = nd;
+    out[6] = nc;
+    free(cand);
+    free(def);
+}
