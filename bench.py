@@ -345,8 +345,12 @@ def ours(args):
         step("fused", 0)
     stream.synchronize()
     fused_name = _ar.ar_last_scan_kernel() or "fused_kernel"
+    with torch.cuda.stream(stream):
+        step("staged", 0)
+    stream.synchronize()
+    ref_name = _ar.ar_last_scan_kernel() or "refine_sum_kernel"   # the specialised or the general refine+SUM
     SEL = "select_tile_kernel+compact_kernel"   # ar_approx_select: two launches (+ memsets)
-    KERNELS = {"staged": ["select_tile_kernel", "compact_kernel", "refine_sum_kernel"]
+    KERNELS = {"staged": ["select_tile_kernel", "compact_kernel", ref_name]
                + (["exclusive_offset_kernel"] if dist_h else []),
                "fused": [fused_name]}
     K = args.steps
@@ -399,7 +403,7 @@ def ours(args):
             ms_total = float(t.item())
         if variant == "staged":
             kern = {SEL: [elapsed(e[0], e[1]) for e in evs],
-                    "refine_sum_kernel": [elapsed(e[2], e[3]) for e in evs]}
+                    ref_name: [elapsed(e[2], e[3]) for e in evs]}
         else:
             kern = {fused_name: [elapsed(e[0], e[1]) for e in evs]}
         res = out.cpu().tolist()
@@ -423,7 +427,7 @@ def ours(args):
     per_kernel_bytes = {
         fused_name: ab["total"],                                            # majors + touched residual/ep sectors
         SEL: ab["scan"] + ab["cand_list_bytes"],                            # majors read + (pos, aux) written
-        "refine_sum_kernel": ab["cand_list_bytes"] + ab["gather"] + 16.0,   # cands read + sector gathers + out
+        ref_name: ab["cand_list_bytes"] + ab["gather"] + 16.0,   # cands read + sector gathers + out
     }
 
     variants = [args.variant] + [v for v in ("fused", "staged") if v != args.variant and not args.only]

@@ -153,11 +153,12 @@ typedef struct {
 const char* ar_status_str(ar_status s);
 const char* ar_last_error(void);     /* thread-local detail of the last failure */
 const char* ar_version(void);
-/* Name of the scan kernel the calling thread's last ar_select_refine_sum or
- * ar_approx_select launched: "fused_rl_kernel" (result-ring one-pass kernel),
- * "fused_kernel" (general one-pass kernel), "select_tile_kernel" (ordered
- * select), "" (none: empty input or an error).  Static storage; for tests and benchmarks that
- * must know which path ran. */
+/* Name of the main kernel the calling thread's last ar_select_refine_sum,
+ * ar_approx_select or ar_refine_sum launched: "fused_rl_kernel" (result-ring
+ * one-pass kernel), "fused_kernel" (general one-pass kernel),
+ * "select_tile_kernel" (ordered select), "refine_sum_sliced_kernel" /
+ * "refine_sum_kernel" (refine + SUM), "" (none: empty input or an error).
+ * Static storage; for tests and benchmarks that must know which path ran. */
 const char* ar_last_scan_kernel(void);
 
 /* --------------------------------------------------- a1: decomposition */
@@ -284,6 +285,39 @@ ar_status ar_sum(const ar_positions* pos, const ar_column* const* cols, int32_t 
  */
 ar_status ar_sum_approximate(const ar_cands* in, const ar_column* const* cols, int32_t ncols,
                              int64_t* out4_dev, void* stream);
+
+/*
+ * MIN / MAX over the exact result (s IV-F, Fig. 6):
+ * select min(Y) / max(Y) from R where <preds>, from the candidate relation
+ * `in` of ar_approx_select over the same `preds`.  "The result of the
+ * approximation of a minimum has to assuredly include the tuple ID of the
+ * actual minimum.  To guarantee this, the error bounds of the applied
+ * selections are propagated to the aggregation": with Y's
+ * majors m (key domain), a definite candidate is certainly in R, so
+ * only candidates with m <= min over definite candidates (MIN; m >= max over
+ * definite candidates for MAX; every candidate when none is definite) can hold
+ * the answer.  Those are refined -- the exact predicates (Alg. 2), then Y's
+ * exact value from its residual ("a join of the candidate set with the input
+ * residuals and the calculation of the minimum").
+ * `col` is any column of the table (it may be a predicate column; its major
+ * is then taken from the carried approximation).  Writes device int64[7]:
+ *   out7[0] = the exact MIN / MAX (a signed column's value as int32; 0 if out7[1] == 0)
+ *   out7[1] = refined rows that satisfy the predicates (>= 1 iff R is not empty)
+ *   out7[2], out7[3] = approximate answer before refinement, lower / upper bound
+ *             (bucket ends; 0, 0 without candidates):
+ *             MIN in [bmin(min_C m), D ? bmax(min_D m) : bmax(max_C m)]
+ *             MAX in [D ? bmin(max_D m) : bmin(min_C m), bmax(max_C m)]
+ *   out7[4] = candidates refined, out7[5] = |definite|, out7[6] = |candidates|
+ * `ws` is a caller-owned device workspace of ar_minmax_ws_bytes() bytes
+ * (initialised by the call).  Four kernel launches on `stream`.
+ * Errors: AR_ERR_INVALID (null pointers, bad mode, predicates that do not
+ * match the candidate relation), AR_ERR_RANGE (workspace too small).
+ */
+#define AR_MIN 0
+#define AR_MAX 1
+size_t ar_minmax_ws_bytes(void);
+ar_status ar_minmax(const ar_cands* in, const ar_pred* preds, int32_t npred, const ar_column* col, int32_t mode,
+                    int64_t* out7_dev, void* ws, size_t ws_bytes, void* stream);
 
 /*
  * Positional projection of one column at the rows of `pos` (the invisible /

@@ -20,6 +20,7 @@ AR_SELECT_CARRY_APPR = 1
 AR_DECOMPOSE_SIGNED, AR_DECOMPOSE_BASE_MIN = 1, 2
 AR_AUX_DEFINITE = 0x80000000
 AR_PROJECT_APPROX, AR_PROJECT_EXACT = 0, 1
+AR_MIN, AR_MAX = 0, 1
 AR_SRS_PDL, AR_SRS_PDL_EARLY_READ = 1, 2
 
 
@@ -77,6 +78,8 @@ SIGNATURES = {
     "ar_sum": (ctypes.c_int, [ctypes.POINTER(Positions), ctypes.POINTER(_P), _I32, _P, _P]),
     "ar_sum_approximate": (ctypes.c_int, [ctypes.POINTER(Cands), ctypes.POINTER(_P), _I32, _P, _P]),
     "ar_project": (ctypes.c_int, [ctypes.POINTER(Positions), _P, _I32, _P, _P]),
+    "ar_minmax_ws_bytes": (_SZ, []),
+    "ar_minmax": (ctypes.c_int, [ctypes.POINTER(Cands), ctypes.POINTER(Pred), _I32, _P, _I32, _P, _P, _SZ, _P]),
     "ar_refine_sum": (ctypes.c_int, [ctypes.POINTER(Cands), ctypes.POINTER(Pred), _I32, ctypes.POINTER(_P), _I32,
                                      _P, _P, _P]),
     "ar_select_refine_sum": (ctypes.c_int, [ctypes.POINTER(Pred), _I32, ctypes.POINTER(_P), _I32, _P, _P]),
@@ -207,6 +210,14 @@ def ar_sum_approximate(cands: Cands, cols, out4_dev, stream):
 
 def ar_project(pos: Positions, col, mode, out_values_dev, stream):
     _call("ar_project", ctypes.byref(pos), col, mode, out_values_dev, stream)
+
+
+def ar_minmax_ws_bytes() -> int:
+    return int(load().ar_minmax_ws_bytes())
+
+
+def ar_minmax(cands: Cands, preds, col, mode, out7_dev, ws, ws_bytes, stream):
+    _call("ar_minmax", ctypes.byref(cands), _preds(preds), len(preds), col, mode, out7_dev, ws, ws_bytes, stream)
 
 
 def ar_refine_sum(cands: Cands, preds, cols, out_sum_dev, out_count_dev, stream):

@@ -203,6 +203,15 @@ def project(pos, col: BWDColumn, exact: bool = True, stream=None) -> torch.Tenso
     return out
 
 
+def minmax(cands: CandidateList, preds, col: BWDColumn, mode: str, out7: torch.Tensor, ws: "Workspace" = None,
+           stream=None):
+    """MIN / MAX of `col` over the refined rows (s IV-F, Fig. 6): out7 = [answer, survivors, approx lower,
+    approx upper, candidates refined, |definite|, |candidates|]."""
+    ws = ws if ws is not None else Workspace(_ar.ar_minmax_ws_bytes(), col.device)
+    _ar.ar_minmax(cands.c, _pred_tuples(preds), col.handle, _ar.AR_MIN if mode == "min" else _ar.AR_MAX,
+                  out7.data_ptr(), ws.ptr, ws.nbytes, _stream(stream))
+
+
 def refine_sum(cands: CandidateList, preds, cols, out_sum: torch.Tensor, out_count: torch.Tensor = None,
                stream=None):
     """Steps a5+a6 fused: out_sum[0] = SUM(prod(cols)) over the refined rows, out_count[0] = their number."""

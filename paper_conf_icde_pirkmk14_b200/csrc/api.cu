@@ -740,7 +740,40 @@ ar_status ar_refine_sum(const ar_cands* in, const ar_pred* preds, int32_t npred,
     const uint64_t max_tiles = ceil_div_u64((uint64_t)std::max<int64_t>(in->capacity, 0), ard::kRefTile);
     if (max_tiles == 0) return AR_OK;
     const int grid = (int)std::min<uint64_t>(max_tiles, (uint64_t)num_sms() * 8);
+    g_last_scan = P.fast_k ? "refine_sum_sliced_kernel" : "refine_sum_kernel";
     return launch_refine_sum(P, grid, s);
+}
+
+// ----------------------------------------------------------- MIN / MAX (s IV-F)
+
+size_t ar_minmax_ws_bytes(void) { return 64; }
+
+ar_status ar_minmax(const ar_cands* in, const ar_pred* preds, int32_t npred, const ar_column* col, int32_t mode,
+                    int64_t* out7_dev, void* ws, size_t ws_bytes, void* stream) {
+    ard::MinMaxParams P;
+    memset(&P, 0, sizeof(P));
+    ar_status st = setup_refine(in, preds, npred, P.r);
+    if (st != AR_OK) return st;
+    if (!out7_dev || !ws || (mode != AR_MIN && mode != AR_MAX)) {
+        set_error("ar_minmax: null output / workspace or mode %d not AR_MIN / AR_MAX", mode);
+        return AR_ERR_INVALID;
+    }
+    if (ws_bytes < ar_minmax_ws_bytes()) {
+        set_error("ar_minmax: workspace %zu < %zu bytes", ws_bytes, ar_minmax_ws_bytes());
+        return AR_ERR_RANGE;
+    }
+    const ar_column* const cols[1] = {col};
+    st = setup_aggs(cols, 1, preds, npred, preds[0].col->d.n, &P.y, 1, true);
+    if (st != AR_OK) return st;
+    P.mode = mode;
+    P.ws = (unsigned int*)ws;
+    P.wc = (unsigned long long*)((char*)ws + 32);
+    P.out7 = (long long*)out7_dev;
+    cudaStream_t s = (cudaStream_t)stream;
+    const int64_t cap = std::max<int64_t>(in->capacity, 1);
+    const int grid = (int)std::min<int64_t>((cap + ard::kRefThreads - 1) / ard::kRefThreads, (int64_t)num_sms() * 8);
+    g_last_scan = "minmax_refine_kernel";
+    return launch_minmax(P, grid, s);
 }
 
 // ----------------------------------------------------------- fused a3+a5+a6

@@ -189,6 +189,16 @@ struct ApproxSumParams {
     unsigned long long* out4;   // [sum_lo, sum_hi, count_lo, count_hi]
 };
 
+// MIN / MAX with the selection's error bounds propagated (s IV-F, Fig. 6)
+struct MinMaxParams {
+    RefParams r;              // candidate relation + predicates (exact re-evaluation)
+    AggCol y;                 // the aggregated column (pred >= 0: its major is in the aux word)
+    int32_t mode;             // AR_MIN / AR_MAX
+    unsigned int* ws;         // [0..3] min/max major over candidates / definite, [4] best exact key (xored)
+    unsigned long long* wc;   // [0] |definite|, [1] rows refined, [2] survivors
+    long long* out7;
+};
+
 // leftjoinapproximate / leftjoinrefine (positional projection)
 struct ProjectParams {
     const uint32_t* pos;
@@ -220,6 +230,7 @@ ar_status launch_refine_sum(const ard::RefParams& P, int grid, cudaStream_t s);
 ar_status launch_sum(const ard::SumParams& P, int grid, cudaStream_t s);
 ar_status launch_approx_sum(const ard::ApproxSumParams& P, int grid, cudaStream_t s);
 ar_status launch_project(const ard::ProjectParams& P, int grid, cudaStream_t s);
+ar_status launch_minmax(const ard::MinMaxParams& P, int grid, cudaStream_t s);
 ar_status launch_decompose_minmax(const uint32_t* col, int64_t n, uint32_t flip, uint32_t* out2, cudaStream_t s);
 ar_status launch_pack_sliced(const uint32_t* col, int64_t n, int shift, uint32_t mask, uint32_t flip, uint32_t base,
                              int w, uint32_t* out, cudaStream_t s);

@@ -299,6 +299,135 @@ __global__ void __launch_bounds__(kRefThreads) sum_kernel(const __grid_constant_
     block_add(sum, P.out_sum);
 }
 
+// MIN / MAX (s IV-F, Fig. 6).  "The result of the
+// approximation of a minimum has to assuredly include the tuple ID of the
+// actual minimum.  To guarantee this, the error bounds of the applied
+// selections are propagated to the aggregation": a definite candidate is
+// certainly in R, so (MIN) nothing whose Y major exceeds the smallest definite
+// major mD can be the minimum.  Three passes over the candidate relation:
+//   minmax_approx_kernel : min / max of Y's major over candidates and over
+//                          definite candidates (the approximate answer);
+//   minmax_refine_kernel : the candidates with major <= mD (MIN; >= MD for MAX;
+//                          every candidate when none is definite) are refined --
+//                          Alg. 2 on the predicates, then Y's residual -- and
+//                          the exact extreme taken ("a join of the candidate set
+//                          with the input residuals and the calculation of the
+//                          minimum");
+//   minmax_final_kernel  : out7 (values mapped back from the key domain).
+__device__ __forceinline__ uint32_t y_major(const MinMaxParams& P, uint32_t pos, uint32_t aux) {
+    const AggCol& y = P.y;
+    if (y.pred >= 0 && P.r.p[y.pred].carried) {
+        const RefPred& p = P.r.p[y.pred];
+        return (aux >> p.ashift) & (p.w == 32 ? 0xffffffffu : ((1u << p.w) - 1u));
+    }
+    return y.w ? major_get(y.major, pos, (int)y.w, (int)y.layout) : 0u;
+}
+
+__global__ void minmax_init_kernel(unsigned int* ws, unsigned long long* wc) {
+    if (threadIdx.x < 5) ws[threadIdx.x] = (threadIdx.x & 1) && threadIdx.x < 4 ? 0u : 0xffffffffu;
+    if (threadIdx.x < 3) wc[threadIdx.x] = 0ull;
+}
+
+__global__ void __launch_bounds__(kRefThreads) minmax_approx_kernel(const __grid_constant__ MinMaxParams P) {
+    const long long count = *P.r.in_count;
+    uint32_t mnC = 0xffffffffu, mxC = 0u, mnD = 0xffffffffu, mxD = 0u;
+    unsigned long long nd = 0;
+    const long long stride = (long long)gridDim.x * kRefThreads;
+    for (long long j = (long long)blockIdx.x * kRefThreads + threadIdx.x; j < count; j += stride) {
+        const uint32_t pos = P.r.in_pos[j], aux = P.r.in_aux[j];
+        const uint32_t m = y_major(P, pos, aux);
+        mnC = min(mnC, m);
+        mxC = max(mxC, m);
+        if (aux & AR_AUX_DEFINITE) {
+            mnD = min(mnD, m);
+            mxD = max(mxD, m);
+            ++nd;
+        }
+    }
+    mnC = __reduce_min_sync(0xffffffffu, mnC);
+    mxC = __reduce_max_sync(0xffffffffu, mxC);
+    mnD = __reduce_min_sync(0xffffffffu, mnD);
+    mxD = __reduce_max_sync(0xffffffffu, mxD);
+#pragma unroll
+    for (int o = 16; o > 0; o >>= 1) nd += __shfl_xor_sync(0xffffffffu, nd, o);
+    if ((threadIdx.x & 31) == 0) {
+        atomicMin(P.ws + 0, mnC);
+        atomicMax(P.ws + 1, mxC);
+        atomicMin(P.ws + 2, mnD);
+        atomicMax(P.ws + 3, mxD);
+        if (nd) atomicAdd(P.wc + 0, nd);
+    }
+}
+
+__global__ void __launch_bounds__(kRefThreads) minmax_refine_kernel(const __grid_constant__ MinMaxParams P) {
+    const long long count = *P.r.in_count;
+    const bool any_def = __ldcg(P.wc + 0) != 0ull;
+    const bool is_min = P.mode == AR_MIN;
+    // refine threshold: MIN keeps m <= (D ? min_D : max_C), MAX keeps m >= (D ? max_D : min_C)
+    const uint32_t thr = is_min ? (any_def ? __ldcg(P.ws + 2) : __ldcg(P.ws + 1))
+                                : (any_def ? __ldcg(P.ws + 3) : __ldcg(P.ws + 0));
+    uint32_t best = 0xffffffffu;   // exact key, complemented for MAX
+    unsigned long long nref = 0, surv = 0;
+    const long long stride = (long long)gridDim.x * kRefThreads;
+    for (long long j = (long long)blockIdx.x * kRefThreads + threadIdx.x; j < count; j += stride) {
+        const uint32_t pos = P.r.in_pos[j], aux = P.r.in_aux[j];
+        const uint32_t m = y_major(P, pos, aux);
+        if (is_min ? m > thr : m < thr) continue;
+        ++nref;
+        if (!refine_keep(P.r, pos, aux)) continue;
+        ++surv;
+        const uint32_t r = P.y.k ? residual_get(P.y.residual, pos, (int)P.y.k, (int)P.y.rlayout) : 0u;
+        const uint32_t key = (P.y.k >= 32 ? r : ((m << P.y.k) | r)) + P.y.base;
+        best = min(best, is_min ? key : ~key);
+    }
+    best = __reduce_min_sync(0xffffffffu, best);
+#pragma unroll
+    for (int o = 16; o > 0; o >>= 1) {
+        nref += __shfl_xor_sync(0xffffffffu, nref, o);
+        surv += __shfl_xor_sync(0xffffffffu, surv, o);
+    }
+    if ((threadIdx.x & 31) == 0) {
+        if (surv) {
+            atomicMin(P.ws + 4, best);
+            atomicAdd(P.wc + 2, surv);
+        }
+        if (nref) atomicAdd(P.wc + 1, nref);
+    }
+}
+
+__device__ __forceinline__ long long key_value(uint32_t key, uint32_t flip) {
+    const uint32_t v = key ^ flip;
+    return flip ? (long long)(int32_t)v : (long long)v;
+}
+
+__global__ void minmax_final_kernel(const __grid_constant__ MinMaxParams P) {
+    if (threadIdx.x != 0) return;
+    const long long nc = *P.r.in_count;
+    const unsigned long long nd = P.wc[0];
+    const bool is_min = P.mode == AR_MIN;
+    const AggCol& y = P.y;
+    const uint64_t two_k = 1ull << y.k;
+    long long lo = 0, hi = 0;
+    if (nc > 0) {
+        const uint64_t mlo = is_min ? P.ws[0] : (nd ? P.ws[3] : P.ws[0]);   // bucket whose bottom bounds it
+        const uint64_t mhi = is_min ? (nd ? P.ws[2] : P.ws[1]) : P.ws[1];   // bucket whose top bounds it
+        const uint64_t klo = (uint64_t)y.base + mlo * two_k;
+        uint64_t khi = (uint64_t)y.base + mhi * two_k + two_k - 1;
+        if (khi > 0xffffffffull) khi = 0xffffffffull;
+        lo = key_value((uint32_t)klo, y.flip);
+        hi = key_value((uint32_t)khi, y.flip);
+    }
+    const unsigned long long surv = P.wc[2];
+    const uint32_t best = is_min ? P.ws[4] : ~P.ws[4];
+    P.out7[0] = surv ? key_value(best, y.flip) : 0;
+    P.out7[1] = (long long)surv;
+    P.out7[2] = lo;
+    P.out7[3] = hi;
+    P.out7[4] = (long long)P.wc[1];
+    P.out7[5] = (long long)nd;
+    P.out7[6] = nc;
+}
+
 // sumapproximate (Fig. 7 bwd.sumapproximate): the approximate
 // answer from the approximation subplan alone, before any residual is read
 // (PAPER.md:360-362, 894-897), as strict error bounds.  With
@@ -404,6 +533,17 @@ ar_status launch_approx_sum(const ard::ApproxSumParams& P, int grid, cudaStream_
 ar_status launch_project(const ard::ProjectParams& P, int grid, cudaStream_t s) {
     ard::project_kernel<<<grid, ard::kRefThreads, 0, s>>>(P);
     AR_CHECK_LAUNCH("project_kernel");
+    return AR_OK;
+}
+ar_status launch_minmax(const ard::MinMaxParams& P, int grid, cudaStream_t s) {
+    ard::minmax_init_kernel<<<1, 32, 0, s>>>(P.ws, P.wc);
+    AR_CHECK_LAUNCH("minmax_init_kernel");
+    ard::minmax_approx_kernel<<<grid, ard::kRefThreads, 0, s>>>(P);
+    AR_CHECK_LAUNCH("minmax_approx_kernel");
+    ard::minmax_refine_kernel<<<grid, ard::kRefThreads, 0, s>>>(P);
+    AR_CHECK_LAUNCH("minmax_refine_kernel");
+    ard::minmax_final_kernel<<<1, 32, 0, s>>>(P);
+    AR_CHECK_LAUNCH("minmax_final_kernel");
     return AR_OK;
 }
 ar_status launch_exclusive_offset(const long long* all_counts, int world, int rank, long long* out,
