@@ -583,7 +583,15 @@ ar_status ar_refine(const ar_cands* in, const ar_pred* preds, int32_t npred, ar_
     P.out_count = (long long*)out->count;
     P.ticket = (unsigned int*)ws;
     P.status = (unsigned long long*)((char*)ws + 16);
-    const int grid = (int)std::min<uint64_t>(max_tiles, (uint64_t)num_sms() * 8);
+    // persistent: every CTA resident (the look-back waits only on running or finished CTAs)
+    static int occ = 0;
+    if (!occ) {
+        cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, (const void*)refine_kernel_fn(), ard::kRefThreads, 0);
+        cudaGetLastError();
+        occ = std::max(occ, 1);
+    }
+    const int grid = (int)std::min<uint64_t>(std::min<uint64_t>(max_tiles, (uint64_t)num_sms() * occ), 640);
+    g_last_scan = "refine_kernel";
     return launch_refine(P, grid, s);
 }
 

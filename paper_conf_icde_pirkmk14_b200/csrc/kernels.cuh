@@ -226,6 +226,7 @@ void retile(ard::SelParams& P, uint32_t tile_rows);   // fused.cu
 ar_status launch_fused_rl(const ard::SelParams& P, const ar_column* const* cols, void* ws, int pdl, bool* launched,
                           cudaStream_t s);
 ar_status launch_refine(const ard::RefParams& P, int grid, cudaStream_t s);
+const void* refine_kernel_fn();
 ar_status launch_refine_sum(const ard::RefParams& P, int grid, cudaStream_t s);
 ar_status launch_sum(const ard::SumParams& P, int grid, cudaStream_t s);
 ar_status launch_approx_sum(const ard::ApproxSumParams& P, int grid, cudaStream_t s);

@@ -52,54 +52,191 @@ __device__ __forceinline__ void load8(const uint32_t* base, uint64_t j0, long lo
     }
 }
 
-__global__ void __launch_bounds__(kRefThreads) refine_kernel(const __grid_constant__ RefParams P) {
-    __shared__ uint32_t st_pos[kRefTile];
+// Batched gathers of 8 candidates' parts (predicated, non-volatile loads: the
+// 8 candidates' loads of one step are in flight together).
+// SLICED part of width w at rows pos[i] where (pred >> i) & 1: w/4 vector steps
+// (a 32-row block's w planes are contiguous; w % 4 == 0 keeps them 16-B aligned),
+// otherwise word by word.
+__device__ __forceinline__ void sliced_batch8(const uint32_t* s, const uint32_t (&pos)[8], uint32_t pred, int w,
+                                              uint32_t (&out)[8]) {
+#pragma unroll
+    for (int i = 0; i < 8; ++i) out[i] = 0u;
+    if ((w & 3) == 0) {
+        for (int q = 0; q < w / 4; ++q) {
+            uint4 a[8];
+#pragma unroll
+            for (int i = 0; i < 8; ++i) a[i] = ld_gather_if4(s + (uint64_t)(pos[i] >> 5) * w + 4 * q, (pred >> i) & 1u);
+#pragma unroll
+            for (int i = 0; i < 8; ++i) {
+                const uint32_t l = pos[i] & 31u;
+                const uint32_t x[4] = {a[i].x, a[i].y, a[i].z, a[i].w};
+                out[i] |= rl::row_bits<4>(x, l) << (4 * q);
+            }
+        }
+    } else {
+        for (int j = 0; j < w; ++j) {
+            uint32_t a[8];
+#pragma unroll
+            for (int i = 0; i < 8; ++i) a[i] = ld_gather_if(s + (uint64_t)(pos[i] >> 5) * w + j, (pred >> i) & 1u);
+#pragma unroll
+            for (int i = 0; i < 8; ++i) out[i] |= ((a[i] >> (pos[i] & 31u)) & 1u) << j;
+        }
+    }
+}
+__device__ __forceinline__ void part_batch8(const uint32_t* s, const uint32_t (&pos)[8], uint32_t pred, int w,
+                                            int layout, uint32_t (&out)[8]) {
+    if (w == 0) {
+#pragma unroll
+        for (int i = 0; i < 8; ++i) out[i] = 0u;
+    } else if (layout == AR_LAYOUT_SLICED) {
+        sliced_batch8(s, pos, pred, w, out);
+    } else {
+#pragma unroll
+        for (int i = 0; i < 8; ++i) out[i] = packed_get_if(s, pos[i], w, (pred >> i) & 1u);
+    }
+}
+
+// Alg. 2 on 8 candidates: definite ones are kept untouched;
+// every non-definite one is joined with its residual (and, when the
+// approximation is not carried, its major) and re-evaluated exactly.
+__device__ __forceinline__ uint32_t refine_batch8(const RefParams& P, const uint32_t (&pos)[8],
+                                                  const uint32_t (&aux)[8], uint32_t valid) {
+    uint32_t def = 0;
+#pragma unroll
+    for (int i = 0; i < 8; ++i) def |= (aux[i] >> 31) << i;
+    def &= valid;
+    uint32_t need = valid & ~def;
+    for (int c = 0; c < P.npred && need; ++c) {
+        const RefPred& p = P.p[c];
+        if (!p.check) continue;
+        uint32_t m[8], r[8];
+        if (p.carried) {
+            const uint32_t mask = p.w == 32 ? 0xffffffffu : ((1u << p.w) - 1u);
+#pragma unroll
+            for (int i = 0; i < 8; ++i) m[i] = (aux[i] >> p.ashift) & mask;
+        } else {
+            part_batch8(p.major, pos, need, (int)p.w, (int)p.layout, m);
+        }
+        part_batch8(p.residual, pos, need, (int)p.k, (int)p.rlayout, r);
+#pragma unroll
+        for (int i = 0; i < 8; ++i) {
+            const uint32_t v = (p.k >= 32 ? r[i] : ((m[i] << p.k) | r[i])) + p.base;
+            if (!(v >= p.lo && v <= p.hi)) need &= ~(1u << i);
+        }
+    }
+    return def | need;
+}
+
+constexpr int kAggPerLane = 20;   // refine_kernel grid <= 32 * kAggPerLane CTAs
+
+// Ordered refine (positions out).  Persistent CTAs, tile t = blockIdx + i *
+// gridDim (2048 candidates), decoupled look-back across tiles (Merrill &
+// Garland) specialised to the round-robin order: a tile's offset is its CTA's
+// previous inclusive prefix plus the aggregates of the gridDim - 1 tiles in
+// between.  Every CTA is resident and walks its tiles in order, so those
+// tiles are done or in progress.  Software-pipelined: a tile's kept positions
+// wait in shared memory while the CTA refines its next tile (whose candidates
+// were loaded one tile ahead), then go out at the resolved offset.
+// Warp 0: exclusive prefix of tile t = this CTA's previous tile's inclusive
+// prefix + the aggregates of the tiles in between (t - G, t).
+__device__ __forceinline__ unsigned long long rr_prefix(const unsigned long long* status, long long t, unsigned lane,
+                                                        unsigned long long prev_incl) {
+    const long long lo = t - (long long)gridDim.x + 1 > 0 ? t - (long long)gridDim.x + 1 : 0;
+    unsigned long long v[kAggPerLane];
+#pragma unroll
+    for (int q = 0; q < kAggPerLane; ++q) {
+        const long long idx = lo + lane + 32 * q;
+        v[q] = idx < t ? ld_relaxed(status + idx) : kFlagAgg;
+    }
+    while (true) {
+        bool ready = true;
+#pragma unroll
+        for (int q = 0; q < kAggPerLane; ++q) ready &= (v[q] >> 62) != 0;
+        if (__all_sync(0xffffffffu, ready)) break;
+        __nanosleep(32);
+#pragma unroll
+        for (int q = 0; q < kAggPerLane; ++q) {
+            const long long idx = lo + lane + 32 * q;
+            if ((v[q] >> 62) == 0) v[q] = ld_relaxed(status + idx);
+        }
+    }
+    unsigned long long sum = 0;
+#pragma unroll
+    for (int q = 0; q < kAggPerLane; ++q) sum += v[q] & kValueMask;
+#pragma unroll
+    for (int o = 16; o > 0; o >>= 1) sum += __shfl_xor_sync(0xffffffffu, sum, o);
+    return prev_incl + sum;
+}
+
+__global__ void __launch_bounds__(kRefThreads, 4) refine_kernel(const __grid_constant__ RefParams P) {
+    __shared__ uint32_t st_pos[2][kRefTile];   // kept positions of the current and the pending tile
     __shared__ uint32_t warp_tot[kRefThreads / 32];
-    __shared__ long long s_tile;
     __shared__ unsigned long long s_off;
     const unsigned warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     const long long count = *P.in_count;
     const long long num_tiles = (count + kRefTile - 1) / kRefTile;
-
-    while (true) {
-        if (threadIdx.x == 0) s_tile = (long long)atomicAdd(P.ticket, 1u);
+    unsigned long long prev_incl = 0;   // warp 0: inclusive prefix of this CTA's last resolved tile
+    long long pend = -1;                // tile whose positions wait in st_pos[pbuf] for their offset
+    uint32_t pend_total = 0, buf = 0;
+    // Write out the pending tile: its predecessors' aggregates were published while this
+    // CTA refined its next tile, so the prefix is normally ready without waiting.
+    auto resolve = [&]() {
+        if (warp == 0) {
+            const unsigned long long prefix = rr_prefix(P.status, pend, lane, prev_incl);
+            prev_incl = prefix + pend_total;
+            if (lane == 0) {
+                s_off = prefix;
+                if (pend == num_tiles - 1) *P.out_count = (long long)(prefix + pend_total);
+            }
+        }
         __syncthreads();
-        const long long t = s_tile;
-        if (t >= num_tiles) break;
+        const unsigned long long off = s_off;
+        const uint32_t* sp = st_pos[buf];   // the pending tile's buffer
+        for (uint32_t j = threadIdx.x; j < pend_total; j += kRefThreads) P.out_pos[off + j] = sp[j];
+        __syncthreads();
+    };
+    uint32_t npos[8], naux[8];
+    if ((long long)blockIdx.x < num_tiles) {
+        const uint64_t j0 = (uint64_t)blockIdx.x * kRefTile + threadIdx.x * kRefPerThread;
+        load8(P.in_pos, j0, count, npos);
+        load8(P.in_aux, j0, count, naux);
+    }
+    for (long long t = blockIdx.x; t < num_tiles; t += gridDim.x) {
         const uint64_t j0 = (uint64_t)t * kRefTile + threadIdx.x * kRefPerThread;
         uint32_t pos[8], aux[8];
-        load8(P.in_pos, j0, count, pos);
-        load8(P.in_aux, j0, count, aux);
-        uint32_t keep = 0;
 #pragma unroll
-        for (int i = 0; i < 8; ++i)
-            if (j0 + i < (uint64_t)count && refine_keep(P, pos[i], aux[i])) keep |= 1u << i;
+        for (int i = 0; i < 8; ++i) {
+            pos[i] = npos[i];
+            aux[i] = naux[i];
+        }
+        if (t + gridDim.x < num_tiles) {
+            const uint64_t j1 = j0 + (uint64_t)gridDim.x * kRefTile;
+            load8(P.in_pos, j1, count, npos);
+            load8(P.in_aux, j1, count, naux);
+        }
+        uint32_t valid = 0;
+#pragma unroll
+        for (int i = 0; i < 8; ++i) valid |= (j0 + i < (uint64_t)count ? 1u : 0u) << i;
+        const uint32_t keep = refine_batch8(P, pos, aux, valid);
 
         const uint32_t cnt = __popc(keep);
         uint32_t total;
         const uint32_t excl = block_excl_scan<kRefThreads>(cnt, warp_tot, total, 1);
-        if (warp == 0) {
-            unsigned long long prefix = 0;
-            if (t == 0) {
-                if (lane == 0) st_relaxed(P.status, kFlagPrefix | total);
-            } else {
-                if (lane == 0) st_relaxed(P.status + t, kFlagAgg | total);
-                prefix = lookback_wide(P.status, t, lane);
-                if (lane == 0) st_relaxed(P.status + t, kFlagPrefix | (prefix + total));
-            }
-            if (lane == 0) {
-                s_off = prefix;
-                if (t == num_tiles - 1) *P.out_count = (long long)(prefix + total);
-            }
-        }
+        if (threadIdx.x == 0) st_relaxed(P.status + t, kFlagAgg | total);   // publish the aggregate at once
         uint32_t o = excl;
+        uint32_t* sp = st_pos[buf];
 #pragma unroll
         for (int i = 0; i < 8; ++i)
-            if (keep & (1u << i)) st_pos[o++] = pos[i];
-        __syncthreads();
-        const unsigned long long off = s_off;
-        for (uint32_t j = threadIdx.x; j < total; j += kRefThreads) P.out_pos[off + j] = st_pos[j];
-        __syncthreads();
+            if (keep & (1u << i)) sp[o++] = pos[i];
+        buf ^= 1u;   // now the pending (previous) tile's buffer
+        if (pend >= 0) resolve();
+        else __syncthreads();
+        pend = t;
+        pend_total = total;
+    }
+    if (pend >= 0) {
+        buf ^= 1u;   // the last tile's buffer
+        resolve();
     }
 }
 
@@ -499,6 +636,7 @@ __global__ void exclusive_offset_kernel(const long long* all, int world, int ran
 
 namespace ar {
 
+const void* refine_kernel_fn() { return (const void*)ard::refine_kernel; }
 ar_status launch_refine(const ard::RefParams& P, int grid, cudaStream_t s) {
     ard::refine_kernel<<<grid, ard::kRefThreads, 0, s>>>(P);
     AR_CHECK_LAUNCH("refine_kernel");

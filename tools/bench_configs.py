@@ -4,8 +4,9 @@
   C3  1 G-row u32 column: major-bit width {8,16,24} x selectivity sweep, positions out
   C5  SF1000-shaped Q6 per GPU share (750 M rows = SF125) with the l_shipdate residual in
       pinned host memory: HBM + host-link rooflines
+  MM  C2 (SF10 Q6 predicates) MIN / MAX(l_extendedprice): ar_approx_select + ar_minmax (s IV-F)
 
-    python tools/bench_configs.py c1|c3|c5 [--reps R]
+    python tools/bench_configs.py c1|c3|c5|mm [--reps R]
 
 One JSON line per point.  Timing as in bench.py: inputs resident, warm-up, CUDA
 events on the launching stream around R back-to-back repetitions, L2 flushed
@@ -79,7 +80,7 @@ def c3(args):
     n = 1_000_000_000
     v = datagen.uniform_u32(3, n)
     flush = torch.empty(512 << 20, dtype=torch.uint8, device="cuda")
-    for M in (8, 16, 24):
+    for M in args.widths:
         col = cu.BWDColumn(v, M)
         k = 32 - M
         w = col.w_major
@@ -88,7 +89,7 @@ def c3(args):
         pos = cu.PositionList(n)
         wr = cu.Workspace(_ar.ar_refine_ws_bytes(n))
         o4 = torch.zeros(4, dtype=torch.int64, device="cuda")
-        for s in (0.0001, 0.001, 0.01, 0.1, 0.5):
+        for s in args.sels:
             lo = 0x1234567
             hi = lo + int(s * 2**32) - 1
             preds = [(col, lo, hi)]
@@ -170,13 +171,48 @@ def c5(args):
         "host_link_frac_staged": host32 / (ms_s / 1e3) / 1e9 / link_gbs}), flush=True)
 
 
+def mm(args):
+    c = datagen.q6_columns(2, 10)
+    n = c["shipdate"].size
+    sd = cu.BWDColumn(c["shipdate"], 24)
+    dc = cu.BWDColumn(c["discount"], 32)
+    qt = cu.BWDColumn(c["quantity"], 32)
+    ep = cu.BWDColumn(c["extprice"], 32, layout=_ar.AR_LAYOUT_PACKED)
+    preds = [(sd, *datagen.Q6_SHIPDATE), (dc, *datagen.Q6_DISCOUNT), (qt, *datagen.Q6_QUANTITY)]
+    cands = cu.CandidateList(n)
+    ws = cu.Workspace(_ar.ar_select_ws_bytes(n))
+    wm = cu.Workspace(_ar.ar_minmax_ws_bytes())
+    o7 = torch.zeros(7, dtype=torch.int64, device="cuda")
+    flush = torch.empty(512 << 20, dtype=torch.uint8, device="cuda")
+    cu.approx_select(preds, cands, ws)
+    torch.cuda.synchronize()
+    pos = cands.positions()
+    for mode in ("min", "max"):
+        ms_sel, _ = timed(lambda: cu.approx_select(preds, cands, ws), args.reps, flush)
+        ms_mm, _ = timed(lambda: cu.minmax(cands, preds, ep, mode, o7, wm), args.reps, flush)
+        torch.cuda.synchronize()
+        r = o7.cpu().tolist()
+        # algorithmic bytes of ar_minmax: candidate list read twice (8 B each), l_extendedprice
+        # sectors at every candidate (the approximate pass needs every candidate's major), and the
+        # residual sectors of the refined non-definite candidates are a few rows (ignored)
+        ep_bytes = 32.0 * sectors(pos, 24, 32)
+        mm_bytes = 2 * 8.0 * pos.size + ep_bytes
+        print(json.dumps({"config": "MM (C2 Q6, %s(l_extendedprice))" % mode.upper(), "rows": n,
+                          "answer": r[0], "survivors": r[1], "approx_bounds": r[2:4], "refined": r[4],
+                          "definite": r[5], "candidates": r[6], "select_us": ms_sel * 1e3, "minmax_us": ms_mm * 1e3,
+                          "rows_per_s": n / ((ms_sel + ms_mm) / 1e3),
+                          "minmax_frac": mm_bytes / (ms_mm / 1e3) / 1e9 / PEAK, "peak_gbs": PEAK}), flush=True)
+
+
 def main():
     ap = argparse.ArgumentParser()
-    ap.add_argument("config", choices=["c1", "c3", "c5"])
+    ap.add_argument("config", choices=["c1", "c3", "c5", "mm"])
     ap.add_argument("--reps", type=int, default=10)
+    ap.add_argument("--widths", type=int, nargs="+", default=[8, 16, 24], help="C3 major bits")
+    ap.add_argument("--sels", type=float, nargs="+", default=[0.0001, 0.001, 0.01, 0.1, 0.5], help="C3 selectivities")
     args = ap.parse_args()
     torch.cuda.set_device(0)
-    {"c1": c1, "c3": c3, "c5": c5}[args.config](args)
+    {"c1": c1, "c3": c3, "c5": c5, "mm": mm}[args.config](args)
 
 
 if __name__ == "__main__":
