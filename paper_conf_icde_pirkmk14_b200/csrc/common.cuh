@@ -248,6 +248,43 @@ __device__ __forceinline__ unsigned long long lookback_wide(const unsigned long 
     }
 }
 
+// Round-robin persistent kernels (tile t = blockIdx + i * gridDim, every CTA
+// resident, tiles walked in order): each tile publishes kFlagAgg | count in
+// status[t] at once; warp 0 of the owner then obtains the exclusive prefix as
+// its CTA's previous inclusive prefix + the aggregates of the gridDim - 1 tiles
+// in between -- no chain of inclusive prefixes.  gridDim <= 32 * kAggPerLane.
+constexpr int kAggPerLane = 20;
+// Warp 0: exclusive prefix of tile t = this CTA's previous tile's inclusive
+// prefix + the aggregates of the tiles in between (t - G, t).
+__device__ __forceinline__ unsigned long long rr_prefix(const unsigned long long* status, long long t, unsigned lane,
+                                                        unsigned long long prev_incl) {
+    const long long lo = t - (long long)gridDim.x + 1 > 0 ? t - (long long)gridDim.x + 1 : 0;
+    unsigned long long v[kAggPerLane];
+#pragma unroll
+    for (int q = 0; q < kAggPerLane; ++q) {
+        const long long idx = lo + lane + 32 * q;
+        v[q] = idx < t ? ld_relaxed(status + idx) : kFlagAgg;
+    }
+    while (true) {
+        bool ready = true;
+#pragma unroll
+        for (int q = 0; q < kAggPerLane; ++q) ready &= (v[q] >> 62) != 0;
+        if (__all_sync(0xffffffffu, ready)) break;
+        __nanosleep(32);
+#pragma unroll
+        for (int q = 0; q < kAggPerLane; ++q) {
+            const long long idx = lo + lane + 32 * q;
+            if ((v[q] >> 62) == 0) v[q] = ld_relaxed(status + idx);
+        }
+    }
+    unsigned long long sum = 0;
+#pragma unroll
+    for (int q = 0; q < kAggPerLane; ++q) sum += v[q] & kValueMask;
+#pragma unroll
+    for (int o = 16; o > 0; o >>= 1) sum += __shfl_xor_sync(0xffffffffu, sum, o);
+    return prev_incl + sum;
+}
+
 // --- value extraction ----------------------------------------------------------
 
 // Gather load of one word.  On B200 a plain scalar load makes L2 fetch a whole

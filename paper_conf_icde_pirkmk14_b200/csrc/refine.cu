@@ -127,8 +127,6 @@ __device__ __forceinline__ uint32_t refine_batch8(const RefParams& P, const uint
     return def | need;
 }
 
-constexpr int kAggPerLane = 20;   // refine_kernel grid <= 32 * kAggPerLane CTAs
-
 // Ordered refine (positions out).  Persistent CTAs, tile t = blockIdx + i *
 // gridDim (2048 candidates), decoupled look-back across tiles (Merrill &
 // Garland) specialised to the round-robin order: a tile's offset is its CTA's
@@ -137,37 +135,6 @@ constexpr int kAggPerLane = 20;   // refine_kernel grid <= 32 * kAggPerLane CTAs
 // tiles are done or in progress.  Software-pipelined: a tile's kept positions
 // wait in shared memory while the CTA refines its next tile (whose candidates
 // were loaded one tile ahead), then go out at the resolved offset.
-// Warp 0: exclusive prefix of tile t = this CTA's previous tile's inclusive
-// prefix + the aggregates of the tiles in between (t - G, t).
-__device__ __forceinline__ unsigned long long rr_prefix(const unsigned long long* status, long long t, unsigned lane,
-                                                        unsigned long long prev_incl) {
-    const long long lo = t - (long long)gridDim.x + 1 > 0 ? t - (long long)gridDim.x + 1 : 0;
-    unsigned long long v[kAggPerLane];
-#pragma unroll
-    for (int q = 0; q < kAggPerLane; ++q) {
-        const long long idx = lo + lane + 32 * q;
-        v[q] = idx < t ? ld_relaxed(status + idx) : kFlagAgg;
-    }
-    while (true) {
-        bool ready = true;
-#pragma unroll
-        for (int q = 0; q < kAggPerLane; ++q) ready &= (v[q] >> 62) != 0;
-        if (__all_sync(0xffffffffu, ready)) break;
-        __nanosleep(32);
-#pragma unroll
-        for (int q = 0; q < kAggPerLane; ++q) {
-            const long long idx = lo + lane + 32 * q;
-            if ((v[q] >> 62) == 0) v[q] = ld_relaxed(status + idx);
-        }
-    }
-    unsigned long long sum = 0;
-#pragma unroll
-    for (int q = 0; q < kAggPerLane; ++q) sum += v[q] & kValueMask;
-#pragma unroll
-    for (int o = 16; o > 0; o >>= 1) sum += __shfl_xor_sync(0xffffffffu, sum, o);
-    return prev_incl + sum;
-}
-
 __global__ void __launch_bounds__(kRefThreads, 4) refine_kernel(const __grid_constant__ RefParams P) {
     __shared__ uint32_t st_pos[2][kRefTile];   // kept positions of the current and the pending tile
     __shared__ uint32_t warp_tot[kRefThreads / 32];

@@ -255,10 +255,7 @@ struct FixedPlanes {
     // approximation tuple: all majors concatenated LSB-first in predicate order
     template <int B>
     __device__ __forceinline__ uint32_t appr(const SelParams&, uint32_t l) const {
-        uint32_t a = 0;
-#pragma unroll
-        for (int p = 0; p < TOTAL; ++p) a |= ((x[B][p] >> l) & 1u) << p;
-        return a;
+        return rl::row_bits<TOTAL>(x[B], l);
     }
 };
 
@@ -877,6 +874,7 @@ struct ShapeList {
         *fn = fused ? E::fused_fn() : E::select_fn(carry);
         return true;
     }
+
 };
 using Shapes = ShapeList<ShapeEntry<4, 4, 6>, ShapeEntry<8>, ShapeEntry<16>, ShapeEntry<24>, ShapeEntry<32>,
                          ShapeEntry<24, 24>>;
