@@ -308,14 +308,15 @@ ar_status ar_sum_approximate(const ar_cands* in, const ar_column* const* cols, i
  *             MIN in [bmin(min_C m), D ? bmax(min_D m) : bmax(max_C m)]
  *             MAX in [D ? bmin(max_D m) : bmin(min_C m), bmax(max_C m)]
  *   out7[4] = candidates refined, out7[5] = |definite|, out7[6] = |candidates|
- * `ws` is a caller-owned device workspace of ar_minmax_ws_bytes() bytes
- * (initialised by the call).  Four kernel launches on `stream`.
+ * `ws` is a caller-owned device workspace of ar_minmax_ws_bytes(in->capacity)
+ * bytes (initialised by the call; it keeps each candidate's Y major between
+ * the approximate and the refine pass).  Four kernel launches on `stream`.
  * Errors: AR_ERR_INVALID (null pointers, bad mode, predicates that do not
  * match the candidate relation), AR_ERR_RANGE (workspace too small).
  */
 #define AR_MIN 0
 #define AR_MAX 1
-size_t ar_minmax_ws_bytes(void);
+size_t ar_minmax_ws_bytes(int64_t capacity);
 ar_status ar_minmax(const ar_cands* in, const ar_pred* preds, int32_t npred, const ar_column* col, int32_t mode,
                     int64_t* out7_dev, void* ws, size_t ws_bytes, void* stream);
 

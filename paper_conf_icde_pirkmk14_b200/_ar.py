@@ -78,7 +78,7 @@ SIGNATURES = {
     "ar_sum": (ctypes.c_int, [ctypes.POINTER(Positions), ctypes.POINTER(_P), _I32, _P, _P]),
     "ar_sum_approximate": (ctypes.c_int, [ctypes.POINTER(Cands), ctypes.POINTER(_P), _I32, _P, _P]),
     "ar_project": (ctypes.c_int, [ctypes.POINTER(Positions), _P, _I32, _P, _P]),
-    "ar_minmax_ws_bytes": (_SZ, []),
+    "ar_minmax_ws_bytes": (_SZ, [_I64]),
     "ar_minmax": (ctypes.c_int, [ctypes.POINTER(Cands), ctypes.POINTER(Pred), _I32, _P, _I32, _P, _P, _SZ, _P]),
     "ar_refine_sum": (ctypes.c_int, [ctypes.POINTER(Cands), ctypes.POINTER(Pred), _I32, ctypes.POINTER(_P), _I32,
                                      _P, _P, _P]),
@@ -212,8 +212,8 @@ def ar_project(pos: Positions, col, mode, out_values_dev, stream):
     _call("ar_project", ctypes.byref(pos), col, mode, out_values_dev, stream)
 
 
-def ar_minmax_ws_bytes() -> int:
-    return int(load().ar_minmax_ws_bytes())
+def ar_minmax_ws_bytes(capacity: int) -> int:
+    return int(load().ar_minmax_ws_bytes(capacity))
 
 
 def ar_minmax(cands: Cands, preds, col, mode, out7_dev, ws, ws_bytes, stream):

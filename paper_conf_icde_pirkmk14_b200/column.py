@@ -207,7 +207,7 @@ def minmax(cands: CandidateList, preds, col: BWDColumn, mode: str, out7: torch.T
            stream=None):
     """MIN / MAX of `col` over the refined rows (s IV-F, Fig. 6): out7 = [answer, survivors, approx lower,
     approx upper, candidates refined, |definite|, |candidates|]."""
-    ws = ws if ws is not None else Workspace(_ar.ar_minmax_ws_bytes(), col.device)
+    ws = ws if ws is not None else Workspace(_ar.ar_minmax_ws_bytes(cands.c.capacity), col.device)
     _ar.ar_minmax(cands.c, _pred_tuples(preds), col.handle, _ar.AR_MIN if mode == "min" else _ar.AR_MAX,
                   out7.data_ptr(), ws.ptr, ws.nbytes, _stream(stream))
 

@@ -754,7 +754,7 @@ ar_status ar_refine_sum(const ar_cands* in, const ar_pred* preds, int32_t npred,
 
 // ----------------------------------------------------------- MIN / MAX (s IV-F)
 
-size_t ar_minmax_ws_bytes(void) { return 64; }
+size_t ar_minmax_ws_bytes(int64_t capacity) { return 64 + 4 * (size_t)std::max<int64_t>(capacity, 0); }
 
 ar_status ar_minmax(const ar_cands* in, const ar_pred* preds, int32_t npred, const ar_column* col, int32_t mode,
                     int64_t* out7_dev, void* ws, size_t ws_bytes, void* stream) {
@@ -766,8 +766,8 @@ ar_status ar_minmax(const ar_cands* in, const ar_pred* preds, int32_t npred, con
         set_error("ar_minmax: null output / workspace or mode %d not AR_MIN / AR_MAX", mode);
         return AR_ERR_INVALID;
     }
-    if (ws_bytes < ar_minmax_ws_bytes()) {
-        set_error("ar_minmax: workspace %zu < %zu bytes", ws_bytes, ar_minmax_ws_bytes());
+    if (ws_bytes < ar_minmax_ws_bytes(in->capacity)) {
+        set_error("ar_minmax: workspace %zu < %zu bytes", ws_bytes, ar_minmax_ws_bytes(in->capacity));
         return AR_ERR_RANGE;
     }
     const ar_column* const cols[1] = {col};
@@ -776,10 +776,11 @@ ar_status ar_minmax(const ar_cands* in, const ar_pred* preds, int32_t npred, con
     P.mode = mode;
     P.ws = (unsigned int*)ws;
     P.wc = (unsigned long long*)((char*)ws + 32);
+    P.ymaj = (uint32_t*)((char*)ws + 64);
     P.out7 = (long long*)out7_dev;
     cudaStream_t s = (cudaStream_t)stream;
     const int64_t cap = std::max<int64_t>(in->capacity, 1);
-    const int grid = (int)std::min<int64_t>((cap + ard::kRefThreads - 1) / ard::kRefThreads, (int64_t)num_sms() * 8);
+    const int grid = (int)std::min<int64_t>((cap + ard::kRefTile - 1) / ard::kRefTile, (int64_t)num_sms() * 8);
     g_last_scan = "minmax_refine_kernel";
     return launch_minmax(P, grid, s);
 }

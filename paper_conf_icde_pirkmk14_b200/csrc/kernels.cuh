@@ -196,6 +196,7 @@ struct MinMaxParams {
     int32_t mode;             // AR_MIN / AR_MAX
     unsigned int* ws;         // [0..3] min/max major over candidates / definite, [4] best exact key (xored)
     unsigned long long* wc;   // [0] |definite|, [1] rows refined, [2] survivors
+    uint32_t* ymaj;           // [capacity] Y's major per candidate (approximate pass -> refine pass)
     long long* out7;
 };
 

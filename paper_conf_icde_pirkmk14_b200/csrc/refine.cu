@@ -410,7 +410,8 @@ __global__ void __launch_bounds__(kRefThreads) sum_kernel(const __grid_constant_
 // certainly in R, so (MIN) nothing whose Y major exceeds the smallest definite
 // major mD can be the minimum.  Three passes over the candidate relation:
 //   minmax_approx_kernel : min / max of Y's major over candidates and over
-//                          definite candidates (the approximate answer);
+//                          definite candidates (the approximate answer); each
+//                          candidate's Y major is kept in the workspace;
 //   minmax_refine_kernel : the candidates with major <= mD (MIN; >= MD for MAX;
 //                          every candidate when none is definite) are refined --
 //                          Alg. 2 on the predicates, then Y's residual -- and
@@ -434,18 +435,36 @@ __global__ void minmax_init_kernel(unsigned int* ws, unsigned long long* wc) {
 
 __global__ void __launch_bounds__(kRefThreads) minmax_approx_kernel(const __grid_constant__ MinMaxParams P) {
     const long long count = *P.r.in_count;
+    const long long num_tiles = (count + kRefTile - 1) / kRefTile;
     uint32_t mnC = 0xffffffffu, mxC = 0u, mnD = 0xffffffffu, mxD = 0u;
     unsigned long long nd = 0;
-    const long long stride = (long long)gridDim.x * kRefThreads;
-    for (long long j = (long long)blockIdx.x * kRefThreads + threadIdx.x; j < count; j += stride) {
-        const uint32_t pos = P.r.in_pos[j], aux = P.r.in_aux[j];
-        const uint32_t m = y_major(P, pos, aux);
-        mnC = min(mnC, m);
-        mxC = max(mxC, m);
-        if (aux & AR_AUX_DEFINITE) {
-            mnD = min(mnD, m);
-            mxD = max(mxD, m);
-            ++nd;
+    const AggCol& y = P.y;
+    const bool carried = y.pred >= 0 && P.r.p[y.pred].carried;
+    for (long long t = blockIdx.x; t < num_tiles; t += gridDim.x) {   // 8 candidates per thread
+        const uint64_t j0 = (uint64_t)t * kRefTile + threadIdx.x * kRefPerThread;
+        uint32_t pos[8], aux[8], m[8];
+        load8(P.r.in_pos, j0, count, pos);
+        load8(P.r.in_aux, j0, count, aux);
+        uint32_t valid = 0;
+#pragma unroll
+        for (int i = 0; i < 8; ++i) valid |= (j0 + i < (uint64_t)count ? 1u : 0u) << i;
+        if (carried) {
+#pragma unroll
+            for (int i = 0; i < 8; ++i) m[i] = y_major(P, pos[i], aux[i]);
+        } else {
+            part_batch8(y.major, pos, valid, (int)y.w, (int)y.layout, m);   // gathers in flight together
+        }
+#pragma unroll
+        for (int i = 0; i < 8; ++i) {
+            if (!((valid >> i) & 1u)) continue;
+            P.ymaj[j0 + i] = m[i];   // the refine pass reads it back sequentially instead of gathering again
+            mnC = min(mnC, m[i]);
+            mxC = max(mxC, m[i]);
+            if (aux[i] & AR_AUX_DEFINITE) {
+                mnD = min(mnD, m[i]);
+                mxD = max(mxD, m[i]);
+                ++nd;
+            }
         }
     }
     mnC = __reduce_min_sync(0xffffffffu, mnC);
@@ -474,9 +493,9 @@ __global__ void __launch_bounds__(kRefThreads) minmax_refine_kernel(const __grid
     unsigned long long nref = 0, surv = 0;
     const long long stride = (long long)gridDim.x * kRefThreads;
     for (long long j = (long long)blockIdx.x * kRefThreads + threadIdx.x; j < count; j += stride) {
-        const uint32_t pos = P.r.in_pos[j], aux = P.r.in_aux[j];
-        const uint32_t m = y_major(P, pos, aux);
+        const uint32_t m = __ldcs(P.ymaj + j);
         if (is_min ? m > thr : m < thr) continue;
+        const uint32_t pos = P.r.in_pos[j], aux = P.r.in_aux[j];
         ++nref;
         if (!refine_keep(P.r, pos, aux)) continue;
         ++surv;

@@ -58,6 +58,7 @@ def test_host_only_entry_points():
     assert _ar.ar_select_ws_bytes(4096) >= 8 * 4096 and _ar.ar_select_ws_bytes(4097) >= 8 * 4097
     assert _ar.ar_refine_ws_bytes(2048) == 16 + 8
     assert _ar.ar_dist_unique_id_bytes() == 128
+    assert _ar.ar_minmax_ws_bytes(100) == 64 + 4 * 100   # header + one Y major per candidate
     assert ctypes.sizeof(_ar.ColumnDesc) == 64
 
 

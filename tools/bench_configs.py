@@ -181,7 +181,7 @@ def mm(args):
     preds = [(sd, *datagen.Q6_SHIPDATE), (dc, *datagen.Q6_DISCOUNT), (qt, *datagen.Q6_QUANTITY)]
     cands = cu.CandidateList(n)
     ws = cu.Workspace(_ar.ar_select_ws_bytes(n))
-    wm = cu.Workspace(_ar.ar_minmax_ws_bytes())
+    wm = cu.Workspace(_ar.ar_minmax_ws_bytes(n))
     o7 = torch.zeros(7, dtype=torch.int64, device="cuda")
     flush = torch.empty(512 << 20, dtype=torch.uint8, device="cuda")
     cu.approx_select(preds, cands, ws)
@@ -192,11 +192,11 @@ def mm(args):
         ms_mm, _ = timed(lambda: cu.minmax(cands, preds, ep, mode, o7, wm), args.reps, flush)
         torch.cuda.synchronize()
         r = o7.cpu().tolist()
-        # algorithmic bytes of ar_minmax: candidate list read twice (8 B each), l_extendedprice
-        # sectors at every candidate (the approximate pass needs every candidate's major), and the
-        # residual sectors of the refined non-definite candidates are a few rows (ignored)
+        # algorithmic bytes of ar_minmax: candidate list read (8 B), l_extendedprice sectors at
+        # every candidate (the approximate pass needs every candidate's major), the kept majors
+        # written and read back (8 B); the refined rows' gathers are a few rows (ignored)
         ep_bytes = 32.0 * sectors(pos, 24, 32)
-        mm_bytes = 2 * 8.0 * pos.size + ep_bytes
+        mm_bytes = 16.0 * pos.size + ep_bytes
         print(json.dumps({"config": "MM (C2 Q6, %s(l_extendedprice))" % mode.upper(), "rows": n,
                           "answer": r[0], "survivors": r[1], "approx_bounds": r[2:4], "refined": r[4],
                           "definite": r[5], "candidates": r[6], "select_us": ms_sel * 1e3, "minmax_us": ms_mm * 1e3,
