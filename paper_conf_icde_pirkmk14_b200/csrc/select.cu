@@ -633,6 +633,18 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_kernel(const __grid_co
         }
         ncand += cnt;
         const bool exact_mode = P.exact_mode != 0;
+        if (P.nagg == 0 && !exact_mode) {
+            // COUNT: a definite candidate is a result (Alg. 2 never touches it) -- counted here,
+            // only the non-definite ones go through the list and the residual gathers
+            cnt = 0;
+#pragma unroll
+            for (int b = 0; b < BPT; ++b) {
+                nres += __popc(dm[b]);
+                cm[b] &= ~dm[b];
+                dm[b] = 0u;
+                cnt += __popc(cm[b]);
+            }
+        }
         if (exact_mode) {
             // a5 in place: exact predicate on major + residual planes of the candidate rows;
             // the list below then holds result rows only (no per-candidate refine pass)
