@@ -93,7 +93,9 @@ def c3(args):
             lo = 0x1234567
             hi = lo + int(s * 2**32) - 1
             preds = [(col, lo, hi)]
-            carry = False            # single predicate: refine gathers the sliced major itself
+            # carry the approximation (4 B per candidate written + read) when many candidates are
+            # non-definite (M = 8: 2/256 of the rows), else let refine gather the few majors it needs
+            carry = M <= 8
 
             def sel():
                 cu.approx_select(preds, cands, ws, carry=carry)
@@ -117,7 +119,7 @@ def c3(args):
             ref_bytes = 8.0 * nc + res_bytes + 4.0 * nr
             rows_s = n / ((ms_sel + ms_ref) / 1e3)
             print(json.dumps({
-                "config": "C3", "rows": n, "major_bits": M, "k": k, "w_major": w, "selectivity": s,
+                "config": "C3", "rows": n, "major_bits": M, "k": k, "w_major": w, "selectivity": s, "carry": carry,
                 "candidates": nc, "definite": nd, "results": nr,
                 "select_ms": ms_sel, "refine_ms": ms_ref, "fused_count_ms": ms_fus,
                 "select_refine_rows_per_s": rows_s,
