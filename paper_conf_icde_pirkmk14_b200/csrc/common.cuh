@@ -287,12 +287,15 @@ __device__ __forceinline__ unsigned long long rr_prefix(const unsigned long long
 
 // --- value extraction ----------------------------------------------------------
 
+#ifndef AR_GHINT
+#define AR_GHINT ".L2::64B"
+#endif
 // Gather load of one word.  On B200 a plain scalar load makes L2 fetch a whole
 // 128-B line from HBM; the .L2::64B prefetch-size hint halves that, which is the
 // smallest gather granularity measured (tools/gather_probe.cu, DESIGN "Gathers").
 __device__ __forceinline__ uint32_t ld_gather(const uint32_t* p) {
     uint32_t v;
-    asm volatile("ld.global.nc.L2::64B.u32 %0, [%1];" : "=r"(v) : "l"(p));   // volatile: never speculated past its guard
+    asm volatile("ld.global.nc" AR_GHINT ".u32 %0, [%1];" : "=r"(v) : "l"(p));   // volatile: never speculated past its guard
     return v;
 }
 
@@ -302,13 +305,13 @@ __device__ __forceinline__ uint32_t ld_gather(const uint32_t* p) {
 // gather from touching memory.  A skipped load returns 0.
 __device__ __forceinline__ uint32_t ld_gather_if(const uint32_t* p, bool pred) {
     uint32_t v = 0;
-    asm("{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %2, 0;\n\t@q ld.global.nc.L2::64B.u32 %0, [%1];\n\t}"
+    asm("{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %2, 0;\n\t@q ld.global.nc" AR_GHINT ".u32 %0, [%1];\n\t}"
         : "+r"(v) : "l"(p), "r"((uint32_t)pred));
     return v;
 }
 __device__ __forceinline__ uint4 ld_gather_if4(const uint32_t* p, bool pred) {   // 16-B aligned
     uint4 v = make_uint4(0, 0, 0, 0);
-    asm("{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %5, 0;\n\t@q ld.global.nc.L2::64B.v4.u32 {%0,%1,%2,%3}, [%4];\n\t}"
+    asm("{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %5, 0;\n\t@q ld.global.nc" AR_GHINT ".v4.u32 {%0,%1,%2,%3}, [%4];\n\t}"
         : "+r"(v.x), "+r"(v.y), "+r"(v.z), "+r"(v.w) : "l"(p), "r"((uint32_t)pred));
     return v;
 }

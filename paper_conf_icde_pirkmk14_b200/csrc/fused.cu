@@ -48,7 +48,7 @@ __device__ __forceinline__ uint32_t stage_value(const SelParams& P, const uint32
 }
 
 __device__ __forceinline__ void cp_async4(uint32_t* dst, const uint32_t* src) {
-    asm volatile("cp.async.ca.shared.global.L2::64B [%0], [%1], 4;" ::"r"(smem_u32(dst)), "l"(src) : "memory");
+    asm volatile("cp.async.ca.shared.global" AR_GHINT " [%0], [%1], 4;" ::"r"(smem_u32(dst)), "l"(src) : "memory");
 }
 __device__ __forceinline__ void cp_async_commit() { asm volatile("cp.async.commit_group;" ::: "memory"); }
 template <int N>
