@@ -87,3 +87,41 @@ def test_gpu_c3_1g_rows_24_8_one_percent(cu):
     assert cands.count() == cpos.size and int(o4[2].item()) == cpos.size and int(o4[3].item()) == int(cdef.sum())
     idx = np.unique(np.linspace(0, cpos.size - 1, 4096).astype(np.int64))
     assert np.array_equal(cands.positions()[idx], cpos[idx])
+
+
+def test_gpu_max_rows_u32_positions(cu):
+    """Maximum size: positions are u32 per column (ar.h), so a column holds < 2^32 rows.  A ragged
+    column of 2^32 - 2^20 - 5 rows (4.29 G; 17 GB of values) through select -> refine -> SUM and
+    the one-pass COUNT: every 64-bit index / offset path past 2^31 and the ragged last tile."""
+    from paper_conf_icde_pirkmk14_b200 import _ar
+    free, _ = torch.cuda.mem_get_info()
+    n = 2**32 - 2**20 - 5
+    if free < 110 * 2**30:
+        pytest.skip("needs ~110 GB of free device memory")
+    v = datagen.uniform_u32(41, n)
+    lo, hi = 0xF0000123, 0xF0000123 + (2**32 // 1000)   # 0.1 %, near the top of the domain
+    col = cu.BWDColumn(v, 24)
+    ref_pos, ref_cnt, ref_sum = oracle.select_sum([v], [lo], [hi], [v], threads=0)
+    cpos, cdef = oracle.approx_select([v], [8], [lo], [hi])
+    preds = [(col, lo, hi)]
+    cands = cu.CandidateList(n)
+    cu.approx_select(preds, cands, cu.Workspace(_ar.ar_select_ws_bytes(n)))
+    torch.cuda.synchronize()
+    got = cands.positions()
+    assert got.size == cpos.size and np.array_equal(got, cpos)
+    assert np.array_equal(cands.definite(), cdef)
+    pos = cu.PositionList(cands.c.capacity)
+    cu.refine(cands, preds, pos, cu.Workspace(_ar.ar_refine_ws_bytes(cands.c.capacity)))
+    s2 = torch.zeros(2, dtype=torch.int64, device="cuda")
+    # SUM of a 32-bit column over up to 2^32 rows could overflow int64: the ABI refuses it (ar.h)
+    with pytest.raises(_ar.ARError, match="AR_ERR_RANGE"):
+        cu.refine_sum(cands, preds, [col], s2[0:1], s2[1:2])
+    cu.refine_sum(cands, preds, [], s2[0:1], s2[1:2])
+    o4 = torch.zeros(4, dtype=torch.int64, device="cuda")
+    cu.select_refine_sum(preds, [], o4)
+    torch.cuda.synchronize()
+    assert np.array_equal(pos.positions(), ref_pos)
+    assert s2.tolist() == [0, ref_cnt]
+    assert oracle.sum_at(ref_pos, [v]) == ref_sum and ref_sum > 0
+    assert o4.tolist() == [0, ref_cnt, cpos.size, int(cdef.sum())]
+    assert ref_pos[-1] > 2**31   # results past 2^31 really exercised
