@@ -19,6 +19,7 @@ Pins (tests/test_oracle_*.py):
   sum_bounds      brute force over every residual of tiny tables, k = 0 collapse to the
                   exact answer, closed forms, containment of the exact answer
   select_minmax   pure-Python brute force on tiny tables, closed forms
+  select_group_sum  Fig. 4's grouped count, pure-Python brute force, closed forms
   minmax_ar       Fig. 6 (the false positive holds the single minimal
                   approximation, the propagated set still holds the true minimum), refined
                   answer == select_minmax, bounds contain it, k = 0 collapse, brute force
@@ -69,6 +70,8 @@ def _load():
         lib.or_sum_bounds.restype = i32
         lib.or_select_minmax.argtypes = [i64, i32, p, p, p, p, p, i32, i32, p]
         lib.or_minmax_ar.argtypes = [i64, i32, p, p, p, p, p, p, i32, u32, i32, i32, p, p]
+        lib.or_select_group_sum.argtypes = [i64, i32, p, p, p, p, i32, i32, p, p, p]
+        lib.or_select_group_sum.restype = i32
         lib.or_threads_default.restype = i32
         _lib = lib
     return _lib
@@ -241,3 +244,24 @@ def minmax_ar(pred_cols, pred_ks, los, his, ycol, y_k: int, mode: str = "min", p
     if flags:
         r["refine_flags"] = fl[:n].astype(bool)
     return r
+
+
+def select_group_sum(pred_cols, los, his, key, ngroups: int, agg_cols=()):
+    """Exact grouped COUNT / product SUM over the selection (s IV-E; Fig. 4 "select count(*) from R where
+    A<5 groupby B"): (sums int64[ngroups], counts int64[ngroups]), group id = key value."""
+    pred_cols = [_u32(c) for c in pred_cols]
+    agg_cols = [_u32(c) for c in agg_cols]
+    key = _u32(key)
+    lo = np.asarray(los, dtype=np.uint32)
+    hi = np.asarray(his, dtype=np.uint32)
+    sums = np.zeros(max(ngroups, 1), dtype=np.int64)
+    cnts = np.zeros(max(ngroups, 1), dtype=np.int64)
+    pc, ac = _ptr_array(pred_cols), _ptr_array(agg_cols)
+    rc = _load().or_select_group_sum(key.size, len(pred_cols), ctypes.cast(pc, ctypes.c_void_p), _ptr(lo), _ptr(hi),
+                                     _ptr(key), ngroups, len(agg_cols), ctypes.cast(ac, ctypes.c_void_p),
+                                     _ptr(sums), _ptr(cnts))
+    if rc == 1:
+        raise OverflowError("a group SUM does not fit in int64")
+    if rc == 2:
+        raise ValueError("a qualifying row has key >= ngroups")
+    return sums[:ngroups], cnts[:ngroups]

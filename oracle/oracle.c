@@ -437,3 +437,40 @@ void or_minmax_ar(int64_t n, int npred, const uint32_t* const* pcols, const int*
     free(cand);
     free(def);
 }
+
+/* ---------------------------------------------------- grouped SUM (s IV-E) */
+
+/*
+ * Exact  select key, count(*), sum(prod_a acols[a]) from R where <conjunction>
+ * group by key  -- the plain definition of a grouped aggregation over the
+ * selection (s IV-E/F; Fig. 4 "select count(*) from R where
+ * A<5 groupby B").  Keys are small non-negative integers
+ * (group id = key value, key < ngroups).  out_cnt[g] = rows of R with key g,
+ * out_sum[g] = their product sum (0 if nagg == 0).  Returns 0, 1 on int64
+ * overflow, 2 if a qualifying row has key >= ngroups.
+ */
+int or_select_group_sum(int64_t n, int npred, const uint32_t* const* pcols, const uint32_t* lo,
+                        const uint32_t* hi, const uint32_t* key, int ngroups, int nagg,
+                        const uint32_t* const* acols, int64_t* out_sum, int64_t* out_cnt) {
+    sel_ctx c;
+    memset(&c, 0, sizeof(c));
+    c.npred = npred; c.pcols = pcols; c.lo = lo; c.hi = hi;
+    __int128* s = (__int128*)calloc((size_t)(ngroups > 0 ? ngroups : 1), sizeof(__int128));
+    for (int g = 0; g < ngroups; ++g) out_cnt[g] = 0;
+    int rc = 0;
+    for (int64_t i = 0; i < n; ++i) {
+        if (!row_qualifies(&c, i)) continue;
+        uint32_t g = key[i];
+        if (g >= (uint32_t)ngroups) { rc = 2; break; }
+        out_cnt[g] += 1;
+        __int128 prod = 1;
+        for (int a = 0; a < nagg; ++a) prod *= (__int128)acols[a][i];
+        if (nagg > 0) s[g] += prod;
+    }
+    for (int g = 0; g < ngroups; ++g) {
+        if (s[g] > (__int128)INT64_MAX) rc = rc ? rc : 1;
+        out_sum[g] = (int64_t)s[g];
+    }
+    free(s);
+    return rc;
+}
