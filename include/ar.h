@@ -72,6 +72,7 @@ typedef enum {
 
 #define AR_MAX_PRED 8          /* predicates per conjunctive select            */
 #define AR_MAX_AGG 2           /* factors of the SUM product    */
+#define AR_MAX_GROUPS 4096     /* groups of ar_refine_group_sum (shared-memory group table) */
 #define AR_MAX_PLANES 64       /* sum of w_major over the predicates of a scan */
 
 /*
@@ -319,6 +320,26 @@ ar_status ar_sum_approximate(const ar_cands* in, const ar_column* const* cols, i
 size_t ar_minmax_ws_bytes(int64_t capacity);
 ar_status ar_minmax(const ar_cands* in, const ar_pred* preds, int32_t npred, const ar_column* col, int32_t mode,
                     int64_t* out7_dev, void* ws, size_t ws_bytes, void* stream);
+
+/*
+ * Grouped COUNT / SUM over the exact result (s IV-E/F):
+ *   select key, count(*), sum(prod_c cols[c]) from R where <preds> group by key
+ * e.g. Fig. 4 "select count(*) from R where A<5 groupby B".
+ * The paper keeps low-cardinality group columns whole on the GPU
+ * (PAPER.md:762-771), so `key` must be a k = 0 unsigned column: its values are
+ * the group ids (no hashing), the approximate pre-grouping is exact, and only
+ * the selection's false positives are eliminated (Alg. 2 on the candidate
+ * relation `in` of ar_approx_select over the same `preds`).  Factors as in
+ * ar_refine_sum (ncols in [0, 2]).  Writes device int64[2 * ngroups]:
+ *   out[g] = SUM over R with key g (0 when ncols == 0), out[ngroups + g] = COUNT.
+ * Errors: AR_ERR_INVALID (null pointers, ngroups outside [1, AR_MAX_GROUPS]),
+ * AR_ERR_UNSUPPORTED (decomposed or signed key), AR_ERR_RANGE (the key's
+ * descriptor admits values >= ngroups: base + 2^w_major - 1 must be < ngroups;
+ * or a SUM that could overflow, as ar_sum).
+ */
+ar_status ar_refine_group_sum(const ar_cands* in, const ar_pred* preds, int32_t npred, const ar_column* key,
+                              const ar_column* const* cols, int32_t ncols, int32_t ngroups, int64_t* out_dev,
+                              void* stream);
 
 /*
  * Positional projection of one column at the rows of `pos` (the invisible /

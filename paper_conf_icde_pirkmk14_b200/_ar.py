@@ -79,6 +79,8 @@ SIGNATURES = {
     "ar_sum_approximate": (ctypes.c_int, [ctypes.POINTER(Cands), ctypes.POINTER(_P), _I32, _P, _P]),
     "ar_project": (ctypes.c_int, [ctypes.POINTER(Positions), _P, _I32, _P, _P]),
     "ar_minmax_ws_bytes": (_SZ, [_I64]),
+    "ar_refine_group_sum": (ctypes.c_int, [ctypes.POINTER(Cands), ctypes.POINTER(Pred), _I32, _P, ctypes.POINTER(_P),
+                                           _I32, _I32, _P, _P]),
     "ar_minmax": (ctypes.c_int, [ctypes.POINTER(Cands), ctypes.POINTER(Pred), _I32, _P, _I32, _P, _P, _SZ, _P]),
     "ar_refine_sum": (ctypes.c_int, [ctypes.POINTER(Cands), ctypes.POINTER(Pred), _I32, ctypes.POINTER(_P), _I32,
                                      _P, _P, _P]),
@@ -218,6 +220,11 @@ def ar_minmax_ws_bytes(capacity: int) -> int:
 
 def ar_minmax(cands: Cands, preds, col, mode, out7_dev, ws, ws_bytes, stream):
     _call("ar_minmax", ctypes.byref(cands), _preds(preds), len(preds), col, mode, out7_dev, ws, ws_bytes, stream)
+
+
+def ar_refine_group_sum(cands: Cands, preds, key, cols, ngroups, out_dev, stream):
+    _call("ar_refine_group_sum", ctypes.byref(cands), _preds(preds), len(preds), key, _handles(cols), len(cols),
+          ngroups, out_dev, stream)
 
 
 def ar_refine_sum(cands: Cands, preds, cols, out_sum_dev, out_count_dev, stream):

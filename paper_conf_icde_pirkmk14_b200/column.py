@@ -212,6 +212,15 @@ def minmax(cands: CandidateList, preds, col: BWDColumn, mode: str, out7: torch.T
                   out7.data_ptr(), ws.ptr, ws.nbytes, _stream(stream))
 
 
+def refine_group_sum(cands: CandidateList, preds, key: BWDColumn, cols, ngroups: int, stream=None) -> torch.Tensor:
+    """Grouped COUNT / SUM over the refined rows (s IV-E/F): returns a device int64 tensor [2, ngroups]
+    (row 0: SUM(prod(cols)) per key value, row 1: COUNT)."""
+    out = torch.empty(2 * ngroups, dtype=torch.int64, device=key.device)
+    _ar.ar_refine_group_sum(cands.c, _pred_tuples(preds), key.handle, [c.handle for c in cols], ngroups,
+                            out.data_ptr(), _stream(stream))
+    return out.view(2, ngroups)
+
+
 def refine_sum(cands: CandidateList, preds, cols, out_sum: torch.Tensor, out_count: torch.Tensor = None,
                stream=None):
     """Steps a5+a6 fused: out_sum[0] = SUM(prod(cols)) over the refined rows, out_count[0] = their number."""

@@ -785,6 +785,51 @@ ar_status ar_minmax(const ar_cands* in, const ar_pred* preds, int32_t npred, con
     return launch_minmax(P, grid, s);
 }
 
+// ----------------------------------------------------------- grouped COUNT / SUM (s IV-E/F)
+
+ar_status ar_refine_group_sum(const ar_cands* in, const ar_pred* preds, int32_t npred, const ar_column* key,
+                              const ar_column* const* cols, int32_t ncols, int32_t ngroups, int64_t* out_dev,
+                              void* stream) {
+    ard::GroupParams P;
+    memset(&P, 0, sizeof(P));
+    ar_status st = setup_refine(in, preds, npred, P.r);
+    if (st != AR_OK) return st;
+    if (!out_dev || !valid_col(key) || ngroups < 1 || ngroups > AR_MAX_GROUPS) {
+        set_error("ar_refine_group_sum: null output / key, or ngroups %d outside [1, %d]", ngroups, AR_MAX_GROUPS);
+        return AR_ERR_INVALID;
+    }
+    const int64_t n = preds[0].col->d.n;
+    if (key->d.n != n) {
+        set_error("ar_refine_group_sum: key column has n != %lld", (long long)n);
+        return AR_ERR_INVALID;
+    }
+    if (key->d.k != 0 || key->d.value_signed) {
+        set_error("ar_refine_group_sum: the group key must be a GPU-resident (k = 0) unsigned column");
+        return AR_ERR_UNSUPPORTED;
+    }
+    // every key value must be a group id: base + 2^w_major - 1 < ngroups (from the descriptor)
+    const uint64_t max_key = (uint64_t)key->d.base + ((1ull << key->d.w_major) - 1ull);
+    if (max_key >= (uint64_t)ngroups) {
+        set_error("ar_refine_group_sum: key values up to %llu need ngroups > %llu", (unsigned long long)max_key,
+                  (unsigned long long)max_key);
+        return AR_ERR_RANGE;
+    }
+    const ar_column* const kc[1] = {key};
+    st = setup_aggs(kc, 1, preds, npred, n, &P.key, 1);
+    if (st != AR_OK) return st;
+    st = setup_aggs(cols, ncols, preds, npred, n, P.r.a, 0);
+    if (st != AR_OK) return st;
+    P.r.nagg = ncols;
+    P.ngroups = ngroups;
+    P.out = (unsigned long long*)out_dev;
+    cudaStream_t s = (cudaStream_t)stream;
+    AR_TRY_CUDA(cudaMemsetAsync(out_dev, 0, 2 * sizeof(int64_t) * (size_t)ngroups, s));
+    const int64_t cap = std::max<int64_t>(in->capacity, 1);
+    const int grid = (int)std::min<int64_t>((cap + ard::kRefTile - 1) / ard::kRefTile, (int64_t)num_sms() * 4);
+    g_last_scan = "group_sum_kernel";
+    return launch_group_sum(P, grid, s);
+}
+
 // ----------------------------------------------------------- fused a3+a5+a6
 
 size_t ar_select_refine_sum_ws_bytes(void) { return kSrsTicketBytes + (size_t)kSrsMaxGrid * 32; }

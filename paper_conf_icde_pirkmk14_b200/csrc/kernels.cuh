@@ -200,6 +200,14 @@ struct MinMaxParams {
     long long* out7;
 };
 
+// grouped COUNT / SUM over the refined rows (s IV-E/F) by a GPU-resident key
+struct GroupParams {
+    RefParams r;              // candidates, predicates, aggregate factors (r.a, r.nagg)
+    AggCol key;               // k == 0, unsigned; group id = key value (< ngroups, host-checked)
+    int32_t ngroups;
+    unsigned long long* out;  // [ngroups] sums, then [ngroups] counts
+};
+
 // leftjoinapproximate / leftjoinrefine (positional projection)
 struct ProjectParams {
     const uint32_t* pos;
@@ -233,6 +241,7 @@ ar_status launch_sum(const ard::SumParams& P, int grid, cudaStream_t s);
 ar_status launch_approx_sum(const ard::ApproxSumParams& P, int grid, cudaStream_t s);
 ar_status launch_project(const ard::ProjectParams& P, int grid, cudaStream_t s);
 ar_status launch_minmax(const ard::MinMaxParams& P, int grid, cudaStream_t s);
+ar_status launch_group_sum(const ard::GroupParams& P, int grid, cudaStream_t s);
 ar_status launch_decompose_minmax(const uint32_t* col, int64_t n, uint32_t flip, uint32_t* out2, cudaStream_t s);
 ar_status launch_pack_sliced(const uint32_t* col, int64_t n, int shift, uint32_t mask, uint32_t flip, uint32_t base,
                              int w, uint32_t* out, cudaStream_t s);

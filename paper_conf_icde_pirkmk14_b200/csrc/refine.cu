@@ -551,6 +551,86 @@ __global__ void minmax_final_kernel(const __grid_constant__ MinMaxParams P) {
     P.out7[6] = nc;
 }
 
+// Grouped COUNT / SUM (s IV-E/F; Fig. 4 "select count(*)
+// from R where A<5 groupby B" with B GPU-resident).  The paper expects group
+// keys to be low-cardinality columns kept whole on the GPU,
+// so the approximate pre-grouping is already exact and only the selection's
+// false positives must be removed before aggregating: 8 candidates per
+// thread are refined (refine_batch8), their keys and factors gathered in one
+// batch, and accumulated into per-CTA group tables in shared memory (the
+// "grouping table"; group id = key value, so no hash probing), flushed with
+// one global atomic per non-empty group and CTA.
+__device__ __forceinline__ void factor_batch8(const RefParams& P, const AggCol& a, const uint32_t (&pos)[8],
+                                              const uint32_t (&aux)[8], uint32_t pred, uint32_t (&v)[8]) {
+    if (a.pred >= 0 && P.p[a.pred].carried && a.k == 0) {
+        const RefPred& p = P.p[a.pred];
+        const uint32_t mask = p.w == 32 ? 0xffffffffu : ((1u << p.w) - 1u);
+#pragma unroll
+        for (int i = 0; i < 8; ++i) v[i] = ((aux[i] >> p.ashift) & mask) + a.base;
+    } else if (a.k == 0) {
+        part_batch8(a.major, pos, pred, (int)a.w, (int)a.layout, v);
+#pragma unroll
+        for (int i = 0; i < 8; ++i) v[i] += a.base;
+    } else {
+#pragma unroll
+        for (int i = 0; i < 8; ++i) v[i] = (pred >> i) & 1u ? agg_value_at(P, a, pos[i], aux[i]) : 0u;
+    }
+}
+
+constexpr int kGroupRepMax = 256;   // up to this many groups every warp gets its own table
+
+__global__ void __launch_bounds__(kRefThreads) group_sum_kernel(const __grid_constant__ GroupParams P) {
+    extern __shared__ unsigned long long gtab_all[];   // per table: [ngroups] sums, [ngroups] counts
+    const int G = P.ngroups;
+    // few groups: one table per warp, so the atomics of a hot group contend within a warp only
+    const int nrep = G <= kGroupRepMax ? kRefThreads / 32 : 1;
+    for (int g = threadIdx.x; g < 2 * G * nrep; g += kRefThreads) gtab_all[g] = 0ull;
+    __syncthreads();
+    unsigned long long* gtab = gtab_all + (nrep > 1 ? (threadIdx.x >> 5) * 2 * G : 0);
+    const long long count = *P.r.in_count;
+    const long long num_tiles = (count + kRefTile - 1) / kRefTile;
+    for (long long t = blockIdx.x; t < num_tiles; t += gridDim.x) {
+        const uint64_t j0 = (uint64_t)t * kRefTile + threadIdx.x * kRefPerThread;
+        uint32_t pos[8], aux[8];
+        load8(P.r.in_pos, j0, count, pos);
+        load8(P.r.in_aux, j0, count, aux);
+        uint32_t valid = 0;
+#pragma unroll
+        for (int i = 0; i < 8; ++i) valid |= (j0 + i < (uint64_t)count ? 1u : 0u) << i;
+        const uint32_t keep = refine_batch8(P.r, pos, aux, valid);
+        if (!keep) continue;
+        uint32_t key[8];
+        factor_batch8(P.r, P.key, pos, aux, keep, key);
+        unsigned long long prod[8];
+#pragma unroll
+        for (int i = 0; i < 8; ++i) prod[i] = 1ull;
+        for (int c = 0; c < P.r.nagg; ++c) {
+            uint32_t v[8];
+            factor_batch8(P.r, P.r.a[c], pos, aux, keep, v);
+#pragma unroll
+            for (int i = 0; i < 8; ++i) prod[i] *= v[i];
+        }
+#pragma unroll
+        for (int i = 0; i < 8; ++i) {
+            if (!((keep >> i) & 1u)) continue;
+            if (P.r.nagg > 0) atomicAdd(gtab + key[i], prod[i]);
+            atomicAdd(gtab + G + key[i], 1ull);
+        }
+    }
+    __syncthreads();
+    for (int g = threadIdx.x; g < G; g += kRefThreads) {
+        unsigned long long sm = 0, c = 0;
+        for (int r = 0; r < nrep; ++r) {
+            sm += gtab_all[r * 2 * G + g];
+            c += gtab_all[r * 2 * G + G + g];
+        }
+        if (c) {
+            if (P.r.nagg > 0) atomicAdd(P.out + g, sm);
+            atomicAdd(P.out + G + g, c);
+        }
+    }
+}
+
 // sumapproximate (Fig. 7 bwd.sumapproximate): the approximate
 // answer from the approximation subplan alone, before any residual is read
 // (PAPER.md:360-362, 894-897), as strict error bounds.  With
@@ -668,6 +748,17 @@ ar_status launch_minmax(const ard::MinMaxParams& P, int grid, cudaStream_t s) {
     AR_CHECK_LAUNCH("minmax_refine_kernel");
     ard::minmax_final_kernel<<<1, 32, 0, s>>>(P);
     AR_CHECK_LAUNCH("minmax_final_kernel");
+    return AR_OK;
+}
+ar_status launch_group_sum(const ard::GroupParams& P, int grid, cudaStream_t s) {
+    const int nrep = P.ngroups <= ard::kGroupRepMax ? ard::kRefThreads / 32 : 1;
+    const size_t smem = (size_t)2 * P.ngroups * nrep * sizeof(unsigned long long);
+    if (smem > 48 * 1024) {
+        AR_TRY_CUDA(cudaFuncSetAttribute((const void*)ard::group_sum_kernel,
+                                         cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem));
+    }
+    ard::group_sum_kernel<<<grid, ard::kRefThreads, smem, s>>>(P);
+    AR_CHECK_LAUNCH("group_sum_kernel");
     return AR_OK;
 }
 ar_status launch_exclusive_offset(const long long* all_counts, int world, int rank, long long* out,

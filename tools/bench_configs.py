@@ -5,8 +5,9 @@
   C5  SF1000-shaped Q6 per GPU share (750 M rows = SF125) with the l_shipdate residual in
       pinned host memory: HBM + host-link rooflines
   MM  C2 (SF10 Q6 predicates) MIN / MAX(l_extendedprice): ar_approx_select + ar_minmax (s IV-F)
+  GRP C2 shipdate + quantity predicates, SUM(l_extendedprice), COUNT group by l_discount (s IV-E)
 
-    python tools/bench_configs.py c1|c3|c5|mm [--reps R]
+    python tools/bench_configs.py c1|c3|c5|mm|grp [--reps R]
 
 One JSON line per point.  Timing as in bench.py: inputs resident, warm-up, CUDA
 events on the launching stream around R back-to-back repetitions, L2 flushed
@@ -206,15 +207,50 @@ def mm(args):
                           "minmax_frac": mm_bytes / (ms_mm / 1e3) / 1e9 / PEAK, "peak_gbs": PEAK}), flush=True)
 
 
+def grp(args):
+    c = datagen.q6_columns(2, 10)
+    n = c["shipdate"].size
+    sd = cu.BWDColumn(c["shipdate"], 24)
+    qt = cu.BWDColumn(c["quantity"], 32)
+    dc = cu.BWDColumn(c["discount"], 32)
+    ep = cu.BWDColumn(c["extprice"], 32, layout=_ar.AR_LAYOUT_PACKED)
+    preds = [(sd, *datagen.Q6_SHIPDATE), (qt, *datagen.Q6_QUANTITY)]
+    cands = cu.CandidateList(n)
+    ws = cu.Workspace(_ar.ar_select_ws_bytes(n))
+    flush = torch.empty(512 << 20, dtype=torch.uint8, device="cuda")
+    cu.approx_select(preds, cands, ws)
+    torch.cuda.synchronize()
+    pos = cands.positions()
+    ms_sel, _ = timed(lambda: cu.approx_select(preds, cands, ws), args.reps, flush)
+    res = {}
+    ms_grp, _ = timed(lambda: res.__setitem__("o", cu.refine_group_sum(cands, preds, dc, [ep], 16)), args.reps, flush)
+    torch.cuda.synchronize()
+    out = res["o"].cpu().numpy()
+    # algorithmic bytes: candidate list (8 B), residual sectors of the non-definite candidates, the
+    # key (l_discount, 4 b) and l_extendedprice sectors at the refined rows, 256 B out
+    sdv = c["shipdate"]
+    other = (c["quantity"] <= 23)
+    major = sdv >> 8
+    nondef = np.nonzero(other & (major >= 2) & (major <= 4) & (major != 3))[0]
+    res_rows = np.nonzero(other & (sdv >= datagen.Q6_SHIPDATE[0]) & (sdv <= datagen.Q6_SHIPDATE[1]))[0]
+    gb = 8.0 * pos.size + 32.0 * sectors(nondef, 8, 32) + 32.0 * sectors(res_rows, 4, 32) \
+        + 32.0 * sectors(res_rows, 24, 32) + 256
+    print(json.dumps({"config": "GRP (C2 shipdate+quantity, SUM(l_extendedprice) GROUP BY l_discount)", "rows": n,
+                      "candidates": int(pos.size), "groups": int((out[1] > 0).sum()), "result_rows": int(out[1].sum()),
+                      "select_us": ms_sel * 1e3, "group_sum_us": ms_grp * 1e3,
+                      "rows_per_s": n / ((ms_sel + ms_grp) / 1e3),
+                      "group_sum_frac": gb / (ms_grp / 1e3) / 1e9 / PEAK, "peak_gbs": PEAK}), flush=True)
+
+
 def main():
     ap = argparse.ArgumentParser()
-    ap.add_argument("config", choices=["c1", "c3", "c5", "mm"])
+    ap.add_argument("config", choices=["c1", "c3", "c5", "mm", "grp"])
     ap.add_argument("--reps", type=int, default=10)
     ap.add_argument("--widths", type=int, nargs="+", default=[8, 16, 24], help="C3 major bits")
     ap.add_argument("--sels", type=float, nargs="+", default=[0.0001, 0.001, 0.01, 0.1, 0.5], help="C3 selectivities")
     args = ap.parse_args()
     torch.cuda.set_device(0)
-    {"c1": c1, "c3": c3, "c5": c5, "mm": mm}[args.config](args)
+    {"c1": c1, "c3": c3, "c5": c5, "mm": mm, "grp": grp}[args.config](args)
 
 
 if __name__ == "__main__":
