@@ -1,8 +1,9 @@
 #!/bin/bash
 # Round measurement on one B200: GPU tests, smoke, the default bench line, the
 # reference (oracle) arm, the ncu launch list of the same bench command (cold,
-# serialised: compare shares), and one full ncu capture of each hot kernel.
-# Outputs land in gpurun_out/; summaries are copied to profiles/ by hand.
+# serialised: compare shares), one full ncu capture of each hot kernel, and the
+# secondary configurations.  Outputs land in gpurun_out/; summaries are copied
+# to profiles/ by hand.
 set -x
 nvidia-smi --query-gpu=name,clocks.sm,clocks.max.sm,clocks.mem,power.draw --format=csv > gpurun_out/smi.txt
 timeout 900 python -m pytest tests -m gpu -q > gpurun_out/gpu_tests.log 2>&1
@@ -14,3 +15,6 @@ timeout 900 ncu --metrics gpu__time_duration.sum --clock-control none --csv --lo
 VARIANTS=fused,staged timeout 900 ncu --set full --clock-control none --import-source on \
     -k regex:"fused_rl_kernel|select_tile_kernel|compact_kernel|refine_sum" -s 3 -c 4 -o gpurun_out/full python tools/profile_step.py \
     > gpurun_out/full.log 2>&1
+for c in mm grp c1 c5 c3; do
+  timeout 900 python tools/bench_configs.py $c --reps 10 >> gpurun_out/configs.jsonl 2>> gpurun_out/configs.err
+done
