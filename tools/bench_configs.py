@@ -111,6 +111,8 @@ def c3(args):
             torch.cuda.synchronize()
             nc, nr = cands.count(), pos.count()
             nd = int(o4[3].item())
+            # two independent GPU paths must agree (staged select -> refine vs the one-pass kernel)
+            consistent = nr == int(o4[1].item()) and nc == int(o4[2].item())
             # algorithmic bytes: majors scanned + candidate list (8 B) + non-definite residual
             # sectors + positions out (4 B)
             nondef = nc - nd
@@ -121,7 +123,7 @@ def c3(args):
             rows_s = n / ((ms_sel + ms_ref) / 1e3)
             print(json.dumps({
                 "config": "C3", "rows": n, "major_bits": M, "k": k, "w_major": w, "selectivity": s, "carry": carry,
-                "candidates": nc, "definite": nd, "results": nr,
+                "candidates": nc, "definite": nd, "results": nr, "staged_equals_one_pass": consistent,
                 "select_ms": ms_sel, "refine_ms": ms_ref, "fused_count_ms": ms_fus,
                 "select_refine_rows_per_s": rows_s,
                 "select_frac": sel_bytes / (ms_sel / 1e3) / 1e9 / PEAK,
