@@ -154,7 +154,7 @@ __device__ __forceinline__ void bar_sync(uint32_t id, uint32_t nthreads) {
     asm volatile("bar.sync %0, %1;" ::"r"(id), "r"(nthreads) : "memory");
 }
 
-// --- 64-bit status words for decoupled look-back.  Each word carries its own
+// --- 64-bit per-tile status words (rr_prefix below).  Each word carries its own
 // flag and value, and no other data is published through it, so relaxed
 // gpu-scope single-copy-atomic accesses are sufficient.
 __device__ __forceinline__ void st_relaxed(unsigned long long* p, unsigned long long v) {
@@ -167,86 +167,7 @@ __device__ __forceinline__ unsigned long long ld_relaxed(const unsigned long lon
 }
 
 constexpr unsigned long long kFlagAgg = 1ull << 62;
-constexpr unsigned long long kFlagPrefix = 2ull << 62;
 constexpr unsigned long long kValueMask = (1ull << 62) - 1;
-
-// Decoupled look-back (Merrill & Garland 2016), run by one full warp for tile
-// `t` (t > 0) whose aggregate is already published: returns the exclusive
-// prefix of all tiles < t.  Lane i inspects tile (t-1-i) of each 32-tile window.
-__device__ __forceinline__ unsigned long long lookback(const unsigned long long* status, long long t,
-                                                       unsigned lane) {
-    unsigned long long excl = 0;
-    long long base = t - 1;
-    while (true) {
-        long long idx = base - (long long)lane;
-        unsigned long long s;
-        while (true) {
-            s = idx >= 0 ? ld_relaxed(status + idx) : kFlagPrefix;  // before tile 0: prefix 0
-            if (__all_sync(0xffffffffu, (s >> 62) != 0)) break;
-            __nanosleep(32);
-        }
-        unsigned prefix_lanes = __ballot_sync(0xffffffffu, (s >> 62) == 2);
-        unsigned long long v = s & kValueMask;
-        if (prefix_lanes) {
-            unsigned first = __ffs(prefix_lanes) - 1;   // nearest tile holding an inclusive prefix
-            if (lane > first) v = 0;
-            for (int o = 16; o > 0; o >>= 1) v += __shfl_xor_sync(0xffffffffu, v, o);
-            return excl + v;
-        }
-        for (int o = 16; o > 0; o >>= 1) v += __shfl_xor_sync(0xffffffffu, v, o);
-        excl += v;
-        base -= 32;
-    }
-}
-
-// Wide variant: each lane inspects kLookV consecutive predecessors, so one
-// round trip covers 32 * kLookV tiles and the prefix frontier advances that
-// many tiles per L2 latency.  Entry (lane, j) is tile base - kLookV*lane - j.
-constexpr int kLookV = 8;
-__device__ __forceinline__ unsigned long long lookback_wide(const unsigned long long* status, long long t,
-                                                            unsigned lane) {
-    unsigned long long excl = 0;
-    long long base = t - 1;
-    while (true) {
-        unsigned long long s[kLookV];
-#pragma unroll
-        for (int j = 0; j < kLookV; ++j) {
-            const long long idx = base - (long long)(kLookV * lane + j);
-            s[j] = idx >= 0 ? ld_relaxed(status + idx) : kFlagPrefix;   // before tile 0: prefix 0
-        }
-        while (true) {
-            bool ready = true;
-#pragma unroll
-            for (int j = 0; j < kLookV; ++j) ready &= (s[j] >> 62) != 0;
-            if (__all_sync(0xffffffffu, ready)) break;
-            __nanosleep(64);
-#pragma unroll
-            for (int j = 0; j < kLookV; ++j) {
-                const long long idx = base - (long long)(kLookV * lane + j);
-                if ((s[j] >> 62) == 0) s[j] = ld_relaxed(status + idx);
-            }
-        }
-        int first_j = kLookV;   // nearest predecessor of this lane holding an inclusive prefix
-#pragma unroll
-        for (int j = kLookV - 1; j >= 0; --j)
-            if ((s[j] >> 62) == 2) first_j = j;
-        const unsigned has = __ballot_sync(0xffffffffu, first_j < kLookV);
-        unsigned long long v = 0;
-        if (has) {
-            const unsigned first_lane = __ffs(has) - 1;
-#pragma unroll
-            for (int j = 0; j < kLookV; ++j)
-                if (lane < first_lane || (lane == first_lane && j <= first_j)) v += s[j] & kValueMask;
-            for (int o = 16; o > 0; o >>= 1) v += __shfl_xor_sync(0xffffffffu, v, o);
-            return excl + v;
-        }
-#pragma unroll
-        for (int j = 0; j < kLookV; ++j) v += s[j] & kValueMask;
-        for (int o = 16; o > 0; o >>= 1) v += __shfl_xor_sync(0xffffffffu, v, o);
-        excl += v;
-        base -= 32 * kLookV;
-    }
-}
 
 // Round-robin persistent kernels (tile t = blockIdx + i * gridDim, every CTA
 // resident, tiles walked in order): each tile publishes kFlagAgg | count in

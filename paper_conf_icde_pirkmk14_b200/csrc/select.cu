@@ -1,30 +1,24 @@
 // select.cu -- step a3: approximate selection + stable compaction over SLICED
-// majors (s IV-B), and the one-pass fused A&R kernel
-// (a3 + a5 + a6).
+// majors (s IV-B), and the general one-pass A&R kernel
+// (a3 + a5 + a6) for shapes the result-ring kernel (fused.cu) does not cover.
 //
-// Structure (both kernels): persistent CTAs, one producer warp + NW consumer
-// warps.  The producer streams tiles (NW * 32 threads * BPT blocks * 32 rows)
-// of every predicate's bit planes into a ring of shared-memory stages with 1-D
-// TMA bulk copies (cp.async.bulk, completion on an mbarrier), so several tiles
-// of HBM traffic are in flight per SM.  Each consumer thread owns BPT
-// consecutive 32-row blocks and evaluates every range predicate on the bit
-// planes with borrow chains: per plane and per bound one 3-input logic op
-// decides 32 rows at once (DESIGN "Kernel a3").
-//
-// Like the paper's operators, which are JIT-generated per data type and
+// Every range predicate is evaluated on the bit planes with borrow chains: per
+// plane and per bound one 3-input logic op decides 32 rows at once (DESIGN
+// s6.2).  Like the paper's operators, which are JIT-generated per data type and
 // decomposition, the kernels are specialised on the
 // decomposition: FixedPlanes<BPT, W...> holds the thread's planes in registers
 // with compile-time widths (tight, unrolled code); DynPlanes<BPT> is the
 // generic runtime-width path for any other shape.
 //
-// select_kernel: ordered compaction.  popc per thread, block scan, decoupled
-// look-back across tiles with a 256-tile window, then the tile's (pos, aux)
-// entries are staged in shared memory in rounds of kStageEntries and written
-// with coalesced stores.  Cooperative launch + round-robin tiles.
+// select_tile_kernel + compact_kernel: one 8192-row tile per CTA (one TMA bulk
+// copy per predicate), stable compaction into the tile's workspace slice, then
+// one warp per tile moves the slice to its final offset (no CTA waits on
+// another CTA; DESIGN s6.2 lists the measured alternatives).
 //
-// fused_kernel: no candidate list in HBM.  Non-definite candidates are refined
-// in place (residual gathers issued kBatch at a time per thread so they
-// overlap), then the SUM factors of the exact rows are gathered the same way.
+// fused_kernel: persistent CTAs, one producer warp streaming tiles into a ring
+// of shared-memory stages (produce_ring), consumer warps compacting candidates
+// into per-warp lists in shared memory; non-definite candidates are refined in
+// place, the SUM factors of the exact rows gathered asynchronously.
 #include <type_traits>
 
 #include "rl_common.cuh"
@@ -337,18 +331,6 @@ struct DynPlanes {
     }
 };
 
-template <class T>
-struct requires_params : std::false_type {};
-template <int BPT>
-struct requires_params<DynPlanes<BPT>> : std::true_type {};
-
-template <class PS, int B>
-__device__ __forceinline__ uint32_t ps_value(const PS& ps, const SelParams& P, int c, uint32_t l) {
-    if constexpr (requires_params<PS>::value)
-        return ps.template value_rt<B>(P, c, l);
-    else
-        return ps.template value_rt<B>(c, l);
-}
 
 // ------------------------------------------------------------ pipeline
 
