@@ -4,10 +4,11 @@
   C3  1 G-row u32 column: major-bit width {8,16,24} x selectivity sweep, positions out
   C5  SF1000-shaped Q6 per GPU share (750 M rows = SF125) with the l_shipdate residual in
       pinned host memory: HBM + host-link rooflines
+  C4  the N = 1 point of C4: TPC-H SF100-shaped Q6 (600 M rows) on one GPU, one pass and staged
   MM  C2 (SF10 Q6 predicates) MIN / MAX(l_extendedprice): ar_approx_select + ar_minmax (s IV-F)
   GRP C2 shipdate + quantity predicates, SUM(l_extendedprice), COUNT group by l_discount (s IV-E)
 
-    python tools/bench_configs.py c1|c3|c5|mm|grp [--reps R]
+    python tools/bench_configs.py c1|c3|c4|c5|mm|grp [--reps R]
 
 One JSON line per point.  Timing as in bench.py: inputs resident, warm-up, CUDA
 events on the launching stream around R back-to-back repetitions, L2 flushed
@@ -176,6 +177,42 @@ def c5(args):
         "host_link_frac_staged": host32 / (ms_s / 1e3) / 1e9 / link_gbs}), flush=True)
 
 
+def c4(args):
+    c = datagen.q6_columns(4, 100)
+    n = c["shipdate"].size
+    sd = cu.BWDColumn(c["shipdate"], 24)
+    dc = cu.BWDColumn(c["discount"], 32)
+    qt = cu.BWDColumn(c["quantity"], 32)
+    ep = cu.BWDColumn(c["extprice"], 32, layout=_ar.AR_LAYOUT_PACKED)
+    preds = [(sd, *datagen.Q6_SHIPDATE), (dc, *datagen.Q6_DISCOUNT), (qt, *datagen.Q6_QUANTITY)]
+    cands = cu.CandidateList(n)
+    ws = cu.Workspace(_ar.ar_select_ws_bytes(n))
+    o4 = torch.zeros(4, dtype=torch.int64, device="cuda")
+    s2 = torch.zeros(2, dtype=torch.int64, device="cuda")
+    srs_ws = cu.SrsWorkspace()
+
+    def staged():
+        cu.approx_select(preds, cands, ws)
+        cu.refine_sum(cands, preds, [ep, dc], s2[0:1], s2[1:2])
+
+    ms_f, mn_f = timed(lambda: cu.select_refine_sum(preds, [ep, dc], o4, ws=srs_ws), args.reps)
+    ms_s, mn_s = timed(staged, args.reps)
+    torch.cuda.synchronize()
+    # algorithmic bytes (DESIGN s6): majors 1.75 B/row + touched residual / l_extendedprice sectors + 8 B
+    sdv = c["shipdate"]
+    oth = (c["discount"] >= 5) & (c["discount"] <= 7) & (c["quantity"] <= 23)
+    major = sdv >> 8
+    nondef = np.nonzero(oth & (major >= 2) & (major <= 4) & (major != 3))[0]
+    res = np.nonzero(oth & (sdv >= datagen.Q6_SHIPDATE[0]) & (sdv <= datagen.Q6_SHIPDATE[1]))[0]
+    alg = n * 14 / 8 + 32.0 * sectors(nondef, 8, 32) + 32.0 * sectors(res, 24, 32) + 8
+    print(json.dumps({"config": "C4 (N=1 point: SF100 Q6, 600 M rows, one GPU)", "rows": n,
+                      "fused_ms": ms_f, "staged_ms": ms_s, "fused_rows_per_s": n / (ms_f / 1e3),
+                      "staged_rows_per_s": n / (ms_s / 1e3), "fused_frac": alg / (ms_f / 1e3) / 1e9 / PEAK,
+                      "parity_staged_equals_one_pass": s2.tolist() == o4[:2].tolist(),
+                      "sum": int(o4[0].item()), "count": int(o4[1].item()), "peak_gbs": PEAK,
+                      "l2": "inputs 3.5 GB >> 126 MB L2 (no flush needed)"}), flush=True)
+
+
 def mm(args):
     c = datagen.q6_columns(2, 10)
     n = c["shipdate"].size
@@ -246,13 +283,13 @@ def grp(args):
 
 def main():
     ap = argparse.ArgumentParser()
-    ap.add_argument("config", choices=["c1", "c3", "c5", "mm", "grp"])
+    ap.add_argument("config", choices=["c1", "c3", "c4", "c5", "mm", "grp"])
     ap.add_argument("--reps", type=int, default=10)
     ap.add_argument("--widths", type=int, nargs="+", default=[8, 16, 24], help="C3 major bits")
     ap.add_argument("--sels", type=float, nargs="+", default=[0.0001, 0.001, 0.01, 0.1, 0.5], help="C3 selectivities")
     args = ap.parse_args()
     torch.cuda.set_device(0)
-    {"c1": c1, "c3": c3, "c5": c5, "mm": mm, "grp": grp}[args.config](args)
+    {"c1": c1, "c3": c3, "c4": c4, "c5": c5, "mm": mm, "grp": grp}[args.config](args)
 
 
 if __name__ == "__main__":
