@@ -507,9 +507,12 @@ def ours(args):
                        "majors (105 MB), ar_select_refine_sum reading the shipdate residual and l_extendedprice "
                        "zero-copy over the host link (only touched 64-B granules), D2H of (SUM, count)"}
 
-    cpu = None
+    cpu = cpu1 = None
     if rank == 0 and world == 1 and not args.no_cpu:
         cpu = run_oracle(cols, rows, args.cpu_seconds)
+        # and single-threaded (the paper's MonetDB baseline ran one thread)
+        cpu1 = run_oracle(cols, rows, 0.0, threads=1)
+        cpu1 = {k: v for k, v in cpu1.items() if k not in ("sum", "count")}
 
     if dist_h:
         _ar.ar_dist_free(dist_h)
@@ -536,7 +539,7 @@ def ours(args):
                       f"({len(copies)} x {bytes_per_copy / 1e6:.0f} MB > 126 MB L2)",
                 "timing": "K steps = one CUDA-graph replay; CUDA events on the launching stream; max over ranks; "
                           "fused step = 1 launch of ar_select_refine_sum_ws (PDL, early input reads)"}),
-            "roofline": head["roofline"], "cpu_baseline": cpu, "e2e": e2e,
+            "roofline": head["roofline"], "cpu_baseline": cpu, "cpu_baseline_single_thread": cpu1, "e2e": e2e,
             "gpu_launches": head["gpu_launches"], "gpu_kernels": head["gpu_kernels"],
             "clocks": sampler.result(),
             "counts": {"candidates": ab["n_cand"], "definite": ab["n_def"], "result": ab["n_result"],
