@@ -27,7 +27,8 @@ def main():
         print("set L2 fetch granularity", os.environ["L2FG"], err, rt.cudaDeviceGetLimit(rt.cudaLimit.cudaLimitMaxL2FetchGranularity))
     cols = datagen.q6_columns(2, sf)
     n = cols["shipdate"].size
-    sd = cu.BWDColumn(cols["shipdate"], 24)
+    # RES_LOC=1: the l_shipdate residual in pinned host memory (the C5 mechanism, read over the host link)
+    sd = cu.BWDColumn(cols["shipdate"], 24, residual_loc=int(os.environ.get("RES_LOC", "0")))
     dc = cu.BWDColumn(cols["discount"], 32)
     qt = cu.BWDColumn(cols["quantity"], 32)
     ep = cu.BWDColumn(cols["extprice"], 32, layout=_ar.AR_LAYOUT_PACKED)
