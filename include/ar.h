@@ -189,7 +189,8 @@ ar_status ar_decompose_plan(const uint32_t* col, int64_t n, int32_t major_bits,
                             void* ws, size_t ws_bytes, ar_column_desc* desc, void* stream);
 
 /*
- * Decompose and pack `col` per `desc`: the major part is written to
+ * bwdecompose (the split of Fig. 2):
+ * decompose and pack `col` per `desc`: the major part is written to
  * `major_buf` (device memory, desc->major_bytes bytes, padding zeroed) and the
  * residual part to `residual_buf` (device memory, or pinned host memory when
  * desc->residual_loc == AR_LOC_HOST_PINNED; desc->residual_bytes bytes).
@@ -360,7 +361,8 @@ ar_status ar_project(const ar_positions* pos, const ar_column* col, int32_t mode
                      void* stream);
 
 /*
- * Fused refine + SUM (a5 + a6): the refinement of ar_refine without
+ * Fused refine + SUM (a5 + a6; SUM(refine) of Fig. 3 / Fig. 7, PAPER.md:333-359,
+ * 884-889, over Alg. 2's refinement): the refinement of ar_refine without
  * materialising positions, then the product SUM of ar_sum over the refined
  * rows.  Aggregated columns that are also predicate columns reuse the carried
  * approximation (and residual) instead of re-gathering.  Writes
@@ -416,6 +418,9 @@ ar_status ar_select_refine_sum_ws(const ar_pred* preds, int32_t npred,
                                   int64_t* out_dev, void* ws, size_t ws_bytes, void* stream);
 
 /* -------------------------------- a4: row-sharded multi-GPU exchange */
+/* Not in the paper, which runs one query per GPU: the build
+ * shards rows across GPUs; rows are independent, so only counts
+ * (for global result offsets) and the SUM are exchanged. */
 
 typedef struct ar_dist ar_dist;
 
