@@ -66,10 +66,10 @@ def _load():
         lib.or_select_sum.restype = i32
         lib.or_sum_at.argtypes = [p, i64, i32, p, p]
         lib.or_sum_at.restype = i32
-        lib.or_sum_bounds.argtypes = [i64, i32, p, p, p, p, p, i32, p, p, p, p]
+        lib.or_sum_bounds.argtypes = [i64, i32, p, p, p, p, p, p, i32, p, p, p, p]
         lib.or_sum_bounds.restype = i32
         lib.or_select_minmax.argtypes = [i64, i32, p, p, p, p, p, i32, i32, p]
-        lib.or_minmax_ar.argtypes = [i64, i32, p, p, p, p, p, p, i32, u32, i32, i32, p, p]
+        lib.or_minmax_ar.argtypes = [i64, i32, p, p, p, p, p, p, p, i32, u32, i32, i32, p, p]
         lib.or_select_group_sum.argtypes = [i64, i32, p, p, p, p, i32, i32, p, p, p]
         lib.or_select_group_sum.restype = i32
         lib.or_threads_default.restype = i32
@@ -89,6 +89,17 @@ def _ptr(a):
 def _ptr_array(arrs):
     arr = (ctypes.c_void_p * max(1, len(arrs)))(*[a.ctypes.data for a in arrs])
     return arr
+
+
+def _signed_preds(pred_cols, los, his, signed):
+    """int32 predicate columns / bounds as their uint32 bit patterns, plus the per-predicate flags
+    (None when every predicate is unsigned)."""
+    if signed is None:
+        return [_u32(c) for c in pred_cols], list(los), list(his), None
+    sg = np.asarray([1 if x else 0 for x in signed], dtype=np.int32)
+    cols = [np.ascontiguousarray(c).view(np.uint32) if np.asarray(c).dtype == np.int32 else _u32(c)
+            for c in pred_cols]
+    return cols, [int(x) & 0xFFFFFFFF for x in los], [int(x) & 0xFFFFFFFF for x in his], sg
 
 
 def default_threads() -> int:
@@ -121,17 +132,24 @@ def paper_f_flags(v, k: int, op: str, x: int):
     return flag.astype(bool)
 
 
-def approx_select(values, ks, los, his, base=None):
+def approx_select(values, ks, los, his, base=None, signed=None):
     """Reference intermediates of the approximate selection (conjunction of predicates):
     returns (cand_positions int64, definite flags at those positions).  Each predicate
-    column is decomposed with its own k; cand/def of a row are the ANDs over predicates."""
+    column is decomposed with its own k; cand/def of a row are the ANDs over predicates.
+    signed[c] true: column c is int32 and its bounds are signed; it is decomposed in the
+    order-preserving key domain d = v ^ 2^31 (DESIGN R8), base[c] in that domain."""
     n = len(values[0])
     cand = np.ones(n, dtype=bool)
     dfn = np.ones(n, dtype=bool)
     for c, v in enumerate(values):
         b = 0 if base is None else base[c]
+        lo, hi = int(los[c]), int(his[c])
+        v = np.asarray(v)
+        if signed is not None and signed[c]:
+            v = np.ascontiguousarray(v).view(np.uint32) ^ np.uint32(0x80000000)
+            lo, hi = (lo & 0xFFFFFFFF) ^ 0x80000000, (hi & 0xFFFFFFFF) ^ 0x80000000
         major, _, _ = decompose(v, ks[c], b)
-        cf, df = bucket_flags(major, ks[c], los[c], his[c], b)
+        cf, df = bucket_flags(major, ks[c], lo, hi, b)
         cand &= cf
         dfn &= df
     pos = np.nonzero(cand)[0].astype(np.int64)
@@ -177,10 +195,12 @@ def sum_at(pos, agg_cols):
     return int(s.value)
 
 
-def sum_bounds(pred_cols, pred_ks, los, his, agg_cols=(), agg_ks=(), pred_bases=None, agg_bases=None):
+def sum_bounds(pred_cols, pred_ks, los, his, agg_cols=(), agg_ks=(), pred_bases=None, agg_bases=None,
+               pred_signed=None):
     """bwd.sumapproximate (Fig. 7; bounds PAPER.md:375-382):
-    (sum_lo, sum_hi, count_lo, count_hi) from the approximation alone."""
-    pred_cols = [_u32(c) for c in pred_cols]
+    (sum_lo, sum_hi, count_lo, count_hi) from the approximation alone.  pred_signed[p]: predicate p's
+    column is int32 (bounds signed, base in the key domain v ^ 2^31)."""
+    pred_cols, los, his, sg = _signed_preds(pred_cols, los, his, pred_signed)
     agg_cols = [_u32(c) for c in agg_cols]
     n = pred_cols[0].size
     npred, nagg = len(pred_cols), len(agg_cols)
@@ -193,7 +213,7 @@ def sum_bounds(pred_cols, pred_ks, los, his, agg_cols=(), agg_ks=(), pred_bases=
     out = np.zeros(4, dtype=np.int64)
     pc, ac = _ptr_array(pred_cols), _ptr_array(agg_cols)
     if _load().or_sum_bounds(n, npred, ctypes.cast(pc, ctypes.c_void_p), _ptr(pks), _ptr(pb), _ptr(lo), _ptr(hi),
-                             nagg, ctypes.cast(ac, ctypes.c_void_p), _ptr(aks), _ptr(ab), _ptr(out)):
+                             _ptr(sg) if sg is not None else None, nagg, ctypes.cast(ac, ctypes.c_void_p), _ptr(aks), _ptr(ab), _ptr(out)):
         raise OverflowError("SUM bound does not fit in int64")
     return tuple(int(x) for x in out)
 
@@ -222,10 +242,11 @@ def select_minmax(pred_cols, los, his, ycol, mode: str = "min", signed=None, y_s
 
 
 def minmax_ar(pred_cols, pred_ks, los, his, ycol, y_k: int, mode: str = "min", pred_bases=None,
-              y_base: int = 0, y_signed: bool = False, flags: bool = False):
+              y_base: int = 0, y_signed: bool = False, flags: bool = False, pred_signed=None):
     """A&R MIN / MAX of s IV-F: dict with the refined answer and survivors,
-    the approximate bounds (lo, hi), |refined|, |D|, |C|, and (flags=True) the refined-row mask."""
-    pred_cols = [_u32(c) for c in pred_cols]
+    the approximate bounds (lo, hi), |refined|, |D|, |C|, and (flags=True) the refined-row mask.
+    pred_signed[p]: predicate p's column is int32 (bounds signed, base in the key domain)."""
+    pred_cols, los, his, sg = _signed_preds(pred_cols, los, his, pred_signed)
     y = np.ascontiguousarray(ycol).view(np.uint32) if np.asarray(ycol).dtype == np.int32 else _u32(ycol)
     n = y.size
     npred = len(pred_cols)
@@ -237,7 +258,7 @@ def minmax_ar(pred_cols, pred_ks, los, his, ycol, y_k: int, mode: str = "min", p
     fl = np.zeros(max(n, 1), dtype=np.uint8)
     pc = _ptr_array(pred_cols)
     _load().or_minmax_ar(n, npred, ctypes.cast(pc, ctypes.c_void_p), _ptr(pks), _ptr(pb), _ptr(lo), _ptr(hi),
-                         _ptr(y), y_k, y_base & 0xFFFFFFFF, 1 if y_signed else 0, 0 if mode == "min" else 1,
+                         _ptr(sg) if sg is not None else None, _ptr(y), y_k, y_base & 0xFFFFFFFF, 1 if y_signed else 0, 0 if mode == "min" else 1,
                          _ptr(out), _ptr(fl) if flags else None)
     r = {"value": int(out[0]), "survivors": int(out[1]), "lo": int(out[2]), "hi": int(out[3]),
          "refined": int(out[4]), "definite": int(out[5]), "candidates": int(out[6])}

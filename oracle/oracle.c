@@ -267,22 +267,28 @@ int or_sum_at(const int64_t* pos, int64_t npos, int nagg, const uint32_t* const*
  *   out[1] = sum over candidate rows of prod_a max(bucket_a)    (>= SUM over R)
  *   out[2] = |definite|,  out[3] = |candidates|
  * pks/pbase: k and base of each predicate column; aks/abase: of each aggregate.
+ * psgn (optional, NULL = all unsigned): psgn[p] = 1 marks an int32 predicate
+ * column; its values and bounds are compared in the order-preserving key
+ * domain d = v ^ 2^31 (DESIGN R8), in which its base and buckets
+ * are defined.  Aggregate factors are unsigned (the ABI's product SUM).
  * Returns 1 if a bound does not fit in int64.
  */
 int or_sum_bounds(int64_t n, int npred, const uint32_t* const* pcols, const int* pks, const uint32_t* pbase,
-                  const uint32_t* lo, const uint32_t* hi, int nagg, const uint32_t* const* acols,
+                  const uint32_t* lo, const uint32_t* hi, const int* psgn, int nagg, const uint32_t* const* acols,
                   const int* aks, const uint32_t* abase, int64_t* out) {
     __int128 slo = 0, shi = 0;
     int64_t ndef = 0, ncand = 0;
     for (int64_t i = 0; i < n; ++i) {
         int cand = 1, def = 1;
         for (int p = 0; p < npred; ++p) {
+            uint32_t flip = (psgn && psgn[p]) ? 0x80000000u : 0u;
+            uint32_t d = pcols[p][i] ^ flip, dlo = lo[p] ^ flip, dhi = hi[p] ^ flip;
             uint64_t two_k = (uint64_t)1 << pks[p];
-            uint64_t m = (uint64_t)(uint32_t)(pcols[p][i] - pbase[p]) / two_k;
+            uint64_t m = (uint64_t)(uint32_t)(d - pbase[p]) / two_k;
             uint64_t first = (uint64_t)pbase[p] + m * two_k;
             uint64_t last = first + two_k - 1;
-            if (!(lo[p] <= hi[p] && first <= hi[p] && last >= lo[p])) cand = 0;
-            if (!(first >= lo[p] && last <= hi[p])) def = 0;
+            if (!(dlo <= dhi && first <= dhi && last >= dlo)) cand = 0;
+            if (!(first >= dlo && last <= dhi)) def = 0;
         }
         if (!cand) continue;
         ++ncand;
@@ -352,7 +358,10 @@ void or_select_minmax(int64_t n, int npred, const uint32_t* const* pcols, const 
  *  3. refinement: "a join of the candidate set with the input residuals and
  *     the calculation of the minimum": the exact predicates
  *     and the exact Y on the set of step 2.
- * pks / pbase: k and base of each predicate column; ky / ybase: of Y.  Bounds
+ * pks / pbase: k and base of each predicate column; ky / ybase: of Y.  psgn
+ * (optional, NULL = all unsigned): psgn[p] = 1 marks an int32 predicate column,
+ * compared -- approximately and exactly -- in the key domain d = v ^ 2^31
+ * (DESIGN R8), in which its base and buckets are defined.  Bounds
  * and the result are values (int32 when ysgn).  out[0] = refined aggregate
  * (0 if no refined row survives), out[1] = survivors of the refinement (>= 1
  * iff R is not empty), out[2] / out[3] = approximate lower / upper bound
@@ -361,8 +370,8 @@ void or_select_minmax(int64_t n, int npred, const uint32_t* const* pcols, const 
  * of step 2.
  */
 void or_minmax_ar(int64_t n, int npred, const uint32_t* const* pcols, const int* pks, const uint32_t* pbase,
-                  const uint32_t* lo, const uint32_t* hi, const uint32_t* ycol, int ky, uint32_t ybase, int ysgn,
-                  int mode, int64_t* out, uint8_t* refine_flag) {
+                  const uint32_t* lo, const uint32_t* hi, const int* psgn, const uint32_t* ycol, int ky,
+                  uint32_t ybase, int ysgn, int mode, int64_t* out, uint8_t* refine_flag) {
     uint32_t flip = ysgn ? 0x80000000u : 0u;
     uint64_t two_ky = (uint64_t)1 << ky;
     uint8_t* cand = (uint8_t*)calloc((size_t)(n > 0 ? n : 1), 1);
@@ -371,12 +380,14 @@ void or_minmax_ar(int64_t n, int npred, const uint32_t* const* pcols, const int*
     for (int64_t i = 0; i < n; ++i) {
         int c = 1, d = 1;
         for (int p = 0; p < npred; ++p) {
+            uint32_t pf = (psgn && psgn[p]) ? 0x80000000u : 0u;
+            uint32_t key = pcols[p][i] ^ pf, klo = lo[p] ^ pf, khi = hi[p] ^ pf;
             uint64_t two_k = (uint64_t)1 << pks[p];
-            uint64_t m = (uint64_t)(uint32_t)(pcols[p][i] - pbase[p]) / two_k;
+            uint64_t m = (uint64_t)(uint32_t)(key - pbase[p]) / two_k;
             uint64_t first = (uint64_t)pbase[p] + m * two_k;
             uint64_t last = first + two_k - 1;
-            if (!(lo[p] <= hi[p] && first <= hi[p] && last >= lo[p])) c = 0;
-            if (!(first >= lo[p] && last <= hi[p])) d = 0;
+            if (!(klo <= khi && first <= khi && last >= klo)) c = 0;
+            if (!(first >= klo && last <= khi)) d = 0;
         }
         cand[i] = (uint8_t)c;
         def[i] = (uint8_t)(c && d);
@@ -417,8 +428,11 @@ void or_minmax_ar(int64_t n, int npred, const uint32_t* const* pcols, const int*
             if (refine_flag) refine_flag[i] = 1;
             ++nref;
             int ok = 1;
-            for (int p = 0; p < npred; ++p)
-                if (!(lo[p] <= pcols[p][i] && pcols[p][i] <= hi[p])) ok = 0;
+            for (int p = 0; p < npred; ++p) {
+                uint32_t pf = (psgn && psgn[p]) ? 0x80000000u : 0u;
+                uint32_t key = pcols[p][i] ^ pf;
+                if (!((lo[p] ^ pf) <= key && key <= (hi[p] ^ pf))) ok = 0;
+            }
             if (!ok) continue;
             int64_t v = ysgn ? (int64_t)(int32_t)ycol[i] : (int64_t)ycol[i];
             if (surv == 0 || (mode == 0 ? v < best : v > best)) best = v;

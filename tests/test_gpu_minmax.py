@@ -24,7 +24,7 @@ def cu():
 def run_minmax(cu, pcols, los, his, ycol, mode, carry=True):
     from paper_conf_icde_pirkmk14_b200 import _ar
     n = pcols[0].n
-    preds = [(c, lo, hi) for c, lo, hi in zip(pcols, los, his)]
+    preds = [(c, lo & 0xFFFFFFFF, hi & 0xFFFFFFFF) for c, lo, hi in zip(pcols, los, his)]
     cands = cu.CandidateList(n)
     cu.approx_select(preds, cands, cu.Workspace(_ar.ar_select_ws_bytes(n)), carry=carry)
     out7 = torch.full((7,), -99, dtype=torch.int64, device="cuda")
@@ -33,10 +33,11 @@ def run_minmax(cu, pcols, los, his, ycol, mode, carry=True):
     return out7.cpu().tolist()
 
 
-def expect(pvals, pcols, los, his, yvals, ycol, mode, y_signed=False):
+def expect(pvals, pcols, los, his, yvals, ycol, mode, y_signed=False, pred_signed=None):
     r = oracle.minmax_ar(pvals, [c.k for c in pcols], los, his, yvals, ycol.k, mode,
-                         pred_bases=[int(c.desc.base) for c in pcols], y_base=int(ycol.desc.base), y_signed=y_signed)
-    exact = oracle.select_minmax(pvals, los, his, yvals, mode, y_signed=y_signed)
+                         pred_bases=[int(c.desc.base) for c in pcols], y_base=int(ycol.desc.base), y_signed=y_signed,
+                         pred_signed=pred_signed)
+    exact = oracle.select_minmax(pvals, los, his, yvals, mode, signed=pred_signed, y_signed=y_signed)
     assert (r["value"], r["survivors"] > 0) == (exact[0], exact[1] > 0)   # A&R reaches the plain answer
     return [r["value"], r["survivors"], r["lo"], r["hi"], r["refined"], r["definite"], r["candidates"]]
 
@@ -98,6 +99,27 @@ def test_gpu_minmax_signed_for_base(cu, mode):
     yc = cu.BWDColumn(s["lon"], 24, signed=True, base="min")
     got = run_minmax(cu, [xc], [100], [350], yc, mode)
     assert got == expect([x], [xc], [100], [350], np.asarray(s["lon"], dtype=np.int32), yc, mode, y_signed=True)
+
+
+@pytest.mark.parametrize("mode", ["min", "max"])
+@pytest.mark.parametrize("n", [4097, 300_001])
+def test_gpu_minmax_signed_predicates(cu, mode, n):
+    # the spatial query's signed lon / lat predicates (FOR base, 24/8) select the rows; MIN / MAX of a
+    # third column and of the signed lon itself (its major carried in the approximation tuple)
+    s = datagen.spatial_columns(14, n)
+    lon, lat = np.asarray(s["lon"], dtype=np.int32), np.asarray(s["lat"], dtype=np.int32)
+    pcols = [cu.BWDColumn(lon, 24, signed=True, base="min"), cu.BWDColumn(lat, 24, signed=True, base="min")]
+    y = datagen.uniform_u32(15, n)
+    yc = cu.BWDColumn(y, 20)
+    # Table I's box, and a box whose longitude range crosses zero (negative lower bound)
+    for los, his in (([datagen.SPATIAL_LON[0], datagen.SPATIAL_LAT[0]], [datagen.SPATIAL_LON[1], datagen.SPATIAL_LAT[1]]),
+                     ([-900_000, 4_000_000], [600_000, 6_000_000])):
+        got = run_minmax(cu, pcols, los, his, yc, mode)
+        assert got == expect([lon, lat], pcols, los, his, y, yc, mode, pred_signed=[True, True])
+        assert got[1] > 0
+        got = run_minmax(cu, pcols, los, his, pcols[0], mode)
+        assert got == expect([lon, lat], pcols, los, his, lon, pcols[0], mode, y_signed=True,
+                             pred_signed=[True, True])
 
 
 def test_gpu_minmax_empty_and_all(cu):
