@@ -205,7 +205,22 @@ ar_status ar_decompose(const uint32_t* col, const ar_column_desc* desc,
                        void* residual_buf, uint64_t residual_buf_bytes,
                        void* stream, ar_column** out);
 
-/* Wrap already-decomposed parts (e.g. a copy of the buffers ar_decompose wrote) in a new handle. */
+/*
+ * Widen a planned descriptor to a stored major width w_major >= desc->w_major
+ * (<= major_bits) and recompute major_bytes.  Row shards of one table are
+ * planned separately but must share one bucket geometry and layout: the
+ * caller takes the global w_M = max over shards (an allreduce-MAX, SURVEY
+ * s8(e)) and widens every shard's descriptor before ar_decompose.  Host only.
+ * Errors: AR_ERR_INVALID (bad desc), AR_ERR_RANGE (w_major outside that range).
+ */
+ar_status ar_decompose_set_width(ar_column_desc* desc, int32_t w_major);
+
+/* Wrap already-decomposed parts (e.g. a copy of the buffers ar_decompose wrote) in a new handle.
+ * Both buffers must be 16-B aligned and hold at least the bytes the descriptor's
+ * geometry needs (n, w_major, k and the layouts; ar_decompose_plan's sizes).
+ * Errors: AR_ERR_INVALID (bad desc, null or misaligned buffer), AR_ERR_RANGE
+ * (major_bytes / residual_bytes below that size), AR_ERR_CUDA (a host-resident
+ * part that is not mapped pinned memory). */
 ar_status ar_column_wrap(const ar_column_desc* desc, const void* major_buf, const void* residual_buf,
                          ar_column** out);
 ar_status ar_column_get_desc(const ar_column* col, ar_column_desc* desc);
@@ -225,11 +240,13 @@ size_t ar_select_ws_bytes(int64_t n);
  * major ranges cand = [lo>>k, hi>>k] (bucket intersects [lo,hi]) and
  * def = [ceil(lo/2^k), floor((hi+1)/2^k) - 1] (bucket inside [lo,hi]), with
  * b = base subtracted first (DESIGN "Readings").  Device side
- * (a3): one pass over the packed majors, stable compaction (warp ballot /
- * popc, block scan, decoupled look-back) into out->pos / out->aux /
- * *out->count.  npred == 0 selects every row.  A predicate with lo > hi makes
- * the result empty (AR_OK).
- * Errors: AR_ERR_INVALID (npred > AR_MAX_PRED, null / mismatched columns,
+ * (a3): one pass over the packed majors, stable compaction (per-tile warp
+ * ballot / popc and block scan into tile slices, then one compaction launch
+ * that places every slice at the prefix of the earlier tiles' counts) into
+ * out->pos / out->aux / *out->count.  At least one predicate is required (a
+ * scan needs a column; [0, 2^32 - 1] keeps every row).  A predicate with
+ * lo > hi makes the result empty (AR_OK).
+ * Errors: AR_ERR_INVALID (npred < 1 or > AR_MAX_PRED, null / mismatched columns,
  * non-SLICED or host-resident majors), AR_ERR_RANGE (capacity < n, ws too
  * small, AR_SELECT_CARRY_APPR with sum of w_major > 31), AR_ERR_UNSUPPORTED
  * (sum of w_major > AR_MAX_PLANES).
@@ -442,6 +459,40 @@ ar_status ar_dist_offsets(ar_dist* d, const int64_t* local_count_dev, int64_t* a
 
 /* In-place ncclAllReduce(int64, sum) of `n` device int64 values (the Q6 SUM and counts). */
 ar_status ar_dist_sum(ar_dist* d, int64_t* values_dev, int32_t n, void* stream);
+
+/*
+ * Shard geometry (host only, no device work): rank `rank` of
+ * `world` owns the contiguous rows [*row0, *row0 + *rows) of an n-row table.
+ * Every shard but the last holds ceil(n / world) rounded up to a multiple of
+ * AR_SHARD_ALIGN_ROWS rows, so each shard's SLICED / PACKED bitstreams start
+ * 16-B aligned; the last shard is ragged and trailing shards may be empty.
+ * Errors: AR_ERR_INVALID (n < 0, rank outside [0, world), null outputs).
+ */
+#define AR_SHARD_ALIGN_ROWS 128
+ar_status ar_dist_shard_range(int64_t n, int32_t world, int32_t rank, int64_t* row0, int64_t* rows);
+
+/*
+ * The prefix step of ar_dist_offsets on its own (device, one launch on
+ * `stream`): from the gathered counts all_counts_dev[world] of every rank,
+ * *global_offset_dev = sum of the counts of ranks < rank and, if total_dev is
+ * not NULL, *total_dev = sum of all counts.  ar_dist_offsets = ncclAllGather +
+ * this kernel.  Errors: AR_ERR_INVALID (null pointers, rank outside [0, world)).
+ */
+ar_status ar_dist_exclusive_offsets(const int64_t* all_counts_dev, int32_t world, int32_t rank,
+                                    int64_t* global_offset_dev, int64_t* total_dev, void* stream);
+
+/*
+ * Place a rank's refined positions in the concatenated, globally ordered
+ * result (device, one launch): out_global[*global_offset_dev + j] =
+ * row0 + local->pos[j] for j < *local->count (int64 global row positions;
+ * row0 from ar_dist_shard_range).  out_global is a caller-owned device buffer
+ * of out_capacity entries -- the whole result on one device, or a rank's view
+ * of a distributed one.  If the slice does not fit, nothing is written and
+ * *overflow_dev (device u32, caller-zeroed) gets bit 0 set.
+ * Errors: AR_ERR_INVALID (null pointers, row0 < 0 or out_capacity < 0).
+ */
+ar_status ar_dist_concat_positions(const ar_positions* local, int64_t row0, const int64_t* global_offset_dev,
+                                   int64_t* out_global, int64_t out_capacity, uint32_t* overflow_dev, void* stream);
 
 void ar_dist_free(ar_dist* d);
 

@@ -94,6 +94,10 @@ SIGNATURES = {
     "ar_dist_offsets": (ctypes.c_int, [_P, _P, _P, _P, _P]),
     "ar_dist_sum": (ctypes.c_int, [_P, _P, _I32, _P]),
     "ar_dist_free": (None, [_P]),
+    "ar_dist_shard_range": (ctypes.c_int, [_I64, _I32, _I32, ctypes.POINTER(_I64), ctypes.POINTER(_I64)]),
+    "ar_dist_exclusive_offsets": (ctypes.c_int, [_P, _I32, _I32, _P, _P, _P]),
+    "ar_dist_concat_positions": (ctypes.c_int, [ctypes.POINTER(Positions), _I64, _P, _P, _I64, _P, _P]),
+    "ar_decompose_set_width": (ctypes.c_int, [ctypes.POINTER(ColumnDesc), _I32]),
 }
 
 _lib = None
@@ -272,3 +276,24 @@ def ar_dist_sum(d, values_dev, n, stream):
 
 def ar_dist_free(d):
     load().ar_dist_free(d)
+
+
+def ar_dist_shard_range(n: int, world: int, rank: int):
+    """(row0, rows) of rank's shard (host only)."""
+    row0, rows = ctypes.c_int64(0), ctypes.c_int64(0)
+    _call("ar_dist_shard_range", n, world, rank, ctypes.byref(row0), ctypes.byref(rows))
+    return int(row0.value), int(rows.value)
+
+
+def ar_dist_exclusive_offsets(all_counts_dev, world, rank, global_offset_dev, total_dev, stream):
+    _call("ar_dist_exclusive_offsets", all_counts_dev, world, rank, global_offset_dev, total_dev, stream)
+
+
+def ar_dist_concat_positions(local: Positions, row0, global_offset_dev, out_global, out_capacity, overflow_dev,
+                             stream):
+    _call("ar_dist_concat_positions", ctypes.byref(local), row0, global_offset_dev, out_global, out_capacity,
+          overflow_dev, stream)
+
+
+def ar_decompose_set_width(desc: ColumnDesc, w_major: int):
+    _call("ar_decompose_set_width", ctypes.byref(desc), w_major)

@@ -36,6 +36,31 @@ int num_sms() {
     return sms;
 }
 
+int current_device() {
+    int dev = 0;
+    if (cudaGetDevice(&dev) != cudaSuccess) {
+        cudaGetLastError();
+        return 0;
+    }
+    return dev;
+}
+
+void opt_in_max_smem(const void* fn) {
+    struct Done { int dev; const void* fn; };
+    static thread_local Done done[128];
+    static thread_local int used = 0;
+    const int dev = current_device();
+    for (int i = 0; i < used; ++i)
+        if (done[i].fn == fn && done[i].dev == dev) return;
+    int max_optin = 227 * 1024;
+    cudaDeviceGetAttribute(&max_optin, cudaDevAttrMaxSharedMemoryPerBlockOptin, dev);
+    cudaFuncAttributes a{};
+    if (cudaFuncGetAttributes(&a, fn) == cudaSuccess)
+        cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, max_optin - (int)a.sharedSizeBytes);
+    cudaGetLastError();   // never leave a sticky error behind for a later launch check
+    if (used < 128) done[used++] = Done{dev, fn};
+}
+
 // Step a2: exact [lo, hi] -> candidate / definite major ranges.
 // In u = v - base units, bucket(m) = [m 2^k, m 2^k + 2^k - 1]:
 //   cand(m) <=> m 2^k <= uhi && m 2^k + 2^k - 1 >= ulo  <=>  ulo >> k <= m <= uhi >> k
@@ -103,18 +128,19 @@ static uint32_t pick_stages_uncached(const void* fn, uint32_t stage_words, bool 
     return 2;
 }
 
-// Memoised per (kernel, stage_words): the occupancy queries stay out of the launch path.
+// Memoised per (device, kernel, stage_words): the occupancy queries stay out of the launch path.
 static uint32_t pick_stages(const void* fn, uint32_t stage_words, bool fused, int* ctas_per_sm) {
-    struct Entry { const void* fn; uint32_t words; uint32_t stages; int occ; };
+    struct Entry { int dev; const void* fn; uint32_t words; uint32_t stages; int occ; };
     static thread_local Entry cache[32];
     static thread_local int used = 0;
+    const int dev = current_device();
     for (int i = 0; i < used; ++i)
-        if (cache[i].fn == fn && cache[i].words == stage_words) {
+        if (cache[i].fn == fn && cache[i].words == stage_words && cache[i].dev == dev) {
             *ctas_per_sm = cache[i].occ;
             return cache[i].stages;
         }
     const uint32_t st = pick_stages_uncached(fn, stage_words, fused, ctas_per_sm);
-    if (used < 32) cache[used++] = Entry{fn, stage_words, st, *ctas_per_sm};
+    if (used < 32) cache[used++] = Entry{dev, fn, stage_words, st, *ctas_per_sm};
     return st;
 }
 
@@ -202,6 +228,22 @@ ar_status ar_decompose_plan(const uint32_t* col, int64_t n, int32_t major_bits, 
     return AR_OK;
 }
 
+static ar_status check_desc(const ar_column_desc* d);
+
+ar_status ar_decompose_set_width(ar_column_desc* desc, int32_t w_major) {
+    ar_status st = check_desc(desc);
+    if (st != AR_OK) return st;
+    if (w_major < desc->w_major || w_major > desc->major_bits) {
+        set_error("ar_decompose_set_width: w_major %d outside [%d (planned), %d (major_bits)]", w_major, desc->w_major,
+                  desc->major_bits);
+        return AR_ERR_RANGE;
+    }
+    desc->w_major = w_major;
+    desc->major_bytes = desc->major_layout == AR_LAYOUT_SLICED ? sliced_bytes(desc->n, w_major)
+                                                                : packed_bytes(desc->n, w_major);
+    return AR_OK;
+}
+
 static ar_status check_desc(const ar_column_desc* d) {
     if (!d || d->n < 0 || d->n >= (int64_t)1 << 32 || d->major_bits < 1 || d->major_bits > 32 ||
         d->k != 32 - d->major_bits || d->w_major < 0 || d->w_major > d->major_bits ||
@@ -209,9 +251,23 @@ static ar_status check_desc(const ar_column_desc* d) {
         (d->residual_loc != AR_LOC_DEVICE && d->residual_loc != AR_LOC_HOST_PINNED) ||
         (d->major_loc != AR_LOC_DEVICE && d->major_loc != AR_LOC_HOST_PINNED) ||
         (d->residual_layout != AR_LAYOUT_SLICED && d->residual_layout != AR_LAYOUT_PACKED) ||
+        (d->residual_layout == AR_LAYOUT_SLICED && d->k > 8) ||
         (d->value_signed != 0 && d->value_signed != 1) || d->reserved != 0) {
         set_error("invalid ar_column_desc");
         return AR_ERR_INVALID;
+    }
+    // the kernels read whole 16-B groups of every part (TMA bulk copies, vector gathers): the
+    // descriptor must promise at least the bytes its geometry implies
+    const uint64_t need_major = d->major_layout == AR_LAYOUT_SLICED ? sliced_bytes(d->n, d->w_major)
+                                                                     : packed_bytes(d->n, d->w_major);
+    const uint64_t need_res = d->k == 0 ? 0
+                              : (d->residual_layout == AR_LAYOUT_SLICED ? sliced_bytes(d->n, d->k)
+                                                                        : packed_bytes(d->n, d->k));
+    if (d->major_bytes < need_major || d->residual_bytes < need_res) {
+        set_error("ar_column_desc: major_bytes %llu / residual_bytes %llu below the %llu / %llu its geometry needs",
+                  (unsigned long long)d->major_bytes, (unsigned long long)d->residual_bytes,
+                  (unsigned long long)need_major, (unsigned long long)need_res);
+        return AR_ERR_RANGE;
     }
     return AR_OK;
 }
@@ -238,6 +294,10 @@ ar_status ar_column_wrap(const ar_column_desc* desc, const void* major_buf, cons
     if (st != AR_OK) return st;
     if (!out || (desc->major_bytes > 0 && !major_buf) || (desc->residual_bytes > 0 && !residual_buf)) {
         set_error("ar_column_wrap: null buffer or output");
+        return AR_ERR_INVALID;
+    }
+    if (((uintptr_t)major_buf & 15u) || ((uintptr_t)residual_buf & 15u)) {
+        set_error("ar_column_wrap: part buffers must be 16-B aligned (TMA bulk copies / vector loads)");
         return AR_ERR_INVALID;
     }
     const uint32_t* res = nullptr;
@@ -581,14 +641,22 @@ ar_status ar_refine(const ar_cands* in, const ar_pred* preds, int32_t npred, ar_
     AR_TRY_CUDA(cudaMemsetAsync(ws, 0, 16 + 8 * max_tiles, s));
     P.out_pos = out->pos;
     P.out_count = (long long*)out->count;
-    P.ticket = (unsigned int*)ws;
-    P.status = (unsigned long long*)((char*)ws + 16);
-    // persistent: every CTA resident (the look-back waits only on running or finished CTAs)
-    static int occ = 0;
+    P.status = (unsigned long long*)((char*)ws + 16);   // [0, 16): reserved
+    // persistent, round-robin tiles whose look-back waits on the tiles of other CTAs: every CTA must be
+    // resident, so the grid is sized from the occupancy on this device and launch_refine launches it
+    // cooperatively (a grid that cannot be co-resident fails with an error instead of hanging)
+    struct Occ { int dev; int occ; };
+    static thread_local Occ occ_cache[16];
+    static thread_local int occ_used = 0;
+    const int dev = current_device();
+    int occ = 0;
+    for (int i = 0; i < occ_used; ++i)
+        if (occ_cache[i].dev == dev) occ = occ_cache[i].occ;
     if (!occ) {
         cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, (const void*)refine_kernel_fn(), ard::kRefThreads, 0);
         cudaGetLastError();
         occ = std::max(occ, 1);
+        if (occ_used < 16) occ_cache[occ_used++] = Occ{dev, occ};
     }
     const int grid = (int)std::min<uint64_t>(std::min<uint64_t>(max_tiles, (uint64_t)num_sms() * occ), 640);
     g_last_scan = "refine_kernel";

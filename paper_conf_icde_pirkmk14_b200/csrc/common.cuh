@@ -25,6 +25,11 @@ namespace ar {
 void set_error(const char* fmt, ...);
 ar_status cuda_fail(cudaError_t e, const char* where);
 int num_sms();
+int current_device();
+// Opt `fn` in to the largest dynamic shared memory it can have on the current
+// device (the opt-in maximum minus its static shared memory), once per
+// (device, kernel) and host thread: function attributes are per device.
+void opt_in_max_smem(const void* fn);
 
 inline uint64_t ceil_div_u64(uint64_t a, uint64_t b) { return (a + b - 1) / b; }
 

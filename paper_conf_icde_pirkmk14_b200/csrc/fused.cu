@@ -462,20 +462,7 @@ ar_status launch_fused_rl(const ard::SelParams& P0, const ar_column* const* cols
     P.rl_ring = (uint32_t)env_ring();
 
     // deepest stage ring (<= 8, >= 3) that keeps 2 CTAs per SM, else 1 CTA with >= 2 stages
-    static thread_local const void* opted[64];
-    static thread_local int nopted = 0;
-    bool seen = false;
-    for (int i = 0; i < nopted; ++i) seen |= opted[i] == k.fn;
-    if (!seen) {
-        int dev = 0, max_optin = 227 * 1024;
-        if (cudaGetDevice(&dev) == cudaSuccess)
-            cudaDeviceGetAttribute(&max_optin, cudaDevAttrMaxSharedMemoryPerBlockOptin, dev);
-        cudaFuncAttributes fa{};   // dynamic + static shared memory <= the opt-in maximum
-        if (cudaFuncGetAttributes(&fa, k.fn) == cudaSuccess) max_optin -= (int)fa.sharedSizeBytes;
-        cudaFuncSetAttribute(k.fn, cudaFuncAttributeMaxDynamicSharedMemorySize, max_optin);
-        cudaGetLastError();
-        if (nopted < 64) opted[nopted++] = k.fn;
-    }
+    opt_in_max_smem(k.fn);
     const int threads = (k.nw + 1) * 32;
     uint32_t stages = 0;
     int occ = 0;

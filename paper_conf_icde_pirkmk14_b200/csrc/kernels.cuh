@@ -247,6 +247,6 @@ ar_status launch_pack_sliced(const uint32_t* col, int64_t n, int shift, uint32_t
                              int w, uint32_t* out, cudaStream_t s);
 ar_status launch_pack_packed(const uint32_t* col, int64_t n, int shift, uint32_t mask, uint32_t flip, uint32_t base,
                              int w, uint64_t out_words, uint32_t* out, cudaStream_t s);
-ar_status launch_exclusive_offset(const long long* all_counts, int world, int rank, long long* out,
+ar_status launch_exclusive_offset(const long long* all_counts, int world, int rank, long long* out, long long* total,
                                   cudaStream_t s);
 }  // namespace ar

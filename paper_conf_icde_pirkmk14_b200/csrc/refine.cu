@@ -692,20 +692,27 @@ __global__ void __launch_bounds__(kRefThreads) project_kernel(const __grid_const
     }
 }
 
-__global__ void exclusive_offset_kernel(const long long* all, int world, int rank, long long* out) {
-    long long s = 0;
-    for (int r = 0; r < rank && r < world; ++r) s += all[r];
-    *out = s;
-}
-
 }  // namespace ard
 
 namespace ar {
 
 const void* refine_kernel_fn() { return (const void*)ard::refine_kernel; }
+// Cooperative: the round-robin look-back (rr_prefix) waits on tiles of other
+// CTAs, so the whole grid must be co-resident; a cooperative launch guarantees
+// that or fails (cudaErrorCooperativeLaunchTooLarge, e.g. under an MPS SM
+// limit or beside a persistent kernel) rather than hanging.
 ar_status launch_refine(const ard::RefParams& P, int grid, cudaStream_t s) {
-    ard::refine_kernel<<<grid, ard::kRefThreads, 0, s>>>(P);
-    AR_CHECK_LAUNCH("refine_kernel");
+    void* args[] = {const_cast<ard::RefParams*>(&P)};
+    cudaLaunchConfig_t cfg = {};
+    cfg.gridDim = dim3(grid);
+    cfg.blockDim = dim3(ard::kRefThreads);
+    cfg.stream = s;
+    cudaLaunchAttribute attr[1];
+    attr[0].id = cudaLaunchAttributeCooperative;
+    attr[0].val.cooperative = 1;
+    cfg.attrs = attr;
+    cfg.numAttrs = 1;
+    AR_TRY_CUDA(cudaLaunchKernelExC(&cfg, (const void*)ard::refine_kernel, args));
     return AR_OK;
 }
 ar_status launch_refine_sum(const ard::RefParams& P, int grid, cudaStream_t s) {
@@ -759,12 +766,6 @@ ar_status launch_group_sum(const ard::GroupParams& P, int grid, cudaStream_t s) 
     }
     ard::group_sum_kernel<<<grid, ard::kRefThreads, smem, s>>>(P);
     AR_CHECK_LAUNCH("group_sum_kernel");
-    return AR_OK;
-}
-ar_status launch_exclusive_offset(const long long* all_counts, int world, int rank, long long* out,
-                                  cudaStream_t s) {
-    ard::exclusive_offset_kernel<<<1, 1, 0, s>>>(all_counts, world, rank, out);
-    AR_CHECK_LAUNCH("exclusive_offset_kernel");
     return AR_OK;
 }
 

@@ -895,21 +895,7 @@ size_t select_smem_bytes(uint32_t stage_words, uint32_t nstages, bool staging) {
     return bytes;
 }
 
-static void set_max_smem(const void* fn) {
-    static thread_local const void* done[64];
-    static thread_local int used = 0;
-    for (int i = 0; i < used; ++i)
-        if (done[i] == fn) return;
-    // opt in to the largest dynamic allocation this kernel can have (227 KB minus its static smem)
-    cudaFuncAttributes a{};
-    int max_optin = 227 * 1024, dev = 0;
-    if (cudaGetDevice(&dev) == cudaSuccess)
-        cudaDeviceGetAttribute(&max_optin, cudaDevAttrMaxSharedMemoryPerBlockOptin, dev);
-    if (cudaFuncGetAttributes(&a, fn) == cudaSuccess)
-        cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, max_optin - (int)a.sharedSizeBytes);
-    cudaGetLastError();   // never leave a sticky error behind for a later launch check
-    if (used < 64) done[used++] = fn;
-}
+static void set_max_smem(const void* fn) { opt_in_max_smem(fn); }
 
 int select_occupancy(const void* fn, size_t smem, bool fused) {
     int blocks = 0;
@@ -918,10 +904,10 @@ int select_occupancy(const void* fn, size_t smem, bool fused) {
     return blocks;
 }
 
-// Cooperative launch for the ordered select: guarantees every CTA of the grid
-// is co-resident, which the round-robin look-back relies on (a CTA never waits
-// on a tile of a CTA that is not running).  The grid is sized from the
-// occupancy calculator.
+// Plain launch of a scan kernel (select_tile_kernel: one tile per CTA, no CTA
+// waits on another; fused_kernel: persistent, tiles handed out round-robin and
+// each CTA's partial SUM / counts added atomically, so neither needs its CTAs
+// co-resident).
 ar_status launch_scan(const void* fn, const ard::SelParams& P, int grid, size_t smem, bool fused, cudaStream_t s) {
     set_max_smem(fn);
     void* args[] = {const_cast<ard::SelParams*>(&P)};
@@ -930,11 +916,6 @@ ar_status launch_scan(const void* fn, const ard::SelParams& P, int grid, size_t 
     cfg.blockDim = dim3(kernel_threads(fused));
     cfg.dynamicSmemBytes = smem;
     cfg.stream = s;
-    cudaLaunchAttribute attr[1];
-    attr[0].id = cudaLaunchAttributeCooperative;
-    attr[0].val.cooperative = 0;
-    cfg.attrs = attr;
-    cfg.numAttrs = 1;
     AR_TRY_CUDA(cudaLaunchKernelExC(&cfg, fn, args));
     return AR_OK;
 }

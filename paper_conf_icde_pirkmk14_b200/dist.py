@@ -12,27 +12,12 @@ from __future__ import annotations
 
 from . import _ar
 
-ALIGN_ROWS = 128
 
-
-def shard_range(n: int, rank: int, world: int, align: int = ALIGN_ROWS):
-    """[start, end) of rank's rows: ceil(n / world) rounded up to `align`, last shard ragged (may be empty)."""
-    if world < 1 or not (0 <= rank < world):
-        raise ValueError("bad rank / world")
-    per = -(-n // world)
-    per = -(-per // align) * align
-    start = min(n, rank * per)
-    end = min(n, start + per)
-    return start, end
-
-
-def exclusive_offsets(counts):
-    """Offsets of each rank's slice in the concatenated result (what ar_dist_offsets computes on device)."""
-    out, run = [], 0
-    for c in counts:
-        out.append(run)
-        run += int(c)
-    return out, run
+def shard_range(n: int, rank: int, world: int):
+    """[start, end) of rank's rows (ar_dist_shard_range: ceil(n / world) rounded up to
+    AR_SHARD_ALIGN_ROWS = 128 rows, last shard ragged, trailing shards may be empty)."""
+    row0, rows = _ar.ar_dist_shard_range(n, world, rank)
+    return row0, row0 + rows
 
 
 class NcclComm:
@@ -48,6 +33,7 @@ class NcclComm:
         self.rank, self.world = rank, world
 
     def offsets(self, local_count_dev, all_counts_dev, global_offset_dev, stream):
+        """ncclAllGather of the local count + the exclusive prefix (ar_dist_offsets)."""
         _ar.ar_dist_offsets(self.handle, local_count_dev, all_counts_dev, global_offset_dev, stream)
 
     def sum(self, values_dev, n, stream):

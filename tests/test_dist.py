@@ -1,6 +1,9 @@
-"""Row sharding (step a4) without a multi-GPU box: shard geometry, offset arithmetic,
-and a world_size-2 gloo run in which each rank evaluates its shard (oracle on CPU)
-and the ranks exchange counts / sums exactly as ar_dist_offsets / ar_dist_sum do."""
+"""Row sharding (step a4) without a multi-GPU box: the library's shard geometry
+(ar_dist_shard_range, a host-only entry point of libar_b200.so), and a
+world_size-2 gloo run in which each rank takes its shard from the library,
+evaluates it (oracle on CPU: no GPU here) and the ranks exchange counts / sums
+as ar_dist_offsets / ar_dist_sum do; the concatenation must equal the
+whole-table oracle."""
 import os
 import socket
 
@@ -10,7 +13,7 @@ import torch.multiprocessing as mp
 
 import datagen
 import oracle
-from paper_conf_icde_pirkmk14_b200.dist import exclusive_offsets, shard_range
+from paper_conf_icde_pirkmk14_b200.dist import shard_range
 
 Q6_LO = [datagen.Q6_SHIPDATE[0], datagen.Q6_DISCOUNT[0], datagen.Q6_QUANTITY[0]]
 Q6_HI = [datagen.Q6_SHIPDATE[1], datagen.Q6_DISCOUNT[1], datagen.Q6_QUANTITY[1]]
@@ -28,9 +31,28 @@ def test_shard_range_partitions(n, world):
     assert prev == n
 
 
-def test_exclusive_offsets():
-    assert exclusive_offsets([3, 0, 5, 2]) == ([0, 3, 3, 8], 10)
-    assert exclusive_offsets([]) == ([], 0)
+def exclusive_offsets(counts):
+    """Offsets of each rank's slice in the concatenated result (test-side arithmetic)."""
+    out, run = [], 0
+    for c in counts:
+        out.append(run)
+        run += int(c)
+    return out, run
+
+
+def test_shard_range_matches_definition():
+    # ceil(n / world) rounded up to 128 rows per shard (SURVEY s8(e)); written out independently
+    for n, world in [(600_000_000, 8), (600_000_000, 3), (1000, 8), (128 * 8 + 1, 8), (5, 4)]:
+        per = -(-(-(-n // world)) // 128) * 128
+        for r in range(world):
+            assert shard_range(n, r, world) == (min(n, r * per), min(n, min(n, r * per) + per))
+
+
+def test_shard_range_rejects_bad_rank():
+    from paper_conf_icde_pirkmk14_b200 import _ar
+    for n, r, w in [(10, 2, 2), (10, -1, 2), (-1, 0, 1), (10, 0, 0)]:
+        with pytest.raises(_ar.ARError):
+            shard_range(n, r, w)
 
 
 def _shard_result(rank, world, n):

@@ -345,3 +345,44 @@ def test_gpu_errors(cu):
     with pytest.raises(_ar.ARError) as e:
         cu.sum_at(cu.PositionList(10), [big, big], s)
     assert e.value.status == _ar.AR_ERR_RANGE
+
+
+def test_gpu_wrap_rejects_short_or_misaligned_buffers(cu):
+    # a descriptor promising fewer bytes than its geometry, or a part buffer that is not 16-B
+    # aligned, is refused at wrap time instead of faulting inside a TMA copy later
+    from paper_conf_icde_pirkmk14_b200 import _ar
+    v = datagen.uniform_u32(10, 5000)
+    a = _col(cu, v, 24)
+    d = _ar.ar_column_get_desc(a.handle)
+    maj, res = a.major.data_ptr(), a.residual.data_ptr()
+    h = _ar.ar_column_wrap(d, maj, res)
+    _ar.ar_column_free(h)
+    for field in ("major_bytes", "residual_bytes"):
+        short = _ar.ar_column_get_desc(a.handle)
+        setattr(short, field, getattr(short, field) - 16)
+        with pytest.raises(_ar.ARError) as e:
+            _ar.ar_column_wrap(short, maj, res)
+        assert e.value.status == _ar.AR_ERR_RANGE
+    with pytest.raises(_ar.ARError) as e:
+        _ar.ar_column_wrap(d, maj + 4, res)
+    assert e.value.status == _ar.AR_ERR_INVALID
+    with pytest.raises(_ar.ARError) as e:
+        _ar.ar_column_wrap(d, maj, res + 8)
+    assert e.value.status == _ar.AR_ERR_INVALID
+
+
+def test_gpu_refine_cooperative_launch(cu):
+    # ar_refine's look-back needs every CTA resident: it is launched cooperatively and sized from
+    # this device's occupancy; a large candidate list (many tiles per CTA) still refines exactly
+    from paper_conf_icde_pirkmk14_b200 import _ar
+    n = 3_000_017
+    v = datagen.uniform_u32(12, n)
+    col = _col(cu, v, 24)
+    lo, hi = 0x10000000, 0xB0000000
+    cands = cu.CandidateList(n)
+    cu.approx_select([(col, lo, hi)], cands, cu.Workspace(_ar.ar_select_ws_bytes(n)))
+    pos = cu.PositionList(n)
+    cu.refine(cands, [(col, lo, hi)], pos, cu.Workspace(_ar.ar_refine_ws_bytes(n)))
+    torch.cuda.synchronize()
+    ref, cnt, _ = oracle.select_sum([v], [lo], [hi])
+    assert pos.count() == cnt and np.array_equal(pos.positions(), ref)
