@@ -42,11 +42,14 @@ class BWDColumn:
     """A bitwise-decomposed column (major part in HBM, residual in HBM or pinned host memory).
 
     signed=True decomposes int32 values in the order-preserving key domain v ^ 0x80000000 (predicate
-    bounds are then int32 values); base="min" is the frame-of-reference prefix base min(key)."""
+    bounds are then int32 values); base="min" is the frame-of-reference prefix base min(key).
+    width_agree: for a row shard of a larger table, a callable mapping this shard's planned stored
+    width w_M to the table's (e.g. an allreduce-MAX over ranks); the descriptor is widened to it
+    (ar_decompose_set_width) so every shard shares one bucket geometry."""
 
     def __init__(self, values, major_bits: int, layout: int = AR_LAYOUT_SLICED,
                  residual_loc: int = AR_LOC_DEVICE, base=0, signed: bool = False, device="cuda", stream=None,
-                 _wrap=None):
+                 width_agree=None, _wrap=None):
         self.device = torch.device(device)
         if _wrap is not None:
             self.desc, self.major, self.residual = _wrap
@@ -60,6 +63,10 @@ class BWDColumn:
         flags = (_ar.AR_DECOMPOSE_SIGNED if signed else 0) | (_ar.AR_DECOMPOSE_BASE_MIN if base == "min" else 0)
         self.desc = _ar.ar_decompose_plan(col.data_ptr() if n else None, n, major_bits, layout, residual_loc,
                                           0 if base == "min" else int(base), flags, ws.data_ptr(), ws.numel(), s)
+        if width_agree is not None:
+            w = int(width_agree(int(self.desc.w_major)))
+            if w != self.desc.w_major:
+                _ar.ar_decompose_set_width(self.desc, w)
         self.major = _nbytes_tensor(self.desc.major_bytes, self.device)
         self.residual = _nbytes_tensor(self.desc.residual_bytes, self.device,
                                        pinned=(residual_loc == AR_LOC_HOST_PINNED))
