@@ -20,6 +20,8 @@ Pins (tests/test_oracle_*.py):
                   exact answer, closed forms, containment of the exact answer
   select_minmax   pure-Python brute force on tiny tables, closed forms
   select_group_sum  Fig. 4's grouped count, pure-Python brute force, closed forms
+  select_group_sum_keys  pure-Python dict grouping on tiny tables, the dense-key special case equals
+                  select_group_sum, one constant key equals select_sum, closed forms
   minmax_ar       Fig. 6 (the false positive holds the single minimal
                   approximation, the propagated set still holds the true minimum), refined
                   answer == select_minmax, bounds contain it, k = 0 collapse, brute force
@@ -72,6 +74,8 @@ def _load():
         lib.or_minmax_ar.argtypes = [i64, i32, p, p, p, p, p, p, p, i32, u32, i32, i32, p, p]
         lib.or_select_group_sum.argtypes = [i64, i32, p, p, p, p, i32, i32, p, p, p]
         lib.or_select_group_sum.restype = i32
+        lib.or_select_group_sum_keys.argtypes = [i64, i32, p, p, p, p, p, i32, p, i64, p, p, p, p]
+        lib.or_select_group_sum_keys.restype = i32
         lib.or_threads_default.restype = i32
         _lib = lib
     return _lib
@@ -286,3 +290,29 @@ def select_group_sum(pred_cols, los, his, key, ngroups: int, agg_cols=()):
     if rc == 2:
         raise ValueError("a qualifying row has key >= ngroups")
     return sums[:ngroups], cnts[:ngroups]
+
+
+def select_group_sum_keys(pred_cols, los, his, key, agg_cols=(), signed=None, max_groups=1 << 20):
+    """Exact grouped COUNT / product SUM over the selection for arbitrary uint32 keys (s IV-E, the plain
+    definition): (keys ascending, counts, sums) of the groups among the qualifying rows."""
+    pred_cols, los, his, sg = _signed_preds(pred_cols, los, his, signed)
+    agg_cols = [_u32(c) for c in agg_cols]
+    key = np.ascontiguousarray(key).view(np.uint32) if np.asarray(key).dtype == np.int32 else _u32(key)
+    lo = np.asarray(los, dtype=np.uint32)
+    hi = np.asarray(his, dtype=np.uint32)
+    cap = max(1, int(max_groups))
+    keys = np.zeros(cap, dtype=np.uint32)
+    cnts = np.zeros(cap, dtype=np.int64)
+    sums = np.zeros(cap, dtype=np.int64)
+    ng = ctypes.c_int64(0)
+    pc, ac = _ptr_array(pred_cols), _ptr_array(agg_cols)
+    rc = _load().or_select_group_sum_keys(key.size, len(pred_cols), ctypes.cast(pc, ctypes.c_void_p), _ptr(lo),
+                                          _ptr(hi), _ptr(sg) if sg is not None else None, _ptr(key),
+                                          len(agg_cols), ctypes.cast(ac, ctypes.c_void_p), cap, _ptr(keys),
+                                          _ptr(cnts), _ptr(sums), ctypes.byref(ng))
+    if rc == 1:
+        raise OverflowError("a group SUM does not fit in int64")
+    if rc == 2:
+        raise ValueError("more groups than max_groups")
+    g = int(ng.value)
+    return keys[:g], cnts[:g], sums[:g]

@@ -488,3 +488,63 @@ int or_select_group_sum(int64_t n, int npred, const uint32_t* const* pcols, cons
     free(s);
     return rc;
 }
+
+/*
+ * Exact  select key, count(*), sum(prod_a acols[a]) from R where <conjunction>
+ * group by key  for ARBITRARY uint32 key values -- the plain definition of a
+ * grouped aggregation (s IV-E/F), with the groups listed in
+ * ascending key order.  Written plainly: the keys of the qualifying rows are
+ * collected and sorted (qsort), duplicates dropped; each qualifying row then
+ * finds its group by binary search and adds to it.  out_key / out_cnt /
+ * out_sum have room for max_groups entries; *ngroups = number of distinct keys
+ * among the qualifying rows.  Returns 0, 1 on int64 overflow of a sum, 2 if
+ * there are more than max_groups groups (outputs then hold the first max_groups).
+ */
+static int or_cmp_u32(const void* a, const void* b) {
+    uint32_t x = *(const uint32_t*)a, y = *(const uint32_t*)b;
+    return x < y ? -1 : (x > y ? 1 : 0);
+}
+
+int or_select_group_sum_keys(int64_t n, int npred, const uint32_t* const* pcols, const uint32_t* lo,
+                             const uint32_t* hi, const int* sgn, const uint32_t* key, int nagg,
+                             const uint32_t* const* acols, int64_t max_groups, uint32_t* out_key,
+                             int64_t* out_cnt, int64_t* out_sum, int64_t* ngroups) {
+    sel_ctx c;
+    memset(&c, 0, sizeof(c));
+    c.npred = npred; c.pcols = pcols; c.lo = lo; c.hi = hi; c.sgn = sgn;
+    uint32_t* keys = (uint32_t*)malloc((size_t)(n > 0 ? n : 1) * sizeof(uint32_t));
+    int64_t m = 0;
+    for (int64_t i = 0; i < n; ++i)
+        if (row_qualifies(&c, i)) keys[m++] = key[i];
+    qsort(keys, (size_t)m, sizeof(uint32_t), or_cmp_u32);
+    int64_t g = 0;
+    for (int64_t i = 0; i < m; ++i)
+        if (i == 0 || keys[i] != keys[i - 1]) keys[g++] = keys[i];
+    *ngroups = g;
+    __int128* s = (__int128*)calloc((size_t)(g > 0 ? g : 1), sizeof(__int128));
+    int64_t* cnt = (int64_t*)calloc((size_t)(g > 0 ? g : 1), sizeof(int64_t));
+    for (int64_t i = 0; i < n; ++i) {
+        if (!row_qualifies(&c, i)) continue;
+        int64_t a = 0, b = g - 1;          /* binary search: keys[a..b] holds key[i] */
+        while (a < b) {
+            int64_t mid = a + (b - a) / 2;
+            if (keys[mid] < key[i]) a = mid + 1; else b = mid;
+        }
+        cnt[a] += 1;
+        __int128 prod = 1;
+        for (int q = 0; q < nagg; ++q) prod *= (__int128)acols[q][i];
+        if (nagg > 0) s[a] += prod;
+    }
+    int rc = 0;
+    for (int64_t j = 0; j < g; ++j) {
+        if (s[j] > (__int128)INT64_MAX) rc = 1;
+        if (j < max_groups) {
+            out_key[j] = keys[j];
+            out_cnt[j] = cnt[j];
+            out_sum[j] = (int64_t)s[j];
+        }
+    }
+    if (g > max_groups) rc = 2;
+    free(keys); free(s); free(cnt);
+    return rc;
+}
