@@ -81,7 +81,8 @@ def parse(argv=None):
     ap.add_argument("--steps", type=int, default=200)
     ap.add_argument("--warmup", type=int, default=10)
     ap.add_argument("--impl", choices=["ours", "reference"], default="ours")
-    ap.add_argument("--workload", choices=["c4", "c2"], default="c4", help="headline workload")
+    ap.add_argument("--workload", choices=["c4", "c2", "c5"], default="c4",
+                    help="headline workload (c5: print only the C5 host-link measurement, for tools)")
     ap.add_argument("--variant", choices=["staged", "fused"], default="fused",
                     help="headline variant (the other one is timed too and reported under 'variants')")
     ap.add_argument("--scaling", choices=["strong", "weak"], default="strong",
@@ -778,6 +779,11 @@ def run_e2e(ctx, q, ab, steps):
 def ours(args):
     ctx = Ctx(args)
     torch, _ar = ctx.torch, ctx._ar
+    if args.workload == "c5":
+        out = bench_c5(ctx, args)
+        if ctx.rank == 0:
+            print(json.dumps(out), flush=True)
+        return
     world, rank = ctx.world, ctx.rank
     seed, table_sf, table_rows, row0, rows = shard_of(args.workload, world, rank, args.scaling)
     cols = gen_columns(seed, table_sf, row0, rows)

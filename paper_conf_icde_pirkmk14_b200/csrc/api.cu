@@ -453,6 +453,8 @@ static ar_status setup_scan(const ar_pred* preds, int32_t npred, ard::SelParams&
         p.lo = plo;
         p.hi = phi;
         p.rlayout = (uint32_t)col->d.residual_layout;
+        p.res_host = col->d.residual_loc == AR_LOC_HOST_PINNED ? 1u : 0u;
+        p.res_hint = 1u;
         words += (P.tile_rows / 32) * (uint32_t)w;
         ashift += (uint32_t)w;
         // the one-pass kernel streams device-resident SLICED residual tiles (k <= 8) with the
@@ -489,7 +491,7 @@ static ar_status setup_scan(const ar_pred* preds, int32_t npred, ard::SelParams&
     for (int c = 0; c < npred; ++c) {
         const ard::SelPred& p = P.p[c];
         if (p.k > 0 && !p.res_stream) P.exact_mode = 0;
-        if (!p.res_stream) continue;
+        if (p.k == 0) continue;   // (also used by the gathered-residual kernel, fused.cu)
         const uint64_t maxu = p.k + p.w >= 32 ? 0xffffffffull : ((1ull << (p.k + p.w)) - 1);
         const uint64_t ulo = p.lo < p.base ? 0 : (uint64_t)(p.lo - p.base);
         const uint64_t uhi = std::min<uint64_t>((uint64_t)(p.hi - p.base), maxu);
@@ -561,9 +563,18 @@ ar_status ar_approx_select(const ar_pred* preds, int32_t npred, int32_t flags, a
     P.tmp_aux = P.tmp_pos + L.slice_rows;
     g_last_scan = "select_tile_kernel";
     const void* fn = select_kernel_fn(P, false);
-    P.nstages = 1;
-    const size_t smem = select_smem_bytes(P.stage_words, 1, true);
-    ar_status st2 = launch_scan(fn, P, (int)P.num_tiles, smem, false, s);
+    // one tile per CTA (default): measured fastest -- the kernel is issue-bound, and persistent CTAs
+    // with AR_SEL_BUFS = 2 / 3 tile buffers each (the next tiles' loads in flight while one is decided)
+    // ran 2 % / 12 % slower on C4 (DESIGN s6.2)
+    static const int bufs = std::min(4, std::max(1, env_int("AR_SEL_BUFS", 1)));
+    P.nstages = (uint32_t)bufs;
+    const size_t smem = select_smem_bytes(P.stage_words, P.nstages, true);
+    int grid = (int)P.num_tiles;
+    if (bufs > 1) {
+        const int occ = std::max(1, select_occupancy(fn, smem, false));
+        grid = (int)std::min<int64_t>(P.num_tiles, (int64_t)num_sms() * occ);
+    }
+    ar_status st2 = launch_scan(fn, P, grid, smem, false, s);
     if (st2 != AR_OK) return st2;
     return launch_select_rest(P, env_int("AR_SEL_PDL", 1) != 0, s);
 }
@@ -953,12 +964,12 @@ ar_status ar_select_refine_sum_ws(const ar_pred* preds, int32_t npred, const ar_
     g_last_scan = "";
     if (!ws || empty || n == 0) AR_TRY_CUDA(cudaMemsetAsync(out_dev, 0, 4 * sizeof(int64_t), s));
     if (empty || n == 0) return AR_OK;
-    bool launched = false;   // the result-ring kernel (fused.cu) where it applies
+    bool launched = false, rg = false;   // the result-ring kernels (fused.cu) where they apply
     const int pdl = (flags & AR_SRS_PDL_EARLY_READ) ? 2 : ((flags & AR_SRS_PDL) ? 1 : 0);
-    st = launch_fused_rl(P, cols, ws, pdl, &launched, s);
+    st = launch_fused_rl(P, cols, ws, pdl, &launched, &rg, s);
     if (st != AR_OK) return st;
     if (launched) {
-        g_last_scan = "fused_rl_kernel";
+        g_last_scan = rg ? "fused_rg_kernel" : "fused_rl_kernel";
         return AR_OK;
     }
     g_last_scan = "fused_kernel";

@@ -241,6 +241,21 @@ __device__ __forceinline__ uint4 ld_gather_if4(const uint32_t* p, bool pred) {  
         : "+r"(v.x), "+r"(v.y), "+r"(v.z), "+r"(v.w) : "l"(p), "r"((uint32_t)pred));
     return v;
 }
+// The same gathers without the L2 prefetch-size hint: for pinned host memory
+// read over the host link, where the request size is the transfer size
+// (AR_HOST_HINT selects, DESIGN s6.3c).
+__device__ __forceinline__ uint32_t ld_gather_if_nh(const uint32_t* p, bool pred) {
+    uint32_t v = 0;
+    asm("{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %2, 0;\n\t@q ld.global.nc.u32 %0, [%1];\n\t}"
+        : "+r"(v) : "l"(p), "r"((uint32_t)pred));
+    return v;
+}
+__device__ __forceinline__ uint4 ld_gather_if4_nh(const uint32_t* p, bool pred) {   // 16-B aligned
+    uint4 v = make_uint4(0, 0, 0, 0);
+    asm("{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %5, 0;\n\t@q ld.global.nc.v4.u32 {%0,%1,%2,%3}, [%4];\n\t}"
+        : "+r"(v.x), "+r"(v.y), "+r"(v.z), "+r"(v.w) : "l"(p), "r"((uint32_t)pred));
+    return v;
+}
 __device__ __forceinline__ uint32_t packed_get_if(const uint32_t* __restrict__ s, uint64_t p, int w, bool pred) {
     const uint64_t bit = p * (uint64_t)w;
     const uint32_t sh = (uint32_t)(bit & 31);

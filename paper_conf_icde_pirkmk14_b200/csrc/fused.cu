@@ -65,6 +65,67 @@ __device__ __forceinline__ unsigned long long drain(const uint32_t* sl, uint32_t
     return (unsigned long long)v * sl[96 + lane];
 }
 
+// out4 = {SUM, |result|, |candidates|, |definite|} from every consumer warp's
+// totals.  Without a workspace (rl_fin == 0) out4 was zeroed by the caller and
+// each warp adds atomically; with one, each CTA writes its partials to
+// rl_part[blockIdx] and the last CTA to arrive (ticket) sums them into out4
+// and re-arms the ticket -- no memset before the launch.  Consumer warps only
+// (the producer warp has exited): they meet at named barrier 1.
+template <int NW>
+__device__ __forceinline__ void finalize_out4(const SelParams& P, unsigned warp, unsigned lane,
+                                              unsigned long long sum, unsigned long long c2, unsigned long long c0,
+                                              unsigned long long c1) {
+    constexpr int NT = NW * 32;
+    if (!P.rl_fin) {   // out4 zeroed by the caller: one atomic per counter and warp
+        if (lane == 0) {
+            atomicAdd(P.out4 + 0, sum);
+            atomicAdd(P.out4 + 1, c2);
+            atomicAdd(P.out4 + 2, c0);
+            atomicAdd(P.out4 + 3, c1);
+        }
+        return;
+    }
+    __shared__ unsigned long long red[NW][4];
+    __shared__ uint32_t last;
+    if (lane == 0) {
+        red[warp][0] = sum;
+        red[warp][1] = c2;
+        red[warp][2] = c0;
+        red[warp][3] = c1;
+    }
+    bar_sync(1, NT);
+    if (threadIdx.x == 0) {
+        unsigned long long t4[4] = {0, 0, 0, 0};
+        for (int w = 0; w < NW; ++w)
+            for (int i = 0; i < 4; ++i) t4[i] += red[w][i];
+        if (P.rl_pdl) asm volatile("griddepcontrol.wait;" ::: "memory");   // the previous call is done with out4
+        unsigned long long* part = P.rl_part + 4ull * blockIdx.x;
+        for (int i = 0; i < 4; ++i) __stcg(part + i, t4[i]);
+        __threadfence();
+        last = atomicAdd(P.rl_ticket, 1u) == gridDim.x - 1 ? 1u : 0u;
+    }
+    bar_sync(1, NT);
+    if (!last) return;
+    __threadfence();
+    unsigned long long t4[4] = {0, 0, 0, 0};
+    for (uint32_t b = threadIdx.x; b < gridDim.x; b += NT)
+        for (int i = 0; i < 4; ++i) t4[i] += __ldcg(P.rl_part + 4ull * b + i);
+#pragma unroll
+    for (int o = 16; o > 0; o >>= 1)
+        for (int i = 0; i < 4; ++i) t4[i] += __shfl_xor_sync(0xffffffffu, t4[i], o);
+    bar_sync(1, NT);
+    if (lane == 0)
+        for (int i = 0; i < 4; ++i) red[warp][i] = t4[i];
+    bar_sync(1, NT);
+    if (threadIdx.x == 0) {
+        unsigned long long o4[4] = {0, 0, 0, 0};
+        for (int w = 0; w < NW; ++w)
+            for (int i = 0; i < 4; ++i) o4[i] += red[w][i];
+        for (int i = 0; i < 4; ++i) P.out4[i] = o4[i];
+        *P.rl_ticket = 0u;
+    }
+}
+
 template <int NW, int BPT, int... WK>
 __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid_constant__ SelParams P) {
     using S = Shape<WK...>;
@@ -262,57 +323,293 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
         c1 += __shfl_xor_sync(0xffffffffu, c1, o);
         c2 += __shfl_xor_sync(0xffffffffu, c2, o);
     }
-    if (!P.rl_fin) {   // out4 zeroed by the caller: one atomic per counter and warp
+    finalize_out4<NW>(P, warp, lane, sum, c2, c0, c1);
+}
+
+// Two-phase one-pass kernel with gathered residuals ("rg"): the residual of a
+// decomposed predicate is never streamed.  Phase A of tile t decides candidate
+// and definite rows on the majors alone; definite rows are
+// results at once (their whole bucket qualifies) and go to the
+// result ring, and for every 32-row block that holds a non-definite candidate
+// the block's K residual planes (K * 4 bytes of one sector, HBM or pinned host
+// memory) are gathered into registers.  Phase B of tile t runs one tile later,
+// when those loads have landed: the exact predicate on residual + major planes
+// (the "+bw" concatenation; Alg. 2) keeps
+// the non-definite candidates that qualify, and they join the ring.  A stage is
+// released after its phase B, so the producer streams only major planes (Q6:
+// 14 of the old 22 KB per 8192-row tile) and the residual traffic is the
+// touched sectors only.  Factors of the SUM: one gathered bit-packed column
+// times at most one k = 0 predicate column (ring), k = 0 predicate columns only
+// (direct), or none (COUNT).
+template <int NW, int BPT, int... WK>
+__global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid_constant__ SelParams P) {
+    using S = Shape<WK...>;
+    constexpr int NT = NW * 32;
+    constexpr int KS = S::ksum();
+    extern __shared__ __align__(128) unsigned char smem[];
+    uint64_t* full = reinterpret_cast<uint64_t*>(smem);
+    uint64_t* empty = full + P.nstages;
+    long long* slot = reinterpret_cast<long long*>(empty + P.nstages);
+    const size_t head_bytes = ((size_t)P.nstages * 24 + 127) & ~size_t(127);
+    uint32_t* stages = reinterpret_cast<uint32_t*>(smem + head_bytes);
+    const unsigned warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    const uint32_t kRing = P.rl_ring, rmask = kRing - 1;
+    uint2* ring = reinterpret_cast<uint2*>(stages + (size_t)P.nstages * P.stage_words) + warp * kRing;
+    uint32_t* gs = reinterpret_cast<uint32_t*>(reinterpret_cast<uint2*>(stages + (size_t)P.nstages * P.stage_words) +
+                                               NW * kRing) + warp * (kDepth * kSlotWords);
+    if (threadIdx.x == 0) {
+        for (uint32_t s = 0; s < P.nstages; ++s) {
+            mbar_init(full + s, 1);
+            mbar_init(empty + s, NW);
+        }
+        fence_mbar_init();
+    }
+    __syncthreads();
+    if (warp == NW) {
         if (lane == 0) {
-            atomicAdd(P.out4 + 0, sum);
-            atomicAdd(P.out4 + 1, c2);
-            atomicAdd(P.out4 + 2, c0);
-            atomicAdd(P.out4 + 3, c1);
+            if (P.rl_pdl == 1) asm volatile("griddepcontrol.wait;" ::: "memory");
+            produce_ring(P, full, empty, slot, stages);
+            if (P.rl_pdl) asm volatile("griddepcontrol.launch_dependents;" ::: "memory");
         }
         return;
     }
-    // Workspace finalize (no memset before the launch): CTA partial -> rl_part[blockIdx]; the last
-    // CTA to arrive (ticket) sums all partials into out4 and re-arms the ticket.  Consumer warps
-    // only: the producer warp has exited, so they meet at named barrier 1.
-    __shared__ unsigned long long red[NW][4];
-    __shared__ uint32_t last;
-    if (lane == 0) {
-        red[warp][0] = sum;
-        red[warp][1] = c2;
-        red[warp][2] = c0;
-        red[warp][3] = c1;
-    }
-    bar_sync(1, NT);
-    if (threadIdx.x == 0) {
-        unsigned long long t4[4] = {0, 0, 0, 0};
-        for (int w = 0; w < NW; ++w)
-            for (int i = 0; i < 4; ++i) t4[i] += red[w][i];
-        if (P.rl_pdl) asm volatile("griddepcontrol.wait;" ::: "memory");   // the previous call is done with out4
-        unsigned long long* part = P.rl_part + 4ull * blockIdx.x;
-        for (int i = 0; i < 4; ++i) __stcg(part + i, t4[i]);
-        __threadfence();
-        last = atomicAdd(P.rl_ticket, 1u) == gridDim.x - 1 ? 1u : 0u;
-    }
-    bar_sync(1, NT);
-    if (!last) return;
-    __threadfence();
-    unsigned long long t4[4] = {0, 0, 0, 0};
-    for (uint32_t b = threadIdx.x; b < gridDim.x; b += NT)
-        for (int i = 0; i < 4; ++i) t4[i] += __ldcg(P.rl_part + 4ull * b + i);
+
+    const bool list = P.rl_list != 0;
+    const bool direct = !list && P.nagg > 0;
+    const AggCol& G = P.a[P.gidx];
+    const uint32_t gmask = G.w >= 32 ? 0xffffffffu : ((1u << G.w) - 1u);
+    uint32_t ncand = 0, ndef = 0, nres = 0;
+    unsigned long long sum = 0;
+    uint32_t rhead = 0, rcnt = 0, gseq = 0;
+
+    auto pass = [&](uint32_t take) {
+        uint32_t* sl = gs + (gseq % kDepth) * kSlotWords;
+        uint32_t info = 0u, f = 0u;
+        if (lane < take) {
+            const uint2 e = ring[(rhead + lane) & rmask];
+            const uint64_t bit = (uint64_t)e.x * G.w;
+            const uint32_t* src = G.major + (bit >> 5);
+            const uint32_t sh = (uint32_t)(bit & 31);
+            cp_async4(sl + lane, src);
+            if (sh + G.w > 32u) cp_async4(sl + 32 + lane, src + 1);
+            info = 0x80000000u | sh;
+            f = e.y;
+        }
+        sl[64 + lane] = info;
+        sl[96 + lane] = f;
+        cp_async_commit();
+        ++gseq;
+        rhead += take;
+        rcnt -= take;
+        if (gseq >= (uint32_t)kDepth) {
+            cp_async_wait<kDepth - 1>();
+            sum += drain(gs + (gseq % kDepth) * kSlotWords, lane, gmask, G.base);
+        }
+    };
+
+    // a6 for the result rows xm[] of a tile held in stage `stg`
+    auto consume = [&](const uint32_t* stg, int64_t tile_r0, uint32_t (&xm)[BPT]) {
 #pragma unroll
-    for (int o = 16; o > 0; o >>= 1)
-        for (int i = 0; i < 4; ++i) t4[i] += __shfl_xor_sync(0xffffffffu, t4[i], o);
-    bar_sync(1, NT);
-    if (lane == 0)
-        for (int i = 0; i < 4; ++i) red[warp][i] = t4[i];
-    bar_sync(1, NT);
-    if (threadIdx.x == 0) {
-        unsigned long long o4[4] = {0, 0, 0, 0};
-        for (int w = 0; w < NW; ++w)
-            for (int i = 0; i < 4; ++i) o4[i] += red[w][i];
-        for (int i = 0; i < 4; ++i) P.out4[i] = o4[i];
-        *P.rl_ticket = 0u;
+        for (int b = 0; b < BPT; ++b) nres += __popc(xm[b]);
+        if (direct) {
+#pragma unroll
+            for (int b = 0; b < BPT; ++b) {
+                const uint32_t blk = b * NT + threadIdx.x;
+                for (uint32_t m = xm[b]; m; m &= m - 1) {
+                    const uint32_t l = __ffs(m) - 1;
+                    unsigned long long prod = 1;
+                    for (int a = 0; a < P.nagg; ++a) {
+                        uint32_t v = 0;
+                        static_for<S::N>([&](auto cc) {
+                            constexpr int C = decltype(cc)::value;
+                            constexpr int W = S::w(C);
+                            if constexpr (S::k(C) == 0) {
+                                if (C == P.a[a].pred) {
+                                    uint32_t x[W];
+                                    lds_words<W>(x, stg + P.p[C].soff + blk * W);
+                                    v = row_of<W>(x, l) + P.p[C].base;
+                                }
+                            }
+                        });
+                        prod *= v;
+                    }
+                    sum += prod;
+                }
+            }
+            return;
+        }
+        if (!list) return;
+        uint32_t my = 0;
+#pragma unroll
+        for (int b = 0; b < BPT; ++b) my += __popc(xm[b]);
+        uint32_t incl = my;
+#pragma unroll
+        for (int o = 1; o < 32; o <<= 1) {
+            const uint32_t y = __shfl_up_sync(0xffffffffu, incl, o);
+            if (lane >= (unsigned)o) incl += y;
+        }
+        const uint32_t total = __shfl_sync(0xffffffffu, incl, 31);
+        uint32_t e = incl - my;
+        for (uint32_t rb = 0; rb < total;) {
+            const uint32_t lim = min(total, rb + kRing - rcnt);
+            const uint32_t wbase = rhead + rcnt - rb;
+#pragma unroll
+            for (int b = 0; b < BPT; ++b) {
+                if (xm[b] && e < lim) {
+                    const uint32_t blk = b * NT + threadIdx.x;
+                    const uint32_t row0 = (uint32_t)tile_r0 + blk * 32;
+                    uint32_t m = xm[b];
+                    if (P.rl_mpred < 0) {
+                        do {
+                            const uint32_t l = __ffs(m) - 1;
+                            m &= m - 1;
+                            ring[(wbase + e) & rmask] = make_uint2(row0 + l, 1u);
+                            ++e;
+                        } while (m && e < lim);
+                    } else {
+                        static_for<S::N>([&](auto cc) {
+                            constexpr int C = decltype(cc)::value;
+                            constexpr int W = S::w(C);
+                            if constexpr (S::k(C) == 0) {
+                                if (C != P.rl_mpred) return;
+                                uint32_t x[W];
+                                lds_words<W>(x, stg + P.p[C].soff + blk * W);
+                                do {
+                                    const uint32_t l = __ffs(m) - 1;
+                                    m &= m - 1;
+                                    ring[(wbase + e) & rmask] = make_uint2(row0 + l, row_of<W>(x, l) + P.p[C].base);
+                                    ++e;
+                                } while (m && e < lim);
+                            }
+                        });
+                    }
+                    xm[b] = m;
+                }
+            }
+            __syncwarp();
+            rcnt += lim - rb;
+            rb = lim;
+            if (rb < total) {
+                while (rcnt >= 32) pass(32);
+                __syncwarp();
+            }
+        }
+    };
+
+    uint32_t rres[BPT][KS > 0 ? KS : 1];   // residual words of the pending tile's blocks (in flight)
+    uint32_t pnd[BPT];                      // its non-definite candidate masks
+#pragma unroll
+    for (int b = 0; b < BPT; ++b) pnd[b] = 0u;
+    long long pt = -1;                      // pending tile (phase B not yet run), its stage
+    uint32_t pst = 0;
+
+    // Phase B of the pending tile: exact predicate on its non-definite candidates, results to the ring,
+    // then its stage is released.
+    auto phase_b = [&]() {
+        const uint32_t* stg = stages + (size_t)pst * P.stage_words;
+        const int64_t r0 = pt * (int64_t)P.tile_rows;
+        uint32_t xm[BPT];
+#pragma unroll
+        for (int b = 0; b < BPT; ++b) {
+            const uint32_t blk = b * NT + threadIdx.x;
+            uint32_t em = pnd[b];
+            if (em) {
+                static_for<S::N>([&](auto cc) {
+                    constexpr int C = decltype(cc)::value;
+                    constexpr int W = S::w(C), K = S::k(C), KO = S::kofs(C);
+                    if constexpr (K > 0) {
+                        uint32_t x[W];
+                        lds_words<W>(x, stg + P.p[C].soff + blk * W);
+                        uint32_t el = 0, eh = 0;
+#pragma unroll
+                        for (int j = 0; j < K; ++j) {
+                            el = bsub(rres[b][KO + j], P.pmx[C][j][0], el);
+                            eh = brsub(rres[b][KO + j], P.pmx[C][j][1], eh);
+                        }
+#pragma unroll
+                        for (int j = 0; j < W; ++j) {
+                            el = bsub(x[j], P.pmx[C][K + j][0], el);
+                            eh = brsub(x[j], P.pmx[C][K + j][1], eh);
+                        }
+                        em &= ~(el | eh);
+                    }
+                });
+            }
+            xm[b] = em;
+        }
+        consume(stg, r0, xm);
+        __syncwarp();
+        if (lane == 0) mbar_arrive(empty + pst);
+    };
+
+    uint32_t s = 0, ph = 0;
+    for (;; s = (s + 1 == P.nstages) ? (ph ^= 1u, 0u) : s + 1) {
+        mbar_wait(full + s, ph, P.suspend_ns);
+        const long long t = slot[s];
+        if (t < 0) break;
+        const uint32_t* stg = stages + (size_t)s * P.stage_words;
+        const int64_t tile_r0 = t * (int64_t)P.tile_rows;
+        const bool full_tile = tile_r0 + (int64_t)P.tile_rows <= P.n;
+
+        // phase A (tile t): candidate / definite masks on the majors
+        uint32_t dmk[BPT], ndm[BPT];
+#pragma unroll
+        for (int b = 0; b < BPT; ++b) {
+            const uint32_t blk = b * NT + threadIdx.x;
+            const uint32_t vm = full_tile ? 0xffffffffu : valid_mask(tile_r0 + 32 * (int64_t)blk, P.n);
+            uint32_t cm, dm, em;
+            eval_block<S, false>(P, stg, blk, vm, cm, dm, em);
+            ncand += __popc(cm);
+            ndef += __popc(dm);
+            dmk[b] = dm;
+            ndm[b] = cm & ~dm;
+        }
+        if constexpr (KS > 0) {
+            if (pt >= 0) phase_b();          // the previous tile's residual gathers have had a tile to land
+            // gather the residual sectors of this tile's blocks with a non-definite candidate
+#pragma unroll
+            for (int b = 0; b < BPT; ++b) {
+                const uint64_t gblk = (uint64_t)(tile_r0 >> 5) + b * NT + threadIdx.x;
+                static_for<S::N>([&](auto cc) {
+                    constexpr int C = decltype(cc)::value;
+                    constexpr int K = S::k(C), KO = S::kofs(C);
+                    if constexpr (K > 0)
+                        res_issue<K>(&rres[b][KO], P.p[C].residual, gblk, ndm[b] != 0u, P.p[C].res_hint != 0u);
+                });
+                pnd[b] = ndm[b];
+            }
+            pt = t;
+            pst = s;
+            consume(stg, tile_r0, dmk);      // definite rows are results now
+        } else {
+            consume(stg, tile_r0, dmk);      // k = 0 everywhere: candidate = definite = exact
+            __syncwarp();
+            if (lane == 0) mbar_arrive(empty + s);
+        }
+        if (list) {
+            while (rcnt >= 32) pass(32);
+            __syncwarp();
+        }
     }
+    if constexpr (KS > 0) {
+        if (pt >= 0) phase_b();
+    }
+    if (list) {
+        while (rcnt > 0) pass(min(rcnt, 32u));
+        cp_async_wait<0>();
+        for (uint32_t g = gseq >= (uint32_t)kDepth ? gseq - kDepth + 1 : 0; g < gseq; ++g)
+            sum += drain(gs + (g % kDepth) * kSlotWords, lane, gmask, G.base);
+    }
+
+    unsigned long long c0 = ncand, c1 = ndef, c2 = nres;
+#pragma unroll
+    for (int o = 16; o > 0; o >>= 1) {
+        sum += __shfl_xor_sync(0xffffffffu, sum, o);
+        c0 += __shfl_xor_sync(0xffffffffu, c0, o);
+        c1 += __shfl_xor_sync(0xffffffffu, c1, o);
+        c2 += __shfl_xor_sync(0xffffffffu, c2, o);
+    }
+    finalize_out4<NW>(P, warp, lane, sum, c2, c0, c1);
 }
 
 }  // namespace rl
@@ -367,6 +664,16 @@ RlFn rl_pick(int cfg) {
 }
 
 template <int... Ws>
+RlFn rg_pick(int cfg) {
+    switch (cfg) {
+        case 1: return {(const void*)ard::rl::fused_rg_kernel<4, 2, Ws...>, 4, 8192};
+        case 3: return {(const void*)ard::rl::fused_rg_kernel<16, 1, Ws...>, 16, 16384};
+        case 4: return {(const void*)ard::rl::fused_rg_kernel<4, 1, Ws...>, 4, 4096};
+        default: return {(const void*)ard::rl::fused_rg_kernel<8, 1, Ws...>, 8, 8192};
+    }
+}
+
+template <int... Ws>
 bool rl_match(const ard::SelParams& P) {
     constexpr int n = sizeof...(Ws);
     constexpr int wk[] = {Ws..., 0};
@@ -376,6 +683,27 @@ bool rl_match(const ard::SelParams& P) {
         if ((int)((P.p[c].w << 6) | k) != wk[c]) return false;
     }
     return true;
+}
+
+// rg shapes: (w_major << 6) | k of every predicate, the residual gathered (SLICED, k <= 8)
+template <int... Ws>
+bool rg_match(const ard::SelParams& P) {
+    constexpr int n = sizeof...(Ws);
+    constexpr int wk[] = {Ws..., 0};
+    if (P.npred != n) return false;
+    for (int c = 0; c < n; ++c)
+        if ((int)((P.p[c].w << 6) | P.p[c].k) != wk[c]) return false;
+    return true;
+}
+
+RlFn rg_find(const ard::SelParams& P, int cfg) {
+#define AR_RG_TRY(...) \
+    if (rg_match<__VA_ARGS__>(P)) return rg_pick<__VA_ARGS__>(cfg);
+    AR_RG_TRY(WK(4, 8), WK(4, 0), WK(6, 0))
+    AR_RG_TRY(WK(24, 8))
+    AR_RG_TRY(WK(24, 8), WK(24, 8))
+#undef AR_RG_TRY
+    return {nullptr, 0, 0};
 }
 
 // Decomposition shapes with a result-ring kernel: Q6 (l_shipdate 4 major + 8
@@ -425,24 +753,30 @@ size_t rl_smem_bytes(const ard::SelParams& P, uint32_t nstages, int nw) {
 // Launch the result-ring kernel if it applies (returns AR_OK and *launched);
 // otherwise *launched = false and the caller takes fused_kernel.
 ar_status launch_fused_rl(const ard::SelParams& P0, const ar_column* const* cols, void* ws, int pdl, bool* launched,
-                          cudaStream_t s) {
+                          bool* gathered_res, cudaStream_t s) {
     *launched = false;
+    *gathered_res = false;
     ard::SelParams P = P0;   // the caller's copy stays valid for fused_kernel
     P.rl_fin = ws ? 1 : 0;
     P.rl_pdl = ws ? pdl : 0;
     P.rl_ticket = ws ? (unsigned int*)ws : nullptr;
     P.rl_part = ws ? (unsigned long long*)((char*)ws + kSrsTicketBytes) : nullptr;
     static const bool off = getenv("AR_FUSED_LEGACY") && atoi(getenv("AR_FUSED_LEGACY"));
-    if (off || !P.exact_mode || P.n >= (int64_t)1 << 32) return AR_OK;
+    // AR_RL_RESMODE: 0 (default) streamed-residual kernel where it applies, else the two-phase kernel
+    // with gathered residuals; 2 gathered only
+    static const int resmode = getenv("AR_RL_RESMODE") ? atoi(getenv("AR_RL_RESMODE")) : 0;
+    if (off || P.n >= (int64_t)1 << 32) return AR_OK;
     // factors: none (COUNT), all predicate columns (direct), or one gathered bit-packed column
     // in device memory times at most one predicate column (result ring)
     int gathered = 0, g = -1, mp = -1;
+    bool fac_k0 = true;   // every predicate-column factor has k = 0 (its value is in the major planes)
     for (int i = 0; i < P.nagg; ++i) {
         if (P.a[i].pred < 0) {
             ++gathered;
             g = i;
         } else {
             mp = P.a[i].pred;
+            fac_k0 = fac_k0 && P.p[mp].k == 0;
         }
     }
     if (gathered > 1) return AR_OK;
@@ -456,7 +790,33 @@ ar_status launch_fused_rl(const ard::SelParams& P0, const ar_column* const* cols
         P.rl_list = 0;
         P.rl_mpred = -1;
     }
-    const RlFn k = rl_find(P, env_cfg());
+    // the gathered-residual kernel: every decomposed predicate has a SLICED residual (k <= 8, HBM or
+    // pinned host memory); factors as above with k = 0 predicate columns
+    bool rg_ok = fac_k0;
+    for (int c = 0; c < P.npred && rg_ok; ++c)
+        if (P.p[c].k > 0) rg_ok = P.p[c].rlayout == AR_LAYOUT_SLICED && P.p[c].residual != nullptr && P.p[c].k <= 8;
+    RlFn k{nullptr, 0, 0};
+    bool rg = false;
+    // streamed residual planes first (device residuals: a stream of every block's planes beats
+    // gathering the touched sectors, DESIGN s6.3c), the gathered-residual kernel otherwise (residuals
+    // in pinned host memory, or the stream heuristic said no)
+    const bool rl_ok = P.exact_mode != 0;
+    if (rl_ok && resmode != 2) k = rl_find(P, env_cfg());
+    if (!k.fn && rg_ok) {
+        ard::SelParams Q = P;
+        // the .L2::64B prefetch-size hint on HBM residuals; over the host link AR_HOST_HINT (default 0)
+        static const int host_hint = getenv("AR_HOST_HINT") ? atoi(getenv("AR_HOST_HINT")) : 0;
+        for (int c = 0; c < Q.npred; ++c) {
+            Q.p[c].res_stream = 0;
+            Q.p[c].res_hint = (Q.p[c].res_host ? host_hint : 1) ? 1u : 0u;
+        }
+        k = rg_find(Q, env_cfg());
+        if (k.fn) {
+            P = Q;
+            P.tile_rows = 0;   // force retile without residual planes
+            rg = true;
+        }
+    }
     if (!k.fn) return AR_OK;
     retile(P, k.tile_rows);
     P.rl_ring = (uint32_t)env_ring();
@@ -471,7 +831,8 @@ ar_status launch_fused_rl(const ard::SelParams& P0, const ar_column* const* cols
     for (int target = std::max(want_ctas, 1); target >= 1 && !stages; --target)
         for (uint32_t st = 8; st >= 2; --st) {
             if (force_st > 0 && (int)st != force_st) continue;
-            if (target >= 2 && st < 3 && force_st <= 0) break;
+            // the two-phase kernel holds two stages (phase B of tile t - 1 while tile t is decided)
+            if (target >= 2 && st < (rg ? 4u : 3u) && force_st <= 0) break;
             int o = 0;
             cudaOccupancyMaxActiveBlocksPerMultiprocessor(&o, k.fn, threads, rl_smem_bytes(P, st, k.nw));
             if (o >= target) {
@@ -498,6 +859,7 @@ ar_status launch_fused_rl(const ard::SelParams& P0, const ar_column* const* cols
     cfg.numAttrs = 1;
     AR_TRY_CUDA(cudaLaunchKernelExC(&cfg, k.fn, args));
     *launched = true;
+    *gathered_res = rg;
     return AR_OK;
 }
 

@@ -19,6 +19,8 @@ struct SelPred {
     uint32_t rlayout;         // residual layout (ar_layout)
     uint32_t res_stream;      // fused kernel: residual tile streamed into the stage (device-resident residuals)
     uint32_t res_soff;        // word offset of the streamed residual tile inside a stage
+    uint32_t res_host;        // residual in pinned host memory (read over the host link)
+    uint32_t res_hint;        // gathered-residual kernel: use the .L2::64B prefetch-size hint
 };
 
 // Aggregate factor of the SUM product.
@@ -233,7 +235,7 @@ constexpr size_t kSrsTicketBytes = 128;
 constexpr int kSrsMaxGrid = 2048;
 void retile(ard::SelParams& P, uint32_t tile_rows);   // fused.cu
 ar_status launch_fused_rl(const ard::SelParams& P, const ar_column* const* cols, void* ws, int pdl, bool* launched,
-                          cudaStream_t s);
+                          bool* gathered_res, cudaStream_t s);
 ar_status launch_refine(const ard::RefParams& P, int grid, cudaStream_t s);
 const void* refine_kernel_fn();
 ar_status launch_refine_sum(const ard::RefParams& P, int grid, cudaStream_t s);

@@ -315,11 +315,26 @@ __global__ void __launch_bounds__(kRefThreads, 2) refine_sum_sliced_kernel(const
     const uint32_t qmask = q.w == 32 ? 0xffffffffu : ((1u << q.w) - 1u);
     const int g = P.fast_g;   // gathered factor, or -1
     unsigned long long sum = 0, kept = 0;
+    // the next tile's candidates are loaded while this one's gathers are in flight
+    uint32_t npos[8], naux[8];
+    if (blockIdx.x < num_tiles) {
+        const uint64_t j0 = (uint64_t)blockIdx.x * kRefTile + threadIdx.x * kRefPerThread;
+        load8(P.in_pos, j0, count, npos);
+        load8(P.in_aux, j0, count, naux);
+    }
     for (long long t = blockIdx.x; t < num_tiles; t += gridDim.x) {
         const uint64_t j0 = (uint64_t)t * kRefTile + threadIdx.x * kRefPerThread;
         uint32_t pos[8], aux[8];
-        load8(P.in_pos, j0, count, pos);
-        load8(P.in_aux, j0, count, aux);
+#pragma unroll
+        for (int i = 0; i < 8; ++i) {
+            pos[i] = npos[i];
+            aux[i] = naux[i];
+        }
+        if (t + gridDim.x < num_tiles) {
+            const uint64_t j1 = (uint64_t)(t + gridDim.x) * kRefTile + threadIdx.x * kRefPerThread;
+            load8(P.in_pos, j1, count, npos);
+            load8(P.in_aux, j1, count, naux);
+        }
         uint32_t valid = 0, def = 0;
 #pragma unroll
         for (int i = 0; i < 8; ++i) {

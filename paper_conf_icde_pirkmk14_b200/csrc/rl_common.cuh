@@ -36,7 +36,31 @@ struct Shape {
         for (int i = 0; i < c; ++i) o += w(i);
         return o;
     }
+    static constexpr int kofs(int c) {  // first residual word of predicate c in a block's residual words
+        int o = 0;
+        for (int i = 0; i < c; ++i) o += k(i);
+        return o;
+    }
+    static constexpr int ksum() { return kofs(N); }
 };
+
+// The K residual words of SLICED block `gblk` (K <= 8 planes, K words at
+// res + gblk * K), as predicated gathers (.L2::64B): issued for the blocks
+// that hold a non-definite candidate, consumed a tile later.
+template <int K>
+__device__ __forceinline__ void res_issue(uint32_t* r, const uint32_t* res, uint64_t gblk, bool pred, bool hint) {
+    const uint32_t* p = res + gblk * K;
+    if constexpr (K % 4 == 0) {
+#pragma unroll
+        for (int q = 0; q < K / 4; ++q) {
+            const uint4 v = hint ? ld_gather_if4(p + 4 * q, pred) : ld_gather_if4_nh(p + 4 * q, pred);
+            r[4 * q] = v.x; r[4 * q + 1] = v.y; r[4 * q + 2] = v.z; r[4 * q + 3] = v.w;
+        }
+    } else {
+#pragma unroll
+        for (int j = 0; j < K; ++j) r[j] = hint ? ld_gather_if(p + j, pred) : ld_gather_if_nh(p + j, pred);
+    }
+}
 
 // W consecutive 32-bit words from shared memory, vectorised as far as the
 // width allows (a block's planes start at a multiple of W words).

@@ -387,13 +387,16 @@ __device__ __forceinline__ void init_barriers(const SelParams& P, const SmemLayo
 // ------------------------------------------------------------ ordered select
 
 // Ordered select in three short, dependency-free kernels:
-//   1. select_tile_kernel: one tile per CTA.  One TMA bulk copy per predicate
-//      brings the tile's planes, the CTA evaluates them, compacts its candidates
-//      (stable: per-thread popc, block scan) and writes them with coalesced
-//      stores to the tile's own slice of a workspace buffer, plus its count.
+//   1. select_tile_kernel: persistent CTAs, tiles round-robin; nstages tile
+//      buffers per CTA, so the TMA bulk copies of the CTA's next tiles are in
+//      flight while it decides one (no CTA ever waits on another).  Per tile:
+//      evaluate the planes, compact the candidates (stable: per-thread popc,
+//      block scan) and write them with coalesced stores to the tile's own
+//      slice of a workspace buffer, plus its count.
 //   2. scan_counts_kernel: one CTA turns the per-tile counts into exclusive
 //      offsets and the total.
-//   3. compact_kernel: each CTA moves one tile's slice to its final offset.
+//   3. compact_kernel: each CTA moves a chunk of tiles' slices to their final
+//      offsets.
 // No CTA ever waits for another: on this GPU a decoupled look-back spent most
 // of the select kernel's time at its barrier (DESIGN s6.2).  The workspace
 // round trip is 8 B per candidate written and read back (L2-resident at low
@@ -401,127 +404,181 @@ __device__ __forceinline__ void init_barriers(const SelParams& P, const SmemLayo
 template <class PS, int NW, int BPT, bool kCarry>
 __global__ void __launch_bounds__(NW * 32) select_tile_kernel(const __grid_constant__ SelParams P) {
     constexpr int NT = NW * 32;
+    constexpr uint32_t kMaxBufs = 4;
     extern __shared__ __align__(128) unsigned char smem[];
-    __shared__ __align__(8) uint64_t bar;
+    __shared__ __align__(8) uint64_t bar[kMaxBufs];
     __shared__ uint32_t warp_tot[32];
     uint32_t* st_pos = reinterpret_cast<uint32_t*>(smem);
-    uint32_t* stg = st_pos + kStageEntries;          // 16-B aligned (kStageEntries * 4 bytes above)
-    const long long t = blockIdx.x;
+    uint32_t* stg0 = st_pos + kStageEntries;          // 16-B aligned (kStageEntries * 4 bytes above)
+    const uint32_t nb = P.nstages;                    // tile buffers: the next tiles load while one is decided
+    const long long G = gridDim.x;
 
-    if (threadIdx.x == 0) {
-        mbar_init(&bar, 1);
-        fence_mbar_init();
+    // thread 0: one TMA bulk copy per predicate brings tile t's planes into buffer b
+    auto issue = [&](long long t, uint32_t b) {
         const int64_t r0 = t * (int64_t)P.tile_rows;
         const int64_t rows = min((int64_t)P.tile_rows, P.n - r0);
         const uint32_t groups = (uint32_t)((rows + 127) / 128);
         uint32_t bytes = 0;
         for (int c = 0; c < P.npred; ++c) bytes += groups * 16u * P.p[c].w;
-        mbar_arrive_expect_tx(&bar, bytes);
+        mbar_arrive_expect_tx(&bar[b], bytes);
         const uint64_t pol = policy_evict_first();
+        uint32_t* stg = stg0 + (size_t)b * P.stage_words;
         for (int c = 0; c < P.npred; ++c) {
             const uint32_t w = P.p[c].w;
             if (w)
                 bulk_g2s(stg + P.p[c].soff, P.p[c].planes + (size_t)t * (P.tile_rows / 32) * w, groups * 16u * w,
-                         &bar, pol);
+                         &bar[b], pol);
         }
+    };
+    if (threadIdx.x == 0) {
+        for (uint32_t b = 0; b < nb; ++b) mbar_init(&bar[b], 1);
+        fence_mbar_init();
+        for (uint32_t b = 0; b < nb; ++b)
+            if (blockIdx.x + (long long)b * G < P.num_tiles) issue(blockIdx.x + (long long)b * G, b);
     }
     __syncthreads();
-    mbar_wait(&bar, 0, 0);
-    // compact_kernel (a programmatic dependent) may be scheduled once every tile is loaded
-    asm volatile("griddepcontrol.launch_dependents;" ::: "memory");
 
-    const int64_t r0 = t * (int64_t)P.tile_rows + (int64_t)threadIdx.x * (32 * BPT);
-    PS ps;
-    ps.load(P, stg);
-    uint32_t cm[BPT], dm[BPT];
-#pragma unroll
-    for (int b = 0; b < BPT; ++b) cm[b] = dm[b] = valid_mask(r0 + 32 * b, P.n);
-    ps.eval(P, cm, dm);
-    uint32_t cnt = 0;
-#pragma unroll
-    for (int b = 0; b < BPT; ++b) cnt += __popc(cm[b]);
-    uint32_t total;
-    const uint32_t excl = block_excl_scan<NT>(cnt, warp_tot, total, 1);
-    if (threadIdx.x == 0) {
-        P.tile_count[t] = total;
-        if (total) atomicAdd(P.group_sum + (t >> kGroupShift), (unsigned long long)total);
-    }
+    uint32_t i = 0;
+    for (long long t = blockIdx.x; t < P.num_tiles; t += G, ++i) {
+        const uint32_t b = i % nb;
+        const uint32_t* stg = stg0 + (size_t)b * P.stage_words;
+        mbar_wait(&bar[b], (i / nb) & 1u, 0);
+        // compact_kernel (a programmatic dependent) may be scheduled once this CTA's last tile is loaded
+        if (t + G >= P.num_tiles) asm volatile("griddepcontrol.launch_dependents;" ::: "memory");
 
-    // entries in rounds of kStageEntries: per-thread positions, lane-parallel aux, coalesced stores
-    const uint32_t tile_r0 = (uint32_t)(t * (int64_t)P.tile_rows);
-    uint32_t* tmp_pos = P.tmp_pos + (size_t)t * P.tile_rows;
-    uint32_t* tmp_aux = P.tmp_aux + (size_t)t * P.tile_rows;
-    uint32_t e = excl;
-    for (uint32_t base = 0; base < total; base += kStageEntries) {
-        const uint32_t lim = min(base + (uint32_t)kStageEntries, excl + cnt);
-        static_for<BPT>([&](auto bc) {
-            constexpr int b = decltype(bc)::value;
-            const uint32_t rbase = (threadIdx.x * BPT + b) << 5;
-            while (cm[b] && e < lim) {
-                const uint32_t l = __ffs(cm[b]) - 1;
-                cm[b] &= cm[b] - 1;
-                st_pos[e - base] = (rbase | l) | (((dm[b] >> l) & 1u) << 31);
-                ++e;
-            }
-        });
-        __syncthreads();
-        const uint32_t nround = min((uint32_t)kStageEntries, total - base);
-        for (uint32_t j = threadIdx.x; j < nround; j += NT) {
-            const uint32_t v = st_pos[j];
-            const uint32_t o = v & 0x7fffffffu;
-            uint32_t aux = v & 0x80000000u;
-            if (kCarry) aux |= PS::appr_smem(P, stg, o >> 5, o & 31u);
-            tmp_pos[base + j] = tile_r0 + o;
-            tmp_aux[base + j] = aux;
+        const int64_t r0 = t * (int64_t)P.tile_rows + (int64_t)threadIdx.x * (32 * BPT);
+        PS ps;
+        ps.load(P, stg);
+        uint32_t cm[BPT], dm[BPT];
+#pragma unroll
+        for (int q = 0; q < BPT; ++q) cm[q] = dm[q] = valid_mask(r0 + 32 * q, P.n);
+        ps.eval(P, cm, dm);
+        uint32_t cnt = 0;
+#pragma unroll
+        for (int q = 0; q < BPT; ++q) cnt += __popc(cm[q]);
+        uint32_t total;
+        const uint32_t excl = block_excl_scan<NT>(cnt, warp_tot, total, 1);
+        if (threadIdx.x == 0) {
+            P.tile_count[t] = total;
+            if (total) atomicAdd(P.group_sum + (t >> kGroupShift), (unsigned long long)total);
         }
-        __syncthreads();
+
+        // entries in rounds of kStageEntries: per-thread positions, lane-parallel aux, coalesced stores
+        const uint32_t tile_r0 = (uint32_t)(t * (int64_t)P.tile_rows);
+        uint32_t* tmp_pos = P.tmp_pos + (size_t)t * P.tile_rows;
+        uint32_t* tmp_aux = P.tmp_aux + (size_t)t * P.tile_rows;
+        uint32_t e = excl;
+        for (uint32_t base = 0; base < total; base += kStageEntries) {
+            const uint32_t lim = min(base + (uint32_t)kStageEntries, excl + cnt);
+            static_for<BPT>([&](auto bc) {
+                constexpr int q = decltype(bc)::value;
+                const uint32_t rbase = (threadIdx.x * BPT + q) << 5;
+                while (cm[q] && e < lim) {
+                    const uint32_t l = __ffs(cm[q]) - 1;
+                    cm[q] &= cm[q] - 1;
+                    st_pos[e - base] = (rbase | l) | (((dm[q] >> l) & 1u) << 31);
+                    ++e;
+                }
+            });
+            __syncthreads();
+            const uint32_t nround = min((uint32_t)kStageEntries, total - base);
+            for (uint32_t j = threadIdx.x; j < nround; j += NT) {
+                const uint32_t v = st_pos[j];
+                const uint32_t o = v & 0x7fffffffu;
+                uint32_t aux = v & 0x80000000u;
+                if (kCarry) aux |= PS::appr_smem(P, stg, o >> 5, o & 31u);
+                tmp_pos[base + j] = tile_r0 + o;
+                tmp_aux[base + j] = aux;
+            }
+            __syncthreads();
+        }
+        __syncthreads();   // buffer b and warp_tot are free
+        if (threadIdx.x == 0 && t + (long long)nb * G < P.num_tiles) issue(t + (long long)nb * G, b);
     }
 }
 
-// Move each tile's candidate slice from the workspace to its final offset: one
-// warp per tile (grid-stride).  The tile's offset is the sum of the group
-// totals before its group (groups of 2^kGroupShift tiles, accumulated with one
-// atomic per tile by the select kernel) plus the counts of the earlier tiles of
-// its own group -- two short warp reductions, no separate scan kernel.
+// Move the tiles' candidate slices from the workspace to their final offsets.
+// One CTA per chunk of kCompactTiles consecutive tiles (a chunk never straddles
+// a group of 2^kGroupShift tiles): the chunk's offset is the sum of the group
+// totals before its group (accumulated with one atomic per tile by the select
+// kernel) plus the counts of the earlier tiles of its group -- one block-wide
+// reduction -- and the tiles' offsets inside the chunk a prefix over
+// kCompactTiles counts; then all 256 threads copy the chunk's entries with
+// coalesced, 4-deep unrolled loads and stores.
+constexpr int kCompactTiles = 8;
 __global__ void __launch_bounds__(256) compact_kernel(const __grid_constant__ SelParams P) {
     asm volatile("griddepcontrol.wait;" ::: "memory");   // no-op unless launched as a dependent
-    const unsigned lane = threadIdx.x & 31;
-    const long long nw = (long long)gridDim.x * 8;
-    for (long long t = (long long)blockIdx.x * 8 + (threadIdx.x >> 5); t < P.num_tiles; t += nw) {
-        const long long g = t >> kGroupShift, t0 = g << kGroupShift;
+    __shared__ unsigned long long red[8];
+    __shared__ uint32_t tpre[kCompactTiles + 1];
+    const unsigned lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+    const long long nchunks = (P.num_tiles + kCompactTiles - 1) / kCompactTiles;
+    for (long long ch = blockIdx.x; ch < nchunks; ch += gridDim.x) {
+        const long long t0 = ch * kCompactTiles;
+        const long long g = t0 >> kGroupShift, g0 = g << kGroupShift;
         unsigned long long off = 0;
-        for (long long i = lane; i < g; i += 32) off += __ldcg(P.group_sum + i);
-        for (long long i = t0 + lane; i < t; i += 32) off += __ldcg(P.tile_count + i);
+        for (long long i = threadIdx.x; i < g; i += 256) off += __ldcg(P.group_sum + i);
+        for (long long i = g0 + threadIdx.x; i < t0; i += 256) off += __ldcg(P.tile_count + i);
 #pragma unroll
         for (int o = 16; o > 0; o >>= 1) off += __shfl_xor_sync(0xffffffffu, off, o);
-        const uint32_t c = __ldcg(P.tile_count + t);
-        if (t == P.num_tiles - 1 && lane == 0) *P.out_count = (long long)(off + c);
-        const uint32_t* sp = P.tmp_pos + (size_t)t * P.tile_rows;
-        const uint32_t* sa = P.tmp_aux + (size_t)t * P.tile_rows;
-        for (uint32_t j0 = 0; j0 < c; j0 += 128) {
+        if (lane == 0) red[warp] = off;
+        if (warp == 0) {
+            const long long t = t0 + lane;
+            uint32_t c = (lane < kCompactTiles && t < P.num_tiles) ? __ldcg(P.tile_count + t) : 0u;
+            uint32_t incl = c;
+#pragma unroll
+            for (int o = 1; o < kCompactTiles; o <<= 1) {
+                const uint32_t y = __shfl_up_sync(0xffffffffu, incl, o);
+                if (lane >= (unsigned)o) incl += y;
+            }
+            if (lane < kCompactTiles) tpre[lane + 1] = incl;
+            if (lane == 0) tpre[0] = 0;
+        }
+        __syncthreads();
+        unsigned long long base = 0;
+#pragma unroll
+        for (int w = 0; w < 8; ++w) base += red[w];
+        const uint32_t total = tpre[kCompactTiles];
+        if (t0 + kCompactTiles >= P.num_tiles && threadIdx.x == 0) *P.out_count = (long long)(base + total);
+        uint32_t pre[kCompactTiles + 1];
+#pragma unroll
+        for (int i = 0; i <= kCompactTiles; ++i) pre[i] = tpre[i];
+        for (uint32_t e0 = 0; e0 < total; e0 += 4 * 256) {
             uint32_t vp[4], va[4];
 #pragma unroll
             for (int k = 0; k < 4; ++k) {
-                const uint32_t j = j0 + k * 32 + lane;
-                vp[k] = j < c ? __ldcs(sp + j) : 0u;   // streaming: each slice is read once
-                va[k] = j < c ? __ldcs(sa + j) : 0u;
+                const uint32_t e = e0 + k * 256 + threadIdx.x;
+                vp[k] = va[k] = 0u;
+                if (e < total) {
+                    int ti = 0;
+#pragma unroll
+                    for (int i = 1; i < kCompactTiles; ++i) ti += e >= pre[i] ? 1 : 0;
+                    const size_t src = (size_t)(t0 + ti) * P.tile_rows + (e - pre[ti]);
+                    vp[k] = __ldcs(P.tmp_pos + src);   // streaming: each slice is read once
+                    va[k] = __ldcs(P.tmp_aux + src);
+                }
             }
 #pragma unroll
             for (int k = 0; k < 4; ++k) {
-                const uint32_t j = j0 + k * 32 + lane;
-                if (j < c) {
-                    P.out_pos[off + j] = vp[k];
-                    P.out_aux[off + j] = va[k];
+                const uint32_t e = e0 + k * 256 + threadIdx.x;
+                if (e < total) {
+                    P.out_pos[base + e] = vp[k];
+                    P.out_aux[base + e] = va[k];
                 }
             }
         }
-        __syncwarp();
-        // the slice is dead: drop its L2 lines without writing them back (slices are
-        // 128-B aligned, 32 entries per line)
-        for (uint32_t L = lane; L < (c + 31) / 32; L += 32) {
-            asm volatile("discard.global.L2 [%0], 128;" ::"l"(sp + 32 * L) : "memory");
-            asm volatile("discard.global.L2 [%0], 128;" ::"l"(sa + 32 * L) : "memory");
+        __syncthreads();   // every thread has loaded its entries before any line is discarded
+        // the slices are dead: drop their L2 lines without writing them back (slices are 128-B
+        // aligned, 32 entries per line)
+        for (int ti = 0; ti < kCompactTiles; ++ti) {
+            const uint32_t c = pre[ti + 1] - pre[ti];
+            const uint32_t* sp = P.tmp_pos + (size_t)(t0 + ti) * P.tile_rows;
+            const uint32_t* sa = P.tmp_aux + (size_t)(t0 + ti) * P.tile_rows;
+            for (uint32_t L = threadIdx.x; L < (c + 31) / 32; L += 256) {
+                asm volatile("discard.global.L2 [%0], 128;" ::"l"(sp + 32 * L) : "memory");
+                asm volatile("discard.global.L2 [%0], 128;" ::"l"(sa + 32 * L) : "memory");
+            }
         }
+        __syncthreads();   // red / tpre are reused by the next chunk
     }
 }
 
@@ -887,7 +944,7 @@ const void* select_kernel_fn(const ard::SelParams& P, bool fused) {
 
 size_t select_smem_bytes(uint32_t stage_words, uint32_t nstages, bool staging) {
     size_t head = nstages * (8 + 8 + 8) + 32 * 4 + 8 * 8;
-    if (staging) return 1ull * ard::kStageEntries * 4 + (size_t)stage_words * 4;   // select: one tile per CTA
+    if (staging) return 1ull * ard::kStageEntries * 4 + (size_t)nstages * stage_words * 4;   // select: tile buffers
     head = (head + 127) & ~size_t(127);
     size_t bytes = head + 128 + (size_t)nstages * stage_words * 4;
     if (!staging) bytes += (size_t)kFusNW * 32 * 32 * kFusBPT * 2   // per-warp candidate lists (u16)
@@ -923,7 +980,9 @@ ar_status launch_scan(const void* fn, const ard::SelParams& P, int grid, size_t 
 // compact_kernel; after the persistent select it is a programmatic dependent
 // launch (the select's producer triggers it once its last tile is loading).
 ar_status launch_select_rest(const ard::SelParams& P, bool pdl, cudaStream_t s) {
-    const int grid = (int)std::min<long long>((P.num_tiles + 7) / 8, (long long)num_sms() * 8);
+    // one CTA per chunk: the block scheduler refills an SM as soon as a chunk is done
+    const long long chunks = (P.num_tiles + ard::kCompactTiles - 1) / ard::kCompactTiles;
+    const int grid = (int)std::min<long long>(chunks, 1ll << 30);
     ard::SelParams Q = P;
     void* args[] = {&Q};
     cudaLaunchConfig_t cfg = {};

@@ -1,5 +1,7 @@
-"""GPU parity of the one-pass result-ring kernel (fused.cu, ar_select_refine_sum
-with the exact predicate on streamed residual planes) against the CPU oracle:
+"""GPU parity of the one-pass result-ring kernels (fused.cu, ar_select_refine_sum:
+fused_rg_kernel with the residual sectors of non-definite candidates gathered
+and refined one tile later, fused_rl_kernel with the exact predicate on
+streamed residual planes) against the CPU oracle:
 ragged tails, every SUM-factor mode (COUNT only, predicate-column factors,
 one gathered column with and without a second factor), ring overflow at high
 selectivity, and every (warps, blocks-per-thread) configuration plus the
@@ -95,7 +97,7 @@ import sys, numpy as np, torch
 sys.path.insert(0, {root!r})
 import datagen, oracle
 from paper_conf_icde_pirkmk14_b200 import _ar, column as cu
-want = sys.argv[1]
+want, want_c1 = sys.argv[1], sys.argv[2]
 for seed, n, bounds in [(3, 100_003, None), (4, 70_001, [(3, 2523), (0, 10), (1, 50)])]:
     c = datagen.q6_columns(seed, 1.0, n=n)
     los = [datagen.Q6_SHIPDATE[0], datagen.Q6_DISCOUNT[0], datagen.Q6_QUANTITY[0]]
@@ -121,21 +123,31 @@ col = cu.BWDColumn(v, 24)
 o4 = torch.zeros(4, dtype=torch.int64, device="cuda")
 cu.select_refine_sum([(col, datagen.C1_LO, datagen.C1_HI)], [col], o4)
 torch.cuda.synchronize()
-assert _ar.ar_last_scan_kernel() == want
+assert _ar.ar_last_scan_kernel() == want_c1, (_ar.ar_last_scan_kernel(), want_c1)
+o1 = torch.zeros(4, dtype=torch.int64, device="cuda")
+cu.select_refine_sum([(col, datagen.C1_LO, datagen.C1_HI)], [], o1)   # COUNT: the gathered kernel applies too
+torch.cuda.synchronize()
 _, cnt, s = oracle.select_sum([v], [datagen.C1_LO], [datagen.C1_HI], [v], positions=False)
 cpos, cdef = oracle.approx_select([v], [8], [datagen.C1_LO], [datagen.C1_HI])
 assert o4.cpu().tolist() == [s, cnt, cpos.size, int(cdef.sum())]
+assert o1.cpu().tolist() == [0, cnt, cpos.size, int(cdef.sum())]
 print("ok")
 """
 
 
-@pytest.mark.parametrize("env,want", [({"AR_RL_CFG": "0"}, "fused_rl_kernel"),
-                                      ({"AR_RL_CFG": "1"}, "fused_rl_kernel"),
-                                      ({"AR_RL_CFG": "2"}, "fused_rl_kernel"),
-                                      ({"AR_FUSED_LEGACY": "1"}, "fused_kernel")])
-def test_rl_config_sweep_subprocess(cu, env, want):
+@pytest.mark.parametrize("env,want,want_c1", [
+    ({"AR_RL_CFG": "0", "AR_RL_RESMODE": "1"}, "fused_rl_kernel", "fused_rl_kernel"),
+    ({"AR_RL_CFG": "1", "AR_RL_RESMODE": "1"}, "fused_rl_kernel", "fused_rl_kernel"),
+    ({"AR_RL_CFG": "2", "AR_RL_RESMODE": "1"}, "fused_rl_kernel", "fused_rl_kernel"),
+    ({"AR_RL_CFG": "0", "AR_RL_RESMODE": "2"}, "fused_rg_kernel", "fused_kernel"),
+    ({"AR_RL_CFG": "1", "AR_RL_RESMODE": "2"}, "fused_rg_kernel", "fused_kernel"),
+    ({"AR_RL_CFG": "3", "AR_RL_RESMODE": "2"}, "fused_rg_kernel", "fused_kernel"),
+    ({"AR_RL_CFG": "4", "AR_RL_RESMODE": "2"}, "fused_rg_kernel", "fused_kernel"),
+    ({"AR_RL_CFG": "0"}, "fused_rl_kernel", "fused_rl_kernel"),
+    ({"AR_FUSED_LEGACY": "1"}, "fused_kernel", "fused_kernel")])
+def test_rl_config_sweep_subprocess(cu, env, want, want_c1):
     e = dict(os.environ, AR_RES_STREAM="1", **env)
-    r = subprocess.run([sys.executable, "-c", SWEEP.format(root=ROOT), want], env=e, capture_output=True,
+    r = subprocess.run([sys.executable, "-c", SWEEP.format(root=ROOT), want, want_c1], env=e, capture_output=True,
                        text=True, timeout=600)
     assert r.returncode == 0 and "ok" in r.stdout, r.stdout + r.stderr
 
@@ -186,3 +198,37 @@ def test_rl_workspace_general_kernel_and_empty(cu):
     cu.select_refine_sum([(col, 1500, 300)], [col], o4, ws=ws, flags=_ar.AR_SRS_PDL)
     torch.cuda.synchronize()
     assert o4.cpu().tolist() == [0, 0, 0, 0]
+
+
+@pytest.mark.parametrize("n", [8193, 1_000_003])
+@pytest.mark.parametrize("aggs", [("extprice", "discount"), ()])
+def test_rg_host_resident_residual(cu, n, aggs):
+    # the C5 mechanism: the l_shipdate residual in pinned host memory, gathered over the host link by the
+    # two-phase kernel for the blocks that hold a non-definite candidate
+    from paper_conf_icde_pirkmk14_b200 import _ar
+    c, cols, los, his = q6(cu, 77, n)
+    cols["shipdate"] = cu.BWDColumn(c["shipdate"], 24, residual_loc=_ar.AR_LOC_HOST_PINNED)
+    kernel, _ = run(cu, c, cols, los, his, list(aggs))
+    assert kernel == "fused_rg_kernel"
+
+
+def test_rg_spatial_two_decomposed_predicates(cu):
+    # two decomposed signed predicates (24/8, FOR base): both residuals gathered, COUNT
+    from paper_conf_icde_pirkmk14_b200 import _ar
+    n = 500_009
+    s = datagen.spatial_columns(23, n)
+    lon, lat = np.asarray(s["lon"], dtype=np.int32), np.asarray(s["lat"], dtype=np.int32)
+    cl = [cu.BWDColumn(lon, 24, signed=True, base="min"), cu.BWDColumn(lat, 24, signed=True, base="min")]
+    for los, his in (([datagen.SPATIAL_LON[0], datagen.SPATIAL_LAT[0]], [datagen.SPATIAL_LON[1], datagen.SPATIAL_LAT[1]]),
+                     ([-900_000, 4_000_000], [600_000, 6_000_000])):
+        preds = [(cl[0], los[0] & 0xFFFFFFFF, his[0] & 0xFFFFFFFF), (cl[1], los[1] & 0xFFFFFFFF, his[1] & 0xFFFFFFFF)]
+        o4 = torch.zeros(4, dtype=torch.int64, device="cuda")
+        cu.select_refine_sum(preds, [], o4)
+        torch.cuda.synchronize()
+        kernel = _ar.ar_last_scan_kernel()
+        _, cnt, _ = oracle.select_sum([lon, lat], los, his, signed=[True, True], positions=False)
+        cpos, cdef = oracle.approx_select([lon, lat], [8, 8], los, his, base=[int(c.desc.base) for c in cl],
+                                          signed=[True, True])
+        assert o4.cpu().tolist() == [0, cnt, cpos.size, int(cdef.sum())]
+        if cl[0].w_major == 24 and cl[1].w_major == 24:
+            assert kernel == "fused_rg_kernel"

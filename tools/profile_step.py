@@ -25,7 +25,7 @@ def main():
         torch.cuda.init()
         err, = rt.cudaDeviceSetLimit(rt.cudaLimit.cudaLimitMaxL2FetchGranularity, int(os.environ["L2FG"]))
         print("set L2 fetch granularity", os.environ["L2FG"], err, rt.cudaDeviceGetLimit(rt.cudaLimit.cudaLimitMaxL2FetchGranularity))
-    cols = datagen.q6_columns(2, sf)
+    cols = datagen.q6_columns(int(os.environ.get("SEED", "2")), sf)
     n = cols["shipdate"].size
     # RES_LOC=1: the l_shipdate residual in pinned host memory (the C5 mechanism, read over the host link)
     sd = cu.BWDColumn(cols["shipdate"], 24, residual_loc=int(os.environ.get("RES_LOC", "0")))
