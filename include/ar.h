@@ -360,6 +360,52 @@ ar_status ar_refine_group_sum(const ar_cands* in, const ar_pred* preds, int32_t 
                               void* stream);
 
 /*
+ * The approximation group operator (s IV-E): "hash-based
+ * grouping to assign group IDs to unique values", the output positionally
+ * aligned with the input.  For each row j < *rows->count at position
+ * rows->pos[j] (e.g. the candidate relation: {cands.pos, cands.count,
+ * cands.capacity}), the grouping value is
+ *   AR_GROUP_APPROX: the approximate value base + (major << k) -- the bucket
+ *                    minimum, a pre-grouping on approximate values (for a k = 0
+ *                    key the exact value);
+ *   AR_GROUP_EXACT : the exact value ((major << k) | residual) + base (reads the
+ *                    residual, device or host-pinned).
+ * Equal values get equal ids; ids are dense (0 .. #groups - 1) in order of
+ * first insertion into a hash table (open addressing) in the caller's
+ * `table` (ar_group_table_bytes(table_slots) bytes of device memory; table_slots
+ * a power of two >= 2 * max_groups; cleared by the call), so the id of a value
+ * depends on scheduling while the value of every id is written to
+ * group_keys_out[id] (device, max_groups entries; a signed column's int32 bits).
+ * gids_out (device, rows->capacity entries) receives the ids; *ngroups_dev
+ * (device int64) the number of distinct values; *overflow_dev (device u32) bit 0
+ * if there were more than max_groups values (ids are then clamped and the
+ * grouping is invalid), bit 1 if the table filled up.  One launch + memsets.
+ * Errors: AR_ERR_INVALID (null pointers, bad mode), AR_ERR_RANGE (table_slots).
+ */
+#define AR_GROUP_APPROX 0
+#define AR_GROUP_EXACT 1
+size_t ar_group_table_bytes(int64_t table_slots);
+ar_status ar_group_ids(const ar_positions* rows, const ar_column* key, int32_t mode, void* table, int64_t table_slots,
+                       int32_t max_groups, uint32_t* gids_out, uint32_t* group_keys_out, int64_t* ngroups_dev,
+                       uint32_t* overflow_dev, void* stream);
+
+/*
+ * Grouped COUNT / SUM over the exact result by the ids of the approximation
+ * group operator (s IV-E/F): as ar_refine_group_sum, but the group of
+ * candidate j is gids[j] (device, aligned with the candidate relation `in`,
+ * e.g. ar_group_ids over {in->pos, in->count}; values < ngroups).  The
+ * refinement eliminates the selection's false positives
+ * before anything is aggregated, so a group whose candidates were all false
+ * positives ends with count 0.  Writes device int64[2 * ngroups]: out[g] = SUM
+ * of prod_c cols[c] over R in group g, out[ngroups + g] = COUNT.
+ * Errors: AR_ERR_INVALID (null pointers, ngroups outside [1, AR_MAX_GROUPS]),
+ * otherwise as ar_refine_sum.
+ */
+ar_status ar_refine_group_sum_ids(const ar_cands* in, const ar_pred* preds, int32_t npred, const uint32_t* gids,
+                                  int32_t ngroups, const ar_column* const* cols, int32_t ncols, int64_t* out_dev,
+                                  void* stream);
+
+/*
  * Positional projection of one column at the rows of `pos` (the invisible /
  * positional join of the A&R plan: bwd.leftjoinapproximate and
  * bwd.leftjoinrefine of Fig. 7; positional joins

@@ -22,6 +22,8 @@ AR_AUX_DEFINITE = 0x80000000
 AR_PROJECT_APPROX, AR_PROJECT_EXACT = 0, 1
 AR_MIN, AR_MAX = 0, 1
 AR_SRS_PDL, AR_SRS_PDL_EARLY_READ = 1, 2
+AR_GROUP_APPROX, AR_GROUP_EXACT = 0, 1
+AR_MAX_GROUPS = 4096
 
 
 class ARError(RuntimeError):
@@ -98,6 +100,10 @@ SIGNATURES = {
     "ar_dist_exclusive_offsets": (ctypes.c_int, [_P, _I32, _I32, _P, _P, _P]),
     "ar_dist_concat_positions": (ctypes.c_int, [ctypes.POINTER(Positions), _I64, _P, _P, _I64, _P, _P]),
     "ar_decompose_set_width": (ctypes.c_int, [ctypes.POINTER(ColumnDesc), _I32]),
+    "ar_group_table_bytes": (_SZ, [_I64]),
+    "ar_group_ids": (ctypes.c_int, [ctypes.POINTER(Positions), _P, _I32, _P, _I64, _I32, _P, _P, _P, _P, _P]),
+    "ar_refine_group_sum_ids": (ctypes.c_int, [ctypes.POINTER(Cands), ctypes.POINTER(Pred), _I32, _P, _I32,
+                                               ctypes.POINTER(_P), _I32, _P, _P]),
 }
 
 _lib = None
@@ -297,3 +303,18 @@ def ar_dist_concat_positions(local: Positions, row0, global_offset_dev, out_glob
 
 def ar_decompose_set_width(desc: ColumnDesc, w_major: int):
     _call("ar_decompose_set_width", ctypes.byref(desc), w_major)
+
+
+def ar_group_table_bytes(slots: int) -> int:
+    return int(load().ar_group_table_bytes(slots))
+
+
+def ar_group_ids(rows: Positions, key, mode, table, table_slots, max_groups, gids_out, group_keys_out, ngroups_dev,
+                 overflow_dev, stream):
+    _call("ar_group_ids", ctypes.byref(rows), key, mode, table, table_slots, max_groups, gids_out, group_keys_out,
+          ngroups_dev, overflow_dev, stream)
+
+
+def ar_refine_group_sum_ids(cands: Cands, preds, gids, ngroups, cols, out_dev, stream):
+    _call("ar_refine_group_sum_ids", ctypes.byref(cands), _preds(preds), len(preds), gids, ngroups, _handles(cols),
+          len(cols), out_dev, stream)

@@ -250,3 +250,52 @@ def SrsWorkspace(device="cuda") -> "Workspace":
     w = Workspace(_ar.ar_select_refine_sum_ws_bytes(), device)
     w.t.zero_()
     return w
+
+
+class Grouping:
+    """Output of the approximation group operator (ar_group_ids, s IV-E): per-row group ids aligned with
+    a position list, the grouping value of every id, the number of groups and the overflow flags."""
+
+    def __init__(self, capacity: int, max_groups: int, device="cuda"):
+        slots = 1
+        while slots < 2 * max_groups:
+            slots <<= 1
+        self.max_groups, self.slots = int(max_groups), slots
+        self.table = torch.empty(max(_ar.ar_group_table_bytes(slots), 16), dtype=torch.uint8, device=device)
+        self.gids = torch.empty(max(int(capacity), 1) + 8, dtype=torch.int32, device=device)
+        self.keys = torch.empty(max_groups, dtype=torch.int32, device=device)
+        self.ngroups_t = torch.zeros(1, dtype=torch.int64, device=device)
+        self.overflow_t = torch.zeros(1, dtype=torch.int32, device=device)
+
+    def ngroups(self) -> int:
+        return int(self.ngroups_t.item())
+
+    def overflow(self) -> int:
+        return int(self.overflow_t.item())
+
+    def group_keys(self) -> np.ndarray:
+        g = min(self.ngroups(), self.max_groups)
+        return self.keys[:g].cpu().numpy().view(np.uint32)
+
+
+def group_ids(rows, key: BWDColumn, grouping: Grouping, exact: bool = False, stream=None) -> Grouping:
+    """The approximation group operator over the rows of a CandidateList or PositionList: hash-assigned
+    dense group ids of the key's approximate (bucket minimum) or exact values, aligned with the rows."""
+    if isinstance(rows, CandidateList):
+        p = Positions(rows.pos.data_ptr(), rows.count_t.data_ptr(), rows.c.capacity)
+    else:
+        p = rows.p
+    _ar.ar_group_ids(p, key.handle, _ar.AR_GROUP_EXACT if exact else _ar.AR_GROUP_APPROX, grouping.table.data_ptr(),
+                     grouping.slots, grouping.max_groups, grouping.gids.data_ptr(), grouping.keys.data_ptr(),
+                     grouping.ngroups_t.data_ptr(), grouping.overflow_t.data_ptr(), _stream(stream))
+    return grouping
+
+
+def refine_group_sum_ids(cands: CandidateList, preds, grouping: Grouping, cols, stream=None) -> torch.Tensor:
+    """Grouped COUNT / SUM over the refined rows by the ids of `grouping` (aligned with `cands`): returns a
+    device int64 tensor [2, max_groups] (row 0: SUM(prod(cols)) per id, row 1: COUNT)."""
+    G = grouping.max_groups
+    out = torch.empty(2 * G, dtype=torch.int64, device=grouping.gids.device)
+    _ar.ar_refine_group_sum_ids(cands.c, _pred_tuples(preds), grouping.gids.data_ptr(), G, [c.handle for c in cols],
+                                out.data_ptr(), _stream(stream))
+    return out.view(2, G)

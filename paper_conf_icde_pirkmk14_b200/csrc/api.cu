@@ -909,6 +909,31 @@ ar_status ar_refine_group_sum(const ar_cands* in, const ar_pred* preds, int32_t 
     return launch_group_sum(P, grid, s);
 }
 
+ar_status ar_refine_group_sum_ids(const ar_cands* in, const ar_pred* preds, int32_t npred, const uint32_t* gids,
+                                  int32_t ngroups, const ar_column* const* cols, int32_t ncols, int64_t* out_dev,
+                                  void* stream) {
+    ard::GroupParams P;
+    memset(&P, 0, sizeof(P));
+    ar_status st = setup_refine(in, preds, npred, P.r);
+    if (st != AR_OK) return st;
+    if (!out_dev || !gids || ngroups < 1 || ngroups > AR_MAX_GROUPS) {
+        set_error("ar_refine_group_sum_ids: null output / ids, or ngroups %d outside [1, %d]", ngroups, AR_MAX_GROUPS);
+        return AR_ERR_INVALID;
+    }
+    st = setup_aggs(cols, ncols, preds, npred, preds[0].col->d.n, P.r.a, 0);
+    if (st != AR_OK) return st;
+    P.r.nagg = ncols;
+    P.gids = gids;
+    P.ngroups = ngroups;
+    P.out = (unsigned long long*)out_dev;
+    cudaStream_t s = (cudaStream_t)stream;
+    AR_TRY_CUDA(cudaMemsetAsync(out_dev, 0, 2 * sizeof(int64_t) * (size_t)ngroups, s));
+    const int64_t cap = std::max<int64_t>(in->capacity, 1);
+    const int grid = (int)std::min<int64_t>((cap + ard::kRefTile - 1) / ard::kRefTile, (int64_t)num_sms() * 4);
+    g_last_scan = "group_sum_kernel";
+    return launch_group_sum(P, grid, s);
+}
+
 // ----------------------------------------------------------- fused a3+a5+a6
 
 size_t ar_select_refine_sum_ws_bytes(void) { return kSrsTicketBytes + (size_t)kSrsMaxGrid * 32; }

@@ -206,6 +206,7 @@ struct MinMaxParams {
 struct GroupParams {
     RefParams r;              // candidates, predicates, aggregate factors (r.a, r.nagg)
     AggCol key;               // k == 0, unsigned; group id = key value (< ngroups, host-checked)
+    const uint32_t* gids;     // or: group id per candidate (aligned with the candidate relation), < ngroups
     int32_t ngroups;
     unsigned long long* out;  // [ngroups] sums, then [ngroups] counts
 };

@@ -615,7 +615,14 @@ __global__ void __launch_bounds__(kRefThreads) group_sum_kernel(const __grid_con
         const uint32_t keep = refine_batch8(P.r, pos, aux, valid);
         if (!keep) continue;
         uint32_t key[8];
-        factor_batch8(P.r, P.key, pos, aux, keep, key);
+        if (P.gids) {   // ids of the approximation group operator, aligned with the candidates
+            uint32_t g8[8];
+            load8(P.gids, j0, count, g8);
+#pragma unroll
+            for (int i = 0; i < 8; ++i) key[i] = g8[i] < (uint32_t)G ? g8[i] : 0u;
+        } else {
+            factor_batch8(P.r, P.key, pos, aux, keep, key);
+        }
         unsigned long long prod[8];
 #pragma unroll
         for (int i = 0; i < 8; ++i) prod[i] = 1ull;

@@ -504,7 +504,7 @@ __global__ void __launch_bounds__(NW * 32) select_tile_kernel(const __grid_const
 // kernel) plus the counts of the earlier tiles of its group -- one block-wide
 // reduction -- and the tiles' offsets inside the chunk a prefix over
 // kCompactTiles counts; then all 256 threads copy the chunk's entries with
-// coalesced, 4-deep unrolled loads and stores.
+// coalesced loads (up to 12 per thread in flight) and stores.
 constexpr int kCompactTiles = 8;
 __global__ void __launch_bounds__(256) compact_kernel(const __grid_constant__ SelParams P) {
     asm volatile("griddepcontrol.wait;" ::: "memory");   // no-op unless launched as a dependent
@@ -542,10 +542,11 @@ __global__ void __launch_bounds__(256) compact_kernel(const __grid_constant__ Se
         uint32_t pre[kCompactTiles + 1];
 #pragma unroll
         for (int i = 0; i <= kCompactTiles; ++i) pre[i] = tpre[i];
-        for (uint32_t e0 = 0; e0 < total; e0 += 4 * 256) {
-            uint32_t vp[4], va[4];
+        constexpr int kDeep = 12;   // a chunk of ~8 tiles at Q6 selectivity is one round: all loads in flight
+        for (uint32_t e0 = 0; e0 < total; e0 += kDeep * 256) {
+            uint32_t vp[kDeep], va[kDeep];
 #pragma unroll
-            for (int k = 0; k < 4; ++k) {
+            for (int k = 0; k < kDeep; ++k) {
                 const uint32_t e = e0 + k * 256 + threadIdx.x;
                 vp[k] = va[k] = 0u;
                 if (e < total) {
@@ -558,7 +559,7 @@ __global__ void __launch_bounds__(256) compact_kernel(const __grid_constant__ Se
                 }
             }
 #pragma unroll
-            for (int k = 0; k < 4; ++k) {
+            for (int k = 0; k < kDeep; ++k) {
                 const uint32_t e = e0 + k * 256 + threadIdx.x;
                 if (e < total) {
                     P.out_pos[base + e] = vp[k];
