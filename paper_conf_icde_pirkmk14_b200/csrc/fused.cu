@@ -496,29 +496,23 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
         }
     };
 
-    // Two pending slots (A, B), used alternately: the residual gathers of tile t land in the slot
-    // that held tile t - 2, whose phase B runs first -- so every gather has two tile periods to
-    // complete (one was not enough on HBM: DESIGN s6.3c) and the consumer holds three stages.
-    struct Pending {
-        uint32_t r[BPT][KS > 0 ? KS : 1];   // residual words of the tile's blocks (in flight)
-        uint32_t nd[BPT];                   // its non-definite candidate masks
-        long long t;                        // the tile (-1: none), its stage
-        uint32_t st;
-    };
-    Pending pa, pb;
-    pa.t = pb.t = -1;
-    pa.st = pb.st = 0;
+    uint32_t rres[BPT][KS > 0 ? KS : 1];   // residual words of the pending tile's blocks (in flight)
+    uint32_t pnd[BPT];                      // its non-definite candidate masks
+#pragma unroll
+    for (int b = 0; b < BPT; ++b) pnd[b] = 0u;
+    long long pt = -1;                      // pending tile (phase B not yet run), its stage
+    uint32_t pst = 0;
 
-    // Phase B of a pending tile: exact predicate on its non-definite candidates, results to the ring,
+    // Phase B of the pending tile: exact predicate on its non-definite candidates, results to the ring,
     // then its stage is released.
-    auto phase_b = [&](Pending& q) {
-        const uint32_t* stg = stages + (size_t)q.st * P.stage_words;
-        const int64_t r0 = q.t * (int64_t)P.tile_rows;
+    auto phase_b = [&]() {
+        const uint32_t* stg = stages + (size_t)pst * P.stage_words;
+        const int64_t r0 = pt * (int64_t)P.tile_rows;
         uint32_t xm[BPT];
 #pragma unroll
         for (int b = 0; b < BPT; ++b) {
             const uint32_t blk = b * NT + threadIdx.x;
-            uint32_t em = q.nd[b];
+            uint32_t em = pnd[b];
             if (em) {
                 static_for<S::N>([&](auto cc) {
                     constexpr int C = decltype(cc)::value;
@@ -529,8 +523,8 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
                         uint32_t el = 0, eh = 0;
 #pragma unroll
                         for (int j = 0; j < K; ++j) {
-                            el = bsub(q.r[b][KO + j], P.pmx[C][j][0], el);
-                            eh = brsub(q.r[b][KO + j], P.pmx[C][j][1], eh);
+                            el = bsub(rres[b][KO + j], P.pmx[C][j][0], el);
+                            eh = brsub(rres[b][KO + j], P.pmx[C][j][1], eh);
                         }
 #pragma unroll
                         for (int j = 0; j < W; ++j) {
@@ -545,17 +539,14 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
         }
         consume(stg, r0, xm);
         __syncwarp();
-        if (lane == 0) mbar_arrive(empty + q.st);
-        q.t = -1;
+        if (lane == 0) mbar_arrive(empty + pst);
     };
 
     uint32_t s = 0, ph = 0;
-    // One tile: wait for its stage, phase A, phase B of the tile two back (slot q), gathers into q.
-    // Returns false at the end of the stream.
-    auto step = [&](Pending& q) -> bool {
+    for (;; s = (s + 1 == P.nstages) ? (ph ^= 1u, 0u) : s + 1) {
         mbar_wait(full + s, ph, P.suspend_ns);
         const long long t = slot[s];
-        if (t < 0) return false;
+        if (t < 0) break;
         const uint32_t* stg = stages + (size_t)s * P.stage_words;
         const int64_t tile_r0 = t * (int64_t)P.tile_rows;
         const bool full_tile = tile_r0 + (int64_t)P.tile_rows <= P.n;
@@ -574,7 +565,8 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
             ndm[b] = cm & ~dm;
         }
         if constexpr (KS > 0) {
-            if (q.t >= 0) phase_b(q);        // tile t - 2: its residual gathers have had two tiles to land
+            if (pt >= 0) phase_b();          // the previous tile's residual gathers have had a tile to land
+            // gather the residual sectors of this tile's blocks with a non-definite candidate
 #pragma unroll
             for (int b = 0; b < BPT; ++b) {
                 const uint64_t gblk = (uint64_t)(tile_r0 >> 5) + b * NT + threadIdx.x;
@@ -582,12 +574,12 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
                     constexpr int C = decltype(cc)::value;
                     constexpr int K = S::k(C), KO = S::kofs(C);
                     if constexpr (K > 0)
-                        res_issue<K>(&q.r[b][KO], P.p[C].residual, gblk, ndm[b] != 0u, P.p[C].res_hint != 0u);
+                        res_issue<K>(&rres[b][KO], P.p[C].residual, gblk, ndm[b] != 0u, P.p[C].res_hint != 0u);
                 });
-                q.nd[b] = ndm[b];
+                pnd[b] = ndm[b];
             }
-            q.t = t;
-            q.st = s;
+            pt = t;
+            pst = s;
             consume(stg, tile_r0, dmk);      // definite rows are results now
         } else {
             consume(stg, tile_r0, dmk);      // k = 0 everywhere: candidate = definite = exact
@@ -598,28 +590,9 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
             while (rcnt >= 32) pass(32);
             __syncwarp();
         }
-        if (++s == P.nstages) {
-            s = 0;
-            ph ^= 1u;
-        }
-        return true;
-    };
-    bool a_next = true;   // slot of the next tile
-    while (true) {
-        if (!step(pa)) break;
-        if (!step(pb)) {
-            a_next = false;
-            break;
-        }
     }
-    if constexpr (KS > 0) {   // the two pending tiles, oldest first
-        if (a_next) {
-            if (pa.t >= 0) phase_b(pa);
-            if (pb.t >= 0) phase_b(pb);
-        } else {
-            if (pb.t >= 0) phase_b(pb);
-            if (pa.t >= 0) phase_b(pa);
-        }
+    if constexpr (KS > 0) {
+        if (pt >= 0) phase_b();
     }
     if (list) {
         while (rcnt > 0) pass(min(rcnt, 32u));
@@ -858,8 +831,8 @@ ar_status launch_fused_rl(const ard::SelParams& P0, const ar_column* const* cols
     for (int target = std::max(want_ctas, 1); target >= 1 && !stages; --target)
         for (uint32_t st = 8; st >= 2; --st) {
             if (force_st > 0 && (int)st != force_st) continue;
-            // the two-phase kernel holds three stages (tiles t - 2, t - 1 pending while t is decided)
-            if (target >= 2 && st < (rg ? 5u : 3u) && force_st <= 0) break;
+            // the two-phase kernel holds two stages (phase B of tile t - 1 while tile t is decided)
+            if (target >= 2 && st < (rg ? 4u : 3u) && force_st <= 0) break;
             int o = 0;
             cudaOccupancyMaxActiveBlocksPerMultiprocessor(&o, k.fn, threads, rl_smem_bytes(P, st, k.nw));
             if (o >= target) {
