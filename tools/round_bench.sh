@@ -1,20 +1,23 @@
 #!/bin/bash
-# Round measurement on one B200: GPU tests, smoke, the default bench line, the
-# reference (oracle) arm, the ncu launch list of the same bench command (cold,
-# serialised: compare shares), one full ncu capture of each hot kernel, and the
-# secondary configurations.  Outputs land in gpurun_out/; summaries are copied
-# to profiles/ by hand.
+# Round measurement on one B200: GPU tests, smoke, the default bench line, the reference (oracle)
+# arm, the ncu launch list of the bench command (cold, serialised: compare shares), full ncu captures
+# of the hot kernels at C4 (the headline) and C2, and the traffic.json they give.  Outputs land in
+# gpurun_out/; summaries are copied to profiles/rNN/ (tools/collect_round.sh).
 set -x
 nvidia-smi --query-gpu=name,clocks.sm,clocks.max.sm,clocks.mem,power.draw --format=csv > gpurun_out/smi.txt
-timeout 900 python -m pytest tests -m gpu -q > gpurun_out/gpu_tests.log 2>&1
+timeout 1200 python -m pytest tests -m gpu -q > gpurun_out/gpu_tests.log 2>&1
 timeout 300 python -c "import __graft_entry__ as g; g.smoke()" > gpurun_out/smoke.log 2>&1
-timeout 600 python bench.py > gpurun_out/bench.json 2> gpurun_out/bench.err
+timeout 900 python bench.py > gpurun_out/bench.json 2> gpurun_out/bench.err
 timeout 300 python bench.py --impl reference --steps 5 --warmup 3 > gpurun_out/bench_ref.json 2> gpurun_out/bench_ref.err
-timeout 900 ncu --metrics gpu__time_duration.sum --clock-control none --csv --log-file gpurun_out/launches.csv \
-    python bench.py --steps 20 --warmup 3 --no-cpu --e2e-steps 0 > gpurun_out/bench_under_ncu.json 2>&1
-VARIANTS=fused,staged timeout 900 ncu --set full --clock-control none --import-source on \
-    -k regex:"fused_rl_kernel|select_tile_kernel|compact_kernel|refine_sum" -s 3 -c 4 -o gpurun_out/full python tools/profile_step.py \
-    > gpurun_out/full.log 2>&1
-for c in mm grp c1 c5 c3; do
-  timeout 900 python tools/bench_configs.py $c --reps 10 >> gpurun_out/configs.jsonl 2>> gpurun_out/configs.err
-done
+timeout 1200 ncu --metrics gpu__time_duration.sum --clock-control none --csv --log-file gpurun_out/launches.csv \
+    python bench.py --steps 20 --warmup 3 --no-cpu --e2e-steps 0 --no-c5 --latency-reps 3 --replays 0 \
+    > gpurun_out/bench_under_ncu.json 2>&1
+SF=100 SEED=4 VARIANTS=fused timeout 900 ncu --set full --clock-control none --import-source on \
+    -k regex:"fused_rl_kernel|fused_rg_kernel" -s 2 -c 1 -o gpurun_out/full_fused_c4 python tools/profile_step.py \
+    > gpurun_out/full_fused_c4.log 2>&1
+SF=100 SEED=4 VARIANTS=staged timeout 900 ncu --set full --clock-control none --import-source on \
+    -k regex:"select_tile_kernel|compact_kernel|refine_sum" -s 3 -c 3 -o gpurun_out/full_staged_c4 python tools/profile_step.py \
+    > gpurun_out/full_staged_c4.log 2>&1
+SF=10 SEED=2 VARIANTS=fused,staged timeout 900 ncu --set full --clock-control none --import-source on \
+    -k regex:"fused_rl_kernel|select_tile_kernel|compact_kernel|refine_sum" -s 3 -c 4 -o gpurun_out/full_c2 python tools/profile_step.py \
+    > gpurun_out/full_c2.log 2>&1
