@@ -13,15 +13,15 @@ def ncu_csv(rep, *args):
 
 def main(rep, kernel_regex=None, top=12):
     rows = ncu_csv(rep, "--page", "raw")
-    hdr = rows[0]
+    hdr, units = rows[0], rows[1]
     for row in rows[2:]:
-        d = dict(zip(hdr, row))
+        d = {h: (f"{v} {u}".strip() if u and h.startswith("dram__bytes") else v) for h, v, u in zip(hdr, row, units)}
         name = d["Kernel Name"]
         if kernel_regex and kernel_regex not in name:
             continue
         f = lambda k: d.get(k, "?")
         print(f"== {name[:60]}  id={f('ID')}")
-        print(f"   time {f('gpu__time_duration.sum')} us  dram rd {f('dram__bytes_read.sum')} MB  wr {f('dram__bytes_write.sum')} MB"
+        print(f"   time {f('gpu__time_duration.sum')} us  dram rd {f('dram__bytes_read.sum')}  wr {f('dram__bytes_write.sum')}"
               f"  dram% {f('gpu__dram_throughput.avg.pct_of_peak_sustained_elapsed')}  issue% {f('smsp__issue_active.avg.pct_of_peak_sustained_active')}"
               f"  warps% {f('sm__warps_active.avg.pct_of_peak_sustained_active')}  inst {f('smsp__inst_executed.sum')}  grid {f('launch__grid_size')}"
               f"  regs {f('launch__registers_per_thread')}")
