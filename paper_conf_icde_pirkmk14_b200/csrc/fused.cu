@@ -128,7 +128,7 @@ __device__ __forceinline__ void finalize_out4(const SelParams& P, unsigned warp,
 
 template <int NW, int BPT, int... WK>
 __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid_constant__ SelParams P) {
-    using S = Shape<WK...>;
+    using S = typename ShapeOf<WK...>::type;
     constexpr int NT = NW * 32;
     extern __shared__ __align__(128) unsigned char smem[];
     uint64_t* full = reinterpret_cast<uint64_t*>(smem);
@@ -214,7 +214,10 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
             const uint32_t blk = b * NT + threadIdx.x;
             const uint32_t vm = full_tile ? 0xffffffffu : valid_mask(tile_r0 + 32 * (int64_t)blk, P.n);
             uint32_t cm, dm, em;
-            eval_block<S, true>(P, stg, blk, vm, cm, dm, em);
+            if constexpr (S::kDynamic)
+                eval_block_dyn(P, stg, blk, vm, cm, dm, em);
+            else
+                eval_block<S, true>(P, stg, blk, vm, cm, dm, em);
             ncand += __popc(cm);
             ndef += __popc(dm);
             nres += __popc(em);
@@ -231,10 +234,14 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
                     unsigned long long prod = 1;
                     for (int a = 0; a < P.nagg; ++a) {
                         uint32_t v = 0;
-                        static_for<S::N>([&](auto cc) {
-                            constexpr int C = decltype(cc)::value;
-                            if (C == P.a[a].pred) v = stage_value<S, C>(P, stg, blk, l);
-                        });
+                        if constexpr (S::kDynamic) {
+                            v = stage_value_dyn(P, stg, P.a[a].pred, blk, l);
+                        } else {
+                            static_for<S::N>([&](auto cc) {
+                                constexpr int C = decltype(cc)::value;
+                                if (C == P.a[a].pred) v = stage_value<S, C>(P, stg, blk, l);
+                            });
+                        }
                         prod *= v;
                     }
                     sum += prod;
@@ -268,6 +275,13 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
                                 const uint32_t l = __ffs(m) - 1;
                                 m &= m - 1;
                                 ring[(wbase + e) & rmask] = make_uint2(row0 + l, 1u);
+                                ++e;
+                            } while (m && e < lim);
+                        } else if constexpr (S::kDynamic) {
+                            do {
+                                const uint32_t l = __ffs(m) - 1;
+                                m &= m - 1;
+                                ring[(wbase + e) & rmask] = make_uint2(row0 + l, stage_value_dyn(P, stg, P.rl_mpred, blk, l));
                                 ++e;
                             } while (m && e < lim);
                         } else {
@@ -720,6 +734,9 @@ RlFn rl_find(const ard::SelParams& P, int cfg) {
     AR_RL_TRY(WK(32, 0))
     AR_RL_TRY(WK(24, 8), WK(24, 8))
 #undef AR_RL_TRY
+    // any other decomposition: the runtime-shape kernel (widths and bounds from the parameters)
+    static const bool no_dyn = getenv("AR_RL_NODYN") && atoi(getenv("AR_RL_NODYN"));
+    if (!no_dyn) return rl_pick<-1>(cfg);
     return {nullptr, 0, 0};
 }
 

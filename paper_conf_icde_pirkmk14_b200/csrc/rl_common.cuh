@@ -22,6 +22,7 @@ __device__ __forceinline__ void static_for(F&& f) {
 // Decomposition shape: per predicate (w_major << 6) | streamed residual width k.
 template <int... WK>
 struct Shape {
+    static constexpr bool kDynamic = false;
     static constexpr int N = sizeof...(WK);
     static constexpr int w(int c) {
         constexpr int a[] = {(WK >> 6)..., 0};
@@ -42,6 +43,22 @@ struct Shape {
         return o;
     }
     static constexpr int ksum() { return kofs(N); }
+};
+
+// Runtime shape (any widths, any number of predicates): the one-pass kernel
+// reads widths, plane offsets and bounds from the parameters.  Selected with
+// the sentinel shape WK = {-1} for decompositions without a compiled shape.
+struct DynShape {
+    static constexpr bool kDynamic = true;
+    static constexpr int N = 0;
+};
+template <int... WK>
+struct ShapeOf {
+    using type = Shape<WK...>;
+};
+template <>
+struct ShapeOf<-1> {
+    using type = DynShape;
 };
 
 // The K residual words of SLICED block `gblk` (K <= 8 planes, K words at
@@ -170,6 +187,68 @@ __device__ __forceinline__ void eval_block(const SelParams& P, const uint32_t* s
             }
         }
     });
+}
+
+// eval_block for a runtime shape: the same borrow chains with the widths and
+// bound masks of the parameters (residual planes streamed where res_stream).
+__device__ __forceinline__ void eval_block_dyn(const SelParams& P, const uint32_t* stg, uint32_t blk, uint32_t vm,
+                                               uint32_t& cm, uint32_t& dm, uint32_t& em) {
+    cm = dm = em = vm;
+    for (int c = 0; c < P.npred; ++c) {
+        const SelPred& p = P.p[c];
+        const uint32_t W = p.w, O = p.ashift;
+        const uint32_t* xp = stg + p.soff + blk * W;
+        uint32_t cl = 0, ch = 0, dl = 0, dh = 0;
+        for (uint32_t j = 0; j < W; ++j) {
+            const uint32_t x = xp[j];
+            cl = bsub(x, P.pm[O + j][0], cl);
+            ch = brsub(x, P.pm[O + j][1], ch);
+            dl = bsub(x, P.pm[O + j][2], dl);
+            dh = brsub(x, P.pm[O + j][3], dh);
+        }
+        const uint32_t cc = ~(cl | ch);
+        cm &= cc;
+        if (p.k == 0) {
+            dm &= cc;
+            em &= cc;
+            continue;
+        }
+        dm &= ~(dl | dh);
+        if (!p.res_stream) {   // the dynamic kernel runs in exact mode only (every residual streamed)
+            em = 0u;
+            continue;
+        }
+        const uint32_t K = p.k;
+        const uint32_t* rp = stg + p.res_soff + blk * K;
+        uint32_t el = 0, eh = 0;
+        for (uint32_t j = 0; j < K; ++j) {
+            const uint32_t r = rp[j];
+            el = bsub(r, P.pmx[c][j][0], el);
+            eh = brsub(r, P.pmx[c][j][1], eh);
+        }
+        for (uint32_t j = 0; j < W; ++j) {
+            const uint32_t x = xp[j];
+            el = bsub(x, P.pmx[c][K + j][0], el);
+            eh = brsub(x, P.pmx[c][K + j][1], eh);
+        }
+        em &= ~(el | eh);
+    }
+}
+
+// Exact value of predicate c's column at row l of block blk from the stage (runtime shape).
+__device__ __forceinline__ uint32_t stage_value_dyn(const SelParams& P, const uint32_t* stg, int c, uint32_t blk,
+                                                    uint32_t l) {
+    const SelPred& p = P.p[c];
+    uint32_t m = 0;
+    const uint32_t* xp = stg + p.soff + blk * p.w;
+    for (uint32_t j = 0; j < p.w; ++j) m |= ((xp[j] >> l) & 1u) << j;
+    if (p.k > 0 && p.res_stream) {
+        uint32_t r = 0;
+        const uint32_t* rp = stg + p.res_soff + blk * p.k;
+        for (uint32_t j = 0; j < p.k; ++j) r |= ((rp[j] >> l) & 1u) << j;
+        return ((m << p.k) | r) + p.base;
+    }
+    return m + p.base;
 }
 
 }  // namespace rl

@@ -550,10 +550,16 @@ __global__ void __launch_bounds__(256) compact_kernel(const __grid_constant__ Se
                 const uint32_t e = e0 + k * 256 + threadIdx.x;
                 vp[k] = va[k] = 0u;
                 if (e < total) {
-                    int ti = 0;
+                    // the tile holding entry e: the last i with pre[i] <= e (selects, no indexed
+                    // register array -- that would go to local memory)
+                    uint32_t ti = 0, tb = 0;
 #pragma unroll
-                    for (int i = 1; i < kCompactTiles; ++i) ti += e >= pre[i] ? 1 : 0;
-                    const size_t src = (size_t)(t0 + ti) * P.tile_rows + (e - pre[ti]);
+                    for (int i = 1; i < kCompactTiles; ++i) {
+                        const bool ge = e >= pre[i];
+                        ti = ge ? (uint32_t)i : ti;
+                        tb = ge ? pre[i] : tb;
+                    }
+                    const size_t src = (size_t)(t0 + ti) * P.tile_rows + (e - tb);
                     vp[k] = __ldcs(P.tmp_pos + src);   // streaming: each slice is read once
                     va[k] = __ldcs(P.tmp_aux + src);
                 }

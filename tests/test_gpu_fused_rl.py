@@ -180,17 +180,17 @@ def test_rl_workspace_and_pdl_back_to_back(cu, flags):
     assert int(ws.t[:4].view(torch.int32).item()) == 0        # ticket left zero
 
 
-def test_rl_workspace_general_kernel_and_empty(cu):
-    # the workspace call on a shape without a result-ring kernel (general fused_kernel) and on an
-    # empty predicate still writes out4 (the output is not accumulated)
+def test_rl_workspace_runtime_shape_and_empty(cu):
+    # the workspace call on a shape without a compiled result-ring shape (the runtime-shape kernel) and
+    # on an empty predicate still writes out4 (the output is not accumulated)
     from paper_conf_icde_pirkmk14_b200 import _ar
-    v = datagen.uniform_u32(5, 100_000, 0, (1 << 11) - 1)      # w_major = 3: no result-ring shape
+    v = datagen.uniform_u32(5, 100_000, 0, (1 << 11) - 1)      # w_major = 3: no compiled shape
     col = cu.BWDColumn(v, 24)
     ws = cu.SrsWorkspace()
     o4 = torch.full((4,), -7, dtype=torch.int64, device="cuda")
     cu.select_refine_sum([(col, 300, 1500)], [col], o4, ws=ws)
     torch.cuda.synchronize()
-    assert _ar.ar_last_scan_kernel() == "fused_kernel"
+    assert _ar.ar_last_scan_kernel() == "fused_rl_kernel"
     _, cnt, s = oracle.select_sum([v], [300], [1500], [v], positions=False)
     cpos, cdef = oracle.approx_select([v], [8], [300], [1500])
     assert o4.cpu().tolist() == [s, cnt, cpos.size, int(cdef.sum())]
@@ -232,3 +232,45 @@ def test_rg_spatial_two_decomposed_predicates(cu):
         assert o4.cpu().tolist() == [0, cnt, cpos.size, int(cdef.sum())]
         if cl[0].w_major == 24 and cl[1].w_major == 24:
             assert kernel == "fused_rg_kernel"
+
+
+@pytest.mark.parametrize("ship_bits", [30, 28, 26, 25, 23])
+@pytest.mark.parametrize("aggs", [("extprice", "discount"), (), ("discount",)])
+def test_rl_runtime_shape_q6_splits(cu, ship_bits, aggs):
+    # other bwdecompose(l_shipdate, M) splits (k = 2..9 residual bits): the runtime-shape result-ring
+    # kernel where the residual planes stream (k <= 8), the general kernel otherwise; identical results
+    from paper_conf_icde_pirkmk14_b200 import _ar
+    n = 300_007
+    c = datagen.q6_columns(57, 1.0, n=n)
+    cols = {"shipdate": cu.BWDColumn(c["shipdate"], ship_bits), "discount": cu.BWDColumn(c["discount"], 32),
+            "quantity": cu.BWDColumn(c["quantity"], 32),
+            "extprice": cu.BWDColumn(c["extprice"], 32, layout=_ar.AR_LAYOUT_PACKED)}
+    los = [datagen.Q6_SHIPDATE[0], datagen.Q6_DISCOUNT[0], datagen.Q6_QUANTITY[0]]
+    his = [datagen.Q6_SHIPDATE[1], datagen.Q6_DISCOUNT[1], datagen.Q6_QUANTITY[1]]
+    preds = [(cols["shipdate"], los[0], his[0]), (cols["discount"], los[1], his[1]),
+             (cols["quantity"], los[2], his[2])]
+    o4 = torch.zeros(4, dtype=torch.int64, device="cuda")
+    cu.select_refine_sum(preds, [cols[a] for a in aggs], o4)
+    torch.cuda.synchronize()
+    values = [c["shipdate"], c["discount"], c["quantity"]]
+    _, cnt, sm = oracle.select_sum(values, los, his, [c[a] for a in aggs], positions=False)
+    cpos, cdef = oracle.approx_select(values, [32 - ship_bits, 0, 0], los, his)
+    assert o4.cpu().tolist() == [sm if aggs else 0, cnt, cpos.size, int(cdef.sum())]
+
+
+def test_rl_runtime_shape_spatial_for_base(cu):
+    # two signed 24/8 predicates with a frame-of-reference base (w_major < 24): runtime shape, COUNT
+    from paper_conf_icde_pirkmk14_b200 import _ar
+    n = 400_021
+    s = datagen.spatial_columns(29, n)
+    lon, lat = np.asarray(s["lon"], dtype=np.int32), np.asarray(s["lat"], dtype=np.int32)
+    cl = [cu.BWDColumn(lon, 24, signed=True, base="min"), cu.BWDColumn(lat, 24, signed=True, base="min")]
+    los, his = [-900_000, 4_000_000], [600_000, 6_000_000]
+    preds = [(cl[0], los[0] & 0xFFFFFFFF, his[0] & 0xFFFFFFFF), (cl[1], los[1] & 0xFFFFFFFF, his[1] & 0xFFFFFFFF)]
+    o4 = torch.zeros(4, dtype=torch.int64, device="cuda")
+    cu.select_refine_sum(preds, [], o4)
+    torch.cuda.synchronize()
+    _, cnt, _ = oracle.select_sum([lon, lat], los, his, signed=[True, True], positions=False)
+    cpos, cdef = oracle.approx_select([lon, lat], [8, 8], los, his, base=[int(c.desc.base) for c in cl],
+                                      signed=[True, True])
+    assert o4.cpu().tolist() == [0, cnt, cpos.size, int(cdef.sum())]
