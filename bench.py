@@ -90,6 +90,10 @@ def parse(argv=None):
     ap.add_argument("--only", action="store_true", help="time the headline variant only (no latency/c2/c5)")
     ap.add_argument("--no-c2", action="store_true")
     ap.add_argument("--no-c5", action="store_true")
+    ap.add_argument("--split", type=int, default=0,
+                    help="c4 / c2: the l_shipdate residual in the split layout with this many high planes apart")
+    ap.add_argument("--c5-split", type=int, default=0,
+                    help="c5: store the l_shipdate residual in the split layout with this many high planes apart")
     ap.add_argument("--latency-reps", type=int, default=30)
     ap.add_argument("--replays", type=int, default=5, help="extra timed replays for the median / min / p90")
     ap.add_argument("--e2e-steps", type=int, default=5)
@@ -306,11 +310,32 @@ def _snake(s):
 
 # -------------------------------------------------------------- algorithmic bytes
 
-def algorithmic_bytes(cols, w_sd=None):
+def split_lo_byte(blk, h):
+    """Byte offset of the low residual planes of 32-row block `blk` in the split layout (ar.h
+    ar_column_desc.residual_split: super-groups of 256 blocks, h high planes then k - h low planes)."""
+    return 4 * ((blk // 256) * (256 * K_SHIP) + 256 * h + (blk % 256) * (K_SHIP - h))
+
+
+def split_hi_byte(blk, h):
+    return 4 * ((blk // 256) * (256 * K_SHIP) + (blk % 256) * h)
+
+
+def _sectors(start, nbytes, gran=SECTOR):
+    """Distinct `gran`-byte units touched by the byte ranges [start, start + nbytes)."""
+    if start.size == 0:
+        return 0
+    return np.unique(np.concatenate([start // gran, (start + nbytes - 1) // gran])).size
+
+
+def algorithmic_bytes(cols, w_sd=None, split=0, high_streamed=True):
     """Bytes the method must move per query: packed scans + sector-granular gathers + output.
     Per column: scanned majors N w / 8; the l_shipdate residual: 32 B per distinct residual sector that holds
     a non-definite candidate; l_extendedprice: 32 B per distinct sector that holds (part of) a result row;
-    each gathered column capped at its size; + 8 B of output.  Computed from the data, not the GPU."""
+    each gathered column capped at its size; + 8 B of output.  Computed from the data, not the GPU.
+    split = h > 0 (the split residual layout, DESIGN s6.3d): with high_streamed (HBM residual, one-pass
+    kernel) the h high planes are a scanned part (N h / 8) and the k - h low planes are gathered for the rows
+    the high planes leave undecided (candidate, not definite at granularity 2^(k-h)); otherwise (residual
+    over the host link) the high planes of every block with a non-definite candidate are gathered too."""
     sd, dc, qt, ep = cols["shipdate"], cols["discount"], cols["quantity"], cols["extprice"]
     rows = sd.size
     if w_sd is None:
@@ -318,29 +343,48 @@ def algorithmic_bytes(cols, w_sd=None):
     w_dc, w_qt, w_ep = int(dc.max()).bit_length(), int(qt.max()).bit_length(), int(ep.max()).bit_length()
     scan = rows * (w_sd + w_dc + w_qt) / 8.0
     lo, hi = PREDS[0]
-    major = sd >> K_SHIP
-    cand_sd = (major >= (lo >> K_SHIP)) & (major <= (hi >> K_SHIP))
-    two_k = 1 << K_SHIP
-    def_sd = (major >= ((lo + two_k - 1) >> K_SHIP)) & (major <= (((hi + 1) >> K_SHIP) - 1))
+
+    def cand_def(kk):   # candidate / definite buckets of l_shipdate at granularity 2^kk
+        m = sd >> kk
+        c = (m >= (lo >> kk)) & (m <= (hi >> kk))
+        d = (m >= ((lo + (1 << kk) - 1) >> kk)) & (m <= (((hi + 1) >> kk) - 1))
+        return c, d
+
+    cand_sd, def_sd = cand_def(K_SHIP)
     other = (dc >= PREDS[1][0]) & (dc <= PREDS[1][1]) & (qt >= PREDS[2][0]) & (qt <= PREDS[2][1])
     cand = cand_sd & other
     nondef = cand & ~def_sd
     result = other & (sd >= lo) & (sd <= hi)
     idx_nd = np.nonzero(nondef)[0].astype(np.int64)
     idx_res = np.nonzero(result)[0].astype(np.int64)
-    # SLICED residual: a 32-row block's k planes are k * 4 B (one 32-B sector at k = 8)
-    res_sectors = np.unique((idx_nd // 32) * (K_SHIP * 4) // SECTOR).size
+    blk_nd = np.unique(idx_nd // 32)
+    if split:
+        kl = K_SHIP - split
+        cf, df = cand_def(kl)
+        blk_und = np.unique(np.nonzero(cf & ~df & other)[0].astype(np.int64) // 32)
+        lo_start = split_lo_byte(blk_und, split)
+        res_sectors = _sectors(lo_start, 4 * kl)
+        res64 = _sectors(lo_start, 4 * kl, 64)
+        if high_streamed:
+            scan += rows * split / 8.0
+        else:
+            hi_start = split_hi_byte(blk_nd, split)
+            res_sectors += _sectors(hi_start, 4 * split)
+            res64 += _sectors(hi_start, 4 * split, 64)
+    else:
+        # SLICED residual: a 32-row block's k planes are k * 4 B (one 32-B sector at k = 8)
+        res_sectors = np.unique(blk_nd * (K_SHIP * 4) // SECTOR).size
+        res64 = np.unique(blk_nd * (K_SHIP * 4) // 64).size
     b0 = idx_res * w_ep                                   # a packed 24-bit value may straddle two sectors
     ep_sectors = np.unique(np.concatenate([b0 // (SECTOR * 8), (b0 + w_ep - 1) // (SECTOR * 8)])).size
     gathered = min(rows * K_SHIP / 8.0, SECTOR * res_sectors) + min(rows * w_ep / 8.0, SECTOR * ep_sectors)
     ncand = int(cand.sum())
-    res64 = np.unique((idx_nd // 32) * (K_SHIP * 4) // 64).size
     ep64 = np.unique(np.concatenate([b0 // (64 * 8), (b0 + w_ep - 1) // (64 * 8)])).size
     return {"scan": scan, "gather": gathered, "residual_gather": SECTOR * res_sectors,
             "ep_gather": SECTOR * ep_sectors, "zero_copy_64": 64.0 * (res64 + ep64),
             "residual_granules_64": 64.0 * res64, "residual_sectors": int(res_sectors), "ep_sectors": int(ep_sectors),
             "total": scan + gathered + 8.0, "n_cand": ncand, "n_def": int((cand & def_sd).sum()),
-            "n_result": int(result.sum()), "cand_list_bytes": 8.0 * ncand,
+            "n_result": int(result.sum()), "cand_list_bytes": 8.0 * ncand, "residual_split": split,
             "widths": {"shipdate_major": w_sd, "discount": w_dc, "quantity": w_qt, "extprice": w_ep}}
 
 
@@ -460,11 +504,11 @@ class Ctx:
 class Q6:
     """One rank's decomposed Q6 columns and the query's predicate / aggregate handles."""
 
-    def __init__(self, ctx, cols, residual_loc=0):
+    def __init__(self, ctx, cols, residual_loc=0, split=0):
         from paper_conf_icde_pirkmk14_b200 import _ar, column as cu
         agree = ctx.allreduce_max_int          # the table's global w_M per column (allreduce-MAX)
         self.sd = cu.BWDColumn(cols["shipdate"], 32 - K_SHIP, residual_loc=residual_loc, device=ctx.dev,
-                               width_agree=agree)
+                               width_agree=agree, split=split)
         self.dc = cu.BWDColumn(cols["discount"], 32, device=ctx.dev, width_agree=agree)
         self.qt = cu.BWDColumn(cols["quantity"], 32, device=ctx.dev, width_agree=agree)
         self.ep = cu.BWDColumn(cols["extprice"], 32, layout=_ar.AR_LAYOUT_PACKED, device=ctx.dev, width_agree=agree)
@@ -707,11 +751,11 @@ def bench_c5(ctx, args):
         except Exception:
             old_aff = None
     cols = gen_columns(seed, table_sf, row0, rows)
-    q = Q6(ctx, cols, residual_loc=1)
+    q = Q6(ctx, cols, residual_loc=1, split=args.c5_split)
     link = measure_h2d(ctx)
     if old_aff:
         os.sched_setaffinity(0, old_aff)
-    ab = algorithmic_bytes(cols, q.sd.w_major)
+    ab = algorithmic_bytes(cols, q.sd.w_major, args.c5_split, high_streamed=False)
     r = Runner(ctx, q, max(3, min(args.steps, 10)))
     runs, kern, res, consistent = r.time_variant("fused", 2, 0)
     ms = runs[0] / r.K
@@ -729,7 +773,7 @@ def bench_c5(ctx, args):
                          "peak_source": "pinned->device cudaMemcpyAsync of 1 GiB on this GPU, best of 5, same run",
                          "algorithmic_host_bytes": host_bytes, "host_bytes_64B_granules": ab["residual_granules_64"]},
            "hbm": {"bytes": hbm_bytes, "gbs": hbm_bytes / (ms / 1e3) / 1e9},
-           "numa_node": node, "gpu_pci": bus, "pinned_on_node": bool(cpus),
+           "numa_node": node, "gpu_pci": bus, "pinned_on_node": bool(cpus), "residual_split": args.c5_split,
            "kernel": r.kernel_names("fused"), "parity": parity}
     del r
     q.free()
@@ -787,11 +831,11 @@ def ours(args):
     world, rank = ctx.world, ctx.rank
     seed, table_sf, table_rows, row0, rows = shard_of(args.workload, world, rank, args.scaling)
     cols = gen_columns(seed, table_sf, row0, rows)
-    q = Q6(ctx, cols)
+    q = Q6(ctx, cols, split=args.split)
     torch.cuda.synchronize()
     K = args.steps
     hbm_peak, peak_src = load_peaks()
-    ab = algorithmic_bytes(cols, q.sd.w_major)
+    ab = algorithmic_bytes(cols, q.sd.w_major, args.split)
     r = Runner(ctx, q, K)
     names = {"fused": r.kernel_names("fused"), "staged": None}
     names["staged"] = r.kernel_names("staged")
@@ -903,7 +947,9 @@ def ours(args):
 
     e2e = None
     if args.e2e_steps > 0:
-        e = run_e2e(ctx, q, ab, args.e2e_steps)
+        # the e2e path reads the residual over the host link (gathered high planes when split)
+        ab_e = ab if not args.split else algorithmic_bytes(cols, q.sd.w_major, args.split, high_streamed=False)
+        e = run_e2e(ctx, q, ab_e, args.e2e_steps)
         e2e = {"value": (table_rows if args.workload == "c4" and args.scaling == "strong" else rows * world)
                * e["steps"] / (e["ms_total"] / 1e3), "unit": UNIT,
                "h2d_bytes_per_step": int(e["h2d_copied"] + e["zero_copy_64"]), "d2h_bytes_per_step": 32,
@@ -922,8 +968,8 @@ def ours(args):
     if not args.only and not args.no_c2 and args.workload != "c2":
         seed2, sf2, trows2, r02, rows2 = shard_of("c2", world, rank)
         cols2 = gen_columns(seed2, sf2, r02, rows2)
-        q2 = Q6(ctx, cols2)
-        ab2 = algorithmic_bytes(cols2, q2.sd.w_major)
+        q2 = Q6(ctx, cols2, split=args.split)
+        ab2 = algorithmic_bytes(cols2, q2.sd.w_major, args.split)
         # C2 (345 MB per copy) is rotated over 3 copies of the decomposed columns so no step hits in L2
         copies = [q2] + [_copy_q6(ctx, q2) for _ in range(2)]
         r2 = RotRunner(ctx, copies, max(args.steps, 200))

@@ -102,7 +102,15 @@ typedef struct {
                                   d = v ^ 0x80000000: u = d - base, and
                                   predicate bounds of ar_pred are int32 bit patterns that
                                   the library maps the same way.  0: uint32 values, d = v. */
-    int32_t reserved;          /* 0 */
+    int32_t residual_split;    /* h, 0 <= h < k: 0 = one SLICED / PACKED residual part.  h > 0
+                                  (SLICED residuals, k <= 8) = the split layout: per
+                                  8192-row super-group (256 blocks of 32 rows) first the h
+                                  high residual planes of its 256 blocks (block-major, h
+                                  words per block: planes k-h .. k-1), then the k - h low
+                                  planes (k - h words per block: planes 0 .. k-h-1); so
+                                  the high bits of a block can be read without its low
+                                  bits (progressive refinement, DESIGN s6.3d).
+                                  residual_bytes = ceil(n / 8192) * 1024 * k.            */
 } ar_column_desc;
 
 typedef struct ar_column ar_column;   /* opaque: desc + part pointers (host object) */
@@ -176,7 +184,9 @@ size_t ar_decompose_ws_bytes(void);
  * of both parts.  SYNCHRONISES `stream` once (the sizing pass).
  * flags: AR_DECOMPOSE_SIGNED   -- int32 values (desc->value_signed);
  *        AR_DECOMPOSE_BASE_MIN -- prefix compression with base = min(d) (the
- *          frame of reference; `base` is ignored).
+ *          frame of reference; `base` is ignored);
+ *        AR_DECOMPOSE_SPLIT(h) -- 1 <= h < k <= 8: the residual in the split
+ *          layout (desc->residual_split = h; AR_ERR_INVALID otherwise).
  * `base` is in the key domain d (d = v ^ 0x80000000 for signed columns).
  * Errors: AR_ERR_INVALID if col == NULL && n > 0, n < 0, n >= 2^32,
  * major_bits outside [1,32], bad layout / location / flags, ws too small or
@@ -184,6 +194,7 @@ size_t ar_decompose_ws_bytes(void);
  */
 #define AR_DECOMPOSE_SIGNED 1
 #define AR_DECOMPOSE_BASE_MIN 2
+#define AR_DECOMPOSE_SPLIT(h) (((h) & 31) << 8)
 ar_status ar_decompose_plan(const uint32_t* col, int64_t n, int32_t major_bits,
                             int32_t major_layout, int32_t residual_loc, uint32_t base, int32_t flags,
                             void* ws, size_t ws_bytes, ar_column_desc* desc, void* stream);

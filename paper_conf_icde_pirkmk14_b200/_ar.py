@@ -18,6 +18,10 @@ AR_LAYOUT_SLICED, AR_LAYOUT_PACKED = 0, 1
 AR_MAX_PRED, AR_MAX_AGG, AR_MAX_PLANES = 8, 2, 64
 AR_SELECT_CARRY_APPR = 1
 AR_DECOMPOSE_SIGNED, AR_DECOMPOSE_BASE_MIN = 1, 2
+
+
+def AR_DECOMPOSE_SPLIT(h: int) -> int:
+    return (h & 31) << 8
 AR_AUX_DEFINITE = 0x80000000
 AR_PROJECT_APPROX, AR_PROJECT_EXACT = 0, 1
 AR_MIN, AR_MAX = 0, 1
@@ -41,7 +45,7 @@ class ColumnDesc(ctypes.Structure):
                 ("w_major", ctypes.c_int32), ("major_layout", ctypes.c_int32), ("residual_loc", ctypes.c_int32),
                 ("base", ctypes.c_uint32), ("major_bytes", ctypes.c_uint64), ("residual_bytes", ctypes.c_uint64),
                 ("major_loc", ctypes.c_int32), ("residual_layout", ctypes.c_int32),
-                ("value_signed", ctypes.c_int32), ("reserved", ctypes.c_int32)]
+                ("value_signed", ctypes.c_int32), ("residual_split", ctypes.c_int32)]
 
 
 class Pred(ctypes.Structure):

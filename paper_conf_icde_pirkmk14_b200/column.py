@@ -45,11 +45,12 @@ class BWDColumn:
     bounds are then int32 values); base="min" is the frame-of-reference prefix base min(key).
     width_agree: for a row shard of a larger table, a callable mapping this shard's planned stored
     width w_M to the table's (e.g. an allreduce-MAX over ranks); the descriptor is widened to it
-    (ar_decompose_set_width) so every shard shares one bucket geometry."""
+    (ar_decompose_set_width) so every shard shares one bucket geometry.
+    split=h: the residual in the split layout, its h high planes stored apart (AR_DECOMPOSE_SPLIT)."""
 
     def __init__(self, values, major_bits: int, layout: int = AR_LAYOUT_SLICED,
                  residual_loc: int = AR_LOC_DEVICE, base=0, signed: bool = False, device="cuda", stream=None,
-                 width_agree=None, _wrap=None):
+                 width_agree=None, split: int = 0, _wrap=None):
         self.device = torch.device(device)
         if _wrap is not None:
             self.desc, self.major, self.residual = _wrap
@@ -60,7 +61,8 @@ class BWDColumn:
         s = _stream(stream)
         ws = torch.empty(_ar.ar_decompose_ws_bytes(), dtype=torch.uint8, device=self.device)
         n = col.numel()
-        flags = (_ar.AR_DECOMPOSE_SIGNED if signed else 0) | (_ar.AR_DECOMPOSE_BASE_MIN if base == "min" else 0)
+        flags = (_ar.AR_DECOMPOSE_SIGNED if signed else 0) | (_ar.AR_DECOMPOSE_BASE_MIN if base == "min" else 0) \
+            | _ar.AR_DECOMPOSE_SPLIT(split)
         self.desc = _ar.ar_decompose_plan(col.data_ptr() if n else None, n, major_bits, layout, residual_loc,
                                           0 if base == "min" else int(base), flags, ws.data_ptr(), ws.numel(), s)
         if width_agree is not None:

@@ -184,7 +184,7 @@ ar_status ar_decompose_plan(const uint32_t* col, int64_t n, int32_t major_bits, 
     }
     if ((major_layout != AR_LAYOUT_SLICED && major_layout != AR_LAYOUT_PACKED) ||
         (residual_loc != AR_LOC_DEVICE && residual_loc != AR_LOC_HOST_PINNED) ||
-        (flags & ~(AR_DECOMPOSE_SIGNED | AR_DECOMPOSE_BASE_MIN)) != 0) {
+        (flags & ~(AR_DECOMPOSE_SIGNED | AR_DECOMPOSE_BASE_MIN | AR_DECOMPOSE_SPLIT(31))) != 0) {
         set_error("ar_decompose_plan: bad layout (%d), residual location (%d) or flags (%d)", major_layout,
                   residual_loc, flags);
         return AR_ERR_INVALID;
@@ -195,6 +195,11 @@ ar_status ar_decompose_plan(const uint32_t* col, int64_t n, int32_t major_bits, 
     }
     cudaStream_t s = (cudaStream_t)stream;
     const int k = 32 - major_bits;
+    const int split = (flags >> 8) & 31;
+    if (split && !(k <= 8 && split < k)) {
+        set_error("ar_decompose_plan: AR_DECOMPOSE_SPLIT(%d) needs 1 <= h < k <= 8 (k = %d)", split, k);
+        return AR_ERR_INVALID;
+    }
     const uint32_t flip = (flags & AR_DECOMPOSE_SIGNED) ? 0x80000000u : 0u;
     uint32_t mm[2] = {0u, 0xffffffffu};   // max(d), min(d)
     if (n > 0) {
@@ -223,7 +228,9 @@ ar_status ar_decompose_plan(const uint32_t* col, int64_t n, int32_t major_bits, 
     desc->base = base;
     desc->major_bytes = major_layout == AR_LAYOUT_SLICED ? sliced_bytes(n, w) : packed_bytes(n, w);
     desc->residual_layout = (k >= 1 && k <= 8) ? AR_LAYOUT_SLICED : AR_LAYOUT_PACKED;
-    desc->residual_bytes = desc->residual_layout == AR_LAYOUT_SLICED ? sliced_bytes(n, k) : packed_bytes(n, k);
+    desc->residual_split = split;
+    desc->residual_bytes = split ? split_bytes(n, k)
+                                 : (desc->residual_layout == AR_LAYOUT_SLICED ? sliced_bytes(n, k) : packed_bytes(n, k));
     desc->value_signed = flip ? 1 : 0;
     return AR_OK;
 }
@@ -252,7 +259,8 @@ static ar_status check_desc(const ar_column_desc* d) {
         (d->major_loc != AR_LOC_DEVICE && d->major_loc != AR_LOC_HOST_PINNED) ||
         (d->residual_layout != AR_LAYOUT_SLICED && d->residual_layout != AR_LAYOUT_PACKED) ||
         (d->residual_layout == AR_LAYOUT_SLICED && d->k > 8) ||
-        (d->value_signed != 0 && d->value_signed != 1) || d->reserved != 0) {
+        (d->value_signed != 0 && d->value_signed != 1) || d->residual_split < 0 ||
+        (d->residual_split > 0 && (d->residual_layout != AR_LAYOUT_SLICED || d->residual_split >= d->k))) {
         set_error("invalid ar_column_desc");
         return AR_ERR_INVALID;
     }
@@ -261,6 +269,7 @@ static ar_status check_desc(const ar_column_desc* d) {
     const uint64_t need_major = d->major_layout == AR_LAYOUT_SLICED ? sliced_bytes(d->n, d->w_major)
                                                                      : packed_bytes(d->n, d->w_major);
     const uint64_t need_res = d->k == 0 ? 0
+                              : d->residual_split ? split_bytes(d->n, d->k)
                               : (d->residual_layout == AR_LAYOUT_SLICED ? sliced_bytes(d->n, d->k)
                                                                         : packed_bytes(d->n, d->k));
     if (d->major_bytes < need_major || d->residual_bytes < need_res) {
@@ -348,7 +357,9 @@ ar_status ar_decompose(const uint32_t* col, const ar_column_desc* desc, void* ma
     }
     if (st == AR_OK && k > 0) {
         uint32_t* rdst = const_cast<uint32_t*>(c->residual);
-        if (desc->residual_layout == AR_LAYOUT_SLICED)
+        if (desc->residual_split)
+            st = launch_pack_split(col, n, k, desc->residual_split, flip, desc->base, rdst, s);
+        else if (desc->residual_layout == AR_LAYOUT_SLICED)
             st = launch_pack_sliced(col, n, 0, (1u << k) - 1u, flip, desc->base, k, rdst, s);
         else
             st = launch_pack_packed(col, n, 0, (1u << k) - 1u, flip, desc->base, k, desc->residual_bytes / 4, rdst,
@@ -452,9 +463,45 @@ static ar_status setup_scan(const ar_pred* preds, int32_t npred, ard::SelParams&
         p.base = col->d.base;
         p.lo = plo;
         p.hi = phi;
-        p.rlayout = (uint32_t)col->d.residual_layout;
+        p.rlayout = rlayout_code(col->d);
         p.res_host = col->d.residual_loc == AR_LOC_HOST_PINNED ? 1u : 0u;
         p.res_hint = 1u;
+        p.rsplit = (uint32_t)col->d.residual_split;
+        if (p.rsplit && !R.empty) {   // progressive refinement: the high residual planes refine the buckets to 2^(k-h)
+            const int kk = k - (int)p.rsplit, ww = w + (int)p.rsplit;
+            const Relaxed Rh = relax(plo, phi, col->d.base, kk, ww);
+            // Fine bucket U of a candidate that is not definite is clo or chi.  The definite bounds are
+            // chosen so that U < dlo <=> U == clo and U > dhi <=> U == chi on those rows (the check code of
+            // the result-ring kernel): the relaxation's when it has a definite bucket, else the empty
+            // [clo + 1, clo] (chi == clo + 1) or [clo + 1, clo - 1] (chi == clo); where clo + 1 or clo - 1
+            // leaves the w + h bits, that code bit is forced through scor.
+            const uint64_t maxf = ww >= 32 ? 0xffffffffull : ((1ull << ww) - 1);
+            uint64_t dlo = Rh.dlo, dhi = Rh.dhi;
+            p.scor = 0;
+            if (!Rh.def_any) {
+                dlo = (uint64_t)Rh.clo + 1;
+                if (dlo > maxf) {
+                    dlo = maxf;
+                    p.scor |= 1u;
+                }
+                if (Rh.chi == Rh.clo) {
+                    if (Rh.clo == 0) {
+                        dhi = 0;
+                        p.scor |= 2u;
+                    } else {
+                        dhi = (uint64_t)Rh.clo - 1;
+                    }
+                } else {
+                    dhi = Rh.clo;
+                }
+            }
+            for (int i = 0; i < ww && i < 32; ++i) {
+                P.pmh[c][i][0] = 0u - ((Rh.clo >> i) & 1u);
+                P.pmh[c][i][1] = 0u - ((Rh.chi >> i) & 1u);
+                P.pmh[c][i][2] = 0u - (uint32_t)((dlo >> i) & 1u);
+                P.pmh[c][i][3] = 0u - (uint32_t)((dhi >> i) & 1u);
+            }
+        }
         words += (P.tile_rows / 32) * (uint32_t)w;
         ashift += (uint32_t)w;
         // the one-pass kernel streams device-resident SLICED residual tiles (k <= 8) with the
@@ -466,7 +513,7 @@ static ar_status setup_scan(const ar_pred* preds, int32_t npred, ard::SelParams&
         // AR_RES_STREAM=0/1 forces the choice.
         bool stream_res = false;
         if (fused && k > 0 && col->d.residual_loc == AR_LOC_DEVICE && col->residual &&
-            col->d.residual_layout == AR_LAYOUT_SLICED && !R.empty) {
+            col->d.residual_layout == AR_LAYOUT_SLICED && col->d.residual_split == 0 && !R.empty) {
             static const int force = env_int("AR_RES_STREAM", -1);
             const double buckets = std::ldexp(1.0, w);
             const double nondef = (double)(R.chi - R.clo + 1) - (R.def_any ? (double)(R.dhi - R.dlo + 1) : 0.0);
@@ -477,6 +524,22 @@ static ar_status setup_scan(const ar_pred* preds, int32_t npred, ard::SelParams&
             p.res_stream = 1;
             p.res_soff = words;
             words += (P.tile_rows / 32) * (uint32_t)k;
+        }
+        // a split residual in HBM: the one-pass kernel streams its h high planes (the fine
+        // buckets decide most rows) and gathers the low planes of the rows they leave undecided
+        if (fused && p.rsplit && col->d.residual_loc == AR_LOC_DEVICE && col->residual && !R.empty &&
+            env_int("AR_SPLIT_STREAM", 1) != 0) {
+            const uint32_t kl = (uint32_t)k - p.rsplit;
+            const uint64_t maxu = (uint64_t)k + w >= 32 ? 0xffffffffull : ((1ull << (k + w)) - 1);
+            const uint64_t ulo = plo < col->d.base ? 0 : (uint64_t)(plo - col->d.base);
+            const uint64_t uhi = std::min<uint64_t>((uint64_t)(phi - col->d.base), maxu);
+            p.sflo = (uint32_t)(ulo >> kl);
+            p.sfhi = (uint32_t)(uhi >> kl);
+            p.sllo = (uint32_t)(ulo & ((1u << kl) - 1u));
+            p.slhi = (uint32_t)(uhi & ((1u << kl) - 1u));
+            p.res_stream = 1;
+            p.res_soff = words;
+            words += (P.tile_rows / 32) * p.rsplit;
         }
     }
     uint32_t planes = 0;
@@ -608,7 +671,7 @@ static ar_status setup_refine(const ar_cands* in, const ar_pred* preds, int32_t 
         const uint32_t flip = col->d.value_signed ? 0x80000000u : 0u;
         p.lo = preds[c].lo ^ flip;   // key domain
         p.hi = preds[c].hi ^ flip;
-        p.rlayout = (uint32_t)col->d.residual_layout;
+        p.rlayout = rlayout_code(col->d);
         p.ashift = ashift;
         p.carried = in->appr_bits > 0 ? 1u : 0u;
         p.check = col->d.k > 0 ? 1u : 0u;
@@ -695,7 +758,7 @@ static ar_status setup_aggs(const ar_column* const* cols, int32_t ncols, const a
         a[i].k = (uint32_t)c->d.k;
         a[i].layout = (uint32_t)c->d.major_layout;
         a[i].base = c->d.base;
-        a[i].rlayout = (uint32_t)c->d.residual_layout;
+        a[i].rlayout = rlayout_code(c->d);
         a[i].flip = c->d.value_signed ? 0x80000000u : 0u;
         if (c->d.value_signed && !allow_signed) {
             set_error("sum: aggregate column %d is signed; the unsigned product SUM does not apply", i);
@@ -999,6 +1062,18 @@ ar_status ar_select_refine_sum_ws(const ar_pred* preds, int32_t npred, const ar_
     }
     g_last_scan = "fused_kernel";
     if (ws) AR_TRY_CUDA(cudaMemsetAsync(out_dev, 0, 4 * sizeof(int64_t), s));   // fused_kernel accumulates
+    bool relay = false;   // fused_kernel gathers split residuals (it streams whole residual planes only)
+    for (int c = 0; c < P.npred; ++c)
+        if (P.p[c].rsplit && P.p[c].res_stream) {
+            P.p[c].res_stream = 0;
+            P.exact_mode = 0;
+            relay = true;
+        }
+    if (relay) {
+        const uint32_t tr = P.tile_rows;
+        P.tile_rows = 0;
+        retile(P, tr);
+    }
     int occ = 1;
     const void* fn = select_kernel_fn(P, true);
     P.nstages = pick_stages(fn, P.stage_words, true, &occ);

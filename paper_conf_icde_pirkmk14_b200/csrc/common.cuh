@@ -15,8 +15,12 @@
 struct ar_column {
     ar_column_desc d;
     const uint32_t* major;      // device pointer (SLICED or PACKED, width d.w_major)
-    const uint32_t* residual;   // device pointer, or device alias of pinned host memory (PACKED, width d.k)
+    const uint32_t* residual;   // device pointer, or device alias of pinned host memory (width d.k)
 };
+
+// Split SLICED residual: 32-row blocks per super-group (8192 rows, one default
+// one-pass tile, so a tile's high planes are one contiguous chunk).
+constexpr int kSplitBlocks = 256;
 
 // ------------------------------------------------------------------ host side
 
@@ -38,6 +42,16 @@ inline uint64_t ceil_div_u64(uint64_t a, uint64_t b) { return (a + b - 1) / b; }
 inline uint64_t sliced_bytes(int64_t n, int w) {
     return w == 0 ? 0 : ceil_div_u64((uint64_t)n, 128) * 16ull * (uint64_t)w;
 }
+// Split SLICED residual (k planes, h of them stored apart): super-groups of
+// kSplitBlocks 32-row blocks, each kSplitBlocks x k words.
+inline uint64_t split_bytes(int64_t n, int k) {
+    return k == 0 ? 0 : ceil_div_u64((uint64_t)n, 32ull * kSplitBlocks) * 4ull * kSplitBlocks * (uint64_t)k;
+}
+// Residual layout code carried to the kernels: ar_layout | (residual_split << 8).
+inline uint32_t rlayout_code(const ar_column_desc& d) {
+    return (uint32_t)d.residual_layout | ((uint32_t)d.residual_split << 8);
+}
+
 // Bytes of a PACKED bitstream of width w: ceil(n*w/32) words + 1 guard word
 // (a straddling value may read word i+1), rounded up to 16 B.
 inline uint64_t packed_bytes(int64_t n, int w) {
@@ -264,13 +278,36 @@ __device__ __forceinline__ uint32_t packed_get_if(const uint32_t* __restrict__ s
     const uint32_t v = __funnelshift_r(lo, hi, sh);
     return w == 32 ? v : (v & ((1u << w) - 1u));
 }
+// Split SLICED residual (layout code AR_LAYOUT_SLICED | h << 8).  Per
+// super-group of kSplitBlocks blocks: the h high planes of its blocks (h words
+// per block, planes k-h .. k-1), then the k - h low planes (k - h words per
+// block, planes 0 .. k-h-1).  So a tile's high planes are one contiguous chunk
+// (streamed) and a block's low planes are k - h consecutive words (gathered).
+__device__ __forceinline__ uint64_t split_hi_word(uint64_t blk, int k, int h) {   // plane k - h of block blk
+    return (blk / kSplitBlocks) * ((uint64_t)kSplitBlocks * k) + (blk % kSplitBlocks) * (uint64_t)h;
+}
+__device__ __forceinline__ uint64_t split_lo_word(uint64_t blk, int k, int h) {   // plane 0 of block blk
+    return (blk / kSplitBlocks) * ((uint64_t)kSplitBlocks * k) + (uint64_t)kSplitBlocks * h +
+           (blk % kSplitBlocks) * (uint64_t)(k - h);
+}
+// word of plane j (bit j of the residual, j < k) of 32-row block blk
+__device__ __forceinline__ uint64_t split_word(uint64_t blk, int k, int h, int j) {
+    return j >= k - h ? split_hi_word(blk, k, h) + (uint64_t)(j - (k - h)) : split_lo_word(blk, k, h) + (uint64_t)j;
+}
+
 // Residual of row p: SLICED blocks of k = 4 / 8 planes (16-B aligned) in one or
-// two vector loads of the block's sector, other widths word by word.
+// two vector loads of the block's sector, other widths (and the split layout)
+// word by word.
 __device__ __forceinline__ uint32_t residual_get_if(const uint32_t* s, uint64_t p, int k, int layout, bool pred) {
-    if (layout != AR_LAYOUT_SLICED) return packed_get_if(s, p, k, pred);
-    const uint32_t* blk = s + (p >> 5) * (uint64_t)k;
+    if ((layout & 0xff) != AR_LAYOUT_SLICED) return packed_get_if(s, p, k, pred);
     const uint32_t l = (uint32_t)(p & 31);
     uint32_t r = 0;
+    const int h = layout >> 8;
+    if (h) {
+        for (int j = 0; j < k; ++j) r |= ((ld_gather_if(s + split_word(p >> 5, k, h, j), pred) >> l) & 1u) << j;
+        return r;
+    }
+    const uint32_t* blk = s + (p >> 5) * (uint64_t)k;
     if (k == 8 || k == 4) {
         const uint4 a = ld_gather_if4(blk, pred);
         r = ((a.x >> l) & 1u) | (((a.y >> l) & 1u) << 1) | (((a.z >> l) & 1u) << 2) | (((a.w >> l) & 1u) << 3);
@@ -295,14 +332,19 @@ __device__ __forceinline__ uint32_t packed_get(const uint32_t* __restrict__ s, u
     if (sh + (uint32_t)w > 32u) v = __funnelshift_r(lo, ld_gather(s + wi + 1), sh);
     return w == 32 ? v : (v & ((1u << w) - 1u));
 }
-// Residual of row p (width k) in either layout, from device memory or from
+// Residual of row p (width k) in any layout, from device memory or from
 // pinned host memory through a mapped pointer.  SLICED (k <= 8): the block's k
-// planes sit in one 32-B sector.
+// planes sit in one 32-B sector; split: its high and low planes in two places.
 __device__ __forceinline__ uint32_t residual_get(const uint32_t* s, uint64_t p, int k, int layout) {
-    if (layout == AR_LAYOUT_SLICED) {
-        const uint32_t* blk = s + (p >> 5) * (uint64_t)k;
+    if ((layout & 0xff) == AR_LAYOUT_SLICED) {
         const uint32_t l = (uint32_t)(p & 31);
+        const int h = layout >> 8;
         uint32_t r = 0;
+        if (h) {
+            for (int j = 0; j < k; ++j) r |= ((ld_gather(s + split_word(p >> 5, k, h, j)) >> l) & 1u) << j;
+            return r;
+        }
+        const uint32_t* blk = s + (p >> 5) * (uint64_t)k;
         for (int j = 0; j < k; ++j) r |= ((ld_gather(blk + j) >> l) & 1u) << j;
         return r;
     }

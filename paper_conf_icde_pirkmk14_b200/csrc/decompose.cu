@@ -68,9 +68,38 @@ __global__ void pack_packed_kernel(const uint32_t* __restrict__ col, int64_t n, 
     }
 }
 
+// Split SLICED residual (k <= 8 planes, h high planes apart): one warp per
+// 32-row block b; plane j (bit j of the residual) goes to its super-group's
+// high-plane area (j >= k - h) or low-plane area.
+__global__ void pack_split_kernel(const uint32_t* __restrict__ col, int64_t n, int k, int h, uint32_t flip,
+                                  uint32_t base, int64_t nblocks, uint32_t* __restrict__ out) {
+    const unsigned lane = threadIdx.x & 31;
+    const int64_t warps = (int64_t)gridDim.x * (blockDim.x / 32);
+    for (int64_t b = (int64_t)blockIdx.x * (blockDim.x / 32) + (threadIdx.x >> 5); b < nblocks; b += warps) {
+        const int64_t row = b * 32 + lane;
+        const uint32_t r = row < n ? (((col[row] ^ flip) - base) & ((1u << k) - 1u)) : 0u;
+        uint32_t mine = 0;
+        for (int j = 0; j < k; ++j) {
+            const uint32_t plane = __ballot_sync(0xffffffffu, (r >> j) & 1u);
+            if ((int)lane == j) mine = plane;
+        }
+        if ((int)lane < k) out[split_word((uint64_t)b, k, h, (int)lane)] = mine;
+    }
+}
+
 }  // namespace ard
 
 namespace ar {
+
+ar_status launch_pack_split(const uint32_t* col, int64_t n, int k, int h, uint32_t flip, uint32_t base, uint32_t* out,
+                            cudaStream_t s) {
+    const int64_t nblocks = (int64_t)ceil_div_u64((uint64_t)n, 32ull * kSplitBlocks) * kSplitBlocks;   // whole super-groups (padding zeroed)
+    if (nblocks == 0) return AR_OK;
+    int grid = (int)std::min<int64_t>((nblocks + 7) / 8, (int64_t)num_sms() * 16);
+    ard::pack_split_kernel<<<grid, 256, 0, s>>>(col, n, k, h, flip, base, nblocks, out);
+    AR_CHECK_LAUNCH("pack_split_kernel");
+    return AR_OK;
+}
 
 ar_status launch_decompose_minmax(const uint32_t* col, int64_t n, uint32_t flip, uint32_t* out2, cudaStream_t s) {
     int grid = (int)std::min<int64_t>((n + 255) / 256, (int64_t)num_sms() * 8);

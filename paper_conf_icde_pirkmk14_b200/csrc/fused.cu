@@ -31,6 +31,8 @@ namespace rl {
 constexpr int kRingDefault = 128;         // result entries (row, factor) per warp (power of two)
 constexpr int kDepth = 4;                 // gather passes in flight per warp
 constexpr int kSlotWords = 4 * 32;        // per pass: lo[32], hi[32], info[32], factor[32]
+// + with a split residual, the KL gathered low-plane words of each lane's row
+__host__ __device__ constexpr int slot_words(int kl) { return kSlotWords + 32 * kl; }
 
 // Exact value of predicate C's column at row l of block blk, from the stage.
 template <class S, int C>
@@ -50,15 +52,41 @@ __device__ __forceinline__ uint32_t stage_value(const SelParams& P, const uint32
 __device__ __forceinline__ void cp_async4(uint32_t* dst, const uint32_t* src) {
     asm volatile("cp.async.ca.shared.global" AR_GHINT " [%0], [%1], 4;" ::"r"(smem_u32(dst)), "l"(src) : "memory");
 }
+__device__ __forceinline__ void cp_async16(uint32_t* dst, const uint32_t* src) {
+    asm volatile("cp.async.cg.shared.global" AR_GHINT " [%0], [%1], 16;" ::"r"(smem_u32(dst)), "l"(src) : "memory");
+}
 __device__ __forceinline__ void cp_async_commit() { asm volatile("cp.async.commit_group;" ::: "memory"); }
 template <int N>
 __device__ __forceinline__ void cp_async_wait() { asm volatile("cp.async.wait_group %0;" ::"n"(N) : "memory"); }
 
+// Low-plane word j of lane `lane` in a slot (KL = 4: one 16-B copy per lane).
+template <int KL>
+__device__ __forceinline__ uint32_t* low_word(uint32_t* sl, uint32_t lane, int j) {
+    return KL == 4 ? sl + kSlotWords + lane * 4 + j : sl + kSlotWords + j * 32 + lane;
+}
+
 // Sum one landed gather slot: this lane's entry (a lane only reads what it copied).
-__device__ __forceinline__ unsigned long long drain(const uint32_t* sl, uint32_t lane, uint32_t gmask,
-                                                    uint32_t gbase) {
+// KL > 0: an entry with a check code (info bits 8-9; bit 0: the row lies in the
+// fine bucket of lo, bit 1: in that of hi) is a row the high residual planes
+// left undecided; its KL low planes (landed with the aggregate) decide it
+// against the low bits of the exact bounds, and a row that qualifies counts
+// in `nchk`.
+template <int KL = 0>
+__device__ __forceinline__ unsigned long long drain(uint32_t* sl, uint32_t lane, uint32_t gmask, uint32_t gbase,
+                                                    const SelPred* sp = nullptr, uint32_t* nchk = nullptr) {
     const uint32_t info = sl[64 + lane];
     if (!(info >> 31)) return 0ull;
+    if constexpr (KL > 0) {
+        const uint32_t code = (info >> 8) & 3u;
+        if (code) {
+            const uint32_t l = (info >> 10) & 31u;
+            uint32_t low = 0;
+#pragma unroll
+            for (int j = 0; j < KL; ++j) low |= ((*low_word<KL>(sl, lane, j) >> l) & 1u) << j;
+            if (((code & 1u) && low < sp->sllo) || ((code & 2u) && low > sp->slhi)) return 0ull;
+            ++*nchk;
+        }
+    }
     // bits of the hi word past the value's width are masked off, so a slot whose
     // value did not straddle (hi word not copied) reads harmless stale data
     const uint32_t v = (__funnelshift_r(sl[lane], sl[32 + lane], info & 31u) & gmask) + gbase;
@@ -130,6 +158,9 @@ template <int NW, int BPT, int... WK>
 __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid_constant__ SelParams P) {
     using S = typename ShapeOf<WK...>::type;
     constexpr int NT = NW * 32;
+    // a split residual (one predicate SP): its high planes are in the stage, its KL low planes are
+    // gathered with the aggregate for the rows they decide
+    constexpr int SP = S::split(), KL = S::kl(), SPi = SP < 0 ? 0 : SP, SW = slot_words(KL);
     extern __shared__ __align__(128) unsigned char smem[];
     uint64_t* full = reinterpret_cast<uint64_t*>(smem);
     uint64_t* empty = full + P.nstages;
@@ -139,8 +170,9 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
     const unsigned warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     const uint32_t kRing = P.rl_ring, rmask = kRing - 1;
     uint2* ring = reinterpret_cast<uint2*>(stages + (size_t)P.nstages * P.stage_words) + warp * kRing;
-    uint32_t* gs = reinterpret_cast<uint32_t*>(reinterpret_cast<uint2*>(stages + (size_t)P.nstages * P.stage_words) +
-                                               NW * kRing) + warp * (kDepth * kSlotWords);
+    uint32_t* gs0 = reinterpret_cast<uint32_t*>(reinterpret_cast<uint2*>(stages + (size_t)P.nstages * P.stage_words) +
+                                                NW * kRing);
+    uint32_t* gs = gs0 + warp * (kDepth * SW);
     if (threadIdx.x == 0) {
         for (uint32_t s = 0; s < P.nstages; ++s) {
             mbar_init(full + s, 1);
@@ -163,16 +195,17 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
     const bool direct = !list && P.nagg > 0;
     const AggCol& G = P.a[P.gidx];
     const uint32_t gmask = G.w >= 32 ? 0xffffffffu : ((1u << G.w) - 1u);
-    uint32_t ncand = 0, ndef = 0, nres = 0;
+    uint32_t ncand = 0, ndef = 0, nres = 0, nchk = 0;
     unsigned long long sum = 0;
     uint32_t rhead = 0, rcnt = 0, gseq = 0;   // warp-uniform ring head / fill and gather passes issued
 
     // One gather pass over the `take` oldest ring entries (take <= 32).
     auto pass = [&](uint32_t take) {
-        uint32_t* sl = gs + (gseq % kDepth) * kSlotWords;
+        uint32_t* sl = gs + (gseq % kDepth) * SW;
         uint32_t info = 0u, f = 0u;
         if (lane < take) {
-            const uint2 e = ring[(rhead + lane) & rmask];
+            const uint32_t ri = (rhead + lane) & rmask;
+            const uint2 e = ring[ri];
             const uint64_t bit = (uint64_t)e.x * G.w;
             const uint32_t* src = G.major + (bit >> 5);
             const uint32_t sh = (uint32_t)(bit & 31);
@@ -180,6 +213,21 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
             if (sh + G.w > 32u) cp_async4(sl + 32 + lane, src + 1);
             info = 0x80000000u | sh;
             f = e.y;
+            if constexpr (KL > 0) {
+                // the check code rides in the top two bits of the factor (host: factors < 2^30)
+                const uint32_t code = e.y >> 30;
+                f = e.y & 0x3fffffffu;
+                if (code) {   // an undecided row: its low residual planes travel with the aggregate
+                    const uint32_t* lp = P.p[SPi].residual + split_lo_word(e.x >> 5, S::k(SPi), S::h(SPi));
+                    if constexpr (KL == 4) {
+                        cp_async16(low_word<KL>(sl, lane, 0), lp);
+                    } else {
+#pragma unroll
+                        for (int j = 0; j < KL; ++j) cp_async4(low_word<KL>(sl, lane, j), lp + j);
+                    }
+                    info |= (code << 8) | ((e.x & 31u) << 10);
+                }
+            }
         }
         sl[64 + lane] = info;
         sl[96 + lane] = f;
@@ -189,7 +237,7 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
         rcnt -= take;
         if (gseq >= (uint32_t)kDepth) {   // sum the pass issued kDepth - 1 passes ago
             cp_async_wait<kDepth - 1>();
-            sum += drain(gs + (gseq % kDepth) * kSlotWords, lane, gmask, G.base);
+            sum += drain<KL>(gs + (gseq % kDepth) * SW, lane, gmask, G.base, &P.p[SPi], &nchk);
         }
     };
 
@@ -208,21 +256,36 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
         const bool full_tile = tile_r0 + (int64_t)P.tile_rows <= P.n;
 
         // a3 + a5: candidate, definite and exact masks of this thread's blocks
-        uint32_t xm[BPT];
+        // result rows (incl. undecided ones); split residual: the undecided rows in the fine bucket
+        // of the lower bound (k0) / of the upper bound (k1) -- the check code, bits 30 / 31 of the entry
+        uint32_t xm[BPT], k0[BPT], k1[BPT];
 #pragma unroll
         for (int b = 0; b < BPT; ++b) {
             const uint32_t blk = b * NT + threadIdx.x;
             const uint32_t vm = full_tile ? 0xffffffffu : valid_mask(tile_r0 + 32 * (int64_t)blk, P.n);
-            uint32_t cm, dm, em;
+            uint32_t cm, dm, em, ul = 0u, uh = 0u;
             if constexpr (S::kDynamic)
                 eval_block_dyn(P, stg, blk, vm, cm, dm, em);
             else
-                eval_block<S, true>(P, stg, blk, vm, cm, dm, em);
+                eval_block<S, true>(P, stg, blk, vm, cm, dm, em, ul, uh);
             ncand += __popc(cm);
             ndef += __popc(dm);
-            nres += __popc(em);
+            const uint32_t xk = em & (ul | uh);
+            nres += __popc(em & ~xk);
             xm[b] = em;
+            if constexpr (KL > 0) {
+                k0[b] = xk & (ul | (0u - (P.p[SPi].scor & 1u)));
+                k1[b] = xk & (uh | (0u - ((P.p[SPi].scor >> 1) & 1u)));
+            } else {
+                k0[b] = k1[b] = 0u;
+            }
         }
+        auto code_at = [&](int b, uint32_t l) -> uint32_t {   // check code << 30 of row l of block b
+            if constexpr (KL > 0)
+                return (((k0[b] >> l) & 1u) << 30) | (((k1[b] >> l) & 1u) << 31);
+            else
+                return 0u;
+        };
 
         if (direct) {
             // a6 without gathers: every factor is a predicate column, its value is in the stage
@@ -274,7 +337,7 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
                             do {
                                 const uint32_t l = __ffs(m) - 1;
                                 m &= m - 1;
-                                ring[(wbase + e) & rmask] = make_uint2(row0 + l, 1u);
+                                ring[(wbase + e) & rmask] = make_uint2(row0 + l, 1u | code_at(b, l));
                                 ++e;
                             } while (m && e < lim);
                         } else if constexpr (S::kDynamic) {
@@ -291,6 +354,7 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
                                 if (C != P.rl_mpred) return;
                                 uint32_t x[W];
                                 lds_words<W>(x, stg + P.p[C].soff + blk * W);
+                                if constexpr (S::h(C) > 0) return;   // never the split column (host-checked)
                                 uint32_t r[K > 0 ? K : 1];
                                 if constexpr (K > 0) lds_words<K>(r, stg + P.p[C].res_soff + blk * K);
                                 do {
@@ -298,7 +362,7 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
                                     m &= m - 1;
                                     uint32_t v = row_of<W>(x, l);
                                     if constexpr (K > 0) v = (v << K) | row_of<K>(r, l);
-                                    ring[(wbase + e) & rmask] = make_uint2(row0 + l, v + P.p[C].base);
+                                    ring[(wbase + e) & rmask] = make_uint2(row0 + l, (v + P.p[C].base) | code_at(b, l));
                                     ++e;
                                 } while (m && e < lim);
                             });
@@ -326,10 +390,10 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
         while (rcnt > 0) pass(min(rcnt, 32u));
         cp_async_wait<0>();
         for (uint32_t g = gseq >= (uint32_t)kDepth ? gseq - kDepth + 1 : 0; g < gseq; ++g)
-            sum += drain(gs + (g % kDepth) * kSlotWords, lane, gmask, G.base);
+            sum += drain<KL>(gs + (g % kDepth) * SW, lane, gmask, G.base, &P.p[SPi], &nchk);
     }
 
-    unsigned long long c0 = ncand, c1 = ndef, c2 = nres;
+    unsigned long long c0 = ncand, c1 = ndef, c2 = nres + nchk;
 #pragma unroll
     for (int o = 16; o > 0; o >>= 1) {
         sum += __shfl_xor_sync(0xffffffffu, sum, o);
@@ -534,6 +598,39 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
                     if constexpr (K > 0) {
                         uint32_t x[W];
                         lds_words<W>(x, stg + P.p[C].soff + blk * W);
+                        const uint32_t H = P.p[C].rsplit;
+                        uint32_t dp = 0u;
+                        if (H) {
+                            // split layout: the high planes (gathered in phase A) refine the bucket to 2^(k-h)
+                            // values; rows decided there need no low planes, the rest gather them now
+                            uint32_t cl = 0, ch = 0, dl = 0, dh = 0;
+#pragma unroll
+                            for (int j = 0; j < K; ++j) {
+                                if (j < K - (int)H) continue;
+                                const uint32_t i = j - (K - H);
+                                cl = bsub(rres[b][KO + j], P.pmh[C][i][0], cl);
+                                ch = brsub(rres[b][KO + j], P.pmh[C][i][1], ch);
+                                dl = bsub(rres[b][KO + j], P.pmh[C][i][2], dl);
+                                dh = brsub(rres[b][KO + j], P.pmh[C][i][3], dh);
+                            }
+#pragma unroll
+                            for (int j = 0; j < W; ++j) {
+                                cl = bsub(x[j], P.pmh[C][H + j][0], cl);
+                                ch = brsub(x[j], P.pmh[C][H + j][1], ch);
+                                dl = bsub(x[j], P.pmh[C][H + j][2], dl);
+                                dh = brsub(x[j], P.pmh[C][H + j][3], dh);
+                            }
+                            dp = em & ~(dl | dh);
+                            em &= ~(cl | ch) & (dl | dh);   // still undecided
+                            const uint64_t gblk = (uint64_t)(r0 >> 5) + blk;
+                            const uint32_t* lo = P.p[C].residual + split_lo_word(gblk, K, (int)H);
+#pragma unroll
+                            for (int j = 0; j < K; ++j) {
+                                if (j >= K - (int)H) continue;
+                                rres[b][KO + j] = P.p[C].res_hint ? ld_gather_if(lo + j, em != 0u)
+                                                                  : ld_gather_if_nh(lo + j, em != 0u);
+                            }
+                        }
                         uint32_t el = 0, eh = 0;
 #pragma unroll
                         for (int j = 0; j < K; ++j) {
@@ -545,7 +642,7 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
                             el = bsub(x[j], P.pmx[C][K + j][0], el);
                             eh = brsub(x[j], P.pmx[C][K + j][1], eh);
                         }
-                        em &= ~(el | eh);
+                        em = dp | (em & ~(el | eh));
                     }
                 });
             }
@@ -572,7 +669,8 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
             const uint32_t blk = b * NT + threadIdx.x;
             const uint32_t vm = full_tile ? 0xffffffffu : valid_mask(tile_r0 + 32 * (int64_t)blk, P.n);
             uint32_t cm, dm, em;
-            eval_block<S, false>(P, stg, blk, vm, cm, dm, em);
+            uint32_t ul, uh;
+            eval_block<S, false>(P, stg, blk, vm, cm, dm, em, ul, uh);
             ncand += __popc(cm);
             ndef += __popc(dm);
             dmk[b] = dm;
@@ -587,8 +685,21 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
                 static_for<S::N>([&](auto cc) {
                     constexpr int C = decltype(cc)::value;
                     constexpr int K = S::k(C), KO = S::kofs(C);
-                    if constexpr (K > 0)
-                        res_issue<K>(&rres[b][KO], P.p[C].residual, gblk, ndm[b] != 0u, P.p[C].res_hint != 0u);
+                    if constexpr (K > 0) {
+                        const uint32_t H = P.p[C].rsplit;
+                        if (H == 0) {
+                            res_issue<K>(&rres[b][KO], P.p[C].residual, gblk, ndm[b] != 0u, P.p[C].res_hint != 0u);
+                        } else {   // split layout: only the block's h high planes now
+                            const uint32_t* hp = P.p[C].residual + split_hi_word(gblk, K, (int)H);
+                            const bool hint = P.p[C].res_hint != 0u;
+#pragma unroll
+                            for (int j = 0; j < K; ++j) {
+                                if (j < K - (int)H) continue;
+                                const uint32_t* q = hp + (j - (K - H));
+                                rres[b][KO + j] = hint ? ld_gather_if(q, ndm[b] != 0u) : ld_gather_if_nh(q, ndm[b] != 0u);
+                            }
+                        }
+                    }
                 });
                 pnd[b] = ndm[b];
             }
@@ -643,9 +754,9 @@ void retile(ard::SelParams& P, uint32_t tile_rows) {
     for (int c = 0; c < P.npred; ++c) {
         P.p[c].soff = words;
         words += (tile_rows / 32) * P.p[c].w;
-        if (P.p[c].res_stream) {
+        if (P.p[c].res_stream) {   // residual planes (a split residual: its high planes)
             P.p[c].res_soff = words;
-            words += (tile_rows / 32) * P.p[c].k;
+            words += (tile_rows / 32) * (P.p[c].rsplit ? P.p[c].rsplit : P.p[c].k);
         }
     }
     P.stage_words = std::max<uint32_t>(words, 4);
@@ -655,6 +766,25 @@ void retile(ard::SelParams& P, uint32_t tile_rows) {
 namespace {
 
 constexpr int WK(int w, int k) { return (w << 6) | k; }
+constexpr int WKH(int w, int k, int h) { return (h << 12) | (w << 6) | k; }   // split residual, h planes streamed
+
+// shape key of predicate c as the result-ring kernel sees it
+inline int rl_key(const ard::SelPred& p) {
+    if (!p.res_stream) return (int)(p.w << 6);
+    return (int)((p.rsplit << 12) | (p.w << 6) | p.k);
+}
+// the predicate whose split residual is streamed (at most one), or -1; its low planes per row
+inline int rl_split(const ard::SelParams& P, uint32_t* kl) {
+    int sp = -1;
+    *kl = 0;
+    for (int c = 0; c < P.npred; ++c)
+        if (P.p[c].res_stream && P.p[c].rsplit) {
+            if (sp >= 0) return -2;
+            sp = c;
+            *kl = P.p[c].k - P.p[c].rsplit;
+        }
+    return sp;
+}
 
 struct RlFn {
     const void* fn;
@@ -692,10 +822,8 @@ bool rl_match(const ard::SelParams& P) {
     constexpr int n = sizeof...(Ws);
     constexpr int wk[] = {Ws..., 0};
     if (P.npred != n) return false;
-    for (int c = 0; c < n; ++c) {
-        const uint32_t k = P.p[c].res_stream ? P.p[c].k : 0u;
-        if ((int)((P.p[c].w << 6) | k) != wk[c]) return false;
-    }
+    for (int c = 0; c < n; ++c)
+        if (rl_key(P.p[c]) != wk[c]) return false;
     return true;
 }
 
@@ -727,6 +855,9 @@ RlFn rl_find(const ard::SelParams& P, int cfg) {
 #define AR_RL_TRY(...) \
     if (rl_match<__VA_ARGS__>(P)) return rl_pick<__VA_ARGS__>(cfg);
     AR_RL_TRY(WK(4, 8), WK(4, 0), WK(6, 0))
+    AR_RL_TRY(WKH(4, 8, 4), WK(4, 0), WK(6, 0))
+    AR_RL_TRY(WKH(4, 8, 3), WK(4, 0), WK(6, 0))
+    AR_RL_TRY(WKH(4, 8, 2), WK(4, 0), WK(6, 0))
     AR_RL_TRY(WK(24, 8))
     AR_RL_TRY(WK(8, 0))
     AR_RL_TRY(WK(16, 0))
@@ -734,9 +865,11 @@ RlFn rl_find(const ard::SelParams& P, int cfg) {
     AR_RL_TRY(WK(32, 0))
     AR_RL_TRY(WK(24, 8), WK(24, 8))
 #undef AR_RL_TRY
-    // any other decomposition: the runtime-shape kernel (widths and bounds from the parameters)
+    // any other decomposition: the runtime-shape kernel (widths and bounds from the parameters;
+    // not for streamed split residuals)
     static const bool no_dyn = getenv("AR_RL_NODYN") && atoi(getenv("AR_RL_NODYN"));
-    if (!no_dyn) return rl_pick<-1>(cfg);
+    uint32_t kl;
+    if (!no_dyn && rl_split(P, &kl) == -1) return rl_pick<-1>(cfg);
     return {nullptr, 0, 0};
 }
 
@@ -759,10 +892,12 @@ int env_ring() {
     return v;
 }
 
-size_t rl_smem_bytes(const ard::SelParams& P, uint32_t nstages, int nw) {
+size_t rl_smem_bytes(const ard::SelParams& P, uint32_t nstages, int nw, bool rg) {
     const size_t head = ((size_t)nstages * 24 + 127) & ~size_t(127);
+    uint32_t kl = 0;
+    if (!rg) rl_split(P, &kl);
     return head + (size_t)nstages * P.stage_words * 4 + (size_t)nw * P.rl_ring * 8 +
-           (size_t)nw * ard::rl::kDepth * ard::rl::kSlotWords * 4;
+           (size_t)nw * ard::rl::kDepth * ard::rl::slot_words((int)kl) * 4;
 }
 
 }  // namespace
@@ -811,13 +946,20 @@ ar_status launch_fused_rl(const ard::SelParams& P0, const ar_column* const* cols
     // pinned host memory); factors as above with k = 0 predicate columns
     bool rg_ok = fac_k0;
     for (int c = 0; c < P.npred && rg_ok; ++c)
-        if (P.p[c].k > 0) rg_ok = P.p[c].rlayout == AR_LAYOUT_SLICED && P.p[c].residual != nullptr && P.p[c].k <= 8;
+        if (P.p[c].k > 0)
+            rg_ok = (P.p[c].rlayout & 0xffu) == AR_LAYOUT_SLICED && P.p[c].residual != nullptr && P.p[c].k <= 8;
     RlFn k{nullptr, 0, 0};
     bool rg = false;
     // streamed residual planes first (device residuals: a stream of every block's planes beats
     // gathering the touched sectors, DESIGN s6.3c), the gathered-residual kernel otherwise (residuals
     // in pinned host memory, or the stream heuristic said no)
-    const bool rl_ok = P.exact_mode != 0;
+    // a streamed split residual needs the result ring (its undecided rows travel with the gathered
+    // aggregate) and must not be the other SUM factor
+    uint32_t kl = 0;
+    const int sp = rl_split(P, &kl);
+    // (the check code rides in the top bits of the other factor, so that factor must stay below 2^30)
+    const bool mp_small = P.rl_mpred < 0 || (P.p[P.rl_mpred].base == 0 && P.p[P.rl_mpred].w + P.p[P.rl_mpred].k <= 30);
+    const bool rl_ok = P.exact_mode != 0 && sp != -2 && (sp < 0 || (P.rl_list && P.rl_mpred != sp && mp_small));
     if (rl_ok && resmode != 2) k = rl_find(P, env_cfg());
     if (!k.fn && rg_ok) {
         ard::SelParams Q = P;
@@ -851,7 +993,7 @@ ar_status launch_fused_rl(const ard::SelParams& P0, const ar_column* const* cols
             // the two-phase kernel holds two stages (phase B of tile t - 1 while tile t is decided)
             if (target >= 2 && st < (rg ? 4u : 3u) && force_st <= 0) break;
             int o = 0;
-            cudaOccupancyMaxActiveBlocksPerMultiprocessor(&o, k.fn, threads, rl_smem_bytes(P, st, k.nw));
+            cudaOccupancyMaxActiveBlocksPerMultiprocessor(&o, k.fn, threads, rl_smem_bytes(P, st, k.nw, rg));
             if (o >= target) {
                 stages = st;
                 occ = o;
@@ -867,7 +1009,7 @@ ar_status launch_fused_rl(const ard::SelParams& P0, const ar_column* const* cols
     cudaLaunchConfig_t cfg = {};
     cfg.gridDim = dim3(grid);
     cfg.blockDim = dim3(threads);
-    cfg.dynamicSmemBytes = rl_smem_bytes(P, stages, k.nw);
+    cfg.dynamicSmemBytes = rl_smem_bytes(P, stages, k.nw, rg);
     cfg.stream = s;
     cudaLaunchAttribute attr[1];
     attr[0].id = cudaLaunchAttributeProgrammaticStreamSerialization;

@@ -135,7 +135,7 @@ ar_status ar_group_ids(const ar_positions* rows, const ar_column* key, int32_t m
     P.key.k = (uint32_t)key->d.k;
     P.key.layout = (uint32_t)key->d.major_layout;
     P.key.base = key->d.base;
-    P.key.rlayout = (uint32_t)key->d.residual_layout;
+    P.key.rlayout = rlayout_code(key->d);
     P.key.flip = key->d.value_signed ? 0x80000000u : 0u;
     P.key.pred = -1;
     P.exact = (mode == AR_GROUP_EXACT && key->d.k > 0) ? 1 : 0;

@@ -21,6 +21,11 @@ struct SelPred {
     uint32_t res_soff;        // word offset of the streamed residual tile inside a stage
     uint32_t res_host;        // residual in pinned host memory (read over the host link)
     uint32_t res_hint;        // gathered-residual kernel: use the .L2::64B prefetch-size hint
+    uint32_t rsplit;          // split residual layout: h high planes stored apart (0: not split)
+    // split residual with its high planes streamed (result-ring kernel): the fine buckets
+    // (u >> (k - h)) of the exact bounds and the low k - h bits of the bounds, u = v - base
+    uint32_t sflo, sfhi, sllo, slhi;
+    uint32_t scor;            // check-code bits forced on every undecided row (edge cases of the pmh encoding)
 };
 
 // Aggregate factor of the SUM product.
@@ -76,6 +81,8 @@ struct SelParams {
     int32_t exact_mode;           // fused: every decomposed predicate has its residual planes streamed, so
                                   // the exact predicate is evaluated on major + residual planes in place
     uint32_t pmx[AR_MAX_PRED][32][2];   // exact bounds, bit i of (lo - base) / (hi - base) as 0 / ~0
+    uint32_t pmh[AR_MAX_PRED][32][4];   // split residuals: candidate lo / hi, definite lo / hi bits of the
+                                        // relaxation at granularity k - h over (major << h | high planes)
     int32_t async_agg;            // fused: the one gathered aggregate column uses asynchronous gathers
     int32_t gidx;                 // index of that column in a[]
     unsigned long long* out4;     // sum, |result|, |cand|, |def|
@@ -120,7 +127,7 @@ __device__ __forceinline__ void produce_ring(const SelParams& P, uint64_t* full,
         uint32_t bytes = 0;
         for (int c = 0; c < P.npred; ++c) {
             bytes += groups * 16u * P.p[c].w;
-            if (P.p[c].res_stream) bytes += groups * 16u * P.p[c].k;
+            if (P.p[c].res_stream) bytes += groups * 16u * (P.p[c].rsplit ? P.p[c].rsplit : P.p[c].k);
         }
         mbar_arrive_expect_tx(full + s, bytes);
         uint32_t* stg = stages + (size_t)s * P.stage_words;
@@ -129,7 +136,19 @@ __device__ __forceinline__ void produce_ring(const SelParams& P, uint64_t* full,
             if (w > 0)
                 bulk_g2s(stg + P.p[c].soff, P.p[c].planes + (size_t)t * blocks_per_tile * w, groups * 16u * w,
                          full + s, pol);
-            if (P.p[c].res_stream) {   // the tile's SLICED residual planes
+            if (P.p[c].res_stream && P.p[c].rsplit) {
+                // split residual: the tile's high planes, one chunk per super-group it covers
+                const uint32_t k = P.p[c].k, h = P.p[c].rsplit, nb = groups * 4u;
+                const uint64_t b0 = (uint64_t)t * blocks_per_tile;
+                for (uint32_t done = 0; done < nb;) {
+                    const uint64_t b = b0 + done;
+                    const uint32_t bb = (uint32_t)(b % kSplitBlocks);
+                    const uint32_t cnt = min(nb - done, (uint32_t)kSplitBlocks - bb);
+                    bulk_g2s(stg + P.p[c].res_soff + done * h, P.p[c].residual + split_hi_word(b, (int)k, (int)h),
+                             cnt * 4u * h, full + s, pol);
+                    done += cnt;
+                }
+            } else if (P.p[c].res_stream) {   // the tile's SLICED residual planes
                 const uint32_t k = P.p[c].k;
                 bulk_g2s(stg + P.p[c].res_soff, P.p[c].residual + (size_t)t * blocks_per_tile * k,
                          groups * 16u * k, full + s, pol);
@@ -248,6 +267,8 @@ ar_status launch_group_sum(const ard::GroupParams& P, int grid, cudaStream_t s);
 ar_status launch_decompose_minmax(const uint32_t* col, int64_t n, uint32_t flip, uint32_t* out2, cudaStream_t s);
 ar_status launch_pack_sliced(const uint32_t* col, int64_t n, int shift, uint32_t mask, uint32_t flip, uint32_t base,
                              int w, uint32_t* out, cudaStream_t s);
+ar_status launch_pack_split(const uint32_t* col, int64_t n, int k, int h, uint32_t flip, uint32_t base, uint32_t* out,
+                            cudaStream_t s);
 ar_status launch_pack_packed(const uint32_t* col, int64_t n, int shift, uint32_t mask, uint32_t flip, uint32_t base,
                              int w, uint64_t out_words, uint32_t* out, cudaStream_t s);
 ar_status launch_exclusive_offset(const long long* all_counts, int world, int rank, long long* out, long long* total,

@@ -90,6 +90,9 @@ __device__ __forceinline__ void part_batch8(const uint32_t* s, const uint32_t (&
         for (int i = 0; i < 8; ++i) out[i] = 0u;
     } else if (layout == AR_LAYOUT_SLICED) {
         sliced_batch8(s, pos, pred, w, out);
+    } else if ((layout & 0xff) == AR_LAYOUT_SLICED) {   // split residual planes
+#pragma unroll
+        for (int i = 0; i < 8; ++i) out[i] = residual_get_if(s, pos[i], w, layout, (pred >> i) & 1u);
     } else {
 #pragma unroll
         for (int i = 0; i < 8; ++i) out[i] = packed_get_if(s, pos[i], w, (pred >> i) & 1u);

@@ -19,19 +19,31 @@ __device__ __forceinline__ void static_for(F&& f) {
     }
 }
 
-// Decomposition shape: per predicate (w_major << 6) | streamed residual width k.
+// Decomposition shape: per predicate (h << 12) | (w_major << 6) | residual
+// width k, h > 0 for a split residual whose h high planes are streamed (the
+// k - h low planes are gathered for the rows the high planes leave undecided).
 template <int... WK>
 struct Shape {
     static constexpr bool kDynamic = false;
     static constexpr int N = sizeof...(WK);
     static constexpr int w(int c) {
-        constexpr int a[] = {(WK >> 6)..., 0};
+        constexpr int a[] = {((WK >> 6) & 63)..., 0};
         return a[c];
     }
     static constexpr int k(int c) {
         constexpr int a[] = {(WK & 63)..., 0};
         return a[c];
     }
+    static constexpr int h(int c) {
+        constexpr int a[] = {((WK >> 12) & 15)..., 0};
+        return a[c];
+    }
+    static constexpr int split() {   // the one predicate with a split residual, or -1
+        for (int i = 0; i < N; ++i)
+            if (h(i) > 0) return i;
+        return -1;
+    }
+    static constexpr int kl() { return split() < 0 ? 0 : k(split()) - h(split()); }   // gathered low planes
     static constexpr int off(int c) {   // global plane index of predicate c (its ashift)
         int o = 0;
         for (int i = 0; i < c; ++i) o += w(i);
@@ -51,6 +63,8 @@ struct Shape {
 struct DynShape {
     static constexpr bool kDynamic = true;
     static constexpr int N = 0;
+    static constexpr int split() { return -1; }   // split residuals need a compiled shape
+    static constexpr int kl() { return 0; }
 };
 template <int... WK>
 struct ShapeOf {
@@ -140,11 +154,18 @@ __device__ __forceinline__ uint32_t row_bits(const uint32_t (&x)[W], uint32_t l)
 // shapes whose residual planes are streamed (K = residual width) -- the exact
 // mask em: one borrow chain over the residual then the major planes (the
 // bitwise concatenation "+bw") against the exact bounds.
-// Without kExact, K > 0 only marks a decomposed predicate.
+// Without kExact, K > 0 only marks a decomposed predicate.  A split residual
+// (H = S::h(C) > 0, its H high planes streamed): em gets the candidate rows of
+// the relaxation at granularity 2^(K-H) over (major << H | high planes), and um
+// the ones of them that are not definite there -- the rows whose K - H low
+// planes decide (progressive refinement, DESIGN s6.3d), as ul | uh: ul = below
+// the fine definite range (fine bucket of the lower bound), uh = above it (that
+// of the upper bound) -- setup_scan encodes the ranges so, see api.cu.
 template <class S, bool kExact>
 __device__ __forceinline__ void eval_block(const SelParams& P, const uint32_t* stg, uint32_t blk, uint32_t vm,
-                                           uint32_t& cm, uint32_t& dm, uint32_t& em) {
+                                           uint32_t& cm, uint32_t& dm, uint32_t& em, uint32_t& ul, uint32_t& uh) {
     cm = dm = em = vm;
+    ul = uh = 0u;
     static_for<S::N>([&](auto cc) {
         constexpr int C = decltype(cc)::value;
         constexpr int W = S::w(C), K = S::k(C), O = S::off(C);
@@ -169,7 +190,29 @@ __device__ __forceinline__ void eval_block(const SelParams& P, const uint32_t* s
                 dh = brsub(x[j], P.pm[O + j][3], dh);
             }
             dm &= ~(dl | dh);
-            if constexpr (kExact) {
+            if constexpr (kExact && S::h(C) > 0) {
+                constexpr int H = S::h(C);
+                uint32_t r[H];
+                lds_words<H>(r, stg + P.p[C].res_soff + blk * H);
+                uint32_t fl = 0, fh = 0, gl = 0, gh = 0;
+#pragma unroll
+                for (int j = 0; j < H; ++j) {
+                    fl = bsub(r[j], P.pmh[C][j][0], fl);
+                    fh = brsub(r[j], P.pmh[C][j][1], fh);
+                    gl = bsub(r[j], P.pmh[C][j][2], gl);
+                    gh = brsub(r[j], P.pmh[C][j][3], gh);
+                }
+#pragma unroll
+                for (int j = 0; j < W; ++j) {
+                    fl = bsub(x[j], P.pmh[C][H + j][0], fl);
+                    fh = brsub(x[j], P.pmh[C][H + j][1], fh);
+                    gl = bsub(x[j], P.pmh[C][H + j][2], gl);
+                    gh = brsub(x[j], P.pmh[C][H + j][3], gh);
+                }
+                em &= ~(fl | fh);
+                ul = gl;
+                uh = gh;
+            } else if constexpr (kExact) {
                 uint32_t r[K];
                 lds_words<K>(r, stg + P.p[C].res_soff + blk * K);
                 uint32_t el = 0, eh = 0;

@@ -907,10 +907,14 @@ struct ShapeEntry {
             if ((int)P.p[c].w != w[c]) return false;
         return true;
     }
-    static const void* select_fn(bool carry) {
-        using PS = ard::FixedPlanes<kSelBPT, Ws...>;
-        return carry ? (const void*)ard::select_tile_kernel<PS, kSelNW, kSelBPT, true>
-                     : (const void*)ard::select_tile_kernel<PS, kSelNW, kSelBPT, false>;
+    template <int BPT>
+    static const void* select_fn_b(bool carry) {
+        using PS = ard::FixedPlanes<BPT, Ws...>;
+        return carry ? (const void*)ard::select_tile_kernel<PS, kSelNW, BPT, true>
+                     : (const void*)ard::select_tile_kernel<PS, kSelNW, BPT, false>;
+    }
+    static const void* select_fn(bool carry, int bpt) {
+        return bpt == 4 ? select_fn_b<4>(carry) : select_fn_b<kSelBPT>(carry);
     }
     static const void* fused_fn() {
         using PS = ard::FixedPlanes<kFusBPT, Ws...>;
@@ -929,7 +933,7 @@ struct ShapeList {
     template <class E>
     static bool try_one(const ard::SelParams& P, bool fused, bool carry, const void** fn) {
         if (!E::match(P)) return false;
-        *fn = fused ? E::fused_fn() : E::select_fn(carry);
+        *fn = fused ? E::fused_fn() : E::select_fn(carry, (int)P.bpt);
         return true;
     }
 
@@ -939,12 +943,17 @@ using Shapes = ShapeList<ShapeEntry<4, 4, 6>, ShapeEntry<8>, ShapeEntry<16>, Sha
 
 int kernel_warps(bool fused) { return fused ? kFusNW : kSelNW; }               // compute warps
 static int kernel_threads(bool fused) { return 32 * (kernel_warps(fused) + (fused ? 1 : 0)); }  // + producer (fused)
-int kernel_bpt(bool fused) { return fused ? kFusBPT : kSelBPT; }
+// blocks of 32 rows per select thread: AR_SEL_BPT = 4 gives 16384-row tiles (compiled shapes only)
+int kernel_bpt(bool fused) {
+    static const int sel_bpt = getenv("AR_SEL_BPT") && atoi(getenv("AR_SEL_BPT")) == 4 ? 4 : kSelBPT;
+    return fused ? kFusBPT : sel_bpt;
+}
 
 const void* select_kernel_fn(const ard::SelParams& P, bool fused) {
     const void* fn = nullptr;
     if (!getenv("AR_FORCE_GENERIC") && Shapes::find(P, fused, P.carry != 0, &fn)) return fn;
     if (fused) return (const void*)ard::fused_kernel<ard::DynPlanes<kFusBPT>, kFusNW, kFusBPT>;
+    if (P.bpt != kSelBPT) return nullptr;   // runtime widths: 2 blocks per thread only
     return P.carry ? (const void*)ard::select_tile_kernel<ard::DynPlanes<kSelBPT>, kSelNW, kSelBPT, true>
                    : (const void*)ard::select_tile_kernel<ard::DynPlanes<kSelBPT>, kSelNW, kSelBPT, false>;
 }

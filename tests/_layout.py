@@ -31,3 +31,21 @@ def unpack_sliced(buf: bytes, n: int, w: int) -> np.ndarray:
     for j in range(w):
         v |= ((words[b * w + j] >> l) & np.uint64(1)) << np.uint64(j)
     return v
+
+
+def unpack_split(buf: bytes, n: int, k: int, h: int) -> np.ndarray:
+    """Split SLICED residual (ar_column_desc.residual_split = h): per 8192-row super-group of 256 blocks,
+    first the h high planes of its blocks (h words per block: planes k-h .. k-1), then the k-h low planes
+    (k-h words per block: planes 0 .. k-h-1); within a word bit l = row 32b+l of block b."""
+    words = np.frombuffer(buf, dtype="<u4").astype(np.uint64)
+    rows = np.arange(n, dtype=np.int64)
+    b, l = rows // 32, (rows % 32).astype(np.uint64)
+    sg, bb = (b // 256) * (256 * k), b % 256
+    v = np.zeros(n, dtype=np.uint64)
+    for j in range(k):
+        if j >= k - h:
+            idx = sg + bb * h + (j - (k - h))
+        else:
+            idx = sg + 256 * h + bb * (k - h) + j
+        v |= ((words[idx] >> l) & np.uint64(1)) << np.uint64(j)
+    return v

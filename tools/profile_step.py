@@ -28,7 +28,8 @@ def main():
     cols = datagen.q6_columns(int(os.environ.get("SEED", "2")), sf)
     n = cols["shipdate"].size
     # RES_LOC=1: the l_shipdate residual in pinned host memory (the C5 mechanism, read over the host link)
-    sd = cu.BWDColumn(cols["shipdate"], 24, residual_loc=int(os.environ.get("RES_LOC", "0")))
+    sd = cu.BWDColumn(cols["shipdate"], 24, residual_loc=int(os.environ.get("RES_LOC", "0")),
+                      split=int(os.environ.get("SPLIT", "0")))
     dc = cu.BWDColumn(cols["discount"], 32)
     qt = cu.BWDColumn(cols["quantity"], 32)
     ep = cu.BWDColumn(cols["extprice"], 32, layout=_ar.AR_LAYOUT_PACKED)
