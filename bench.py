@@ -92,7 +92,7 @@ def parse(argv=None):
     ap.add_argument("--no-c5", action="store_true")
     ap.add_argument("--split", type=int, default=0,
                     help="c4 / c2: the l_shipdate residual in the split layout with this many high planes apart")
-    ap.add_argument("--c5-split", type=int, default=0,
+    ap.add_argument("--c5-split", type=int, default=4,
                     help="c5: store the l_shipdate residual in the split layout with this many high planes apart")
     ap.add_argument("--latency-reps", type=int, default=30)
     ap.add_argument("--replays", type=int, default=5, help="extra timed replays for the median / min / p90")

@@ -527,8 +527,7 @@ static ar_status setup_scan(const ar_pred* preds, int32_t npred, ard::SelParams&
         }
         // a split residual in HBM: the one-pass kernel streams its h high planes (the fine
         // buckets decide most rows) and gathers the low planes of the rows they leave undecided
-        if (fused && p.rsplit && col->d.residual_loc == AR_LOC_DEVICE && col->residual && !R.empty &&
-            env_int("AR_SPLIT_STREAM", 1) != 0) {
+        if (p.rsplit && !R.empty) {   // the low bits of the exact bounds (check entries of the one-pass kernels)
             const uint32_t kl = (uint32_t)k - p.rsplit;
             const uint64_t maxu = (uint64_t)k + w >= 32 ? 0xffffffffull : ((1ull << (k + w)) - 1);
             const uint64_t ulo = plo < col->d.base ? 0 : (uint64_t)(plo - col->d.base);
@@ -537,6 +536,9 @@ static ar_status setup_scan(const ar_pred* preds, int32_t npred, ard::SelParams&
             p.sfhi = (uint32_t)(uhi >> kl);
             p.sllo = (uint32_t)(ulo & ((1u << kl) - 1u));
             p.slhi = (uint32_t)(uhi & ((1u << kl) - 1u));
+        }
+        if (fused && p.rsplit && col->d.residual_loc == AR_LOC_DEVICE && col->residual && !R.empty &&
+            env_int("AR_SPLIT_STREAM", 1) != 0) {
             p.res_stream = 1;
             p.res_soff = words;
             words += (P.tile_rows / 32) * p.rsplit;

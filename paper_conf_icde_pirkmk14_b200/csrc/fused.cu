@@ -172,7 +172,8 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
     uint2* ring = reinterpret_cast<uint2*>(stages + (size_t)P.nstages * P.stage_words) + warp * kRing;
     uint32_t* gs0 = reinterpret_cast<uint32_t*>(reinterpret_cast<uint2*>(stages + (size_t)P.nstages * P.stage_words) +
                                                 NW * kRing);
-    uint32_t* gs = gs0 + warp * (kDepth * SW);
+    const uint32_t depth = P.rl_depth, dmask = depth - 1;   // gather passes in flight per warp (4 or 8)
+    uint32_t* gs = gs0 + warp * (depth * SW);
     if (threadIdx.x == 0) {
         for (uint32_t s = 0; s < P.nstages; ++s) {
             mbar_init(full + s, 1);
@@ -201,7 +202,7 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
 
     // One gather pass over the `take` oldest ring entries (take <= 32).
     auto pass = [&](uint32_t take) {
-        uint32_t* sl = gs + (gseq % kDepth) * SW;
+        uint32_t* sl = gs + (gseq & dmask) * SW;
         uint32_t info = 0u, f = 0u;
         if (lane < take) {
             const uint32_t ri = (rhead + lane) & rmask;
@@ -235,9 +236,12 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
         ++gseq;
         rhead += take;
         rcnt -= take;
-        if (gseq >= (uint32_t)kDepth) {   // sum the pass issued kDepth - 1 passes ago
-            cp_async_wait<kDepth - 1>();
-            sum += drain<KL>(gs + (gseq % kDepth) * SW, lane, gmask, G.base, &P.p[SPi], &nchk);
+        if (gseq >= depth) {   // sum the pass issued depth - 1 passes ago
+            if (depth == 8)
+                cp_async_wait<7>();
+            else
+                cp_async_wait<kDepth - 1>();
+            sum += drain<KL>(gs + (gseq & dmask) * SW, lane, gmask, G.base, &P.p[SPi], &nchk);
         }
     };
 
@@ -389,8 +393,8 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
     if (list) {   // the ring's tail, then every pass still in flight
         while (rcnt > 0) pass(min(rcnt, 32u));
         cp_async_wait<0>();
-        for (uint32_t g = gseq >= (uint32_t)kDepth ? gseq - kDepth + 1 : 0; g < gseq; ++g)
-            sum += drain<KL>(gs + (g % kDepth) * SW, lane, gmask, G.base, &P.p[SPi], &nchk);
+        for (uint32_t g = gseq >= depth ? gseq - depth + 1 : 0; g < gseq; ++g)
+            sum += drain<KL>(gs + (g & dmask) * SW, lane, gmask, G.base, &P.p[SPi], &nchk);
     }
 
     unsigned long long c0 = ncand, c1 = ndef, c2 = nres + nchk;
@@ -424,6 +428,9 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
     using S = Shape<WK...>;
     constexpr int NT = NW * 32;
     constexpr int KS = S::ksum();
+    // a compiled split residual (predicate SP): rows its high planes leave undecided go to the ring as check
+    // entries and their KL low planes are gathered with the aggregate (no synchronous gather)
+    constexpr int SP = S::split(), KL = S::kl(), SPi = SP < 0 ? 0 : SP, SW = slot_words(KL);
     extern __shared__ __align__(128) unsigned char smem[];
     uint64_t* full = reinterpret_cast<uint64_t*>(smem);
     uint64_t* empty = full + P.nstages;
@@ -434,7 +441,7 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
     const uint32_t kRing = P.rl_ring, rmask = kRing - 1;
     uint2* ring = reinterpret_cast<uint2*>(stages + (size_t)P.nstages * P.stage_words) + warp * kRing;
     uint32_t* gs = reinterpret_cast<uint32_t*>(reinterpret_cast<uint2*>(stages + (size_t)P.nstages * P.stage_words) +
-                                               NW * kRing) + warp * (kDepth * kSlotWords);
+                                               NW * kRing) + warp * (kDepth * SW);
     if (threadIdx.x == 0) {
         for (uint32_t s = 0; s < P.nstages; ++s) {
             mbar_init(full + s, 1);
@@ -456,12 +463,12 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
     const bool direct = !list && P.nagg > 0;
     const AggCol& G = P.a[P.gidx];
     const uint32_t gmask = G.w >= 32 ? 0xffffffffu : ((1u << G.w) - 1u);
-    uint32_t ncand = 0, ndef = 0, nres = 0;
+    uint32_t ncand = 0, ndef = 0, nres = 0, nchk = 0;
     unsigned long long sum = 0;
     uint32_t rhead = 0, rcnt = 0, gseq = 0;
 
     auto pass = [&](uint32_t take) {
-        uint32_t* sl = gs + (gseq % kDepth) * kSlotWords;
+        uint32_t* sl = gs + (gseq % kDepth) * SW;
         uint32_t info = 0u, f = 0u;
         if (lane < take) {
             const uint2 e = ring[(rhead + lane) & rmask];
@@ -472,6 +479,20 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
             if (sh + G.w > 32u) cp_async4(sl + 32 + lane, src + 1);
             info = 0x80000000u | sh;
             f = e.y;
+            if constexpr (KL > 0) {
+                const uint32_t code = e.y >> 30;   // check code (host: factors < 2^30)
+                f = e.y & 0x3fffffffu;
+                if (code) {
+                    const uint32_t* lp = P.p[SPi].residual + split_lo_word(e.x >> 5, S::k(SPi), S::h(SPi));
+                    if constexpr (KL == 4) {
+                        cp_async16(low_word<KL>(sl, lane, 0), lp);
+                    } else {
+#pragma unroll
+                        for (int j = 0; j < KL; ++j) cp_async4(low_word<KL>(sl, lane, j), lp + j);
+                    }
+                    info |= (code << 8) | ((e.x & 31u) << 10);
+                }
+            }
         }
         sl[64 + lane] = info;
         sl[96 + lane] = f;
@@ -481,14 +502,22 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
         rcnt -= take;
         if (gseq >= (uint32_t)kDepth) {
             cp_async_wait<kDepth - 1>();
-            sum += drain(gs + (gseq % kDepth) * kSlotWords, lane, gmask, G.base);
+            sum += drain<KL>(gs + (gseq % kDepth) * SW, lane, gmask, G.base, &P.p[SPi], &nchk);
         }
     };
 
-    // a6 for the result rows xm[] of a tile held in stage `stg`
-    auto consume = [&](const uint32_t* stg, int64_t tile_r0, uint32_t (&xm)[BPT]) {
+    // a6 for the result rows xm[] of a tile held in stage `stg`; ck0 / ck1: rows of xm that are check
+    // entries (split residual, list mode) in the fine bucket of the lower / upper bound
+    auto consume = [&](const uint32_t* stg, int64_t tile_r0, uint32_t (&xm)[BPT], const uint32_t (&ck0)[BPT],
+                       const uint32_t (&ck1)[BPT]) {
 #pragma unroll
-        for (int b = 0; b < BPT; ++b) nres += __popc(xm[b]);
+        for (int b = 0; b < BPT; ++b) nres += __popc(xm[b] & ~(ck0[b] | ck1[b]));   // check rows count when drained
+        auto code_at = [&](int b, uint32_t l) -> uint32_t {   // check code << 30 of row l of block b
+            if constexpr (KL > 0)
+                return (((ck0[b] >> l) & 1u) << 30) | (((ck1[b] >> l) & 1u) << 31);
+            else
+                return 0u;
+        };
         if (direct) {
 #pragma unroll
             for (int b = 0; b < BPT; ++b) {
@@ -541,7 +570,7 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
                         do {
                             const uint32_t l = __ffs(m) - 1;
                             m &= m - 1;
-                            ring[(wbase + e) & rmask] = make_uint2(row0 + l, 1u);
+                            ring[(wbase + e) & rmask] = make_uint2(row0 + l, 1u | code_at(b, l));
                             ++e;
                         } while (m && e < lim);
                     } else {
@@ -555,7 +584,8 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
                                 do {
                                     const uint32_t l = __ffs(m) - 1;
                                     m &= m - 1;
-                                    ring[(wbase + e) & rmask] = make_uint2(row0 + l, row_of<W>(x, l) + P.p[C].base);
+                                    ring[(wbase + e) & rmask] =
+                                        make_uint2(row0 + l, (row_of<W>(x, l) + P.p[C].base) | code_at(b, l));
                                     ++e;
                                 } while (m && e < lim);
                             }
@@ -586,16 +616,44 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
     auto phase_b = [&]() {
         const uint32_t* stg = stages + (size_t)pst * P.stage_words;
         const int64_t r0 = pt * (int64_t)P.tile_rows;
-        uint32_t xm[BPT];
+        uint32_t xm[BPT], xk0[BPT], xk1[BPT];
 #pragma unroll
         for (int b = 0; b < BPT; ++b) {
             const uint32_t blk = b * NT + threadIdx.x;
-            uint32_t em = pnd[b];
+            uint32_t em = pnd[b], u0 = 0u, u1 = 0u;
             if (em) {
                 static_for<S::N>([&](auto cc) {
                     constexpr int C = decltype(cc)::value;
                     constexpr int W = S::w(C), K = S::k(C), KO = S::kofs(C);
-                    if constexpr (K > 0) {
+                    if constexpr (K > 0 && S::h(C) > 0) {
+                        // compiled split residual: the high planes (gathered in phase A) give the relaxation at
+                        // granularity 2^(K-H); its definite rows are results, its undecided ones check entries
+                        // whose code (fine bucket of lo / of hi) the pass turns into a low-plane gather
+                        constexpr int H = S::h(C);
+                        uint32_t x[W];
+                        lds_words<W>(x, stg + P.p[C].soff + blk * W);
+                        uint32_t fl = 0, fh = 0, gl = 0, gh = 0;
+#pragma unroll
+                        for (int j = K - H; j < K; ++j) {
+                            fl = bsub(rres[b][KO + j], P.pmh[C][j - (K - H)][0], fl);
+                            fh = brsub(rres[b][KO + j], P.pmh[C][j - (K - H)][1], fh);
+                            gl = bsub(rres[b][KO + j], P.pmh[C][j - (K - H)][2], gl);
+                            gh = brsub(rres[b][KO + j], P.pmh[C][j - (K - H)][3], gh);
+                        }
+#pragma unroll
+                        for (int j = 0; j < W; ++j) {
+                            fl = bsub(x[j], P.pmh[C][H + j][0], fl);
+                            fh = brsub(x[j], P.pmh[C][H + j][1], fh);
+                            gl = bsub(x[j], P.pmh[C][H + j][2], gl);
+                            gh = brsub(x[j], P.pmh[C][H + j][3], gh);
+                        }
+                        em &= ~(fl | fh);
+                        u0 = gl | (0u - (P.p[C].scor & 1u));
+                        u1 = gh | (0u - ((P.p[C].scor >> 1) & 1u));
+                        const uint32_t und = gl | gh;
+                        u0 &= und;
+                        u1 &= und;
+                    } else if constexpr (K > 0) {
                         uint32_t x[W];
                         lds_words<W>(x, stg + P.p[C].soff + blk * W);
                         const uint32_t H = P.p[C].rsplit;
@@ -647,12 +705,17 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
                 });
             }
             xm[b] = em;
+            xk0[b] = em & u0;
+            xk1[b] = em & u1;
         }
-        consume(stg, r0, xm);
+        consume(stg, r0, xm, xk0, xk1);
         __syncwarp();
         if (lane == 0) mbar_arrive(empty + pst);
     };
 
+    uint32_t zero[BPT];
+#pragma unroll
+    for (int b = 0; b < BPT; ++b) zero[b] = 0u;
     uint32_t s = 0, ph = 0;
     for (;; s = (s + 1 == P.nstages) ? (ph ^= 1u, 0u) : s + 1) {
         mbar_wait(full + s, ph, P.suspend_ns);
@@ -705,9 +768,9 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
             }
             pt = t;
             pst = s;
-            consume(stg, tile_r0, dmk);      // definite rows are results now
+            consume(stg, tile_r0, dmk, zero, zero);   // definite rows are results now
         } else {
-            consume(stg, tile_r0, dmk);      // k = 0 everywhere: candidate = definite = exact
+            consume(stg, tile_r0, dmk, zero, zero);   // k = 0 everywhere: candidate = definite = exact
             __syncwarp();
             if (lane == 0) mbar_arrive(empty + s);
         }
@@ -723,10 +786,10 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
         while (rcnt > 0) pass(min(rcnt, 32u));
         cp_async_wait<0>();
         for (uint32_t g = gseq >= (uint32_t)kDepth ? gseq - kDepth + 1 : 0; g < gseq; ++g)
-            sum += drain(gs + (g % kDepth) * kSlotWords, lane, gmask, G.base);
+            sum += drain<KL>(gs + (g % kDepth) * SW, lane, gmask, G.base, &P.p[SPi], &nchk);
     }
 
-    unsigned long long c0 = ncand, c1 = ndef, c2 = nres;
+    unsigned long long c0 = ncand, c1 = ndef, c2 = nres + nchk;
 #pragma unroll
     for (int o = 16; o > 0; o >>= 1) {
         sum += __shfl_xor_sync(0xffffffffu, sum, o);
@@ -827,20 +890,39 @@ bool rl_match(const ard::SelParams& P) {
     return true;
 }
 
-// rg shapes: (w_major << 6) | k of every predicate, the residual gathered (SLICED, k <= 8)
+// rg shapes: (w_major << 6) | k of every predicate, the residual gathered (SLICED, k <= 8); a split
+// residual carries its h (<< 12) when its undecided rows can be check entries of the result ring (list
+// mode, the other factor below 2^30; rg_split_ok), otherwise it is matched as unsplit (runtime h,
+// synchronous low-plane gathers)
 template <int... Ws>
-bool rg_match(const ard::SelParams& P) {
+bool rg_match(const ard::SelParams& P, bool split_ok) {
     constexpr int n = sizeof...(Ws);
     constexpr int wk[] = {Ws..., 0};
     if (P.npred != n) return false;
-    for (int c = 0; c < n; ++c)
-        if ((int)((P.p[c].w << 6) | P.p[c].k) != wk[c]) return false;
+    for (int c = 0; c < n; ++c) {
+        const uint32_t h = split_ok ? P.p[c].rsplit : 0u;
+        if ((int)((h << 12) | (P.p[c].w << 6) | P.p[c].k) != wk[c]) return false;
+    }
     return true;
+}
+inline bool rg_split_ok(const ard::SelParams& P) {
+    int ns = 0;
+    for (int c = 0; c < P.npred; ++c) ns += P.p[c].rsplit ? 1 : 0;
+    const bool mp_small =
+        P.rl_mpred < 0 || (P.p[P.rl_mpred].base == 0 && P.p[P.rl_mpred].w + P.p[P.rl_mpred].k <= 30);
+    return ns == 1 && P.rl_list && mp_small;
 }
 
 RlFn rg_find(const ard::SelParams& P, int cfg) {
+    const bool sok = rg_split_ok(P);
 #define AR_RG_TRY(...) \
-    if (rg_match<__VA_ARGS__>(P)) return rg_pick<__VA_ARGS__>(cfg);
+    if (rg_match<__VA_ARGS__>(P, sok)) return rg_pick<__VA_ARGS__>(cfg);
+    AR_RG_TRY(WKH(4, 8, 4), WK(4, 0), WK(6, 0))
+    AR_RG_TRY(WKH(4, 8, 3), WK(4, 0), WK(6, 0))
+    AR_RG_TRY(WKH(4, 8, 2), WK(4, 0), WK(6, 0))
+#undef AR_RG_TRY
+#define AR_RG_TRY(...) \
+    if (rg_match<__VA_ARGS__>(P, false)) return rg_pick<__VA_ARGS__>(cfg);
     AR_RG_TRY(WK(4, 8), WK(4, 0), WK(6, 0))
     AR_RG_TRY(WK(24, 8))
     AR_RG_TRY(WK(24, 8), WK(24, 8))
@@ -895,9 +977,14 @@ int env_ring() {
 size_t rl_smem_bytes(const ard::SelParams& P, uint32_t nstages, int nw, bool rg) {
     const size_t head = ((size_t)nstages * 24 + 127) & ~size_t(127);
     uint32_t kl = 0;
-    if (!rg) rl_split(P, &kl);
+    if (!rg) {
+        rl_split(P, &kl);
+    } else if (rg_split_ok(P)) {   // a compiled split shape uses KL low-plane words per slot lane
+        for (int c = 0; c < P.npred; ++c)
+            if (P.p[c].rsplit) kl = P.p[c].k - P.p[c].rsplit;
+    }
     return head + (size_t)nstages * P.stage_words * 4 + (size_t)nw * P.rl_ring * 8 +
-           (size_t)nw * ard::rl::kDepth * ard::rl::slot_words((int)kl) * 4;
+           (size_t)nw * (rg ? ard::rl::kDepth : P.rl_depth) * ard::rl::slot_words((int)kl) * 4;
 }
 
 }  // namespace
@@ -979,6 +1066,8 @@ ar_status launch_fused_rl(const ard::SelParams& P0, const ar_column* const* cols
     if (!k.fn) return AR_OK;
     retile(P, k.tile_rows);
     P.rl_ring = (uint32_t)env_ring();
+    static const int depth_env = getenv("AR_RL_DEPTH") ? atoi(getenv("AR_RL_DEPTH")) : 4;
+    P.rl_depth = depth_env == 8 ? 8u : 4u;
 
     // deepest stage ring (<= 8, >= 3) that keeps 2 CTAs per SM, else 1 CTA with >= 2 stages
     opt_in_max_smem(k.fn);
@@ -987,8 +1076,11 @@ ar_status launch_fused_rl(const ard::SelParams& P0, const ar_column* const* cols
     int occ = 0;
     static const int force_st = getenv("AR_STAGES") ? atoi(getenv("AR_STAGES")) : 0;
     static const int want_ctas = getenv("AR_RL_CTAS") ? atoi(getenv("AR_RL_CTAS")) : 2;
+    // the result-ring kernel runs 3 stages (deeper rings measured slower at C4 / C2: the stream's extra
+    // TMA requests delay the aggregate gathers, DESIGN s6.3); the two-phase kernel up to 8
+    const uint32_t max_st = rg ? 8u : 3u;
     for (int target = std::max(want_ctas, 1); target >= 1 && !stages; --target)
-        for (uint32_t st = 8; st >= 2; --st) {
+        for (uint32_t st = force_st > 0 ? 8u : max_st; st >= 2; --st) {
             if (force_st > 0 && (int)st != force_st) continue;
             // the two-phase kernel holds two stages (phase B of tile t - 1 while tile t is decided)
             if (target >= 2 && st < (rg ? 4u : 3u) && force_st <= 0) break;

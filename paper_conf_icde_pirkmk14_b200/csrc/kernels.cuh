@@ -90,6 +90,7 @@ struct SelParams {
     int32_t rl_list;              // 1: one gathered SUM factor, rows queued in the warp result ring
     int32_t rl_mpred;             // predicate whose exact value is the other SUM factor, or -1
     uint32_t rl_ring;             // result-ring entries per warp (power of two)
+    uint32_t rl_depth;            // gather passes in flight per warp (4 or 8)
     int32_t rl_fin;               // 1: finalize out4 through rl_part / rl_ticket (no memset before the launch)
     int32_t rl_pdl;               // programmatic dependent launch: 1 = wait before reading inputs, 2 = read
                                   // inputs at once (caller: the previous kernel does not write them)

@@ -119,16 +119,19 @@ def test_gpu_split_general_kernel_and_spatial(cu):
 @pytest.mark.parametrize("h", [2, 3, 4])
 @pytest.mark.parametrize("bounds", [(731, 1095), (800, 805), (768, 1023), (0, 0xFFFFFFFF), (1, 2526), (1000, 1000),
                                     (1024, 1040), (2520, 5000), (1, 5), (3, 20), (2500, 2510), (0, 0)])
-def test_gpu_split_stream_bounds(cu, h, bounds):
-    """The streamed-high-planes result-ring kernel at bound placements the check code must get right: both
-    bounds inside one fine bucket (code 3), bucket-aligned bounds (no undecided rows), the whole domain, a
-    point predicate, a bound past the data; 8192-row tiles with a ragged tail."""
+@pytest.mark.parametrize("loc", [0, 1])
+def test_gpu_split_stream_bounds(cu, h, bounds, loc):
+    """Check entries of the split residual at bound placements the check code must get right: both bounds
+    inside one fine bucket (code 3), bucket-aligned bounds (no undecided rows), the whole domain, a point
+    predicate, a bound past the data; 8192-row tiles with a ragged tail.  HBM residual: the result-ring
+    kernel streaming the high planes; pinned host residual: the gathered-residual kernel (high planes
+    gathered in phase A, low planes with the aggregate)."""
     from paper_conf_icde_pirkmk14_b200 import _ar
     n = 3 * 8192 + 77_777
     c = datagen.q6_columns(90 + h, 1.0, n=n)
     vals = [c["shipdate"], c["discount"], c["quantity"]]
     los, his = [bounds[0], LOS[1], LOS[2]], [bounds[1], HIS[1], HIS[2]]
-    sd = cu.BWDColumn(vals[0], 24, split=h)
+    sd = cu.BWDColumn(vals[0], 24, split=h, residual_loc=loc)
     dc, qt = cu.BWDColumn(vals[1], 32), cu.BWDColumn(vals[2], 32)
     ep = cu.BWDColumn(c["extprice"], 32, layout=_ar.AR_LAYOUT_PACKED)
     preds = [(sd, los[0], his[0]), (dc, los[1], his[1]), (qt, los[2], his[2])]
@@ -138,7 +141,7 @@ def test_gpu_split_stream_bounds(cu, h, bounds):
         o4 = torch.zeros(4, dtype=torch.int64, device="cuda")
         cu.select_refine_sum(preds, aggs, o4)
         torch.cuda.synchronize()
-        assert _ar.ar_last_scan_kernel() == "fused_rl_kernel"
+        assert _ar.ar_last_scan_kernel() == ("fused_rl_kernel" if loc == 0 else "fused_rg_kernel")
         if want is None:
             _, _, want = oracle.select_sum(vals, los, his, [c["extprice"]], positions=False)
         assert o4.cpu().tolist() == [want, ref_cnt, cpos.size, int(cdef.sum())]
