@@ -133,6 +133,31 @@ __device__ __forceinline__ void mbar_wait(uint64_t* bar, uint32_t parity, uint32
     }
 }
 
+// The same on a shared-window address (smem_u32 of the barrier computed once by
+// the caller: the generic -> shared conversion is several instructions).
+__device__ __forceinline__ void mbar_wait_a(uint32_t bar, uint32_t parity, uint32_t hint_ns) {
+    if (hint_ns) {
+        asm volatile(
+            "{\n\t.reg .pred p;\n"
+            "AR_WAIT_%=:\n\t"
+            "mbarrier.try_wait.parity.shared::cta.b64 p, [%0], %1, %2;\n\t"
+            "@!p bra AR_WAIT_%=;\n}" ::"r"(bar),
+            "r"(parity), "r"(hint_ns)
+            : "memory");
+    } else {
+        asm volatile(
+            "{\n\t.reg .pred p;\n"
+            "AR_WAIT_%=:\n\t"
+            "mbarrier.try_wait.parity.shared::cta.b64 p, [%0], %1;\n\t"
+            "@!p bra AR_WAIT_%=;\n}" ::"r"(bar),
+            "r"(parity)
+            : "memory");
+    }
+}
+__device__ __forceinline__ void mbar_arrive_a(uint32_t bar) {
+    asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(bar) : "memory");
+}
+
 // Wait with an exponential __nanosleep back-off between probes: for a lone
 // producer lane, whose spinning would otherwise take issue slots from the
 // consumer warps of its SM.

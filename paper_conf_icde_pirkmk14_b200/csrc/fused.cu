@@ -52,6 +52,12 @@ __device__ __forceinline__ uint32_t stage_value(const SelParams& P, const uint32
 __device__ __forceinline__ void cp_async4(uint32_t* dst, const uint32_t* src) {
     asm volatile("cp.async.ca.shared.global" AR_GHINT " [%0], [%1], 4;" ::"r"(smem_u32(dst)), "l"(src) : "memory");
 }
+__device__ __forceinline__ void cp_async4_a(uint32_t dst, const uint32_t* src) {   // dst: shared-window address
+    asm volatile("cp.async.ca.shared.global" AR_GHINT " [%0], [%1], 4;" ::"r"(dst), "l"(src) : "memory");
+}
+__device__ __forceinline__ void cp_async16_a(uint32_t dst, const uint32_t* src) {
+    asm volatile("cp.async.cg.shared.global" AR_GHINT " [%0], [%1], 16;" ::"r"(dst), "l"(src) : "memory");
+}
 __device__ __forceinline__ void cp_async16(uint32_t* dst, const uint32_t* src) {
     asm volatile("cp.async.cg.shared.global" AR_GHINT " [%0], [%1], 16;" ::"r"(smem_u32(dst)), "l"(src) : "memory");
 }
@@ -174,6 +180,8 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
                                                 NW * kRing);
     const uint32_t depth = P.rl_depth, dmask = depth - 1;   // gather passes in flight per warp (4 or 8)
     uint32_t* gs = gs0 + warp * (depth * SW);
+    // shared-window addresses, converted once (the conversion is several instructions)
+    const uint32_t gs_a = smem_u32(gs), full_a = smem_u32(full), empty_a = smem_u32(empty);
     if (threadIdx.x == 0) {
         for (uint32_t s = 0; s < P.nstages; ++s) {
             mbar_init(full + s, 1);
@@ -203,6 +211,7 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
     // One gather pass over the `take` oldest ring entries (take <= 32).
     auto pass = [&](uint32_t take) {
         uint32_t* sl = gs + (gseq & dmask) * SW;
+        const uint32_t sl_a = gs_a + (gseq & dmask) * (SW * 4);
         uint32_t info = 0u, f = 0u;
         if (lane < take) {
             const uint32_t ri = (rhead + lane) & rmask;
@@ -210,8 +219,8 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
             const uint64_t bit = (uint64_t)e.x * G.w;
             const uint32_t* src = G.major + (bit >> 5);
             const uint32_t sh = (uint32_t)(bit & 31);
-            cp_async4(sl + lane, src);
-            if (sh + G.w > 32u) cp_async4(sl + 32 + lane, src + 1);
+            cp_async4_a(sl_a + lane * 4, src);
+            if (sh + G.w > 32u) cp_async4_a(sl_a + (32 + lane) * 4, src + 1);
             info = 0x80000000u | sh;
             f = e.y;
             if constexpr (KL > 0) {
@@ -221,10 +230,10 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
                 if (code) {   // an undecided row: its low residual planes travel with the aggregate
                     const uint32_t* lp = P.p[SPi].residual + split_lo_word(e.x >> 5, S::k(SPi), S::h(SPi));
                     if constexpr (KL == 4) {
-                        cp_async16(low_word<KL>(sl, lane, 0), lp);
+                        cp_async16_a(sl_a + (kSlotWords + lane * 4) * 4, lp);
                     } else {
 #pragma unroll
-                        for (int j = 0; j < KL; ++j) cp_async4(low_word<KL>(sl, lane, j), lp + j);
+                        for (int j = 0; j < KL; ++j) cp_async4_a(sl_a + (kSlotWords + j * 32 + lane) * 4, lp + j);
                     }
                     info |= (code << 8) | ((e.x & 31u) << 10);
                 }
@@ -247,13 +256,13 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
 
     uint32_t s = 0, ph = 0;
     for (;; s = (s + 1 == P.nstages) ? (ph ^= 1u, 0u) : s + 1) {
-        mbar_wait(full + s, ph, P.suspend_ns);
+        mbar_wait_a(full_a + 8 * s, ph, P.suspend_ns);
         const long long t = slot[s];
         if (t < 0) break;
         const uint32_t* stg = stages + (size_t)s * P.stage_words;
         if (P.debug == 7) {   // experiment: the TMA stream alone (no evaluation)
             __syncwarp();
-            if (lane == 0) mbar_arrive(empty + s);
+            if (lane == 0) mbar_arrive_a(empty_a + 8 * s);
             continue;
         }
         const int64_t tile_r0 = t * (int64_t)P.tile_rows;
@@ -364,8 +373,8 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
                                 do {
                                     const uint32_t l = __ffs(m) - 1;
                                     m &= m - 1;
-                                    uint32_t v = row_of<W>(x, l);
-                                    if constexpr (K > 0) v = (v << K) | row_of<K>(r, l);
+                                    uint32_t v = row_bits<W>(x, l);
+                                    if constexpr (K > 0) v = (v << K) | row_bits<K>(r, l);
                                     ring[(wbase + e) & rmask] = make_uint2(row0 + l, (v + P.p[C].base) | code_at(b, l));
                                     ++e;
                                 } while (m && e < lim);
@@ -384,7 +393,7 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rl_kernel(const __grid
             }
         }
         __syncwarp();
-        if (lane == 0) mbar_arrive(empty + s);   // the stage is no longer read
+        if (lane == 0) mbar_arrive_a(empty_a + 8 * s);   // the stage is no longer read
         if (list) {
             while (rcnt >= 32) pass(32);
             __syncwarp();
@@ -585,7 +594,7 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
                                     const uint32_t l = __ffs(m) - 1;
                                     m &= m - 1;
                                     ring[(wbase + e) & rmask] =
-                                        make_uint2(row0 + l, (row_of<W>(x, l) + P.p[C].base) | code_at(b, l));
+                                        make_uint2(row0 + l, (row_bits<W>(x, l) + P.p[C].base) | code_at(b, l));
                                     ++e;
                                 } while (m && e < lim);
                             }

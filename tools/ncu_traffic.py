@@ -48,8 +48,9 @@ def short(name):
 
 def main():
     wl, reps = sys.argv[1], sys.argv[2:]
-    commit = subprocess.run(["git", "rev-parse", "--short", "HEAD"], cwd=ROOT, capture_output=True,
-                            text=True).stdout.strip()
+    # the GPU box has no .git: the caller passes the commit in COMMIT
+    commit = os.environ.get("COMMIT") or subprocess.run(["git", "rev-parse", "--short", "HEAD"], cwd=ROOT,
+                                                        capture_output=True, text=True).stdout.strip()
     acc = {}
     for rep in reps:
         for k in kernels(rep):
@@ -73,7 +74,7 @@ def main():
             "read_per_launch": e1["read_per_launch"] + e2["read_per_launch"],
             "write_per_launch": e1["write_per_launch"] + e2["write_per_launch"],
             "us_per_launch_cold": e1["us_per_launch_cold"] + e2["us_per_launch_cold"], "source": src}
-    path = os.path.join(ROOT, "profiles", "traffic.json")
+    path = os.environ.get("TRAFFIC_JSON") or os.path.join(ROOT, "profiles", "traffic.json")
     allt = {}
     if os.path.exists(path):
         try:
