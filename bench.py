@@ -249,6 +249,8 @@ class ClockSampler:
 
     def __init__(self, index):
         self.samples, self.reasons, self.stop_flag = [], set(), False
+        self.mem, self.power = [], []
+        self.index = index
         self.ok = False
         try:
             import pynvml
@@ -273,6 +275,8 @@ class ClockSampler:
         while not self.stop_flag:
             try:
                 self.samples.append(nv.nvmlDeviceGetClockInfo(self.h, nv.NVML_CLOCK_SM))
+                self.mem.append(nv.nvmlDeviceGetClockInfo(self.h, nv.NVML_CLOCK_MEM))
+                self.power.append(nv.nvmlDeviceGetPowerUsage(self.h) / 1000.0)
                 r = nv.nvmlDeviceGetCurrentClocksEventReasons(self.h)
                 for bit, name in names.items():
                     if bit and (r & bit) == bit and name not in ("None", "GpuIdle"):
@@ -298,6 +302,8 @@ class ClockSampler:
             return {"sm_mhz": None, "sm_max_mhz": getattr(self, "max_mhz", None), "reasons": [],
                     "samples": 0, "source": "nvml"}
         return {"sm_mhz": statistics.median(self.samples), "sm_max_mhz": self.max_mhz,
+                "mem_mhz": statistics.median(self.mem) if self.mem else None,
+                "power_w_median": statistics.median(self.power) if self.power else None,
                 "reasons": sorted(self.reasons), "samples": len(self.samples), "source": "nvml"}
 
 
@@ -649,7 +655,15 @@ class Runner:
                 g_warm.replay()
                 ctx.stream.synchronize()
                 ctx.barrier()
-                cm = sampler if (sampler is not None and r == 0) else _Null()
+                # run 0 is the headline (its clocks are the line's); the replays get their own sampler
+                if sampler is not None and r == 0:
+                    cm = sampler
+                elif sampler is not None:
+                    if getattr(sampler, "replay_sampler", None) is None:
+                        sampler.replay_sampler = ClockSampler(sampler.index)
+                    cm = sampler.replay_sampler
+                else:
+                    cm = _Null()
                 with cm:
                     ctx.rec(t0)
                     g_timed.replay()
@@ -867,7 +881,8 @@ def ours(args):
             "value": rows * world * K / (ms_total / 1e3) if args.workload != "c4" or args.scaling == "weak"
             else table_rows * K / (ms_total / 1e3),
             "ms_per_step": ms_step, "result": res, "steps_consistent": consistent,
-            "ms_per_step_replays": dist_stats([x / K for x in runs]),
+            "ms_per_step_replays": dict(dist_stats([x / K for x in runs]) or {},
+                                        runs=[round(x / K, 5) for x in runs]),
             "roofline": {"bound": "hbm", "achieved": achieved, "peak": hbm_peak, "unit": "GB/s",
                          "frac": achieved / hbm_peak, "traffic": (tr or {}).get("bytes_per_launch"),
                          "traffic_source": (tr or {}).get("source"),
@@ -1024,6 +1039,7 @@ def ours(args):
             "roofline": head["roofline"], "cpu_baseline": cpu, "cpu_baseline_single_thread": cpu1, "e2e": e2e,
             "gpu_launches": head["gpu_launches"], "gpu_kernels": head["gpu_kernels"],
             "clocks": sampler.result(),
+            "clocks_replays": sampler.replay_sampler.result() if getattr(sampler, "replay_sampler", None) else None,
             "ms_per_step_replays": head["ms_per_step_replays"],
             "latency": latency,
             "counts": {"candidates": ab["n_cand"], "definite": ab["n_def"], "result": ab["n_result"],

@@ -4,7 +4,7 @@
 # of the hot kernels at C4 (the headline) and C2, and the traffic.json they give.  Outputs land in
 # gpurun_out/; summaries are copied to profiles/rNN/ (tools/collect_round.sh).
 set -x
-nvidia-smi --query-gpu=name,clocks.sm,clocks.max.sm,clocks.mem,power.draw --format=csv > gpurun_out/smi.txt
+nvidia-smi --query-gpu=name,clocks.sm,clocks.max.sm,clocks.mem,power.draw,power.limit,enforced.power.limit --format=csv > gpurun_out/smi.txt
 timeout 1200 python -m pytest tests -m gpu -q > gpurun_out/gpu_tests.log 2>&1
 timeout 300 python -c "import __graft_entry__ as g; g.smoke()" > gpurun_out/smoke.log 2>&1
 timeout 900 python bench.py > gpurun_out/bench.json 2> gpurun_out/bench.err
