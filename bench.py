@@ -795,13 +795,14 @@ def bench_c5(ctx, args):
     return out
 
 
-def run_e2e(ctx, q, ab, steps):
+def run_e2e(ctx, q, ab, steps, sd_host=None):
     """The same metric end to end through the C ABI with HOST buffers: the decomposed table at rest in
     pinned host memory; every step copies the scanned majors H2D, ar_select_refine_sum reads the shipdate
     residual and l_extendedprice zero-copy over the host link (only touched sectors), and the (SUM, count)
     result is copied D2H (after the SUM allreduce when G > 1)."""
     torch, _ar = ctx.torch, ctx._ar
-    sd_e = q.sd.copy(residual_loc=_ar.AR_LOC_HOST_PINNED)
+    # sd_host: the l_shipdate column decomposed with its residual in pinned host memory (split layout)
+    sd_e = sd_host if sd_host is not None else q.sd.copy(residual_loc=_ar.AR_LOC_HOST_PINNED)
     dc_e, qt_e = q.dc.copy(), q.qt.copy()
     ep_e = q.ep.copy(major_loc=_ar.AR_LOC_HOST_PINNED)
     host_src = [(q.sd.major.cpu().pin_memory(), sd_e.major), (q.dc.major.cpu().pin_memory(), dc_e.major),
@@ -962,16 +963,22 @@ def ours(args):
 
     e2e = None
     if args.e2e_steps > 0:
-        # the e2e path reads the residual over the host link (gathered high planes when split)
-        ab_e = ab if not args.split else algorithmic_bytes(cols, q.sd.w_major, args.split, high_streamed=False)
-        e = run_e2e(ctx, q, ab_e, args.e2e_steps)
+        # the e2e path reads the residual over the host link: there the split layout (--c5-split high
+        # planes apart, as C5) is the faster one (DESIGN s6.3d)
+        from paper_conf_icde_pirkmk14_b200 import column as cu
+        hsplit = args.c5_split
+        sd_host = cu.BWDColumn(cols["shipdate"], 32 - K_SHIP, residual_loc=_ar.AR_LOC_HOST_PINNED, device=ctx.dev,
+                               width_agree=ctx.allreduce_max_int, split=hsplit)
+        ab_e = algorithmic_bytes(cols, sd_host.w_major, hsplit, high_streamed=False)
+        e = run_e2e(ctx, q, ab_e, args.e2e_steps, sd_host=sd_host)
         e2e = {"value": (table_rows if args.workload == "c4" and args.scaling == "strong" else rows * world)
                * e["steps"] / (e["ms_total"] / 1e3), "unit": UNIT,
                "h2d_bytes_per_step": int(e["h2d_copied"] + e["zero_copy_64"]), "d2h_bytes_per_step": 32,
                "h2d_copied_bytes": int(e["h2d_copied"]), "h2d_zero_copy_bytes_64B": int(e["zero_copy_64"]),
                "ms_per_step": e["ms_total"] / e["steps"], "result_matches_device_run": e["result"][:2] == head["result"][:2],
                "path": "decomposed table in pinned host memory; per step: cudaMemcpyAsync H2D of the scanned majors, "
-                       "ar_select_refine_sum reading the shipdate residual and l_extendedprice zero-copy over the host "
+                       "ar_select_refine_sum reading the shipdate residual (split layout, "
+                       f"{hsplit} high planes apart) and l_extendedprice zero-copy over the host "
                        "link (only touched 64-B granules), [SUM allreduce,] D2H of (SUM, count, |cand|, |def|)"}
 
     del r

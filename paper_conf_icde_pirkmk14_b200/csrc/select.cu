@@ -503,9 +503,10 @@ __global__ void __launch_bounds__(NW * 32) select_tile_kernel(const __grid_const
 // totals before its group (accumulated with one atomic per tile by the select
 // kernel) plus the counts of the earlier tiles of its group -- one block-wide
 // reduction -- and the tiles' offsets inside the chunk a prefix over
-// kCompactTiles counts; then all 256 threads copy the chunk's entries with
-// coalesced loads (up to 12 per thread in flight) and stores.
-constexpr int kCompactTiles = 8;
+// kCompactTiles counts.  Then warp w copies tile w of the chunk on its own:
+// a contiguous slice to a contiguous destination, up to kDeep entries per lane
+// in flight, and drops the slice's L2 lines once its lanes have loaded them.
+constexpr int kCompactTiles = 8;   // = warps per CTA
 __global__ void __launch_bounds__(256) compact_kernel(const __grid_constant__ SelParams P) {
     asm volatile("griddepcontrol.wait;" ::: "memory");   // no-op unless launched as a dependent
     __shared__ unsigned long long red[8];
@@ -537,53 +538,40 @@ __global__ void __launch_bounds__(256) compact_kernel(const __grid_constant__ Se
         unsigned long long base = 0;
 #pragma unroll
         for (int w = 0; w < 8; ++w) base += red[w];
-        const uint32_t total = tpre[kCompactTiles];
-        if (t0 + kCompactTiles >= P.num_tiles && threadIdx.x == 0) *P.out_count = (long long)(base + total);
-        uint32_t pre[kCompactTiles + 1];
-#pragma unroll
-        for (int i = 0; i <= kCompactTiles; ++i) pre[i] = tpre[i];
-        constexpr int kDeep = 12;   // a chunk of ~8 tiles at Q6 selectivity is one round: all loads in flight
-        for (uint32_t e0 = 0; e0 < total; e0 += kDeep * 256) {
+        if (t0 + kCompactTiles >= P.num_tiles && threadIdx.x == 0) *P.out_count = (long long)(base + tpre[kCompactTiles]);
+        // warp `warp` copies tile t0 + warp
+        const uint32_t c = tpre[warp + 1] - tpre[warp];
+        const size_t so = (size_t)(t0 + warp) * P.tile_rows;
+        const uint32_t* sp = P.tmp_pos + so;
+        const uint32_t* sa = P.tmp_aux + so;
+        uint32_t* dp = P.out_pos + base + tpre[warp];
+        uint32_t* da = P.out_aux + base + tpre[warp];
+        constexpr int kDeep = 16;   // a tile at Q6 selectivity (~330 candidates) is one round
+        for (uint32_t e0 = 0; e0 < c; e0 += kDeep * 32) {
             uint32_t vp[kDeep], va[kDeep];
 #pragma unroll
             for (int k = 0; k < kDeep; ++k) {
-                const uint32_t e = e0 + k * 256 + threadIdx.x;
-                vp[k] = va[k] = 0u;
-                if (e < total) {
-                    // the tile holding entry e: the last i with pre[i] <= e (selects, no indexed
-                    // register array -- that would go to local memory)
-                    uint32_t ti = 0, tb = 0;
-#pragma unroll
-                    for (int i = 1; i < kCompactTiles; ++i) {
-                        const bool ge = e >= pre[i];
-                        ti = ge ? (uint32_t)i : ti;
-                        tb = ge ? pre[i] : tb;
-                    }
-                    const size_t src = (size_t)(t0 + ti) * P.tile_rows + (e - tb);
-                    vp[k] = __ldcs(P.tmp_pos + src);   // streaming: each slice is read once
-                    va[k] = __ldcs(P.tmp_aux + src);
+                const uint32_t e = e0 + k * 32 + lane;
+                if (e < c) {
+                    vp[k] = __ldcs(sp + e);   // streaming: each slice is read once
+                    va[k] = __ldcs(sa + e);
                 }
             }
 #pragma unroll
             for (int k = 0; k < kDeep; ++k) {
-                const uint32_t e = e0 + k * 256 + threadIdx.x;
-                if (e < total) {
-                    P.out_pos[base + e] = vp[k];
-                    P.out_aux[base + e] = va[k];
+                const uint32_t e = e0 + k * 32 + lane;
+                if (e < c) {
+                    dp[e] = vp[k];
+                    da[e] = va[k];
                 }
             }
         }
-        __syncthreads();   // every thread has loaded its entries before any line is discarded
-        // the slices are dead: drop their L2 lines without writing them back (slices are 128-B
-        // aligned, 32 entries per line)
-        for (int ti = 0; ti < kCompactTiles; ++ti) {
-            const uint32_t c = pre[ti + 1] - pre[ti];
-            const uint32_t* sp = P.tmp_pos + (size_t)(t0 + ti) * P.tile_rows;
-            const uint32_t* sa = P.tmp_aux + (size_t)(t0 + ti) * P.tile_rows;
-            for (uint32_t L = threadIdx.x; L < (c + 31) / 32; L += 256) {
-                asm volatile("discard.global.L2 [%0], 128;" ::"l"(sp + 32 * L) : "memory");
-                asm volatile("discard.global.L2 [%0], 128;" ::"l"(sa + 32 * L) : "memory");
-            }
+        __syncwarp();   // every lane has loaded its entries before the slice's lines are dropped
+        // the slice is dead: drop its L2 lines without writing them back (slices are 128-B aligned,
+        // 32 entries per line)
+        for (uint32_t L = lane; L < (c + 31) / 32; L += 32) {
+            asm volatile("discard.global.L2 [%0], 128;" ::"l"(sp + 32 * L) : "memory");
+            asm volatile("discard.global.L2 [%0], 128;" ::"l"(sa + 32 * L) : "memory");
         }
         __syncthreads();   // red / tpre are reused by the next chunk
     }

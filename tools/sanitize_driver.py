@@ -1,7 +1,8 @@
 """Small-size driver for compute-sanitizer (racecheck / synccheck / memcheck): one call of every
 hot-path entry point on Q6-shaped data, each result checked against the oracle so a run that
 skipped a kernel cannot pass silently.  Kernel selection knobs are environment variables read
-once per process (AR_RL_RESMODE, AR_FUSED_LEGACY, AR_SEL_BUFS), so tools/sanitize.sh runs this
+once per process (AR_RL_RESMODE, AR_FUSED_LEGACY, AR_SEL_BUFS; SPLIT = the l_shipdate residual in the
+split layout with that many high planes apart), so tools/sanitize.sh runs this
 driver once per configuration.
 
     compute-sanitizer --tool racecheck python tools/sanitize_driver.py
@@ -27,7 +28,7 @@ def main():
     his = [datagen.Q6_SHIPDATE[1], datagen.Q6_DISCOUNT[1], datagen.Q6_QUANTITY[1]]
     vals = [c["shipdate"], c["discount"], c["quantity"]]
     res_loc = int(os.environ.get("RES_LOC", "0"))
-    sd = cu.BWDColumn(c["shipdate"], 24, residual_loc=res_loc)
+    sd = cu.BWDColumn(c["shipdate"], 24, residual_loc=res_loc, split=int(os.environ.get("SPLIT", "0")))
     dc, qt = cu.BWDColumn(c["discount"], 32), cu.BWDColumn(c["quantity"], 32)
     ep = cu.BWDColumn(c["extprice"], 32, layout=_ar.AR_LAYOUT_PACKED)
     preds = [(sd, los[0], his[0]), (dc, los[1], his[1]), (qt, los[2], his[2])]
