@@ -49,7 +49,10 @@ constexpr int kSelWarps = 4;                      // consumer warps per CTA
 constexpr int kSelThreads = kSelWarps * 32;       // each consumer thread owns BPT consecutive 32-row blocks
 constexpr int kSelMinTileRows = kSelThreads * 32; // tile rows = 4096 * BPT (BPT in {1, 2, 4})
 constexpr int kStageEntries = 2048;
-constexpr int kGroupShift = 8;                    // select: 256 tiles per offset group
+#ifndef AR_GROUP_SHIFT
+#define AR_GROUP_SHIFT 8
+#endif
+constexpr int kGroupShift = AR_GROUP_SHIFT;       // select: 2^kGroupShift tiles per offset group
 
 struct SelParams {
     SelPred p[AR_MAX_PRED];
