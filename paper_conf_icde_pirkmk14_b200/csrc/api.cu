@@ -566,14 +566,49 @@ static ar_status setup_scan(const ar_pred* preds, int32_t npred, ard::SelParams&
         }
     }
     for (int c = 0; c < npred; ++c) {
-        const ard::SelPred& p = P.p[c];
+        ard::SelPred& p = P.p[c];
+        // Mode 2 (no definite bucket): an empty definite range chosen so that, on a non-definite
+        // candidate, "below it" <=> major == clo and "above it" <=> major == chi -- [clo + 1, clo]
+        // (chi == clo + 1) or [clo + 1, clo - 1] (chi == clo) -- the check code of the
+        // gathered-residual kernel's bit-packed residuals (as for split residuals, setup_scan above);
+        // where clo + 1 / clo - 1 leaves the w bits, that code bit is forced through scor.  Mode 1:
+        // the relaxation's own definite range has the property.
+        uint64_t dlo = p.dlo, dhi = p.dhi;
+        if (p.mode == 2) {
+            const uint64_t maxm = p.w >= 32 ? 0xffffffffull : ((1ull << p.w) - 1);
+            const uint32_t scor0 = p.k > 8 ? 0u : p.scor;
+            uint32_t scor = 0;
+            dlo = (uint64_t)p.clo + 1;
+            if (dlo > maxm) {
+                dlo = maxm;
+                scor |= 1u;
+            }
+            if (p.chi == p.clo) {
+                if (p.clo == 0) {
+                    dhi = 0;
+                    scor |= 2u;
+                } else {
+                    dhi = (uint64_t)p.clo - 1;
+                }
+            } else {
+                dhi = p.clo;
+            }
+            if (p.k > 8) p.scor = scor; else p.scor = scor0;
+        }
         for (uint32_t j = 0; j < p.w; ++j) {
             uint32_t* m = P.pm[p.ashift + j];
             m[0] = 0u - ((p.clo >> j) & 1u);
             m[1] = 0u - ((p.chi >> j) & 1u);
-            // mode 2 (no definite bucket): an empty definite range, lo = 2^w - 1 > hi = 0
-            m[2] = p.mode == 2 ? ~0u : 0u - ((p.dlo >> j) & 1u);
-            m[3] = p.mode == 2 ? 0u : 0u - ((p.dhi >> j) & 1u);
+            m[2] = 0u - (uint32_t)((dlo >> j) & 1u);
+            m[3] = 0u - (uint32_t)((dhi >> j) & 1u);
+        }
+        if (p.k > 8 && p.mode != 0) {   // bit-packed residual: the low k bits of the exact bounds (check entries)
+            const uint64_t maxu = (uint64_t)p.k + p.w >= 32 ? 0xffffffffull : ((1ull << (p.k + p.w)) - 1);
+            const uint64_t ulo = p.lo < p.base ? 0 : (uint64_t)(p.lo - p.base);
+            const uint64_t uhi = std::min<uint64_t>((uint64_t)(p.hi - p.base), maxu);
+            const uint64_t km = p.k >= 32 ? 0xffffffffull : ((1ull << p.k) - 1);
+            p.sllo = (uint32_t)(ulo & km);
+            p.slhi = (uint32_t)(uhi & km);
         }
     }
     P.npred = npred;

@@ -77,9 +77,15 @@ __device__ __forceinline__ uint32_t* low_word(uint32_t* sl, uint32_t lane, int j
 // left undecided; its KL low planes (landed with the aggregate) decide it
 // against the low bits of the exact bounds, and a row that qualifies counts
 // in `nchk`.
-template <int KL = 0>
+// KP > 0 (gathered-residual kernel): the check entries are the non-definite
+// candidates of a predicate with a bit-packed KP-bit residual; its two landed
+// words and bit offset (info bits 10-14) give the residual, tested the same
+// way (the candidate's bucket is that of lo or of hi).  has_g = false (COUNT):
+// the ring holds check entries only and nothing is summed.
+template <int KL = 0, int KP = 0>
 __device__ __forceinline__ unsigned long long drain(uint32_t* sl, uint32_t lane, uint32_t gmask, uint32_t gbase,
-                                                    const SelPred* sp = nullptr, uint32_t* nchk = nullptr) {
+                                                    const SelPred* sp = nullptr, uint32_t* nchk = nullptr,
+                                                    bool has_g = true) {
     const uint32_t info = sl[64 + lane];
     if (!(info >> 31)) return 0ull;
     if constexpr (KL > 0) {
@@ -92,6 +98,16 @@ __device__ __forceinline__ unsigned long long drain(uint32_t* sl, uint32_t lane,
             if (((code & 1u) && low < sp->sllo) || ((code & 2u) && low > sp->slhi)) return 0ull;
             ++*nchk;
         }
+    }
+    if constexpr (KP > 0) {
+        const uint32_t code = (info >> 8) & 3u;
+        if (code) {
+            const uint32_t r = __funnelshift_r(*low_word<2>(sl, lane, 0), *low_word<2>(sl, lane, 1), (info >> 10) & 31u) &
+                               (KP >= 32 ? 0xffffffffu : ((1u << KP) - 1u));
+            if (((code & 1u) && r < sp->sllo) || ((code & 2u) && r > sp->slhi)) return 0ull;
+            ++*nchk;
+        }
+        if (!has_g) return 0ull;
     }
     // bits of the hi word past the value's width are masked off, so a slot whose
     // value did not straddle (hi word not copied) reads harmless stale data
@@ -439,7 +455,13 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
     constexpr int KS = S::ksum();
     // a compiled split residual (predicate SP): rows its high planes leave undecided go to the ring as check
     // entries and their KL low planes are gathered with the aggregate (no synchronous gather)
-    constexpr int SP = S::split(), KL = S::kl(), SPi = SP < 0 ? 0 : SP, SW = slot_words(KL);
+    constexpr int SP = S::split(), KL = S::kl(), SPi = SP < 0 ? 0 : SP;
+    // a bit-packed residual (predicate PC, k > 8, the query's only decomposed predicate): its non-definite
+    // candidates go to the ring as check entries, their residual (1-2 words) gathered with the aggregate
+    constexpr int PC = S::pk(), PCi = PC < 0 ? 0 : PC, KP = PC < 0 ? 0 : S::k(PCi);
+    constexpr int CKi = SP >= 0 ? SPi : PCi;                  // the predicate whose check entries the ring holds
+    constexpr bool kChk = KL > 0 || KP > 0;
+    constexpr int SW = slot_words(KL > 0 ? KL : (KP > 0 ? 2 : 0));
     extern __shared__ __align__(128) unsigned char smem[];
     uint64_t* full = reinterpret_cast<uint64_t*>(smem);
     uint64_t* empty = full + P.nstages;
@@ -470,6 +492,8 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
 
     const bool list = P.rl_list != 0;
     const bool direct = !list && P.nagg > 0;
+    const bool cring = KP > 0 && P.nagg == 0;   // COUNT with packed check entries: a ring of check entries only
+    const bool ring_on = list || cring;
     const AggCol& G = P.a[P.gidx];
     const uint32_t gmask = G.w >= 32 ? 0xffffffffu : ((1u << G.w) - 1u);
     uint32_t ncand = 0, ndef = 0, nres = 0, nchk = 0;
@@ -481,13 +505,28 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
         uint32_t info = 0u, f = 0u;
         if (lane < take) {
             const uint2 e = ring[(rhead + lane) & rmask];
-            const uint64_t bit = (uint64_t)e.x * G.w;
-            const uint32_t* src = G.major + (bit >> 5);
-            const uint32_t sh = (uint32_t)(bit & 31);
-            cp_async4(sl + lane, src);
-            if (sh + G.w > 32u) cp_async4(sl + 32 + lane, src + 1);
-            info = 0x80000000u | sh;
+            info = 0x80000000u;
+            if (list) {
+                const uint64_t bit = (uint64_t)e.x * G.w;
+                const uint32_t* src = G.major + (bit >> 5);
+                const uint32_t sh = (uint32_t)(bit & 31);
+                cp_async4(sl + lane, src);
+                if (sh + G.w > 32u) cp_async4(sl + 32 + lane, src + 1);
+                info |= sh;
+            }
             f = e.y;
+            if constexpr (KP > 0) {
+                const uint32_t code = e.y >> 30;   // check code (host: factors < 2^30)
+                f = e.y & 0x3fffffffu;
+                if (code) {   // the candidate's bit-packed residual: bits [row * KP, row * KP + KP)
+                    const uint64_t rb = (uint64_t)e.x * KP;
+                    const uint32_t* rp = P.p[PCi].residual + (rb >> 5);
+                    const uint32_t rsh = (uint32_t)(rb & 31);
+                    cp_async4(low_word<2>(sl, lane, 0), rp);
+                    if (rsh + KP > 32u) cp_async4(low_word<2>(sl, lane, 1), rp + 1);
+                    info |= (code << 8) | (rsh << 10);
+                }
+            }
             if constexpr (KL > 0) {
                 const uint32_t code = e.y >> 30;   // check code (host: factors < 2^30)
                 f = e.y & 0x3fffffffu;
@@ -511,7 +550,7 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
         rcnt -= take;
         if (gseq >= (uint32_t)kDepth) {
             cp_async_wait<kDepth - 1>();
-            sum += drain<KL>(gs + (gseq % kDepth) * SW, lane, gmask, G.base, &P.p[SPi], &nchk);
+            sum += drain<KL, KP>(gs + (gseq % kDepth) * SW, lane, gmask, G.base, &P.p[CKi], &nchk, list);
         }
     };
 
@@ -522,7 +561,7 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
 #pragma unroll
         for (int b = 0; b < BPT; ++b) nres += __popc(xm[b] & ~(ck0[b] | ck1[b]));   // check rows count when drained
         auto code_at = [&](int b, uint32_t l) -> uint32_t {   // check code << 30 of row l of block b
-            if constexpr (KL > 0)
+            if constexpr (kChk)
                 return (((ck0[b] >> l) & 1u) << 30) | (((ck1[b] >> l) & 1u) << 31);
             else
                 return 0u;
@@ -554,7 +593,7 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
             }
             return;
         }
-        if (!list) return;
+        if (!ring_on) return;
         uint32_t my = 0;
 #pragma unroll
         for (int b = 0; b < BPT; ++b) my += __popc(xm[b]);
@@ -662,7 +701,7 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
                         const uint32_t und = gl | gh;
                         u0 &= und;
                         u1 &= und;
-                    } else if constexpr (K > 0) {
+                    } else if constexpr (K > 0 && K <= 8) {
                         uint32_t x[W];
                         lds_words<W>(x, stg + P.p[C].soff + blk * W);
                         const uint32_t H = P.p[C].rsplit;
@@ -735,7 +774,7 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
         const bool full_tile = tile_r0 + (int64_t)P.tile_rows <= P.n;
 
         // phase A (tile t): candidate / definite masks on the majors
-        uint32_t dmk[BPT], ndm[BPT];
+        uint32_t dmk[BPT], ndm[BPT], ul_[BPT], uh_[BPT];
 #pragma unroll
         for (int b = 0; b < BPT; ++b) {
             const uint32_t blk = b * NT + threadIdx.x;
@@ -743,12 +782,29 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
             uint32_t cm, dm, em;
             uint32_t ul, uh;
             eval_block<S, false>(P, stg, blk, vm, cm, dm, em, ul, uh);
+            ul_[b] = ul;
+            uh_[b] = uh;
             ncand += __popc(cm);
             ndef += __popc(dm);
             dmk[b] = dm;
             ndm[b] = cm & ~dm;
         }
-        if constexpr (KS > 0) {
+        if constexpr (KP > 0) {
+            // bit-packed residual: definite rows are results, non-definite candidates check entries whose
+            // code (bucket of lo / of hi) the pass turns into a residual gather (Alg. 2 on those rows only)
+            uint32_t xm[BPT], k0[BPT], k1[BPT];
+#pragma unroll
+            for (int b = 0; b < BPT; ++b) {
+                const uint32_t nd = ndm[b];
+                k0[b] = nd & (ul_[b] | (0u - (P.p[PCi].scor & 1u)));
+                k1[b] = nd & (uh_[b] | (0u - ((P.p[PCi].scor >> 1) & 1u)));
+                xm[b] = cring ? nd : (dmk[b] | nd);
+                if (cring) nres += __popc(dmk[b]);   // COUNT: definite rows never enter the ring
+            }
+            consume(stg, tile_r0, xm, k0, k1);
+            __syncwarp();
+            if (lane == 0) mbar_arrive(empty + s);
+        } else if constexpr (KS > 0) {
             if (pt >= 0) phase_b();          // the previous tile's residual gathers have had a tile to land
             // gather the residual sectors of this tile's blocks with a non-definite candidate
 #pragma unroll
@@ -757,7 +813,7 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
                 static_for<S::N>([&](auto cc) {
                     constexpr int C = decltype(cc)::value;
                     constexpr int K = S::k(C), KO = S::kofs(C);
-                    if constexpr (K > 0) {
+                    if constexpr (K > 0 && K <= 8) {
                         const uint32_t H = P.p[C].rsplit;
                         if (H == 0) {
                             res_issue<K>(&rres[b][KO], P.p[C].residual, gblk, ndm[b] != 0u, P.p[C].res_hint != 0u);
@@ -783,7 +839,7 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
             __syncwarp();
             if (lane == 0) mbar_arrive(empty + s);
         }
-        if (list) {
+        if (ring_on) {
             while (rcnt >= 32) pass(32);
             __syncwarp();
         }
@@ -791,11 +847,11 @@ __global__ void __launch_bounds__((NW + 1) * 32, 2) fused_rg_kernel(const __grid
     if constexpr (KS > 0) {
         if (pt >= 0) phase_b();
     }
-    if (list) {
+    if (ring_on) {
         while (rcnt > 0) pass(min(rcnt, 32u));
         cp_async_wait<0>();
         for (uint32_t g = gseq >= (uint32_t)kDepth ? gseq - kDepth + 1 : 0; g < gseq; ++g)
-            sum += drain<KL>(gs + (g % kDepth) * SW, lane, gmask, G.base, &P.p[SPi], &nchk);
+            sum += drain<KL, KP>(gs + (g % kDepth) * SW, lane, gmask, G.base, &P.p[CKi], &nchk, list);
     }
 
     unsigned long long c0 = ncand, c1 = ndef, c2 = nres + nchk;
@@ -914,6 +970,18 @@ bool rg_match(const ard::SelParams& P, bool split_ok) {
     }
     return true;
 }
+// a bit-packed residual (k > 8) as check entries of the gathered-residual kernel: the query's only
+// decomposed predicate, SUM through the result ring with the other factor below 2^30, or COUNT
+inline bool rg_packed_ok(const ard::SelParams& P) {
+    int nk = 0, np = 0;
+    for (int c = 0; c < P.npred; ++c) {
+        nk += P.p[c].k > 0 ? 1 : 0;
+        np += (P.p[c].k > 8 && P.p[c].residual != nullptr) ? 1 : 0;
+    }
+    const bool mp_small =
+        P.rl_mpred < 0 || (P.p[P.rl_mpred].base == 0 && P.p[P.rl_mpred].w + P.p[P.rl_mpred].k <= 30);
+    return nk == 1 && np == 1 && ((P.rl_list && mp_small) || P.nagg == 0);
+}
 inline bool rg_split_ok(const ard::SelParams& P) {
     int ns = 0;
     for (int c = 0; c < P.npred; ++c) ns += P.p[c].rsplit ? 1 : 0;
@@ -935,6 +1003,14 @@ RlFn rg_find(const ard::SelParams& P, int cfg) {
     AR_RG_TRY(WK(4, 8), WK(4, 0), WK(6, 0))
     AR_RG_TRY(WK(24, 8))
     AR_RG_TRY(WK(24, 8), WK(24, 8))
+#undef AR_RG_TRY
+    // bit-packed residuals (C3 at M = 8 / 16 / 12, BASELINE configs[2]) as check entries
+#define AR_RG_TRY(...) \
+    if (pok && rg_match<__VA_ARGS__>(P, false)) return rg_pick<__VA_ARGS__>(cfg);
+    const bool pok = rg_packed_ok(P);
+    AR_RG_TRY(WK(8, 24))
+    AR_RG_TRY(WK(16, 16))
+    AR_RG_TRY(WK(12, 20))
 #undef AR_RG_TRY
     return {nullptr, 0, 0};
 }
@@ -991,6 +1067,8 @@ size_t rl_smem_bytes(const ard::SelParams& P, uint32_t nstages, int nw, bool rg)
     } else if (rg_split_ok(P)) {   // a compiled split shape uses KL low-plane words per slot lane
         for (int c = 0; c < P.npred; ++c)
             if (P.p[c].rsplit) kl = P.p[c].k - P.p[c].rsplit;
+    } else if (rg_packed_ok(P)) {   // packed check entries: two residual words per slot lane
+        kl = 2;
     }
     return head + (size_t)nstages * P.stage_words * 4 + (size_t)nw * P.rl_ring * 8 +
            (size_t)nw * (rg ? ard::rl::kDepth : P.rl_depth) * ard::rl::slot_words((int)kl) * 4;
@@ -1044,6 +1122,7 @@ ar_status launch_fused_rl(const ard::SelParams& P0, const ar_column* const* cols
     for (int c = 0; c < P.npred && rg_ok; ++c)
         if (P.p[c].k > 0)
             rg_ok = (P.p[c].rlayout & 0xffu) == AR_LAYOUT_SLICED && P.p[c].residual != nullptr && P.p[c].k <= 8;
+    if (!rg_ok && fac_k0 && rg_packed_ok(P)) rg_ok = true;   // bit-packed residual: check entries
     RlFn k{nullptr, 0, 0};
     bool rg = false;
     // streamed residual planes first (device residuals: a stream of every block's planes beats

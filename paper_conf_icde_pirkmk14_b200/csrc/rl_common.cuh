@@ -44,14 +44,20 @@ struct Shape {
         return -1;
     }
     static constexpr int kl() { return split() < 0 ? 0 : k(split()) - h(split()); }   // gathered low planes
+    static constexpr int pk() {      // the one predicate with a bit-packed residual (k > 8), or -1
+        for (int i = 0; i < N; ++i)
+            if (k(i) > 8) return i;
+        return -1;
+    }
+    static constexpr int rk(int c) { return k(c) <= 8 ? k(c) : 0; }   // SLICED residual words per block
     static constexpr int off(int c) {   // global plane index of predicate c (its ashift)
         int o = 0;
         for (int i = 0; i < c; ++i) o += w(i);
         return o;
     }
-    static constexpr int kofs(int c) {  // first residual word of predicate c in a block's residual words
+    static constexpr int kofs(int c) {  // first SLICED residual word of predicate c in a block's residual words
         int o = 0;
-        for (int i = 0; i < c; ++i) o += k(i);
+        for (int i = 0; i < c; ++i) o += rk(i);
         return o;
     }
     static constexpr int ksum() { return kofs(N); }
@@ -63,8 +69,9 @@ struct Shape {
 struct DynShape {
     static constexpr bool kDynamic = true;
     static constexpr int N = 0;
-    static constexpr int split() { return -1; }   // split residuals need a compiled shape
+    static constexpr int split() { return -1; }   // split / packed residuals need a compiled shape
     static constexpr int kl() { return 0; }
+    static constexpr int pk() { return -1; }
 };
 template <int... WK>
 struct ShapeOf {
@@ -190,6 +197,10 @@ __device__ __forceinline__ void eval_block(const SelParams& P, const uint32_t* s
                 dh = brsub(x[j], P.pm[O + j][3], dh);
             }
             dm &= ~(dl | dh);
+            if constexpr (K > 8) {   // bit-packed residual (gathered-residual kernel): the check code bits
+                ul = dl;
+                uh = dh;
+            }
             if constexpr (kExact && S::h(C) > 0) {
                 constexpr int H = S::h(C);
                 uint32_t r[H];
