@@ -1157,33 +1157,63 @@ ar_status launch_fused_rl(const ard::SelParams& P0, const ar_column* const* cols
     static const int depth_env = getenv("AR_RL_DEPTH") ? atoi(getenv("AR_RL_DEPTH")) : 4;
     P.rl_depth = depth_env == 8 ? 8u : 4u;
 
-    // deepest stage ring (<= 8, >= 3) that keeps 2 CTAs per SM, else 1 CTA with >= 2 stages
-    opt_in_max_smem(k.fn);
-    const int threads = (k.nw + 1) * 32;
-    uint32_t stages = 0;
-    int occ = 0;
+    // deepest stage ring (<= max_st) that keeps `want` CTAs per SM, else fewer CTAs with >= 2 stages
     static const int force_st = getenv("AR_STAGES") ? atoi(getenv("AR_STAGES")) : 0;
     static const int want_ctas = getenv("AR_RL_CTAS") ? atoi(getenv("AR_RL_CTAS")) : 2;
     // the result-ring kernel runs 3 stages (deeper rings measured slower at C4 / C2: the stream's extra
     // TMA requests delay the aggregate gathers, DESIGN s6.3); the two-phase kernel up to 8
     const uint32_t max_st = rg ? 8u : 3u;
-    for (int target = std::max(want_ctas, 1); target >= 1 && !stages; --target)
-        for (uint32_t st = force_st > 0 ? 8u : max_st; st >= 2; --st) {
-            if (force_st > 0 && (int)st != force_st) continue;
-            // the two-phase kernel holds two stages (phase B of tile t - 1 while tile t is decided)
-            if (target >= 2 && st < (rg ? 4u : 3u) && force_st <= 0) break;
-            int o = 0;
-            cudaOccupancyMaxActiveBlocksPerMultiprocessor(&o, k.fn, threads, rl_smem_bytes(P, st, k.nw, rg));
-            if (o >= target) {
-                stages = st;
-                occ = o;
-                break;
+    auto fit = [&](const RlFn& kk, const ard::SelParams& PP, int want, uint32_t* st_out, int* occ_out) {
+        opt_in_max_smem(kk.fn);
+        const int thr = (kk.nw + 1) * 32;
+        *st_out = 0;
+        *occ_out = 0;
+        for (int target = std::max(want, 1); target >= 1 && !*st_out; --target)
+            for (uint32_t st = force_st > 0 ? 8u : max_st; st >= 2; --st) {
+                if (force_st > 0 && (int)st != force_st) continue;
+                // the two-phase kernel holds two stages (phase B of tile t - 1 while tile t is decided)
+                if (target >= 2 && st < (rg ? 4u : 3u) && force_st <= 0) break;
+                int o = 0;
+                cudaOccupancyMaxActiveBlocksPerMultiprocessor(&o, kk.fn, thr, rl_smem_bytes(PP, st, kk.nw, rg));
+                if (o >= target) {
+                    *st_out = st;
+                    *occ_out = std::min(o, std::max(want, 1));
+                    break;
+                }
+            }
+        cudaGetLastError();
+    };
+    uint32_t stages = 0;
+    int occ = 0;
+    fit(k, P, want_ctas, &stages, &occ);
+    // wide stages (e.g. a 24/8 column: 32 planes = 32 KB per 8192-row tile) leave one 8-warp CTA per SM:
+    // then 4-warp CTAs on 4096-row tiles, as many as fit (C3 at M = 24: 0.495 vs 0.562 ms), unless
+    // AR_RL_CFG chose the configuration
+    if (!getenv("AR_RL_CFG") && occ < 2) {
+        ard::SelParams P4 = P;
+        const RlFn k4 = rg ? rg_find(P4, 4) : rl_find(P4, 4);
+        if (k4.fn) {
+            retile(P4, k4.tile_rows);
+            uint32_t st4 = 0;
+            int occ4 = 0;
+            fit(k4, P4, 3, &st4, &occ4);
+            // at equal resident warps the smaller tiles win too (two pipelines per SM, finer tail)
+            if (st4 && occ4 * k4.nw >= occ * k.nw) {
+                k = k4;
+                P = P4;
+                stages = st4;
+                occ = occ4;
             }
         }
-    cudaGetLastError();
+    }
+    const int threads = (k.nw + 1) * 32;
+    static const bool dbg = getenv("AR_DEBUG_LAUNCH") != nullptr;
+    if (dbg)
+        fprintf(stderr, "launch_fused_rl: %s nw=%d tile=%u stages=%u ctas/SM=%d smem=%zu\n", rg ? "rg" : "rl", k.nw,
+                k.tile_rows, stages, occ, rl_smem_bytes(P, stages ? stages : 1, k.nw, rg));
     if (!stages) return AR_OK;
     P.nstages = stages;
-    const int grid = (int)std::min<int64_t>(P.num_tiles, (int64_t)num_sms() * std::min(occ, std::max(want_ctas, 1)));
+    const int grid = (int)std::min<int64_t>(P.num_tiles, (int64_t)num_sms() * occ);
     if (ws && grid > kSrsMaxGrid) return AR_OK;
     void* args[] = {&P};
     cudaLaunchConfig_t cfg = {};

@@ -83,6 +83,18 @@ def main():
     got = {int(keys[i]): int(gs[1, i].item()) for i in range(gr.ngroups()) if gs[1, i].item() > 0}
     k2, c2, _ = oracle.select_group_sum_keys(vals, los, his, c["quantity"])
     assert got == dict(zip(k2.tolist(), c2.tolist()))
+
+    # one pass over a bit-packed residual (k = 24, C3 at M = 8): check entries, COUNT and SUM
+    v = datagen.uniform_u32(91, n)
+    col = cu.BWDColumn(v, 8)
+    lo, hi = 0x5A5A5A37, 0x5A5A5A37 + (1 << 32) // 100
+    _, pc, ps = oracle.select_sum([v], [lo], [hi], [c["extprice"]], positions=False)
+    pcp, pcd = oracle.approx_select([v], [24], [lo], [hi])
+    for aggs, want in (([], 0), ([ep], ps)):
+        cu.select_refine_sum([(col, lo, hi)], aggs, o4)
+        torch.cuda.synchronize()
+        assert o4.tolist() == [want, pc, pcp.size, int(pcd.sum())], o4.tolist()
+    ran.append(_ar.ar_last_scan_kernel() + "(packed)")
     print("sanitize driver ok:", ",".join(ran), flush=True)
 
 
