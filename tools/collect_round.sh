@@ -10,7 +10,7 @@ tail -3 gpurun_out/gpu_tests.log > profiles/$R/gpu_tests_tail.txt
 cat gpurun_out/smoke.log > profiles/$R/smoke.txt
 cp gpurun_out/launches.csv profiles/$R/launches.csv
 cp gpurun_out/round/launches_summary.txt profiles/$R/launches_summary.txt
-for rep in full_fused_c4 full_staged_c4 full_c2; do
+for rep in full_fused_c4 full_staged_c4 full_c2 full_refine_c4; do
   cp gpurun_out/round/ncu_$rep.txt profiles/$R/ncu_$rep.txt
 done
 cp gpurun_out/round/traffic.json profiles/traffic.json

@@ -37,6 +37,8 @@ def main():
     cands = cu.CandidateList(n)
     ws = cu.Workspace(_ar.ar_select_ws_bytes(n))
     out = torch.zeros(4, dtype=torch.int64, device="cuda")
+    pos = cu.PositionList(n) if "refine" in variants else None
+    wr = cu.Workspace(_ar.ar_refine_ws_bytes(n)) if "refine" in variants else None
     flush = torch.empty(512 * 1024 * 1024, dtype=torch.uint8, device="cuda")
     for v in variants:
         for _ in range(steps):
@@ -44,6 +46,10 @@ def main():
             if v == "staged":
                 cu.approx_select(preds, cands, ws, carry=True)
                 cu.refine_sum(cands, preds, [ep, dc], out[0:1], out[1:2])
+            elif v == "refine":   # a5 as its own step: ordered positions out (ar_refine)
+                cu.approx_select(preds, cands, ws, carry=True)
+                cu.refine(cands, preds, pos, wr)
+                out[1] = pos.count_t[0]
             else:
                 cu.select_refine_sum(preds, [ep, dc], out)
         torch.cuda.synchronize()

@@ -18,6 +18,9 @@ SF=100 SEED=4 VARIANTS=fused timeout 900 ncu --set full --clock-control none --i
 SF=100 SEED=4 VARIANTS=staged timeout 900 ncu --set full --clock-control none --import-source on \
     -k regex:"select_tile_kernel|compact_kernel|refine_sum" -s 3 -c 3 -o gpurun_out/full_staged_c4 python tools/profile_step.py \
     > gpurun_out/full_staged_c4.log 2>&1
+SF=100 SEED=4 VARIANTS=refine timeout 900 ncu --set full --clock-control none --import-source on \
+    -k regex:"refine_kernel" -s 1 -c 1 -o gpurun_out/full_refine_c4 python tools/profile_step.py \
+    > gpurun_out/full_refine_c4.log 2>&1
 SF=10 SEED=2 VARIANTS=fused,staged timeout 900 ncu --set full --clock-control none --import-source on \
     -k regex:"fused_rl_kernel|select_tile_kernel|compact_kernel|refine_sum" -s 3 -c 4 -o gpurun_out/full_c2 python tools/profile_step.py \
     > gpurun_out/full_c2.log 2>&1
@@ -25,11 +28,11 @@ SF=10 SEED=2 VARIANTS=fused,staged timeout 900 ncu --set full --clock-control no
 # summary and traffic.json (bench.py reads profiles/traffic.json; tools/collect_round.sh installs it);
 # only the C4 fused report is kept
 mkdir -p gpurun_out/round
-for rep in full_fused_c4 full_staged_c4 full_c2; do
+for rep in full_fused_c4 full_staged_c4 full_c2 full_refine_c4; do
   python tools/ncu_summary.py gpurun_out/$rep.ncu-rep > gpurun_out/round/ncu_$rep.txt 2>&1
 done
 cp profiles/traffic.json gpurun_out/round/traffic.json 2>/dev/null
 TRAFFIC_JSON=gpurun_out/round/traffic.json python tools/ncu_traffic.py c4 gpurun_out/full_fused_c4.ncu-rep gpurun_out/full_staged_c4.ncu-rep > /dev/null
 TRAFFIC_JSON=gpurun_out/round/traffic.json python tools/ncu_traffic.py c2 gpurun_out/full_c2.ncu-rep > /dev/null
 python tools/launch_summary.py gpurun_out/launches.csv "python bench.py --steps 20 --warmup 3 --no-cpu --e2e-steps 0 --no-c5 --latency-reps 3 --replays 0" > gpurun_out/round/launches_summary.txt 2>&1
-rm -f gpurun_out/full_staged_c4.ncu-rep gpurun_out/full_c2.ncu-rep
+rm -f gpurun_out/full_staged_c4.ncu-rep gpurun_out/full_c2.ncu-rep gpurun_out/full_refine_c4.ncu-rep
