@@ -38,8 +38,8 @@ def _bounds(k):
     ]
 
 
-@pytest.mark.parametrize("major_bits", [8, 12, 16])
-def test_gpu_packed_check_entries(cu, major_bits):
+@pytest.mark.parametrize("major_bits,loc", [(8, 0), (12, 0), (16, 0), (8, 1), (16, 1)])
+def test_gpu_packed_check_entries(cu, major_bits, loc):
     from paper_conf_icde_pirkmk14_b200 import _ar
     k = 32 - major_bits
     n = 5 * 8192 + 3333
@@ -48,7 +48,7 @@ def test_gpu_packed_check_entries(cu, major_bits):
     # plant rows at the bucket edges the bounds below test (the data must reach the first / last bucket)
     v[:40] = np.arange(40, dtype=np.uint32) * 3
     v[40:80] = (np.uint64(2**32 - 1) - np.arange(40, dtype=np.uint64) * 3).astype(np.uint32)
-    col = cu.BWDColumn(v, major_bits)
+    col = cu.BWDColumn(v, major_bits, residual_loc=loc)   # loc 1: the residual read over the host link
     assert col.desc.k == k and col.desc.w_major == major_bits
     ag = cu.BWDColumn(agg, 32, layout=_ar.AR_LAYOUT_PACKED)
     for lo, hi in _bounds(k):
