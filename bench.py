@@ -575,6 +575,7 @@ class Runner:
                 ctx.rec(ev[0], external=True)
             _ar.ar_approx_select(q.preds, _ar.AR_SELECT_CARRY_APPR, self.cands.c, self.ws_sel.ptr,
                                  self.ws_sel.nbytes, ctx.s_ptr)
+            self.select_kernel = _ar.ar_last_scan_kernel()
             if ev is not None:
                 ctx.rec(ev[1], external=True)
             if ctx.dist_h:       # candidate-count allgather + prefix (a4), overlapping the refine
@@ -879,12 +880,13 @@ def ours(args):
     r = Runner(ctx, q, K)
     names = {"fused": r.kernel_names("fused"), "staged": None}
     names["staged"] = r.kernel_names("staged")
-    KERNELS = {"staged": ["select_tile_kernel", "compact_kernel", names["staged"] or "refine_sum_kernel"],
+    sel_kernels = (["select_rr_kernel"] if getattr(r, "select_kernel", "") == "select_rr_kernel"
+                   else ["select_tile_kernel", "compact_kernel"])
+    KERNELS = {"staged": sel_kernels + [names["staged"] or "refine_sum_kernel"],
                "fused": [names["fused"] or "fused_kernel"]}
     per_kernel_bytes = {"fused": ab["total"], "select": ab["scan"] + ab["cand_list_bytes"],
                         "refine_sum": ab["cand_list_bytes"] + ab["gather"] + 16.0}
-    kname = {"fused": KERNELS["fused"][0], "select": "select_tile_kernel+compact_kernel",
-             "refine_sum": KERNELS["staged"][2]}
+    kname = {"fused": KERNELS["fused"][0], "select": "+".join(sel_kernels), "refine_sum": KERNELS["staged"][-1]}
 
     variants = [args.variant] + [v for v in ("fused", "staged") if v != args.variant and not args.only]
     sampler = ClockSampler(torch.cuda.current_device() if "CUDA_VISIBLE_DEVICES" not in os.environ else ctx.local)

@@ -165,7 +165,8 @@ const char* ar_version(void);
 /* Name of the main kernel the calling thread's last ar_select_refine_sum,
  * ar_approx_select or ar_refine_sum launched: "fused_rl_kernel" (result-ring
  * one-pass kernel), "fused_kernel" (general one-pass kernel),
- * "select_tile_kernel" (ordered select), "refine_sum_sliced_kernel" /
+ * "select_rr_kernel" / "select_tile_kernel" (ordered select),
+ * "refine_sum_sliced_kernel" /
  * "refine_sum_kernel" (refine + SUM), "" (none: empty input or an error).
  * Static storage; for tests and benchmarks that must know which path ran. */
 const char* ar_last_scan_kernel(void);

@@ -656,6 +656,27 @@ ar_status ar_approx_select(const ar_pred* preds, int32_t npred, int32_t flags, a
     // workspace (sel_ws): group sums and tile counts (zeroed), tile slices
     const SelWs L = sel_ws(n);
     char* base = (char*)(((uintptr_t)ws + 127) & ~uintptr_t(127));
+    // one-kernel ordered select (default): round-robin look-back over per-tile counts (status words,
+    // zeroed), entries written once at their final offsets -- no tile slices, no compaction
+    static const int rr = env_int("AR_SEL_RR", 1);
+    const void* rr_fn = rr ? select_rr_kernel_fn(P) : nullptr;
+    if (rr_fn) {
+        static const int rr_bufs = std::min(4, std::max(1, env_int("AR_SEL_RR_BUFS", 1)));
+        P.nstages = (uint32_t)rr_bufs;
+        P.status = (unsigned long long*)base;
+        AR_TRY_CUDA(cudaMemsetAsync(base, 0, 8 * (size_t)P.num_tiles, s));
+        const size_t smem = select_rr_smem_bytes(P.stage_words, P.nstages);
+        const int occ = select_occupancy(rr_fn, smem, false);
+        if (occ > 0) {
+            static const int rr_ctas = env_int("AR_SEL_RR_CTAS", 0);   // CTAs per SM (0: as many as fit)
+            const int per_sm = rr_ctas > 0 ? std::min(rr_ctas, occ) : occ;
+            static const int max_grid = env_int("AR_SEL_RR_GRID", 0);   // tests: force several rounds
+            int grid = (int)std::min<int64_t>(P.num_tiles, (int64_t)num_sms() * per_sm);
+            if (max_grid > 0) grid = std::min(grid, max_grid);
+            g_last_scan = "select_rr_kernel";
+            return launch_select_rr(rr_fn, P, grid, smem, s);
+        }
+    }
     P.group_sum = (unsigned long long*)base;
     P.tile_count = (uint32_t*)(base + 8 * L.groups);
     AR_TRY_CUDA(cudaMemsetAsync(base, 0, L.counts_bytes, s));

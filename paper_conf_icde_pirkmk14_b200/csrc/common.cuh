@@ -211,6 +211,7 @@ __device__ __forceinline__ unsigned long long ld_relaxed(const unsigned long lon
 }
 
 constexpr unsigned long long kFlagAgg = 1ull << 62;
+constexpr unsigned long long kFlagInc = 1ull << 63;   // inclusive prefix (select_rr_kernel)
 constexpr unsigned long long kValueMask = (1ull << 62) - 1;
 
 // Round-robin persistent kernels (tile t = blockIdx + i * gridDim, every CTA

@@ -49,6 +49,7 @@ constexpr int kSelWarps = 4;                      // consumer warps per CTA
 constexpr int kSelThreads = kSelWarps * 32;       // each consumer thread owns BPT consecutive 32-row blocks
 constexpr int kSelMinTileRows = kSelThreads * 32; // tile rows = 4096 * BPT (BPT in {1, 2, 4})
 constexpr int kStageEntries = 2048;
+constexpr int kRrEntries = 512;    // select_rr_kernel: staged entries per tile buffer (denser tiles resolve at once)
 #ifndef AR_GROUP_SHIFT
 #define AR_GROUP_SHIFT 8
 #endif
@@ -251,6 +252,9 @@ size_t select_smem_bytes(uint32_t stage_words, uint32_t nstages, bool staging);
 int kernel_warps(bool fused);
 int kernel_bpt(bool fused);
 const void* select_kernel_fn(const ard::SelParams& P, bool fused);
+const void* select_rr_kernel_fn(const ard::SelParams& P);
+size_t select_rr_smem_bytes(uint32_t stage_words, uint32_t nstages);
+ar_status launch_select_rr(const void* fn, const ard::SelParams& P, int grid, size_t smem, cudaStream_t s);
 int select_occupancy(const void* fn, size_t smem, bool fused);
 ar_status launch_scan(const void* fn, const ard::SelParams& P, int grid, size_t smem, bool fused, cudaStream_t s);
 ar_status launch_select_rest(const ard::SelParams& P, bool pdl, cudaStream_t s);

@@ -440,18 +440,24 @@ __global__ void __launch_bounds__(NW * 32) select_tile_kernel(const __grid_const
 
     uint32_t i = 0;
     for (long long t = blockIdx.x; t < P.num_tiles; t += G, ++i) {
-        const uint32_t b = i % nb;
+        // one tile per CTA (nb == 1, the default): no buffer rotation
+        const uint32_t b = nb == 1 ? 0u : i % nb;
         const uint32_t* stg = stg0 + (size_t)b * P.stage_words;
-        mbar_wait(&bar[b], (i / nb) & 1u, 0);
+        mbar_wait(&bar[b], nb == 1 ? (i & 1u) : ((i / nb) & 1u), 0);
         // compact_kernel (a programmatic dependent) may be scheduled once this CTA's last tile is loaded
-        if (t + G >= P.num_tiles) asm volatile("griddepcontrol.launch_dependents;" ::: "memory");
+        if (G == P.num_tiles || t + G >= P.num_tiles) asm volatile("griddepcontrol.launch_dependents;" ::: "memory");
 
-        const int64_t r0 = t * (int64_t)P.tile_rows + (int64_t)threadIdx.x * (32 * BPT);
         PS ps;
         ps.load(P, stg);
         uint32_t cm[BPT], dm[BPT];
+        if ((t + 1) * (int64_t)P.tile_rows <= P.n) {   // a full tile: every row valid
 #pragma unroll
-        for (int q = 0; q < BPT; ++q) cm[q] = dm[q] = valid_mask(r0 + 32 * q, P.n);
+            for (int q = 0; q < BPT; ++q) cm[q] = dm[q] = 0xffffffffu;
+        } else {
+            const int64_t r0 = t * (int64_t)P.tile_rows + (int64_t)threadIdx.x * (32 * BPT);
+#pragma unroll
+            for (int q = 0; q < BPT; ++q) cm[q] = dm[q] = valid_mask(r0 + 32 * q, P.n);
+        }
         ps.eval(P, cm, dm);
         uint32_t cnt = 0;
 #pragma unroll
@@ -497,6 +503,201 @@ __global__ void __launch_bounds__(NW * 32) select_tile_kernel(const __grid_const
     }
 }
 
+#ifndef AR_RR_MINB
+#define AR_RR_MINB 10   // CTAs per SM the register budget must allow (occupancy is what the kernel needs)
+#endif
+// Ordered select in ONE kernel, no workspace round trip: persistent CTAs (all
+// co-resident: cooperative launch), tiles round-robin, nb TMA tile buffers per
+// CTA.  Per tile the CTA evaluates the planes, publishes its candidate count
+// (status[t] = kFlagAgg | count) at once and stages the tile's (position, aux)
+// entries in shared memory; the entries then wait there while the CTA decides
+// its next tile, and go out at their final offset, found by a decoupled
+// look-back (Merrill & Garland) that normally ends at an already resolved
+// neighbour (kFlagInc | inclusive prefix).  A tile with more than kRrEntries
+// candidates resolves its offset at once and writes in rounds.
+template <class PS, int NW, int BPT, bool kCarry>
+__global__ void __launch_bounds__(NW * 32, AR_RR_MINB) select_rr_kernel(const __grid_constant__ SelParams P) {
+    constexpr int NT = NW * 32;
+    constexpr uint32_t kMaxBufs = 4;
+    extern __shared__ __align__(128) unsigned char smem[];
+    __shared__ __align__(8) uint64_t bar[kMaxBufs];
+    __shared__ uint32_t warp_tot[32];
+    __shared__ unsigned long long s_off;
+    // staged entries: the row inside the tile (15 bits) | definite << 15, and the aux word
+    uint32_t* st_aux = reinterpret_cast<uint32_t*>(smem);                 // [2][kRrEntries]
+    uint16_t* st_row = reinterpret_cast<uint16_t*>(st_aux + 2 * kRrEntries);   // [2][kRrEntries]
+    uint32_t* stg0 = reinterpret_cast<uint32_t*>(st_row + 2 * kRrEntries);     // nb tile buffers
+    const uint32_t nb = P.nstages;
+    const long long G = gridDim.x;
+    const unsigned warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+
+    auto issue = [&](long long t, uint32_t b) {
+        const int64_t r0 = t * (int64_t)P.tile_rows;
+        const int64_t rows = min((int64_t)P.tile_rows, P.n - r0);
+        const uint32_t groups = (uint32_t)((rows + 127) / 128);
+        uint32_t bytes = 0;
+        for (int c = 0; c < P.npred; ++c) bytes += groups * 16u * P.p[c].w;
+        mbar_arrive_expect_tx(&bar[b], bytes);
+        const uint64_t pol = policy_evict_first();
+        uint32_t* stg = stg0 + (size_t)b * P.stage_words;
+        for (int c = 0; c < P.npred; ++c) {
+            const uint32_t w = P.p[c].w;
+            if (w)
+                bulk_g2s(stg + P.p[c].soff, P.p[c].planes + (size_t)t * (P.tile_rows / 32) * w, groups * 16u * w,
+                         &bar[b], pol);
+        }
+    };
+    if (threadIdx.x == 0) {
+        for (uint32_t b = 0; b < nb; ++b) mbar_init(&bar[b], 1);
+        fence_mbar_init();
+        for (uint32_t b = 0; b < nb; ++b)
+            if (blockIdx.x + (long long)b * G < P.num_tiles) issue(blockIdx.x + (long long)b * G, b);
+    }
+    __syncthreads();
+
+    long long pend = -1;                // tile whose entries wait in st_*[pbuf] for their offset
+    uint32_t pend_total = 0, pbuf = 0;
+    // Exclusive prefix of tile t by decoupled look-back (warp 0): one window of the 32 preceding
+    // status words per step; a tile that is already resolved carries its inclusive prefix
+    // (kFlagInc) and ends the walk, otherwise its count is added and the walk goes on.  Counts
+    // are published right after each tile's evaluation, a round before its entries are
+    // resolved, so the window is normally complete and ends at a resolved neighbour.
+    auto lookback = [&](long long t, uint32_t total) {   // warp 0 only; every lane gets the prefix
+        unsigned long long excl = 0;
+        long long idx = t - 1;
+        while (idx >= 0) {
+            const long long j = idx - (long long)lane;
+            unsigned long long v = j >= 0 ? ld_relaxed(P.status + j) : (kFlagInc | 0ull);
+            while (!__all_sync(0xffffffffu, (v >> 62) != 0)) {
+                __nanosleep(32);
+                if ((v >> 62) == 0) v = ld_relaxed(P.status + j);
+            }
+            const unsigned inc = __ballot_sync(0xffffffffu, (v >> 63) != 0);
+            const unsigned upto = inc ? (__ffs(inc) - 1) : 31u;   // lanes 0..upto contribute
+            unsigned long long x = lane <= upto ? (v & kValueMask) : 0ull;
+#pragma unroll
+            for (int o = 16; o > 0; o >>= 1) x += __shfl_xor_sync(0xffffffffu, x, o);
+            excl += x;
+            if (inc) break;
+            idx -= 32;
+        }
+        if (lane == 0) {
+            st_relaxed(P.status + t, kFlagInc | (excl + total));
+            if (t == P.num_tiles - 1) *P.out_count = (long long)(excl + total);
+        }
+        return excl;
+    };
+    // Warp 0 writes out the pending tile while the other warps go on to the next tile (their
+    // next block-scan barrier waits for it, so the buffer is free before it is restaged).
+    auto resolve_w0 = [&]() {
+        const unsigned long long off = lookback(pend, pend_total);
+        const uint16_t* sp = st_row + pbuf * kRrEntries;
+        const uint32_t* sa = st_aux + pbuf * kRrEntries;
+        const uint32_t r0 = (uint32_t)(pend * (int64_t)P.tile_rows);
+        for (uint32_t j = lane; j < pend_total; j += 32) {
+            P.out_pos[off + j] = r0 + (sp[j] & 0x7fffu);
+            P.out_aux[off + j] = sa[j];
+        }
+    };
+
+    uint32_t i = 0, cb = 0;   // cb: staging buffer of the current tile
+    for (long long t = blockIdx.x; t < P.num_tiles; t += G, ++i) {
+        const uint32_t b = nb == 1 ? 0u : i % nb;
+        const uint32_t* stg = stg0 + (size_t)b * P.stage_words;
+        mbar_wait(&bar[b], nb == 1 ? (i & 1u) : ((i / nb) & 1u), 0);
+
+        PS ps;
+        ps.load(P, stg);
+        uint32_t cm[BPT], dm[BPT];
+        if ((t + 1) * (int64_t)P.tile_rows <= P.n) {
+#pragma unroll
+            for (int q = 0; q < BPT; ++q) cm[q] = dm[q] = 0xffffffffu;
+        } else {
+            const int64_t r0 = t * (int64_t)P.tile_rows + (int64_t)threadIdx.x * (32 * BPT);
+#pragma unroll
+            for (int q = 0; q < BPT; ++q) cm[q] = dm[q] = valid_mask(r0 + 32 * q, P.n);
+        }
+        ps.eval(P, cm, dm);
+        uint32_t cnt = 0;
+#pragma unroll
+        for (int q = 0; q < BPT; ++q) cnt += __popc(cm[q]);
+        uint32_t total;
+        const uint32_t excl = block_excl_scan<NT>(cnt, warp_tot, total, 1);
+        if (threadIdx.x == 0) st_relaxed(P.status + t, kFlagAgg | total);   // publish the count at once
+        const uint32_t tile_r0 = (uint32_t)(t * (int64_t)P.tile_rows);
+
+        if (total <= (uint32_t)kRrEntries) {
+            // stage this tile's entries in buffer cb (the pending tile holds the other one)
+            uint16_t* sp = st_row + cb * kRrEntries;
+            uint32_t* sa = st_aux + cb * kRrEntries;
+            uint32_t e = excl;
+            static_for<BPT>([&](auto bc) {
+                constexpr int q = decltype(bc)::value;
+                const uint32_t rbase = (threadIdx.x * BPT + q) << 5;
+                for (uint32_t m = cm[q]; m; m &= m - 1) {
+                    const uint32_t l = __ffs(m) - 1;
+                    sp[e++] = (uint16_t)((rbase | l) | (((dm[q] >> l) & 1u) << 15));
+                }
+            });
+            __syncthreads();
+            for (uint32_t j = threadIdx.x; j < total; j += NT) {
+                const uint32_t v = sp[j];
+                const uint32_t o = v & 0x7fffu;
+                uint32_t aux = (v >> 15) << 31;
+                if (kCarry) aux |= PS::appr_smem(P, stg, o >> 5, o & 31u);
+                sa[j] = aux;
+            }
+            __syncthreads();   // stage b is free; entries staged
+            if (threadIdx.x == 0 && t + (long long)nb * G < P.num_tiles) issue(t + (long long)nb * G, b);
+            if (warp == 0 && pend >= 0) resolve_w0();
+            pend = t;
+            pend_total = total;
+            pbuf = cb;
+            cb ^= 1u;
+        } else {
+            // a dense tile: resolve the pending one, then this one's offset now; write in rounds
+            if (warp == 0) {
+                if (pend >= 0) resolve_w0();
+                const unsigned long long o = lookback(t, total);
+                if (lane == 0) s_off = o;
+            }
+            pend = -1;
+            __syncthreads();
+            const unsigned long long off = s_off;
+            uint16_t* sp = st_row + cb * kRrEntries;
+            uint32_t e = excl;
+            for (uint32_t base = 0; base < total; base += kRrEntries) {
+                const uint32_t lim = min(base + (uint32_t)kRrEntries, excl + cnt);
+                static_for<BPT>([&](auto bc) {
+                    constexpr int q = decltype(bc)::value;
+                    const uint32_t rbase = (threadIdx.x * BPT + q) << 5;
+                    while (cm[q] && e < lim) {
+                        const uint32_t l = __ffs(cm[q]) - 1;
+                        cm[q] &= cm[q] - 1;
+                        sp[e - base] = (uint16_t)((rbase | l) | (((dm[q] >> l) & 1u) << 15));
+                        ++e;
+                    }
+                });
+                __syncthreads();
+                const uint32_t nround = min((uint32_t)kRrEntries, total - base);
+                for (uint32_t j = threadIdx.x; j < nround; j += NT) {
+                    const uint32_t v = sp[j];
+                    const uint32_t o = v & 0x7fffu;
+                    uint32_t aux = (v >> 15) << 31;
+                    if (kCarry) aux |= PS::appr_smem(P, stg, o >> 5, o & 31u);
+                    P.out_pos[off + base + j] = tile_r0 + o;
+                    P.out_aux[off + base + j] = aux;
+                }
+                __syncthreads();
+            }
+            if (threadIdx.x == 0 && t + (long long)nb * G < P.num_tiles) issue(t + (long long)nb * G, b);
+        }
+    }
+    if (warp == 0 && pend >= 0) resolve_w0();
+    // the refine kernel (a programmatic dependent, if launched as one) may start
+    asm volatile("griddepcontrol.launch_dependents;" ::: "memory");
+}
+
 // Move the tiles' candidate slices from the workspace to their final offsets.
 // One CTA per chunk of kCompactTiles consecutive tiles (a chunk never straddles
 // a group of 2^kGroupShift tiles): the chunk's offset is the sum of the group
@@ -507,7 +708,7 @@ __global__ void __launch_bounds__(NW * 32) select_tile_kernel(const __grid_const
 // a contiguous slice to a contiguous destination, up to kDeep entries per lane
 // in flight, and drops the slice's L2 lines once its lanes have loaded them.
 constexpr int kCompactTiles = 8;   // = warps per CTA
-__global__ void __launch_bounds__(256) compact_kernel(const __grid_constant__ SelParams P) {
+__global__ void __launch_bounds__(256, 4) compact_kernel(const __grid_constant__ SelParams P) {
     asm volatile("griddepcontrol.wait;" ::: "memory");   // no-op unless launched as a dependent
     __shared__ unsigned long long red[8];
     __shared__ uint32_t tpre[kCompactTiles + 1];
@@ -517,8 +718,8 @@ __global__ void __launch_bounds__(256) compact_kernel(const __grid_constant__ Se
         const long long t0 = ch * kCompactTiles;
         const long long g = t0 >> kGroupShift, g0 = g << kGroupShift;
         unsigned long long off = 0;
-        for (long long i = threadIdx.x; i < g; i += 256) off += __ldcg(P.group_sum + i);
-        for (long long i = g0 + threadIdx.x; i < t0; i += 256) off += __ldcg(P.tile_count + i);
+        for (int i = (int)threadIdx.x; i < (int)g; i += 256) off += __ldcg(P.group_sum + i);
+        for (int i = (int)threadIdx.x; i < (int)(t0 - g0); i += 256) off += __ldcg(P.tile_count + g0 + i);
 #pragma unroll
         for (int o = 16; o > 0; o >>= 1) off += __shfl_xor_sync(0xffffffffu, off, o);
         if (lane == 0) red[warp] = off;
@@ -904,6 +1105,11 @@ struct ShapeEntry {
     static const void* select_fn(bool carry, int bpt) {
         return bpt == 4 ? select_fn_b<4>(carry) : select_fn_b<kSelBPT>(carry);
     }
+    static const void* select_rr_fn(bool carry) {
+        using PS = ard::FixedPlanes<kSelBPT, Ws...>;
+        return carry ? (const void*)ard::select_rr_kernel<PS, kSelNW, kSelBPT, true>
+                     : (const void*)ard::select_rr_kernel<PS, kSelNW, kSelBPT, false>;
+    }
     static const void* fused_fn() {
         using PS = ard::FixedPlanes<kFusBPT, Ws...>;
         return (const void*)ard::fused_kernel<PS, kFusNW, kFusBPT>;
@@ -917,6 +1123,9 @@ template <class... Es>
 struct ShapeList {
     static bool find(const ard::SelParams& P, bool fused, bool carry, const void** fn) {
         return (try_one<Es>(P, fused, carry, fn) || ...);
+    }
+    static bool find_rr(const ard::SelParams& P, bool carry, const void** fn) {
+        return ((Es::match(P) ? (*fn = Es::select_rr_fn(carry), true) : false) || ...);
     }
     template <class E>
     static bool try_one(const ard::SelParams& P, bool fused, bool carry, const void** fn) {
@@ -944,6 +1153,36 @@ const void* select_kernel_fn(const ard::SelParams& P, bool fused) {
     if (P.bpt != kSelBPT) return nullptr;   // runtime widths: 2 blocks per thread only
     return P.carry ? (const void*)ard::select_tile_kernel<ard::DynPlanes<kSelBPT>, kSelNW, kSelBPT, true>
                    : (const void*)ard::select_tile_kernel<ard::DynPlanes<kSelBPT>, kSelNW, kSelBPT, false>;
+}
+
+// The one-kernel ordered select (select_rr_kernel) for this shape: compiled shapes, else runtime widths.
+const void* select_rr_kernel_fn(const ard::SelParams& P) {
+    const void* fn = nullptr;
+    if (P.bpt != kSelBPT) return nullptr;
+    if (!getenv("AR_FORCE_GENERIC") && Shapes::find_rr(P, P.carry != 0, &fn)) return fn;
+    return P.carry ? (const void*)ard::select_rr_kernel<ard::DynPlanes<kSelBPT>, kSelNW, kSelBPT, true>
+                   : (const void*)ard::select_rr_kernel<ard::DynPlanes<kSelBPT>, kSelNW, kSelBPT, false>;
+}
+size_t select_rr_smem_bytes(uint32_t stage_words, uint32_t nstages) {
+    return 2ull * ard::kRrEntries * (4 + 2) + (size_t)nstages * stage_words * 4;
+}
+// Cooperative launch: the look-back waits on other CTAs' tiles, so every CTA must be
+// resident; a grid that cannot be fails with an error instead of hanging.
+ar_status launch_select_rr(const void* fn, const ard::SelParams& P, int grid, size_t smem, cudaStream_t s) {
+    opt_in_max_smem(fn);
+    void* args[] = {const_cast<ard::SelParams*>(&P)};
+    cudaLaunchConfig_t cfg = {};
+    cfg.gridDim = dim3(grid);
+    cfg.blockDim = dim3(kernel_threads(false));
+    cfg.dynamicSmemBytes = smem;
+    cfg.stream = s;
+    cudaLaunchAttribute attr[1];
+    attr[0].id = cudaLaunchAttributeCooperative;
+    attr[0].val.cooperative = 1;
+    cfg.attrs = attr;
+    cfg.numAttrs = 1;
+    AR_TRY_CUDA(cudaLaunchKernelExC(&cfg, fn, args));
+    return AR_OK;
 }
 
 size_t select_smem_bytes(uint32_t stage_words, uint32_t nstages, bool staging) {

@@ -89,3 +89,23 @@ def hot_blocks(rep, kernel_regex, top=14, key="inst"):
     for b in sorted(blocks, key=k)[:top]:
         print(f"   {b[0]:9.0f} x{b[1]:4d} = {b[0] * b[1] / tot * 100:5.1f}% inst {b[3] / tws * 100:5.1f}% stall"
               f" @{b[2]}: {' | '.join(b[4][:7])[:170]}")
+
+
+def hot_src(rep, kernel_regex, top=30):
+    """Per CUDA source line (all files): instructions executed and stall samples (-lineinfo + --import-source)."""
+    rows = ncu_csv(rep, "--page", "source", "-k", f"regex:{kernel_regex}", "--launch-count", "1",
+                   "--print-source", "cuda,sass")
+    fname, hdr, lines = "?", None, []
+    for x in rows:
+        if len(x) == 2 and x[0] == "File Path":
+            fname = x[1].rsplit("/", 1)[-1]
+        elif "Instructions Executed" in x:
+            hdr = x
+        elif hdr and len(x) == len(hdr) and x[0] not in ("", "-"):
+            lines.append((fname, x[0], x[1], float(x[hdr.index("Instructions Executed")] or 0),
+                          float(x[hdr.index("Warp Stall Sampling (All Samples)")] or 0)))
+    tot = sum(l[3] for l in lines) or 1
+    tws = sum(l[4] for l in lines) or 1
+    print(f"   instructions {tot:.0f}, stall samples {tws:.0f}")
+    for f, ln, src, ie, ws in sorted(lines, key=lambda l: -l[3])[:top]:
+        print(f"   {ie / tot * 100:5.1f}% inst {ws / tws * 100:5.1f}% stall  {f}:{ln:<5} {src.strip()[:100]}")

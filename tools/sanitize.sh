@@ -6,7 +6,7 @@
 # gpurun_out/sanitize_*.txt.  CFGS="name:ENV=V,ENV=V name2:..." restricts the configurations.
 out=gpurun_out
 for tool in racecheck synccheck memcheck; do
-  for cfg in ${CFGS:-"base:" "rg:AR_RL_RESMODE=2" "host:RES_LOC=1" "legacy:AR_FUSED_LEGACY=1" "selbufs:AR_SEL_BUFS=2" "split:SPLIT=4" "splithost:SPLIT=4 RES_LOC=1" "split3host:SPLIT=3 RES_LOC=1"}; do
+  for cfg in ${CFGS:-"base:" "rg:AR_RL_RESMODE=2" "host:RES_LOC=1" "legacy:AR_FUSED_LEGACY=1" "seltile:AR_SEL_RR=0" "selbufs:AR_SEL_RR=0,AR_SEL_BUFS=2" "selrr3:AR_SEL_RR_GRID=3" "split:SPLIT=4" "splithost:SPLIT=4 RES_LOC=1" "split3host:SPLIT=3 RES_LOC=1"}; do
     name=${cfg%%:*}; envs=${cfg#*:}; envs=${envs//,/ }
     extra=""
     [ "$tool" = "racecheck" ] && extra="--racecheck-report all"
