@@ -16,13 +16,13 @@ SF=100 SEED=4 VARIANTS=fused timeout 900 ncu --set full --clock-control none --i
     -k regex:"fused_rl_kernel|fused_rg_kernel" -s 2 -c 1 -o gpurun_out/full_fused_c4 python tools/profile_step.py \
     > gpurun_out/full_fused_c4.log 2>&1
 SF=100 SEED=4 VARIANTS=staged timeout 900 ncu --set full --clock-control none --import-source on \
-    -k regex:"select_tile_kernel|compact_kernel|refine_sum" -s 3 -c 3 -o gpurun_out/full_staged_c4 python tools/profile_step.py \
+    -k regex:"select_rr_kernel|select_tile_kernel|compact_kernel|refine_sum" -s 2 -c 2 -o gpurun_out/full_staged_c4 python tools/profile_step.py \
     > gpurun_out/full_staged_c4.log 2>&1
 SF=100 SEED=4 VARIANTS=refine timeout 900 ncu --set full --clock-control none --import-source on \
     -k regex:"refine_kernel" -s 1 -c 1 -o gpurun_out/full_refine_c4 python tools/profile_step.py \
     > gpurun_out/full_refine_c4.log 2>&1
 SF=10 SEED=2 VARIANTS=fused,staged timeout 900 ncu --set full --clock-control none --import-source on \
-    -k regex:"fused_rl_kernel|select_tile_kernel|compact_kernel|refine_sum" -s 3 -c 4 -o gpurun_out/full_c2 python tools/profile_step.py \
+    -k regex:"fused_rl_kernel|select_rr_kernel|select_tile_kernel|compact_kernel|refine_sum" -s 3 -c 3 -o gpurun_out/full_c2 python tools/profile_step.py \
     > gpurun_out/full_c2.log 2>&1
 # summaries on the box (gpurun merges at most 64 MiB of gpurun_out/ back): ncu summaries, the launch-list
 # summary and traffic.json (bench.py reads profiles/traffic.json; tools/collect_round.sh installs it);
