@@ -658,13 +658,31 @@ ar_status ar_approx_select(const ar_pred* preds, int32_t npred, int32_t flags, a
     char* base = (char*)(((uintptr_t)ws + 127) & ~uintptr_t(127));
     // one-kernel ordered select (default): round-robin look-back over per-tile counts (status words,
     // zeroed), entries written once at their final offsets -- no tile slices, no compaction
+    // AR_SEL_RR: 0 = never, 2 = always, 1 (default) = when a tile's major planes total >= kRrMinPlanes
+    // words per block and the candidate major ranges cover at most kRrEntries / tile_rows of the major
+    // domains (product over predicates): with narrower planes the per-tile look-back does not
+    // amortise, and tiles past the staging buffer take the slower dense paths (C3 at 8 planes 0.385
+    // vs 0.352 ms, at 10 % selectivity 1.39 vs 1.10 ms; Q6: 0.329 vs 0.346 ms; DESIGN s6.2).  Both
+    // kernels give the same result; this only picks the faster one.
     static const int rr = env_int("AR_SEL_RR", 1);
-    const void* rr_fn = rr ? select_rr_kernel_fn(P) : nullptr;
+    uint32_t planes = 0;
+    double frac = 1.0;
+    for (int c = 0; c < npred; ++c) {
+        const ard::SelPred& p = P.p[c];
+        planes += p.w;
+        frac *= p.w >= 32 ? ((double)p.chi - p.clo + 1.0) / 4294967296.0
+                          : ((double)p.chi - p.clo + 1.0) / (double)(1ull << p.w);
+    }
+    const bool use_rr = rr == 2 || (rr == 1 && planes >= (uint32_t)ard::kRrMinPlanes &&
+                                     frac * P.tile_rows <= (double)ard::kRrEntries);
+    const void* rr_fn = use_rr ? select_rr_kernel_fn(P) : nullptr;
     if (rr_fn) {
         static const int rr_bufs = std::min(4, std::max(1, env_int("AR_SEL_RR_BUFS", 1)));
         P.nstages = (uint32_t)rr_bufs;
-        P.status = (unsigned long long*)base;
+        P.status = (unsigned long long*)base;   // 8 * num_tiles <= L.counts_bytes
         AR_TRY_CUDA(cudaMemsetAsync(base, 0, 8 * (size_t)P.num_tiles, s));
+        P.tmp_pos = (uint32_t*)(base + L.tmp_off);   // slices of dense tiles (> kRrEntries candidates)
+        P.tmp_aux = P.tmp_pos + L.slice_rows;
         const size_t smem = select_rr_smem_bytes(P.stage_words, P.nstages);
         const int occ = select_occupancy(rr_fn, smem, false);
         if (occ > 0) {

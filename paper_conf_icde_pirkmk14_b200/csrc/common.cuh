@@ -251,6 +251,36 @@ __device__ __forceinline__ unsigned long long rr_prefix(const unsigned long long
     return prev_incl + sum;
 }
 
+// Warp-wide decoupled look-back (Merrill & Garland) over per-tile status words:
+// exclusive prefix of tile t from the windows of the 32 preceding words, each
+// either a count (kFlagAgg, published right after the tile is decided) or an
+// inclusive prefix (kFlagInc, published when the tile is resolved); the walk
+// ends at the first inclusive prefix.  Lane 0 publishes t's inclusive prefix.
+// Every lane returns the exclusive prefix.  Waits only for counts.
+__device__ __forceinline__ unsigned long long lookback_inclusive(unsigned long long* status, long long t,
+                                                                 unsigned long long total, unsigned lane) {
+    unsigned long long excl = 0;
+    long long idx = t - 1;
+    while (idx >= 0) {
+        const long long j = idx - (long long)lane;
+        unsigned long long v = j >= 0 ? ld_relaxed(status + j) : kFlagInc;
+        while (!__all_sync(0xffffffffu, (v >> 62) != 0)) {
+            __nanosleep(32);
+            if ((v >> 62) == 0) v = ld_relaxed(status + j);
+        }
+        const unsigned inc = __ballot_sync(0xffffffffu, (v >> 63) != 0);
+        const unsigned upto = inc ? (__ffs(inc) - 1) : 31u;   // lanes 0..upto contribute
+        unsigned long long x = lane <= upto ? (v & kValueMask) : 0ull;
+#pragma unroll
+        for (int o = 16; o > 0; o >>= 1) x += __shfl_xor_sync(0xffffffffu, x, o);
+        excl += x;
+        if (inc) break;
+        idx -= 32;
+    }
+    if (lane == 0) st_relaxed(status + t, kFlagInc | (excl + total));
+    return excl;
+}
+
 // --- value extraction ----------------------------------------------------------
 
 #ifndef AR_GHINT

@@ -49,7 +49,10 @@ constexpr int kSelWarps = 4;                      // consumer warps per CTA
 constexpr int kSelThreads = kSelWarps * 32;       // each consumer thread owns BPT consecutive 32-row blocks
 constexpr int kSelMinTileRows = kSelThreads * 32; // tile rows = 4096 * BPT (BPT in {1, 2, 4})
 constexpr int kStageEntries = 2048;
-constexpr int kRrEntries = 512;    // select_rr_kernel: staged entries per tile buffer (denser tiles resolve at once)
+constexpr int kRrEntries = 512; 
+constexpr int kRrMinPlanes = 12;      // ar_approx_select: select_rr_kernel for wider tiles (AR_SEL_RR=1)
+constexpr int kRrSyncEntries = 2048;   // select_rr_kernel: denser tiles resolve at once and write directly
+   // select_rr_kernel: staged entries per tile buffer (denser tiles resolve at once)
 #ifndef AR_GROUP_SHIFT
 #define AR_GROUP_SHIFT 8
 #endif

@@ -132,12 +132,12 @@ __device__ __forceinline__ uint32_t refine_batch8(const RefParams& P, const uint
 
 // Ordered refine (positions out).  Persistent CTAs, tile t = blockIdx + i *
 // gridDim (2048 candidates), decoupled look-back across tiles (Merrill &
-// Garland) specialised to the round-robin order: a tile's offset is its CTA's
-// previous inclusive prefix plus the aggregates of the gridDim - 1 tiles in
-// between.  Every CTA is resident and walks its tiles in order, so those
-// tiles are done or in progress.  Software-pipelined: a tile's kept positions
+// Garland, lookback_inclusive): each tile publishes its count at once and its
+// inclusive prefix when resolved.  Software-pipelined: a tile's kept positions
 // wait in shared memory while the CTA refines its next tile (whose candidates
-// were loaded one tile ahead), then go out at the resolved offset.
+// were loaded one tile ahead), then go out at the resolved offset -- a round
+// after the counts around it were published, so the walk is short.  Every CTA
+// is resident (cooperative launch), so the counts waited for always come.
 __global__ void __launch_bounds__(kRefThreads, 4) refine_kernel(const __grid_constant__ RefParams P) {
     __shared__ uint32_t st_pos[2][kRefTile];   // kept positions of the current and the pending tile
     __shared__ uint32_t warp_tot[kRefThreads / 32];
@@ -145,15 +145,13 @@ __global__ void __launch_bounds__(kRefThreads, 4) refine_kernel(const __grid_con
     const unsigned warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     const long long count = *P.in_count;
     const long long num_tiles = (count + kRefTile - 1) / kRefTile;
-    unsigned long long prev_incl = 0;   // warp 0: inclusive prefix of this CTA's last resolved tile
     long long pend = -1;                // tile whose positions wait in st_pos[pbuf] for their offset
     uint32_t pend_total = 0, buf = 0;
     // Write out the pending tile: its predecessors' aggregates were published while this
     // CTA refined its next tile, so the prefix is normally ready without waiting.
     auto resolve = [&]() {
         if (warp == 0) {
-            const unsigned long long prefix = rr_prefix(P.status, pend, lane, prev_incl);
-            prev_incl = prefix + pend_total;
+            const unsigned long long prefix = lookback_inclusive(P.status, pend, pend_total, lane);
             if (lane == 0) {
                 s_off = prefix;
                 if (pend == num_tiles - 1) *P.out_count = (long long)(prefix + pend_total);
@@ -317,6 +315,12 @@ __global__ void __launch_bounds__(kRefThreads, 2) refine_sum_sliced_kernel(const
     const RefPred& q = P.p[P.fast_chk];
     const uint32_t qmask = q.w == 32 ? 0xffffffffu : ((1u << q.w) - 1u);
     const int g = P.fast_g;   // gathered factor, or -1
+    // two factors, one gathered and one carried predicate column (Q6): its shift / mask / base once
+    const int f2 = (P.nagg == 2 && g >= 0) ? 1 - g : -1;
+    const uint32_t f2_sh = f2 >= 0 ? P.p[P.a[f2].pred].ashift : 0u;
+    const uint32_t f2_w = f2 >= 0 ? P.p[P.a[f2].pred].w : 0u;
+    const uint32_t f2_mask = f2_w >= 32 ? 0xffffffffu : ((1u << f2_w) - 1u);
+    const uint32_t f2_base = f2 >= 0 ? P.a[f2].base : 0u;
     unsigned long long sum = 0, kept = 0;
     // the next tile's candidates are loaded while this one's gathers are in flight
     uint32_t npos[8], naux[8];
@@ -384,6 +388,12 @@ __global__ void __launch_bounds__(kRefThreads, 2) refine_sum_sliced_kernel(const
                 const uint32_t v = packed_get_if(a.major, pos[i], (int)a.w, (late >> i) & 1u);
                 gv[i] = ((late >> i) & 1u ? v : gv[i]) + a.base;
             }
+        }
+        if (f2 >= 0) {   // Q6: the gathered factor times one carried predicate column (shift / mask hoisted)
+#pragma unroll
+            for (int i = 0; i < 8; ++i)
+                if ((keep >> i) & 1u) sum += (unsigned long long)gv[i] * (((aux[i] >> f2_sh) & f2_mask) + f2_base);
+            continue;
         }
 #pragma unroll
         for (int i = 0; i < 8; ++i) {
@@ -722,7 +732,7 @@ __global__ void __launch_bounds__(kRefThreads) project_kernel(const __grid_const
 namespace ar {
 
 const void* refine_kernel_fn() { return (const void*)ard::refine_kernel; }
-// Cooperative: the round-robin look-back (rr_prefix) waits on tiles of other
+// Cooperative: the look-back (lookback_inclusive) waits on tiles of other
 // CTAs, so the whole grid must be co-resident; a cooperative launch guarantees
 // that or fails (cudaErrorCooperativeLaunchTooLarge, e.g. under an MPS SM
 // limit or beside a persistent kernel) rather than hanging.

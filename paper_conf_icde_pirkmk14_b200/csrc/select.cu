@@ -557,34 +557,15 @@ __global__ void __launch_bounds__(NW * 32, AR_RR_MINB) select_rr_kernel(const __
 
     long long pend = -1;                // tile whose entries wait in st_*[pbuf] for their offset
     uint32_t pend_total = 0, pbuf = 0;
+    bool pend_dense = false;            // its entries are in its workspace slice, not in shared memory
     // Exclusive prefix of tile t by decoupled look-back (warp 0): one window of the 32 preceding
     // status words per step; a tile that is already resolved carries its inclusive prefix
     // (kFlagInc) and ends the walk, otherwise its count is added and the walk goes on.  Counts
     // are published right after each tile's evaluation, a round before its entries are
     // resolved, so the window is normally complete and ends at a resolved neighbour.
     auto lookback = [&](long long t, uint32_t total) {   // warp 0 only; every lane gets the prefix
-        unsigned long long excl = 0;
-        long long idx = t - 1;
-        while (idx >= 0) {
-            const long long j = idx - (long long)lane;
-            unsigned long long v = j >= 0 ? ld_relaxed(P.status + j) : (kFlagInc | 0ull);
-            while (!__all_sync(0xffffffffu, (v >> 62) != 0)) {
-                __nanosleep(32);
-                if ((v >> 62) == 0) v = ld_relaxed(P.status + j);
-            }
-            const unsigned inc = __ballot_sync(0xffffffffu, (v >> 63) != 0);
-            const unsigned upto = inc ? (__ffs(inc) - 1) : 31u;   // lanes 0..upto contribute
-            unsigned long long x = lane <= upto ? (v & kValueMask) : 0ull;
-#pragma unroll
-            for (int o = 16; o > 0; o >>= 1) x += __shfl_xor_sync(0xffffffffu, x, o);
-            excl += x;
-            if (inc) break;
-            idx -= 32;
-        }
-        if (lane == 0) {
-            st_relaxed(P.status + t, kFlagInc | (excl + total));
-            if (t == P.num_tiles - 1) *P.out_count = (long long)(excl + total);
-        }
+        const unsigned long long excl = lookback_inclusive(P.status, t, total, lane);
+        if (lane == 0 && t == P.num_tiles - 1) *P.out_count = (long long)(excl + total);
         return excl;
     };
     // Warp 0 writes out the pending tile while the other warps go on to the next tile (their
@@ -626,38 +607,28 @@ __global__ void __launch_bounds__(NW * 32, AR_RR_MINB) select_rr_kernel(const __
         if (threadIdx.x == 0) st_relaxed(P.status + t, kFlagAgg | total);   // publish the count at once
         const uint32_t tile_r0 = (uint32_t)(t * (int64_t)P.tile_rows);
 
-        if (total <= (uint32_t)kRrEntries) {
-            // stage this tile's entries in buffer cb (the pending tile holds the other one)
-            uint16_t* sp = st_row + cb * kRrEntries;
-            uint32_t* sa = st_aux + cb * kRrEntries;
-            uint32_t e = excl;
-            static_for<BPT>([&](auto bc) {
-                constexpr int q = decltype(bc)::value;
-                const uint32_t rbase = (threadIdx.x * BPT + q) << 5;
-                for (uint32_t m = cm[q]; m; m &= m - 1) {
-                    const uint32_t l = __ffs(m) - 1;
-                    sp[e++] = (uint16_t)((rbase | l) | (((dm[q] >> l) & 1u) << 15));
+        const bool dense = total > (uint32_t)kRrEntries;
+        if (total > (uint32_t)kRrSyncEntries) {
+            // a very dense tile: resolve the pending one and this one's offset now, write in rounds
+            // straight to the output (the writes dwarf the look-back; a workspace round trip would not)
+            if (pend >= 0 && !pend_dense) {
+                if (warp == 0) resolve_w0();
+            } else if (pend >= 0) {
+                if (warp == 0) {
+                    const unsigned long long o = lookback(pend, pend_total);
+                    if (lane == 0) s_off = o;
                 }
-            });
-            __syncthreads();
-            for (uint32_t j = threadIdx.x; j < total; j += NT) {
-                const uint32_t v = sp[j];
-                const uint32_t o = v & 0x7fffu;
-                uint32_t aux = (v >> 15) << 31;
-                if (kCarry) aux |= PS::appr_smem(P, stg, o >> 5, o & 31u);
-                sa[j] = aux;
+                __syncthreads();
+                const unsigned long long off = s_off;
+                const uint32_t* tp = P.tmp_pos + (size_t)pend * P.tile_rows;
+                const uint32_t* ta = P.tmp_aux + (size_t)pend * P.tile_rows;
+                for (uint32_t j = threadIdx.x; j < pend_total; j += NT) {
+                    P.out_pos[off + j] = __ldcs(tp + j);
+                    P.out_aux[off + j] = __ldcs(ta + j);
+                }
+                __syncthreads();   // every thread has read s_off
             }
-            __syncthreads();   // stage b is free; entries staged
-            if (threadIdx.x == 0 && t + (long long)nb * G < P.num_tiles) issue(t + (long long)nb * G, b);
-            if (warp == 0 && pend >= 0) resolve_w0();
-            pend = t;
-            pend_total = total;
-            pbuf = cb;
-            cb ^= 1u;
-        } else {
-            // a dense tile: resolve the pending one, then this one's offset now; write in rounds
             if (warp == 0) {
-                if (pend >= 0) resolve_w0();
                 const unsigned long long o = lookback(t, total);
                 if (lane == 0) s_off = o;
             }
@@ -691,9 +662,108 @@ __global__ void __launch_bounds__(NW * 32, AR_RR_MINB) select_rr_kernel(const __
                 __syncthreads();
             }
             if (threadIdx.x == 0 && t + (long long)nb * G < P.num_tiles) issue(t + (long long)nb * G, b);
+            continue;
+        }
+        if (!dense) {
+            // stage this tile's entries in buffer cb (the pending tile holds the other one)
+            uint16_t* sp = st_row + cb * kRrEntries;
+            uint32_t* sa = st_aux + cb * kRrEntries;
+            uint32_t e = excl;
+            static_for<BPT>([&](auto bc) {
+                constexpr int q = decltype(bc)::value;
+                const uint32_t rbase = (threadIdx.x * BPT + q) << 5;
+                for (uint32_t m = cm[q]; m; m &= m - 1) {
+                    const uint32_t l = __ffs(m) - 1;
+                    sp[e++] = (uint16_t)((rbase | l) | (((dm[q] >> l) & 1u) << 15));
+                }
+            });
+            __syncthreads();
+            for (uint32_t j = threadIdx.x; j < total; j += NT) {
+                const uint32_t v = sp[j];
+                const uint32_t o = v & 0x7fffu;
+                uint32_t aux = (v >> 15) << 31;
+                if (kCarry) aux |= PS::appr_smem(P, stg, o >> 5, o & 31u);
+                sa[j] = aux;
+            }
+        } else {
+            // a dense tile: its entries go, in rounds through buffer cb, to the tile's own workspace
+            // slice (tile-local order); they are copied to their final offset when resolved
+            uint16_t* sp = st_row + cb * kRrEntries;
+            uint32_t* tp = P.tmp_pos + (size_t)t * P.tile_rows;
+            uint32_t* ta = P.tmp_aux + (size_t)t * P.tile_rows;
+            uint32_t e = excl;
+            for (uint32_t base = 0; base < total; base += kRrEntries) {
+                const uint32_t lim = min(base + (uint32_t)kRrEntries, excl + cnt);
+                static_for<BPT>([&](auto bc) {
+                    constexpr int q = decltype(bc)::value;
+                    const uint32_t rbase = (threadIdx.x * BPT + q) << 5;
+                    while (cm[q] && e < lim) {
+                        const uint32_t l = __ffs(cm[q]) - 1;
+                        cm[q] &= cm[q] - 1;
+                        sp[e - base] = (uint16_t)((rbase | l) | (((dm[q] >> l) & 1u) << 15));
+                        ++e;
+                    }
+                });
+                __syncthreads();
+                const uint32_t nround = min((uint32_t)kRrEntries, total - base);
+                for (uint32_t j = threadIdx.x; j < nround; j += NT) {
+                    const uint32_t v = sp[j];
+                    const uint32_t o = v & 0x7fffu;
+                    uint32_t aux = (v >> 15) << 31;
+                    if (kCarry) aux |= PS::appr_smem(P, stg, o >> 5, o & 31u);
+                    tp[base + j] = tile_r0 + o;
+                    ta[base + j] = aux;
+                }
+                if (base + kRrEntries < total) __syncthreads();   // sp is refilled by the next round
+            }
+        }
+        __syncthreads();   // stage b is free; entries staged
+        if (threadIdx.x == 0 && t + (long long)nb * G < P.num_tiles) issue(t + (long long)nb * G, b);
+        // resolve the pending tile (a round after its count was published: the look-back is short)
+        if (pend >= 0) {
+            if (!pend_dense) {
+                if (warp == 0) resolve_w0();
+            } else {   // a dense pending tile: warp 0 finds the offset, the whole CTA copies its slice
+                if (warp == 0) {
+                    const unsigned long long o = lookback(pend, pend_total);
+                    if (lane == 0) s_off = o;
+                }
+                __syncthreads();
+                const unsigned long long off = s_off;
+                const uint32_t* tp = P.tmp_pos + (size_t)pend * P.tile_rows;
+                const uint32_t* ta = P.tmp_aux + (size_t)pend * P.tile_rows;
+                for (uint32_t j = threadIdx.x; j < pend_total; j += NT) {
+                    P.out_pos[off + j] = __ldcs(tp + j);
+                    P.out_aux[off + j] = __ldcs(ta + j);
+                }
+            }
+        }
+        pend = t;
+        pend_total = total;
+        pend_dense = dense;
+        if (!dense) {
+            pbuf = cb;
+            cb ^= 1u;
         }
     }
-    if (warp == 0 && pend >= 0) resolve_w0();
+    if (pend >= 0) {   // the last tile
+        if (!pend_dense) {
+            if (warp == 0) resolve_w0();
+        } else {
+            if (warp == 0) {
+                const unsigned long long o = lookback(pend, pend_total);
+                if (lane == 0) s_off = o;
+            }
+            __syncthreads();
+            const unsigned long long off = s_off;
+            const uint32_t* tp = P.tmp_pos + (size_t)pend * P.tile_rows;
+            const uint32_t* ta = P.tmp_aux + (size_t)pend * P.tile_rows;
+            for (uint32_t j = threadIdx.x; j < pend_total; j += NT) {
+                P.out_pos[off + j] = __ldcs(tp + j);
+                P.out_aux[off + j] = __ldcs(ta + j);
+            }
+        }
+    }
     // the refine kernel (a programmatic dependent, if launched as one) may start
     asm volatile("griddepcontrol.launch_dependents;" ::: "memory");
 }
@@ -708,7 +778,7 @@ __global__ void __launch_bounds__(NW * 32, AR_RR_MINB) select_rr_kernel(const __
 // a contiguous slice to a contiguous destination, up to kDeep entries per lane
 // in flight, and drops the slice's L2 lines once its lanes have loaded them.
 constexpr int kCompactTiles = 8;   // = warps per CTA
-__global__ void __launch_bounds__(256, 4) compact_kernel(const __grid_constant__ SelParams P) {
+__global__ void __launch_bounds__(256) compact_kernel(const __grid_constant__ SelParams P) {
     asm volatile("griddepcontrol.wait;" ::: "memory");   // no-op unless launched as a dependent
     __shared__ unsigned long long red[8];
     __shared__ uint32_t tpre[kCompactTiles + 1];

@@ -95,8 +95,35 @@ def test_staged_q6_sizes(cu, n, k):
     [(5000, 6000), (0, 10), (0, 60)],     # no row qualifies
 ])
 def test_staged_bound_placements(cu, bounds):
+    # default kernel choice: dense placements go to the tile kernel + compaction
     sel, ref, ncand, res = staged(cu, 6_000_001, 90, 8, ["extprice", "discount"], bounds=bounds)
-    assert (sel == "select_rr_kernel" or (ncand == 0 and sel == "")) and ncand >= res
+    assert sel in ("select_rr_kernel", "select_tile_kernel") or (ncand == 0 and sel == "")
+    assert ncand >= res
+
+
+BOUNDS = [[(3, 2523), (0, 10), (1, 50)], [(0, 2600), (0, 10), (0, 5)], [(1000, 1000), (0, 10), (0, 60)],
+          [(768, 1023), (5, 7), (0, 23)], [(5000, 6000), (0, 10), (0, 60)]]
+
+
+@pytest.mark.parametrize("grid", ["0", "3"])
+def test_rr_dense_paths_in_subprocess(grid):
+    """AR_SEL_RR=2: the one-kernel select on every bound placement -- tiles staged in shared memory,
+    through workspace slices (513-2048 candidates) and resolved at once (> 2048) -- with the whole
+    grid and with 3 CTAs (many look-back rounds)."""
+    code = (
+        "import sys; sys.path.insert(0, %r); sys.path.insert(0, %r)\n"
+        "import test_gpu_staged as t\n"
+        "from paper_conf_icde_pirkmk14_b200 import column as cu\n"
+        "for b in t.BOUNDS:\n"
+        "    sel, _, ncand, res = t.staged(cu, 6_000_001, 90, 8, ['extprice', 'discount'], bounds=b)\n"
+        "    assert sel == 'select_rr_kernel' or (ncand == 0 and sel == ''), sel\n"
+        "print('ok')\n" % (ROOT, os.path.join(ROOT, "tests")))
+    env = {**os.environ, "AR_SEL_RR": "2"}
+    if grid != "0":
+        env["AR_SEL_RR_GRID"] = grid
+    r = subprocess.run([sys.executable, "-c", code], cwd=ROOT, capture_output=True, text=True, timeout=900,
+                       env=env)
+    assert r.returncode == 0 and "ok" in r.stdout, r.stderr[-3000:]
 
 
 @pytest.mark.parametrize("aggs", [(), ("discount",), ("discount", "quantity"), ("extprice",),
@@ -130,7 +157,7 @@ def test_staged_rr_grids_in_subprocess(env):
         "sel, _, _, _ = t.staged(cu, 6_000_001, 90, 8, ['extprice'], bounds=[(0, 2600), (0, 10), (0, 5)])\n"
         "print('ok')\n" % (ROOT, os.path.join(ROOT, "tests")))
     r = subprocess.run([sys.executable, "-c", code], cwd=ROOT, capture_output=True, text=True, timeout=900,
-                       env={**os.environ, **env})
+                       env={**os.environ, "AR_SEL_RR": "2", **env})
     assert r.returncode == 0 and "ok" in r.stdout, r.stderr[-3000:]
 
 
@@ -148,4 +175,23 @@ def test_tile_kernel_and_compaction_in_subprocess():
         "print('ok')\n" % (ROOT, os.path.join(ROOT, "tests")))
     r = subprocess.run([sys.executable, "-c", code], cwd=ROOT, capture_output=True, text=True, timeout=900,
                        env={**os.environ, "AR_SEL_RR": "0"})
+    assert r.returncode == 0 and "ok" in r.stdout, r.stderr[-3000:]
+
+
+def test_rr_forced_on_narrow_planes_in_subprocess():
+    """AR_SEL_RR=2: the one-kernel select also on shapes the default leaves to the tile kernel
+    (fewer than 12 major planes), compared with the oracle by test_gpu_parity's checker."""
+    code = (
+        "import sys; sys.path.insert(0, %r); sys.path.insert(0, %r)\n"
+        "import numpy as np, datagen, torch\n"
+        "import test_gpu_parity as tp\n"
+        "from paper_conf_icde_pirkmk14_b200 import column as cu, _ar\n"
+        "for n, k, lo, hi in ((100_003, 24, 1 << 29, 3 << 29), (3_000_017, 24, 5 << 24, 5 << 24),\n"
+        "                     (3_000_017, 28, 0, 1 << 31), (70_001, 16, 12345, 2 ** 32 - 7)):\n"
+        "    v = datagen.uniform_u32(n + k, n)\n"
+        "    tp.check_select(cu, [v], [k], [lo], [hi])\n"
+        "    assert _ar.ar_last_scan_kernel() == 'select_rr_kernel', _ar.ar_last_scan_kernel()\n"
+        "print('ok')\n" % (ROOT, os.path.join(ROOT, "tests")))
+    r = subprocess.run([sys.executable, "-c", code], cwd=ROOT, capture_output=True, text=True, timeout=900,
+                       env={**os.environ, "AR_SEL_RR": "2"})
     assert r.returncode == 0 and "ok" in r.stdout, r.stderr[-3000:]
