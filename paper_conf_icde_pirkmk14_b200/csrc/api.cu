@@ -795,22 +795,41 @@ ar_status ar_refine(const ar_cands* in, const ar_pred* preds, int32_t npred, ar_
     // persistent, round-robin tiles whose look-back waits on the tiles of other CTAs: every CTA must be
     // resident, so the grid is sized from the occupancy on this device and launch_refine launches it
     // cooperatively (a grid that cannot be co-resident fails with an error instead of hanging)
-    struct Occ { int dev; int occ; };
+    // the wide instance when a checked predicate has an unsplit SLICED 8-plane residual (its two 16-B
+    // halves gathered together, 2 CTAs per SM); the 4-CTA instance otherwise
+    // and at most 8 candidate buckets (so a good share of the candidates is in the two boundary
+    // buckets and needs its residual: Q6's l_shipdate has 3; C3 at 24 major bits has thousands, nearly
+    // all definite, and runs faster with 4 CTAs per SM -- DESIGN s6.4)
+    bool wide = false;
+    for (int c = 0; c < P.npred; ++c) {
+        const ard::RefPred& p = P.p[c];
+        if (!p.check || p.rlayout != AR_LAYOUT_SLICED || p.k != 8) continue;
+        const uint32_t blo = (p.lo - p.base) >> 8, bhi = (p.hi - p.base) >> 8;
+        if (bhi >= blo && bhi - blo < 8) wide = true;
+    }
+    static const int wide_env = env_int("AR_REFINE_WIDE", 1);
+    wide = wide && wide_env != 0;
+    struct Occ { int dev; int occ[2]; };
     static thread_local Occ occ_cache[16];
     static thread_local int occ_used = 0;
     const int dev = current_device();
-    int occ = 0;
+    int* occp = nullptr;
     for (int i = 0; i < occ_used; ++i)
-        if (occ_cache[i].dev == dev) occ = occ_cache[i].occ;
+        if (occ_cache[i].dev == dev) occp = occ_cache[i].occ;
+    if (!occp && occ_used < 16) {
+        occ_cache[occ_used] = Occ{dev, {0, 0}};
+        occp = occ_cache[occ_used++].occ;
+    }
+    int occ = occp ? occp[wide] : 0;
     if (!occ) {
-        cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, (const void*)refine_kernel_fn(), ard::kRefThreads, 0);
+        cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, refine_kernel_fn(wide), ard::kRefThreads, 0);
         cudaGetLastError();
         occ = std::max(occ, 1);
-        if (occ_used < 16) occ_cache[occ_used++] = Occ{dev, occ};
+        if (occp) occp[wide] = occ;
     }
-    const int grid = (int)std::min<uint64_t>(std::min<uint64_t>(max_tiles, (uint64_t)num_sms() * occ), 640);
+    const int grid = (int)std::min<uint64_t>(max_tiles, (uint64_t)num_sms() * occ);
     g_last_scan = "refine_kernel";
-    return launch_refine(P, grid, s);
+    return launch_refine(P, grid, wide, s);
 }
 
 // ------------------------------------------------------------------ a6

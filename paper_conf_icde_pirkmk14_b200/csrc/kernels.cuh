@@ -181,6 +181,7 @@ struct RefPred {
 constexpr int kRefThreads = 256;
 constexpr int kRefPerThread = 8;
 constexpr int kRefTile = kRefThreads * kRefPerThread;   // 2048 candidates per tile
+constexpr int kRefWarpCopy = kRefTile;   // refine_kernel: a pending tile with more kept positions is copied out by the CTA (never: measured slower at C4)
 
 struct RefParams {
     RefPred p[AR_MAX_PRED];
@@ -267,8 +268,8 @@ constexpr int kSrsMaxGrid = 2048;
 void retile(ard::SelParams& P, uint32_t tile_rows);   // fused.cu
 ar_status launch_fused_rl(const ard::SelParams& P, const ar_column* const* cols, void* ws, int pdl, bool* launched,
                           bool* gathered_res, cudaStream_t s);
-ar_status launch_refine(const ard::RefParams& P, int grid, cudaStream_t s);
-const void* refine_kernel_fn();
+ar_status launch_refine(const ard::RefParams& P, int grid, bool wide, cudaStream_t s);
+const void* refine_kernel_fn(bool wide);
 ar_status launch_refine_sum(const ard::RefParams& P, int grid, cudaStream_t s);
 ar_status launch_sum(const ard::SumParams& P, int grid, cudaStream_t s);
 ar_status launch_approx_sum(const ard::ApproxSumParams& P, int grid, cudaStream_t s);

@@ -57,11 +57,24 @@ __device__ __forceinline__ void load8(const uint32_t* base, uint64_t j0, long lo
 // SLICED part of width w at rows pos[i] where (pred >> i) & 1: w/4 vector steps
 // (a 32-row block's w planes are contiguous; w % 4 == 0 keeps them 16-B aligned),
 // otherwise word by word.
+template <bool kWide = false>   // kWide: the w == 8 case with both 16-B halves in flight (128 registers)
 __device__ __forceinline__ void sliced_batch8(const uint32_t* s, const uint32_t (&pos)[8], uint32_t pred, int w,
                                               uint32_t (&out)[8]) {
 #pragma unroll
     for (int i = 0; i < 8; ++i) out[i] = 0u;
-    if ((w & 3) == 0) {
+    if (kWide && w == 8) {   // both 16-B halves of every block in flight together (one gather latency, not two)
+        uint4 a[8], b[8];
+#pragma unroll
+        for (int i = 0; i < 8; ++i) {
+            a[i] = ld_gather_if4(s + (uint64_t)(pos[i] >> 5) * 8, (pred >> i) & 1u);
+            b[i] = ld_gather_if4(s + (uint64_t)(pos[i] >> 5) * 8 + 4, (pred >> i) & 1u);
+        }
+#pragma unroll
+        for (int i = 0; i < 8; ++i) {
+            const uint32_t x[8] = {a[i].x, a[i].y, a[i].z, a[i].w, b[i].x, b[i].y, b[i].z, b[i].w};
+            out[i] = rl::row_bits<8>(x, pos[i] & 31u);
+        }
+    } else if ((w & 3) == 0) {
         for (int q = 0; q < w / 4; ++q) {
             uint4 a[8];
 #pragma unroll
@@ -83,13 +96,14 @@ __device__ __forceinline__ void sliced_batch8(const uint32_t* s, const uint32_t 
         }
     }
 }
+template <bool kWide = false>
 __device__ __forceinline__ void part_batch8(const uint32_t* s, const uint32_t (&pos)[8], uint32_t pred, int w,
                                             int layout, uint32_t (&out)[8]) {
     if (w == 0) {
 #pragma unroll
         for (int i = 0; i < 8; ++i) out[i] = 0u;
     } else if (layout == AR_LAYOUT_SLICED) {
-        sliced_batch8(s, pos, pred, w, out);
+        sliced_batch8<kWide>(s, pos, pred, w, out);
     } else if ((layout & 0xff) == AR_LAYOUT_SLICED) {   // split residual planes
 #pragma unroll
         for (int i = 0; i < 8; ++i) out[i] = residual_get_if(s, pos[i], w, layout, (pred >> i) & 1u);
@@ -102,6 +116,7 @@ __device__ __forceinline__ void part_batch8(const uint32_t* s, const uint32_t (&
 // Alg. 2 on 8 candidates: definite ones are kept untouched;
 // every non-definite one is joined with its residual (and, when the
 // approximation is not carried, its major) and re-evaluated exactly.
+template <bool kWide = false>
 __device__ __forceinline__ uint32_t refine_batch8(const RefParams& P, const uint32_t (&pos)[8],
                                                   const uint32_t (&aux)[8], uint32_t valid) {
     uint32_t def = 0;
@@ -120,7 +135,7 @@ __device__ __forceinline__ uint32_t refine_batch8(const RefParams& P, const uint
         } else {
             part_batch8(p.major, pos, need, (int)p.w, (int)p.layout, m);
         }
-        part_batch8(p.residual, pos, need, (int)p.k, (int)p.rlayout, r);
+        part_batch8<kWide>(p.residual, pos, need, (int)p.k, (int)p.rlayout, r);
 #pragma unroll
         for (int i = 0; i < 8; ++i) {
             const uint32_t v = (p.k >= 32 ? r[i] : ((m[i] << p.k) | r[i])) + p.base;
@@ -138,18 +153,38 @@ __device__ __forceinline__ uint32_t refine_batch8(const RefParams& P, const uint
 // were loaded one tile ahead), then go out at the resolved offset -- a round
 // after the counts around it were published, so the walk is short.  Every CTA
 // is resident (cooperative launch), so the counts waited for always come.
-__global__ void __launch_bounds__(kRefThreads, 4) refine_kernel(const __grid_constant__ RefParams P) {
+// kWide (a checked predicate with an unsplit SLICED 8-plane residual): both 16-B
+// halves of every candidate's residual block in flight together -- one gather
+// latency per tile instead of two -- at 128 registers (2 CTAs per SM); the
+// other shapes keep 4 CTAs per SM.
+template <bool kWide>
+__global__ void __launch_bounds__(kRefThreads, kWide ? 2 : 4) refine_kernel(const __grid_constant__ RefParams P) {
     __shared__ uint32_t st_pos[2][kRefTile];   // kept positions of the current and the pending tile
-    __shared__ uint32_t warp_tot[kRefThreads / 32];
+    // two sets of warp totals, by tile parity: no barrier follows a tile's block scan, so the next
+    // tile's scan must not overwrite totals a slower warp may still be reading
+    __shared__ uint32_t warp_tot[2][kRefThreads / 32];
     __shared__ unsigned long long s_off;
     const unsigned warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     const long long count = *P.in_count;
     const long long num_tiles = (count + kRefTile - 1) / kRefTile;
     long long pend = -1;                // tile whose positions wait in st_pos[pbuf] for their offset
-    uint32_t pend_total = 0, buf = 0;
-    // Write out the pending tile: its predecessors' aggregates were published while this
-    // CTA refined its next tile, so the prefix is normally ready without waiting.
+    uint32_t pend_total = 0, cb = 0, pbuf = 0;
+    // Warp 0 writes out the pending tile while the other warps refine the next one (their next
+    // block-scan barrier waits for it, which also orders the buffer's reuse): its neighbours'
+    // counts were published while this CTA refined, so the look-back is normally short.
+    auto resolve_w0 = [&]() {
+        const unsigned long long prefix = lookback_inclusive(P.status, pend, pend_total, lane);
+        if (lane == 0 && pend == num_tiles - 1) *P.out_count = (long long)(prefix + pend_total);
+        const uint32_t* sp = st_pos[pbuf];
+        for (uint32_t j = lane; j < pend_total; j += 32) P.out_pos[prefix + j] = sp[j];
+    };
+    // A pending tile with many kept positions is copied out by the whole CTA (warp 0 alone would
+    // hold the CTA up at the next barrier for longer than the barrier here costs).
     auto resolve = [&]() {
+        if (pend_total <= (uint32_t)kRefWarpCopy) {
+            if (warp == 0) resolve_w0();
+            return;
+        }
         if (warp == 0) {
             const unsigned long long prefix = lookback_inclusive(P.status, pend, pend_total, lane);
             if (lane == 0) {
@@ -159,9 +194,8 @@ __global__ void __launch_bounds__(kRefThreads, 4) refine_kernel(const __grid_con
         }
         __syncthreads();
         const unsigned long long off = s_off;
-        const uint32_t* sp = st_pos[buf];   // the pending tile's buffer
+        const uint32_t* sp = st_pos[pbuf];
         for (uint32_t j = threadIdx.x; j < pend_total; j += kRefThreads) P.out_pos[off + j] = sp[j];
-        __syncthreads();
     };
     uint32_t npos[8], naux[8];
     if ((long long)blockIdx.x < num_tiles) {
@@ -185,27 +219,25 @@ __global__ void __launch_bounds__(kRefThreads, 4) refine_kernel(const __grid_con
         uint32_t valid = 0;
 #pragma unroll
         for (int i = 0; i < 8; ++i) valid |= (j0 + i < (uint64_t)count ? 1u : 0u) << i;
-        const uint32_t keep = refine_batch8(P, pos, aux, valid);
+        const uint32_t keep = refine_batch8<kWide>(P, pos, aux, valid);
 
         const uint32_t cnt = __popc(keep);
         uint32_t total;
-        const uint32_t excl = block_excl_scan<kRefThreads>(cnt, warp_tot, total, 1);
-        if (threadIdx.x == 0) st_relaxed(P.status + t, kFlagAgg | total);   // publish the aggregate at once
+        const uint32_t excl = block_excl_scan<kRefThreads>(cnt, warp_tot[cb], total, 1);
+        if (threadIdx.x == 0) st_relaxed(P.status + t, kFlagAgg | total);   // publish the count at once
         uint32_t o = excl;
-        uint32_t* sp = st_pos[buf];
+        uint32_t* sp = st_pos[cb];
 #pragma unroll
         for (int i = 0; i < 8; ++i)
             if (keep & (1u << i)) sp[o++] = pos[i];
-        buf ^= 1u;   // now the pending (previous) tile's buffer
         if (pend >= 0) resolve();
-        else __syncthreads();
         pend = t;
         pend_total = total;
+        pbuf = cb;
+        cb ^= 1u;
     }
-    if (pend >= 0) {
-        buf ^= 1u;   // the last tile's buffer
-        resolve();
-    }
+    __syncthreads();   // the last tile's positions are staged
+    if (pend >= 0) resolve();
 }
 
 template <typename T>
@@ -731,12 +763,14 @@ __global__ void __launch_bounds__(kRefThreads) project_kernel(const __grid_const
 
 namespace ar {
 
-const void* refine_kernel_fn() { return (const void*)ard::refine_kernel; }
+const void* refine_kernel_fn(bool wide) {
+    return wide ? (const void*)ard::refine_kernel<true> : (const void*)ard::refine_kernel<false>;
+}
 // Cooperative: the look-back (lookback_inclusive) waits on tiles of other
 // CTAs, so the whole grid must be co-resident; a cooperative launch guarantees
 // that or fails (cudaErrorCooperativeLaunchTooLarge, e.g. under an MPS SM
 // limit or beside a persistent kernel) rather than hanging.
-ar_status launch_refine(const ard::RefParams& P, int grid, cudaStream_t s) {
+ar_status launch_refine(const ard::RefParams& P, int grid, bool wide, cudaStream_t s) {
     void* args[] = {const_cast<ard::RefParams*>(&P)};
     cudaLaunchConfig_t cfg = {};
     cfg.gridDim = dim3(grid);
@@ -747,7 +781,7 @@ ar_status launch_refine(const ard::RefParams& P, int grid, cudaStream_t s) {
     attr[0].val.cooperative = 1;
     cfg.attrs = attr;
     cfg.numAttrs = 1;
-    AR_TRY_CUDA(cudaLaunchKernelExC(&cfg, (const void*)ard::refine_kernel, args));
+    AR_TRY_CUDA(cudaLaunchKernelExC(&cfg, refine_kernel_fn(wide), args));
     return AR_OK;
 }
 ar_status launch_refine_sum(const ard::RefParams& P, int grid, cudaStream_t s) {

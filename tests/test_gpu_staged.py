@@ -195,3 +195,27 @@ def test_rr_forced_on_narrow_planes_in_subprocess():
     r = subprocess.run([sys.executable, "-c", code], cwd=ROOT, capture_output=True, text=True, timeout=900,
                        env={**os.environ, "AR_SEL_RR": "2"})
     assert r.returncode == 0 and "ok" in r.stdout, r.stderr[-3000:]
+
+
+@pytest.mark.parametrize("bounds", [None, [(3, 2523), (0, 10), (1, 50)], [(0, 2600), (0, 10), (0, 5)],
+                                    [(1000, 1000), (0, 10), (0, 60)]])
+def test_ordered_refine_positions(cu, bounds):
+    """ar_refine (a5, positions out; refine_kernel: warp 0 resolves a tile's offset by look-back a
+    round later while the CTA refines the next one): ascending exact positions equal to the oracle's,
+    up to ~3000 tiles of 2048 candidates (several rounds of the ~600-CTA grid)."""
+    from paper_conf_icde_pirkmk14_b200 import _ar
+    n = 6_000_001
+    c = datagen.q6_columns(95, 1.0, n=n)
+    b = bounds or Q6
+    los, his = [x[0] for x in b], [x[1] for x in b]
+    cols = [cu.BWDColumn(c["shipdate"], 24), cu.BWDColumn(c["discount"], 32), cu.BWDColumn(c["quantity"], 32)]
+    preds = list(zip(cols, los, his))
+    cands = cu.CandidateList(n)
+    cu.approx_select(preds, cands, cu.Workspace(_ar.ar_select_ws_bytes(n)), carry=True)
+    out = cu.PositionList(n)
+    cu.refine(cands, preds, out, cu.Workspace(_ar.ar_refine_ws_bytes(n)))
+    torch.cuda.synchronize()
+    assert _ar.ar_last_scan_kernel() == "refine_kernel"
+    ref_pos, ref_cnt, _ = oracle.select_sum([c["shipdate"], c["discount"], c["quantity"]], los, his)
+    assert out.count() == ref_cnt
+    assert np.array_equal(out.positions(), ref_pos)
