@@ -252,10 +252,15 @@ size_t ar_select_ws_bytes(int64_t n);
  * major ranges cand = [lo>>k, hi>>k] (bucket intersects [lo,hi]) and
  * def = [ceil(lo/2^k), floor((hi+1)/2^k) - 1] (bucket inside [lo,hi]), with
  * b = base subtracted first (DESIGN "Readings").  Device side
- * (a3): one pass over the packed majors, stable compaction (per-tile warp
- * ballot / popc and block scan into tile slices, then one compaction launch
- * that places every slice at the prefix of the earlier tiles' counts) into
- * out->pos / out->aux / *out->count.  At least one predicate is required (a
+ * (a3): one pass over the packed majors with stable compaction into
+ * out->pos / out->aux / *out->count: per tile a popc + block scan, and either
+ * (select_rr_kernel, the default for wide sparse scans) the tile's entries
+ * written once at the offset a decoupled look-back over the per-tile counts
+ * gives, or (select_tile_kernel) tile slices in the workspace that one
+ * compaction launch places at the prefix of the earlier tiles' counts.  The
+ * workspace holds the per-tile counts / status words and the slices; the
+ * one-kernel select launches cooperatively (AR_ERR_CUDA if its grid cannot be
+ * co-resident).  At least one predicate is required (a
  * scan needs a column; [0, 2^32 - 1] keeps every row).  A predicate with
  * lo > hi makes the result empty (AR_OK).
  * Errors: AR_ERR_INVALID (npred < 1 or > AR_MAX_PRED, null / mismatched columns,
