@@ -639,7 +639,7 @@ __device__ __forceinline__ void factor_batch8(const RefParams& P, const AggCol& 
 
 constexpr int kGroupRepMax = 256;   // up to this many groups every warp gets its own table
 
-__global__ void __launch_bounds__(kRefThreads) group_sum_kernel(const __grid_constant__ GroupParams P) {
+__global__ void __launch_bounds__(kRefThreads, 2) group_sum_kernel(const __grid_constant__ GroupParams P) {
     extern __shared__ unsigned long long gtab_all[];   // per table: [ngroups] sums, [ngroups] counts
     const int G = P.ngroups;
     // few groups: one table per warp, so the atomics of a hot group contend within a warp only
@@ -657,7 +657,7 @@ __global__ void __launch_bounds__(kRefThreads) group_sum_kernel(const __grid_con
         uint32_t valid = 0;
 #pragma unroll
         for (int i = 0; i < 8; ++i) valid |= (j0 + i < (uint64_t)count ? 1u : 0u) << i;
-        const uint32_t keep = refine_batch8(P.r, pos, aux, valid);
+        const uint32_t keep = refine_batch8<true>(P.r, pos, aux, valid);   // 8-plane residual halves together
         if (!keep) continue;
         uint32_t key[8];
         if (P.gids) {   // ids of the approximation group operator, aligned with the candidates
