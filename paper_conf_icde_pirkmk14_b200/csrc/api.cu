@@ -646,9 +646,11 @@ ar_status ar_approx_select(const ar_pred* preds, int32_t npred, int32_t flags, a
     }
     out->appr_bits = carry ? (int32_t)std::max<uint32_t>(abits, 1) : 0;
     cudaStream_t s = (cudaStream_t)stream;
-    AR_TRY_CUDA(cudaMemsetAsync(out->count, 0, sizeof(int64_t), s));
     g_last_scan = "";
-    if (empty || n == 0) return AR_OK;
+    if (empty || n == 0) {   // no kernel runs: the count is set here (otherwise the kernels write it)
+        AR_TRY_CUDA(cudaMemsetAsync(out->count, 0, sizeof(int64_t), s));
+        return AR_OK;
+    }
     P.carry = carry ? 1 : 0;
     P.out_pos = out->pos;
     P.out_aux = out->aux;
@@ -980,8 +982,12 @@ ar_status ar_refine_sum(const ar_cands* in, const ar_pred* preds, int32_t npred,
         if (ok) P.fast_k = (int32_t)P.p[P.fast_chk].k;
     }
     cudaStream_t s = (cudaStream_t)stream;
-    if (out_sum_dev) AR_TRY_CUDA(cudaMemsetAsync(out_sum_dev, 0, sizeof(int64_t), s));
-    if (out_count_dev) AR_TRY_CUDA(cudaMemsetAsync(out_count_dev, 0, sizeof(int64_t), s));
+    if (out_sum_dev && out_count_dev == out_sum_dev + 1) {   // adjacent outputs: one memset node
+        AR_TRY_CUDA(cudaMemsetAsync(out_sum_dev, 0, 2 * sizeof(int64_t), s));
+    } else {
+        if (out_sum_dev) AR_TRY_CUDA(cudaMemsetAsync(out_sum_dev, 0, sizeof(int64_t), s));
+        if (out_count_dev) AR_TRY_CUDA(cudaMemsetAsync(out_count_dev, 0, sizeof(int64_t), s));
+    }
     const uint64_t max_tiles = ceil_div_u64((uint64_t)std::max<int64_t>(in->capacity, 0), ard::kRefTile);
     if (max_tiles == 0) return AR_OK;
     const int grid = (int)std::min<uint64_t>(max_tiles, (uint64_t)num_sms() * 8);
